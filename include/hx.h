@@ -1,0 +1,208 @@
+/*
+ * hx.h — C-ABI of libhx, the B200-native hot path of HetExchange (Chrysogelos et al.,
+ * PVLDB 12(5) 2019): the fused GPU pipeline that runs a Star Schema Benchmark query —
+ * scan lineorder → filter → probe k dimension hash tables → group-by aggregate — plus the
+ * operators that spread it over GPUs (router, mem-move, broadcast, union-router merge).
+ *
+ * Citations are PAPER.md line ranges (the paper's text) with the section they fall in.
+ * All entry points return an int status (HX_OK = 0, negative on error) and never throw;
+ * hx_last_error() returns a thread-local message for the last failure of this thread.
+ * Plain pointers and sizes only: no torch (or other framework) types cross this boundary.
+ * Device pointers are CUDA device (or UVA) addresses; `stream` arguments are cudaStream_t
+ * passed as void*. One hx_ctx drives ONE GPU (one process per GPU; §4.2
+ * "pipeline template ... instantiated" per device).
+ *
+ * Asynchrony: every call that launches device work enqueues it on the context stream and
+ * returns without synchronising, EXCEPT hx_ht_info, hx_merge_aggregates, hx_profile_read
+ * and hx_ht_broadcast (the latter waits for the HT size on the root), which synchronise
+ * that stream. Nothing on the path copies device results to the host before the merge.
+ */
+#ifndef HX_H
+#define HX_H
+#include <stddef.h>
+#include <stdint.h>
+
+#ifdef __cplusplus
+extern "C" {
+#endif
+
+/* ---- status codes ------------------------------------------------------------------- */
+enum {
+  HX_OK = 0,
+  HX_EINVAL = -1,        /* null / inconsistent argument                                   */
+  HX_ECUDA = -2,         /* a CUDA runtime call failed (message in hx_last_error)         */
+  HX_ENCCL = -3,         /* an NCCL call failed, or no communicator for a collective      */
+  HX_ENOMEM = -4,        /* device or pinned host allocation failed                        */
+  HX_ECAPACITY = -5,     /* group count beyond HX_MAX_GROUPS, or too many columns          */
+  HX_EDUPKEY = -6,       /* a dimension primary key occurs twice among the filtered rows   */
+  HX_EUNSUPPORTED = -7   /* a configuration this build does not implement                 */
+};
+const char* hx_last_error(void);
+
+/* ---- context (one GPU) ------------------------------------------------------------- */
+typedef struct hx_ctx hx_ctx;
+/* Binds CUDA device `device`. `stream` (cudaStream_t) is the stream all work is enqueued on;
+   NULL makes the library create a non-blocking stream it owns. *out owned by the library. */
+int hx_init(int device, void* stream, hx_ctx** out);
+int hx_finalize(hx_ctx* ctx);
+int hx_ctx_stream(hx_ctx* ctx, void** stream);
+/* Number of SMs and resident K1 CTAs per SM chosen for this device (for reporting). */
+int hx_ctx_info(hx_ctx* ctx, int* n_sms, int* k1_ctas_per_sm);
+
+/* ---- communicator (NCCL over NVLink/NVSwitch; one rank per GPU) ------------------- */
+/* The 128-byte ncclUniqueId, created on rank 0 and shipped to the others by the caller
+   (e.g. torch.distributed). hx_comm_init is collective over all `nranks` ranks. */
+int hx_comm_unique_id(void* id128);
+int hx_comm_init(hx_ctx* ctx, int nranks, int rank, const void* id128);
+int hx_comm_info(hx_ctx* ctx, int* rank, int* nranks);
+
+/* ---- router: segmenter + range / round-robin policy (§8(a) a2) ---------------------
+ * PAPER.md:469-473 §3.1 (the segmenter splits the input into block-shaped partitions; the
+ * router routes block handles to consumer instances while load-balancing)
+ * (round-robin/range policies), Listing 1 pipeline 6. A block handle is a
+ * row range plus the consumer it is routed to (handles, not data).
+ * Blocks are [b*block_rows, min((b+1)*block_rows, n_rows)); HX_POLICY_RANGE gives each part
+ * a contiguous run of whole blocks (balanced to within one block), HX_POLICY_ROUND_ROBIN
+ * routes block b to part b % n_parts. Invariant: the blocks are disjoint and cover
+ * [0, n_rows). n_rows may be 0 (no blocks). */
+enum { HX_POLICY_RANGE = 0, HX_POLICY_ROUND_ROBIN = 1 };
+typedef struct { int64_t row_begin, row_end; int32_t part; int32_t reserved; } hx_block;
+typedef struct hx_partition hx_partition;
+int hx_router_partition(int64_t n_rows, int n_parts, int64_t block_rows, int policy,
+                        hx_partition** out);
+/* *blocks points into library memory valid until hx_partition_free. */
+int hx_partition_info(const hx_partition* p, int64_t* n_blocks, const hx_block** blocks);
+/* Rows routed to `part` (sum of its blocks). */
+int hx_partition_rows(const hx_partition* p, int part, int64_t* n_rows);
+int hx_partition_free(hx_partition* p);
+
+/* ---- columns: mem-move into HBM (§8(a) a1) -----------------------------------------
+ * PAPER.md:500-520 §3.2 (mem-move moves each block to the consumer's memory, or only
+ * forwards the handle when the data is already local), §6.1 (tables
+ * partitioned over the GPUs; dimension columns broadcast to every GPU).
+ * A column is `n_rows` int32 values (SoA), identified by `col_id` (ssbgen.h column ids).
+ * `data` is a host or device (UVA) pointer, caller-owned, alive until the call's work
+ * completes (HX_PLACE_COPY) or for the table's lifetime (HX_PLACE_VIEW).
+ *   part == NULL   : all rows (replicated dimension tables).
+ *   part != NULL   : only the blocks the router gave to `part_index`, concatenated in
+ *                    block order (the rows this GPU owns).
+ *   HX_PLACE_COPY  : library-owned device columns (cudaMemcpyAsync on the ctx stream,
+ *                    H2D or D2D by UVA); base pointers 256-byte aligned.
+ *   HX_PLACE_VIEW  : no copy; every `data` must be device memory and the selected rows one
+ *                    contiguous range (always true for part == NULL).
+ *   HX_PLACE_HOST_PINNED : no copy; `data` must be page-locked host memory; K1 then streams
+ *                    blocks over PCIe through a device staging ring (mem-move, §8(a) a8).
+ * All columns of one table must have the same number of rows. At most HX_MAX_COLS. */
+enum { HX_PLACE_COPY = 0, HX_PLACE_VIEW = 1, HX_PLACE_HOST_PINNED = 2 };
+#define HX_MAX_COLS 16
+typedef struct { int32_t col_id; int32_t reserved; const int32_t* data; int64_t n_rows; } hx_col;
+typedef struct hx_table hx_table;
+int hx_load_columns(hx_ctx* ctx, const hx_col* cols, int n_cols, const hx_partition* part,
+                    int part_index, int placement, hx_table** out);
+int hx_table_info(const hx_table* t, int64_t* n_rows, int* n_cols);
+/* A view of rows [row_begin, row_end) of `t` (no copy; lifetime bounded by `t`). */
+int hx_table_slice(const hx_table* t, int64_t row_begin, int64_t row_end, hx_table** out);
+int hx_table_free(hx_table* t);
+
+/* ---- dimension filter + hash-table build (§8(a) a3, kernel K2) ----------------------
+ * PAPER.md:1160-1163 §6.1 (broadcast-hash-join plans: the build side is the filtered
+ * dimension), §4.3 (the hash table is operator state owned by the memory
+ * manager), PAPER.md:231-233 (build-phase atomics).
+ * Rows of `dim` passing the AND of `preds` (range lo <= v <= hi, or v IN in[0..n_in)) are
+ * inserted as key -> rank into an open-addressing table in HBM (linear probing, 8-byte
+ * slots {int32 key, int32 rank}, capacity the power of two >= 2*n_pass, min 16), built
+ * with warp-cooperative CAS inserts. If group_col >= 0 its values must lie in
+ * [group_lo, group_hi]; rank = position of the row's group code among the DISTINCT codes
+ * of the passing rows in ascending order (dense ranks; rank_to_code recovers the code).
+ * group_col < 0: membership only, rank 0, one rank.
+ * Asynchronous and sync-free: the passing count, capacity and rank count live on the
+ * device, so a query's builds, K1 and merge enqueue without a host round trip.
+ * Errors detected on the device (duplicate key among passing rows, group code out of
+ * range) are reported by hx_ht_info / hx_merge_aggregates as HX_EDUPKEY / HX_EINVAL. */
+enum { HX_PRED_RANGE = 0, HX_PRED_IN = 1 };
+typedef struct {
+  int32_t col_id;
+  int32_t kind;       /* HX_PRED_RANGE | HX_PRED_IN */
+  int32_t lo, hi;     /* RANGE: lo <= v <= hi (inclusive) */
+  int32_t n_in;       /* IN: 1..4 values */
+  int32_t in[4];
+} hx_pred;
+typedef struct hx_ht hx_ht;
+int hx_build_dim_ht(hx_ctx* ctx, const hx_table* dim, int32_t key_col, const hx_pred* preds,
+                    int n_preds, int32_t group_col, int32_t group_lo, int32_t group_hi,
+                    hx_ht** out);
+/* Synchronises, then reports the table: passing keys, slots in use, distinct group codes,
+   rank->code map (caller array of >= n_ranks entries, may be NULL) and HX_OK / the error
+   the build detected. Any out pointer may be NULL. */
+int hx_ht_info(hx_ht* ht, int64_t* n_keys, int64_t* n_slots, int32_t* n_ranks,
+               int32_t* rank_to_code);
+/* Mem-move broadcast of a built table from rank `root` to every rank (§8(a) a4;
+   PAPER.md:530-537 §3.2 multicast is mem-move's job). Collective: every
+   rank calls it; non-root ranks pass a table from hx_build_dim_ht over the same dimension
+   (any preds — its contents are replaced). Requires hx_comm_init. */
+int hx_ht_broadcast(hx_ctx* ctx, hx_ht* ht, int root);
+int hx_ht_free(hx_ht* ht);
+
+/* ---- fused scan → filter → probe×k → aggregate (§8(a) a5, kernel K1) ----------------
+ * PAPER.md:859-869 Listing 1 pipeline 9 (grid-stride unpack, predicate, thread-local
+ * accumulator, neighbourhood reduce, leader atomic add to the pipeline state),
+ * PAPER.md:919-926, 937-951 §4.1/Fig. 3 (GPU provider: grid-wide thread ids, worker-scoped
+ * atomics), §6.1 (SSB query shapes: 1, 3, 3, 4 joins), PAPER.md:240-244,
+ * 285-290 (fused pipelines, no materialisation).
+ * For every row of `fact`: all `preds` (fact columns) must hold; then for each join in
+ * array order the row's FK value is probed in hts[join_ht] (miss drops the row); the
+ * measure is  a (HX_AGG_SUM), a*b (HX_AGG_SUM_MUL) or a-b (HX_AGG_SUM_SUB), formed in
+ * int64; the group index is the mixed radix of the ranks of the joins listed in gdim_join
+ * (first = most significant). SUM (int64, two's complement, exact) and COUNT are added
+ * to the agg's group arrays. n_gdims == 0 gives one ungrouped total.
+ * The result accumulates into a NEW hx_agg (zeroed on the device first). Asynchronous. */
+enum { HX_AGG_SUM = 0, HX_AGG_SUM_MUL = 1, HX_AGG_SUM_SUB = 2 };
+#define HX_MAX_PREDS 3
+#define HX_MAX_JOINS 4
+#define HX_MAX_GDIMS 3
+#define HX_MAX_GROUPS (1 << 26)
+typedef struct {
+  int32_t n_preds;
+  hx_pred preds[HX_MAX_PREDS];           /* on fact columns (col_id = fact column id)     */
+  int32_t n_joins;
+  int32_t join_fk_col[HX_MAX_JOINS];     /* fact FK column id of each join                */
+  int32_t join_ht[HX_MAX_JOINS];         /* index into hts[]; probe order = array order   */
+  int32_t agg_op;                        /* HX_AGG_*                                       */
+  int32_t agg_a, agg_b;                  /* fact column ids of the measure operands        */
+  int32_t n_gdims;
+  int32_t gdim_join[HX_MAX_GDIMS];       /* joins whose ranks form the group key           */
+} hx_query_shape;
+typedef struct hx_agg hx_agg;
+int hx_pipeline_probe_agg(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* shape,
+                          hx_ht* const* hts, int n_hts, hx_agg** out);
+/* Accumulate another fact table (e.g. the next block of this GPU) into an existing agg. */
+int hx_pipeline_probe_agg_into(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* shape,
+                               hx_ht* const* hts, int n_hts, hx_agg* agg);
+
+/* ---- merge partial aggregates + finalize (§8(a) a6, a7) ----------------------------
+ * PAPER.md:485-488 §3.1 (a local reduction per device, then the union router gathers the
+ * partial results into one global aggregation), PAPER.md:927-936 (pipelines 8, 3 → 2).
+ * With a communicator of > 1 ranks the per-GPU group arrays are summed with
+ * ncclAllReduce (root < 0) or ncclReduce to `root` over NVLink; then the (merged) arrays
+ * are copied to the host and finalised: groups with count 0 are dropped (a query without
+ * GROUP BY always yields its one row), and each group index is decoded back to the
+ * dictionary codes of its group columns (keys[i*n_gdims + g], in gdim order).
+ * Writes at most `cap` rows; *n_rows = rows produced (HX_ECAPACITY if > cap, with
+ * *n_rows set to the required count). Synchronises. Non-root ranks of a reduce get
+ * *n_rows = 0. Returns HX_EDUPKEY / HX_EINVAL if a build it depends on failed. */
+int hx_merge_aggregates(hx_ctx* ctx, hx_agg* agg, int root, int64_t* sums, int64_t* counts,
+                        int32_t* keys, int64_t cap, int64_t* n_rows);
+int hx_agg_free(hx_agg* agg);
+
+/* ---- measurement ------------------------------------------------------------------
+ * When enabled, CUDA events bracket every K1 launch on the ctx stream. hx_profile_read
+ * synchronises and returns the summed K1 device time (ms), launch count and algorithmic
+ * bytes (rows x 4 B x distinct fact columns the shape references), then resets if asked. */
+int hx_profile_enable(hx_ctx* ctx, int on);
+int hx_profile_read(hx_ctx* ctx, double* k1_ms, int64_t* k1_launches, int64_t* k1_bytes,
+                    int reset);
+
+#ifdef __cplusplus
+}
+#endif
+#endif /* HX_H */

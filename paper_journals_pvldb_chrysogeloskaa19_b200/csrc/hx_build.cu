@@ -1,0 +1,255 @@
+// hx_build.cu — K2: dimension filter + open-addressing hash-table build (§8(a) a3).
+//
+// PAPER.md:1160-1163 §6.1: Proteus runs SSB with broadcast-hash-join plans; the build side
+// of each join is the filtered dimension. PAPER.md:1019-1022 §4.3: the hash table is
+// operator state allocated by the device-local memory manager. PAPER.md:231-233: the build
+// phase needs atomics. The paper does not describe its table layout (R15), so
+// this is a B200-first design:
+//   * one HBM allocation per table (header, dense-rank maps, slot array) so the fused
+//     probe kernel sees one L2-friendly region;
+//   * 8-byte slots {int32 key, int32 rank} written with one 64-bit CAS, linear probing,
+//     capacity = next pow2 >= 2 * passing rows (load factor <= 0.5), Fibonacci hashing;
+//   * sizing happens ON THE DEVICE (count kernel -> rank kernel writes log2cap), so a query
+//     enqueues build -> probe -> merge with no host round trip (CUDA-graph capturable);
+//   * inserts are warp-cooperative: the warp takes one pending key at a time and inspects
+//     32 consecutive slots with one coalesced load + ballot, CAS-ing the first empty one.
+#include <cub/block/block_scan.cuh>
+
+#include "hx_internal.cuh"
+
+namespace hx {
+
+namespace {
+
+constexpr unsigned kFull = 0xFFFFFFFFu;
+
+struct BuildParams {
+  const int32_t* key;
+  const int32_t* group;                // nullptr: membership only
+  const int32_t* pcol[HX_MAX_PREDS];
+  DevPred preds[HX_MAX_PREDS];
+  int32_t n_preds;
+  int64_t n_rows;
+  HtHeader* hdr;
+  int32_t* c2r;
+  int32_t* r2c;
+  unsigned long long* slots;
+  int32_t group_lo, domain, max_log2cap;
+};
+
+__device__ __forceinline__ bool row_pass(const BuildParams& p, int64_t i) {
+  bool ok = true;
+#pragma unroll
+  for (int k = 0; k < HX_MAX_PREDS; ++k)
+    if (k < p.n_preds) ok = ok && pred_pass(p.preds[k], __ldg(p.pcol[k] + i));
+  return ok;
+}
+
+// Count passing rows; flag the group codes present among them.
+__global__ void k2_filter_mark(BuildParams p) {
+  int local = 0;
+  const int64_t stride = (int64_t)gridDim.x * blockDim.x;
+  for (int64_t i = (int64_t)blockIdx.x * blockDim.x + threadIdx.x; i < p.n_rows; i += stride) {
+    if (!row_pass(p, i)) continue;
+    ++local;
+    if (p.group) {
+      int32_t code = __ldg(p.group + i) - p.group_lo;
+      if (code < 0 || code >= p.domain)
+        atomicExch(&p.hdr->error, HX_EINVAL);
+      else
+        p.c2r[code] = 1;  // benign race: every writer stores 1
+    }
+  }
+#pragma unroll
+  for (int o = 16; o > 0; o >>= 1) local += __shfl_xor_sync(kFull, local, o);
+  if ((threadIdx.x & 31) == 0 && local) atomicAdd(&p.hdr->n_keys, local);
+}
+
+// One CTA: dense ranks of the present group codes (exclusive scan of the flags), rank->code
+// map, and the table capacity from the passing count.
+__global__ void k2_rank(BuildParams p) {
+  using Scan = cub::BlockScan<int, 1024>;
+  __shared__ typename Scan::TempStorage tmp;
+  __shared__ int running;
+  if (threadIdx.x == 0) running = 0;
+  __syncthreads();
+  if (p.group) {
+    for (int base = 0; base < p.domain; base += 1024) {
+      int code = base + threadIdx.x;
+      int flag = code < p.domain ? p.c2r[code] : 0;
+      int excl, total;
+      Scan(tmp).ExclusiveSum(flag, excl, total);
+      int rank = running + excl;
+      if (flag) {
+        p.c2r[code] = rank;
+        p.r2c[rank] = code + p.group_lo;
+      }
+      __syncthreads();
+      if (threadIdx.x == 0) running += total;
+      __syncthreads();
+    }
+  }
+  if (threadIdx.x == 0) {
+    int n = p.hdr->n_keys;
+    int lg = kMinLog2Cap;
+    while (lg < p.max_log2cap && (1ll << lg) < 2ll * n) ++lg;
+    p.hdr->log2cap = lg;
+    p.hdr->n_ranks = p.group ? running : 1;
+    p.hdr->max_log2cap = p.max_log2cap;
+    p.hdr->group_lo = p.group_lo;
+    p.hdr->domain = p.domain;
+  }
+}
+
+// Empty the slots in use (the capacity is only known on the device).
+__global__ void k2_clear(BuildParams p) {
+  const int64_t cap = 1ll << p.hdr->log2cap;
+  const int64_t stride = (int64_t)gridDim.x * blockDim.x;
+  for (int64_t i = (int64_t)blockIdx.x * blockDim.x + threadIdx.x; i < cap; i += stride)
+    p.slots[i] = kEmptySlot;
+}
+
+// Warp-cooperative linear-probing insert of every passing row.
+__global__ void k2_insert(BuildParams p) {
+  const int lane = threadIdx.x & 31;
+  const int log2cap = p.hdr->log2cap;
+  const uint32_t mask = (1u << log2cap) - 1u;
+  const int64_t stride = (int64_t)gridDim.x * blockDim.x;
+  for (int64_t base = (int64_t)blockIdx.x * blockDim.x + (threadIdx.x & ~31); base < p.n_rows;
+       base += stride) {
+    const int64_t i = base + lane;
+    bool has = i < p.n_rows && row_pass(p, i);
+    int32_t key = 0, rank = 0;
+    if (has) {
+      key = __ldg(p.key + i);
+      if (p.group) {
+        int32_t code = __ldg(p.group + i) - p.group_lo;
+        has = code >= 0 && code < p.domain;  // out-of-range codes were flagged by the filter
+        if (has) rank = p.c2r[code];
+      }
+    }
+    unsigned pending = __ballot_sync(kFull, has);
+    while (pending) {
+      const int leader = __ffs(pending) - 1;
+      pending &= pending - 1;
+      const int32_t k = __shfl_sync(kFull, key, leader);
+      const int32_t r = __shfl_sync(kFull, rank, leader);
+      const unsigned long long packed =
+          ((unsigned long long)(uint32_t)r << 32) | (unsigned long long)(uint32_t)k;
+      const uint32_t home = ht_home(k, log2cap);
+      bool done = false;
+      for (uint32_t off = 0; !done && off <= mask; off += 32) {
+        const uint32_t s = (home + off + lane) & mask;
+        const unsigned long long v = __ldcg(p.slots + s);
+        unsigned mk = __ballot_sync(kFull, v != kEmptySlot && (int32_t)(uint32_t)v == k);
+        unsigned any = mk | __ballot_sync(kFull, v == kEmptySlot);
+        while (any) {
+          const int f = __ffs(any) - 1;
+          if (mk & (1u << f)) {  // the key is already present: duplicate primary key
+            if (lane == 0) atomicExch(&p.hdr->error, HX_EDUPKEY);
+            done = true;
+            break;
+          }
+          unsigned long long old = 0;
+          if (lane == f) old = atomicCAS(p.slots + ((home + off + f) & mask), kEmptySlot, packed);
+          old = __shfl_sync(kFull, old, f);
+          if (old == kEmptySlot) {
+            done = true;
+            break;
+          }
+          if ((int32_t)(uint32_t)old == k) {  // a concurrent insert of the same key won
+            if (lane == 0) atomicExch(&p.hdr->error, HX_EDUPKEY);
+            done = true;
+            break;
+          }
+          any &= ~(1u << f);  // taken by another key: try the next free slot of the window
+        }
+      }
+    }
+  }
+}
+
+int ceil_log2(int64_t x) {
+  int l = 0;
+  while ((1ll << l) < x) ++l;
+  return l;
+}
+
+}  // namespace
+
+int build_dim_ht(hx_ctx* ctx, const hx_table* dim, int32_t key_col, const hx_pred* preds,
+                 int n_preds, int32_t group_col, int32_t group_lo, int32_t group_hi,
+                 hx_ht** out) {
+  HX_REQUIRE(ctx && dim && out, HX_EINVAL, "hx_build_dim_ht: null argument");
+  HX_REQUIRE(n_preds >= 0 && n_preds <= HX_MAX_PREDS && (n_preds == 0 || preds), HX_EINVAL,
+             "hx_build_dim_ht: bad predicate list");
+  HX_REQUIRE(dim->placement != HX_PLACE_HOST_PINNED, HX_EUNSUPPORTED,
+             "hx_build_dim_ht: dimension tables must be device resident");
+  HX_REQUIRE(dim->n_rows < (1ll << 30), HX_ECAPACITY, "hx_build_dim_ht: dimension too large");
+  BuildParams p{};
+  p.key = table_col(dim, key_col);
+  HX_REQUIRE(table_has_col(dim, key_col), HX_EINVAL, "hx_build_dim_ht: key column not in table");
+  p.n_preds = n_preds;
+  for (int k = 0; k < n_preds; ++k) {
+    p.pcol[k] = table_col(dim, preds[k].col_id);
+    HX_REQUIRE(table_has_col(dim, preds[k].col_id), HX_EINVAL, "hx_build_dim_ht: predicate column not in table");
+    HX_REQUIRE(preds[k].kind == HX_PRED_RANGE ||
+                   (preds[k].kind == HX_PRED_IN && preds[k].n_in >= 1 && preds[k].n_in <= 4),
+               HX_EINVAL, "hx_build_dim_ht: bad predicate");
+    p.preds[k] = DevPred{k, preds[k].kind, preds[k].lo, preds[k].hi, preds[k].n_in,
+                         {preds[k].in[0], preds[k].in[1], preds[k].in[2], preds[k].in[3]}};
+  }
+  int64_t domain = 1;
+  if (group_col >= 0) {
+    p.group = table_col(dim, group_col);
+    HX_REQUIRE(table_has_col(dim, group_col), HX_EINVAL, "hx_build_dim_ht: group column not in table");
+    HX_REQUIRE(group_hi >= group_lo && (int64_t)group_hi - group_lo < (1 << 24), HX_EINVAL,
+               "hx_build_dim_ht: bad group code range");
+    domain = (int64_t)group_hi - group_lo + 1;
+  }
+  p.n_rows = dim->n_rows;
+  p.group_lo = group_lo;
+  p.domain = (int32_t)domain;
+  p.max_log2cap = std::max(kMinLog2Cap, ceil_log2(2 * std::max<int64_t>(dim->n_rows, 1)));
+
+  hx_ht* ht = new hx_ht();
+  ht->ctx = ctx;
+  ht->domain = (int32_t)domain;
+  ht->group_lo = group_lo;
+  ht->has_group = group_col >= 0;
+  ht->max_log2cap = p.max_log2cap;
+  ht->dim_rows = dim->n_rows;
+  const size_t maps = (sizeof(HtHeader) + 2 * domain * sizeof(int32_t) + 255) & ~size_t(255);
+  ht->bytes = maps + (size_t(1) << p.max_log2cap) * sizeof(unsigned long long);
+  cudaError_t e = cudaMallocAsync(&ht->base, ht->bytes, ctx->stream);
+  if (e != cudaSuccess) {
+    delete ht;
+    return cuda_fail(e, "cudaMallocAsync(hash table)", __FILE__, __LINE__);
+  }
+  ht->hdr = reinterpret_cast<HtHeader*>(ht->base);
+  ht->code_to_rank = reinterpret_cast<int32_t*>(ht->hdr + 1);
+  ht->rank_to_code = ht->code_to_rank + domain;
+  ht->slots = reinterpret_cast<unsigned long long*>(static_cast<char*>(ht->base) + maps);
+  p.hdr = ht->hdr;
+  p.c2r = ht->code_to_rank;
+  p.r2c = ht->rank_to_code;
+  p.slots = ht->slots;
+  *out = ht;
+
+  HX_CK(cudaMemsetAsync(ht->base, 0, sizeof(HtHeader) + domain * sizeof(int32_t), ctx->stream));
+  const int64_t want = (dim->n_rows + 255) / 256;
+  const int grid = (int)std::max<int64_t>(1, std::min<int64_t>(want, (int64_t)ctx->n_sms * 8));
+  k2_filter_mark<<<grid, 256, 0, ctx->stream>>>(p);
+  HX_CK_LAUNCH("k2_filter_mark");
+  k2_rank<<<1, 1024, 0, ctx->stream>>>(p);
+  HX_CK_LAUNCH("k2_rank");
+  const int64_t slots_max = int64_t(1) << p.max_log2cap;
+  const int cgrid = (int)std::min<int64_t>((slots_max + 255) / 256, (int64_t)ctx->n_sms * 16);
+  k2_clear<<<cgrid, 256, 0, ctx->stream>>>(p);
+  HX_CK_LAUNCH("k2_clear");
+  k2_insert<<<grid, 256, 0, ctx->stream>>>(p);
+  HX_CK_LAUNCH("k2_insert");
+  return HX_OK;
+}
+
+}  // namespace hx

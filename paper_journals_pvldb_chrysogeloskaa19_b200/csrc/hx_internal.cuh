@@ -1,0 +1,152 @@
+// hx_internal.cuh — shared definitions of libhx (the product path). Not part of the C-ABI.
+#pragma once
+#include <cuda_runtime.h>
+#include <nccl.h>
+#include <stdint.h>
+
+#include <string>
+#include <vector>
+
+#include "hx.h"
+
+namespace hx {
+
+// ---- error plumbing (hx_last_error) ----------------------------------------------------
+void set_error(const std::string& msg);
+int fail(int code, const std::string& msg);
+int cuda_fail(cudaError_t e, const char* what, const char* file, int line);
+
+#define HX_CK(call)                                                   \
+  do {                                                                \
+    cudaError_t _e = (call);                                          \
+    if (_e != cudaSuccess) return ::hx::cuda_fail(_e, #call, __FILE__, __LINE__); \
+  } while (0)
+#define HX_CK_LAUNCH(what) HX_CK(cudaGetLastError())
+#define HX_REQUIRE(cond, code, msg) \
+  do {                              \
+    if (!(cond)) return ::hx::fail((code), (msg)); \
+  } while (0)
+
+// ---- hash table layout (one device allocation per table) ------------------------------
+// [HtHeader | code_to_rank[domain] | rank_to_code[domain] | pad to 256 | slots[max_cap]]
+constexpr uint64_t kEmptySlot = 0xFFFFFFFFFFFFFFFFull;
+constexpr int kMinLog2Cap = 4;
+
+struct HtHeader {
+  int32_t log2cap;   // device-written by the rank kernel
+  int32_t n_keys;    // passing dimension rows (atomic counter in the filter kernel)
+  int32_t n_ranks;   // distinct group codes among passing rows (1 if no group column)
+  int32_t error;     // 0 ok, HX_EDUPKEY, HX_EINVAL (group code out of range)
+  int32_t max_log2cap;
+  int32_t group_lo;
+  int32_t domain;
+  int32_t n_inserted;
+};
+
+// Multiplicative (Fibonacci) hashing: the top log2cap bits of key * 2^32/phi.
+__host__ __device__ __forceinline__ uint32_t ht_home(int32_t key, int log2cap) {
+  return ((uint32_t)key * 2654435769u) >> (32 - log2cap);
+}
+
+// Device-side predicate (a copy of hx_pred with the column resolved to a pointer or a
+// staged-column index).
+struct DevPred {
+  int32_t c;      // column index (table column or staged column)
+  int32_t kind;
+  int32_t lo, hi;
+  int32_t n_in;
+  int32_t in[4];
+};
+
+__device__ __forceinline__ bool pred_pass(const DevPred& p, int32_t v) {
+  if (p.kind == HX_PRED_RANGE) return v >= p.lo && v <= p.hi;
+  bool r = false;
+#pragma unroll
+  for (int i = 0; i < 4; ++i) r |= (i < p.n_in) && v == p.in[i];
+  return r;
+}
+
+}  // namespace hx
+
+// ---- library objects (opaque in hx.h) ----------------------------------------------------
+struct hx_ctx {
+  int device = 0;
+  cudaStream_t stream = nullptr;
+  bool own_stream = false;
+  int n_sms = 0;
+  int k1_ctas_per_sm = 0;
+  ncclComm_t comm = nullptr;
+  int rank = 0, nranks = 1;
+  // K1 profiling: event pairs around each launch
+  bool prof_on = false;
+  std::vector<std::pair<cudaEvent_t, cudaEvent_t>> prof_events;
+  std::vector<cudaEvent_t> event_pool;
+  int64_t prof_launches = 0, prof_bytes = 0;
+  double prof_ms = 0.0;
+};
+
+struct hx_partition {
+  int64_t n_rows = 0, block_rows = 0;
+  int n_parts = 0, policy = 0;
+  std::vector<hx_block> blocks;
+};
+
+struct hx_table {
+  hx_ctx* ctx = nullptr;
+  int n_cols = 0;
+  int32_t col_id[HX_MAX_COLS];
+  int32_t* dev[HX_MAX_COLS];       // device (or pinned host) base of each column
+  int64_t n_rows = 0;
+  int placement = HX_PLACE_COPY;
+  bool owned = false;              // columns allocated by the library
+  const hx_table* parent = nullptr;
+};
+
+struct hx_ht {
+  hx_ctx* ctx = nullptr;
+  void* base = nullptr;            // the single device allocation
+  size_t bytes = 0;
+  hx::HtHeader* hdr = nullptr;
+  int32_t* code_to_rank = nullptr;
+  int32_t* rank_to_code = nullptr;
+  unsigned long long* slots = nullptr;
+  int32_t max_log2cap = 0;
+  int32_t domain = 1;              // group code range size (1 when no group column)
+  int32_t group_lo = 0;
+  bool has_group = false;
+  int64_t dim_rows = 0;
+};
+
+struct hx_agg {
+  hx_ctx* ctx = nullptr;
+  void* base = nullptr;
+  unsigned long long* sums = nullptr;   // [cap_groups]
+  unsigned long long* cnts = nullptr;   // [cap_groups]
+  struct AggMeta* meta = nullptr;       // device
+  int64_t cap_groups = 1;               // host-known upper bound of n_groups
+  int n_gdims = 0;
+  const hx_ht* gdim_ht[HX_MAX_GDIMS] = {nullptr, nullptr, nullptr};
+  std::vector<const hx_ht*> deps;       // every HT the pipeline probed (error check)
+};
+
+// Device-computed group layout of one pipeline (written by the prepare kernel).
+struct AggMeta {
+  long long n_groups;
+  int32_t jstride[HX_MAX_JOINS];   // per join: stride of its rank in the group index (0 = none)
+  int32_t n_ranks[HX_MAX_GDIMS];
+  int32_t error;
+  int32_t pad;
+};
+
+namespace hx {
+// launchers implemented in hx_build.cu / hx_probe.cu
+int build_dim_ht(hx_ctx* ctx, const hx_table* dim, int32_t key_col, const hx_pred* preds,
+                 int n_preds, int32_t group_col, int32_t group_lo, int32_t group_hi,
+                 hx_ht** out);
+int probe_agg(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* shape,
+              hx_ht* const* hts, int n_hts, hx_agg* agg, bool fresh);
+int k1_occupancy(hx_ctx* ctx);
+const int32_t* table_col(const hx_table* t, int32_t col_id);
+bool table_has_col(const hx_table* t, int32_t col_id);
+cudaEvent_t pooled_event(hx_ctx* ctx);
+}  // namespace hx

@@ -1,0 +1,568 @@
+// hx_probe.cu — K1: the fused scan -> filter -> probe x k -> group-by aggregate pipeline
+// (§8(a) a5), the one hot loop of HetExchange's GPU execution of an SSB query.
+//
+// What it computes follows Listing 1 pipeline 9: every GPU thread walks
+// its share of the block (unpack), evaluates the predicate (filter), accumulates into a
+// thread-local value, reduces over its neighbourhood and the neighbourhood leader adds the
+// result to the pipeline state with one atomic (reduce; Fig. 3). SSB
+// pipelines add the broadcast-hash-join probes between filter and reduce
+// and a GROUP BY (the paper does not describe its group-by; R17).
+//
+// How (B200-first, not the paper's 2019 LLVM-generated sm_61 code):
+//   * persistent CTAs (grid = SMs x resident CTAs), each with one PRODUCER warp that
+//     streams lineorder tiles (T rows x the query's columns) from HBM into a shared-memory
+//     ring with cp.async.bulk (the TMA bulk-copy engine) completing on mbarriers, L2
+//     evict-first; and 8 CONSUMER warps that process a tile while the next S-1 are in
+//     flight (mem-move's "prefetch to the consumer's local memory", done
+//     at tile granularity inside the kernel);
+//   * each consumer thread owns R rows of the tile (strided by 256 -> conflict-free LDS) and
+//     runs the pipeline stage-wise across them: predicates, then for each join the R
+//     hash probes are issued together (R independent L2 loads in flight) before any is
+//     checked; rows die as soon as a predicate or probe fails;
+//   * hash tables are read with L2 evict-last hints so the scan does not evict them;
+//   * GROUP BY: a dense per-CTA shared-memory table (int64 SUM, int32 COUNT) indexed by the
+//     mixed radix of the probed dimensions' dense ranks, flushed with one global atomic per
+//     non-empty group per CTA; ungrouped queries reduce warp -> CTA -> one global atomic.
+#include <algorithm>
+
+#include "hx_internal.cuh"
+
+namespace hx {
+
+namespace {
+
+constexpr unsigned kFull = 0xFFFFFFFFu;
+constexpr int kConsumerWarps = 8;
+constexpr int kConsumers = kConsumerWarps * 32;
+constexpr int kThreads = kConsumers + 32;  // + one producer warp
+constexpr int kRowsPerThread = 8;          // R
+constexpr int kTileRows = kConsumers * kRowsPerThread;  // T = 2048
+constexpr int kMaxStageCols = 8;
+constexpr int kSmemGroups = 1024;          // per-CTA group table capacity
+
+struct JoinDev {
+  int32_t c;                               // staged column of the FK
+  const unsigned long long* slots;
+  const HtHeader* hdr;
+};
+
+struct K1Params {
+  const int32_t* col[kMaxStageCols];       // staged fact columns (table base + head offset)
+  int32_t n_cols;
+  int32_t stages;
+  int64_t n_rows;                          // rows after the head
+  int64_t n_tiles;
+  const int32_t* head_col[kMaxStageCols];  // misaligned head rows (read directly)
+  int32_t head_rows;                       // 0..3
+  int32_t n_preds;
+  DevPred preds[HX_MAX_PREDS];
+  JoinDev joins[HX_MAX_JOINS];
+  int32_t agg_op, agg_a, agg_b;
+  const AggMeta* meta;
+  unsigned long long* g_sum;
+  unsigned long long* g_cnt;
+  int32_t smem_groups;                     // 0 for ungrouped instances
+};
+
+// ---- PTX helpers: mbarrier, bulk copy, cache policies -------------------------------------
+__device__ __forceinline__ uint32_t smem_u32(const void* p) {
+  return (uint32_t)__cvta_generic_to_shared(p);
+}
+__device__ __forceinline__ void mbar_init(uint64_t* bar, uint32_t count) {
+  asm volatile("mbarrier.init.shared::cta.b64 [%0], %1;" ::"r"(smem_u32(bar)), "r"(count));
+}
+__device__ __forceinline__ void mbar_arrive_expect_tx(uint64_t* bar, uint32_t bytes) {
+  asm volatile("mbarrier.arrive.expect_tx.shared::cta.b64 _, [%0], %1;" ::"r"(smem_u32(bar)),
+               "r"(bytes)
+               : "memory");
+}
+__device__ __forceinline__ void mbar_arrive(uint64_t* bar) {
+  asm volatile("mbarrier.arrive.shared::cta.b64 _, [%0];" ::"r"(smem_u32(bar)) : "memory");
+}
+__device__ __forceinline__ void mbar_wait(uint64_t* bar, uint32_t parity) {
+  asm volatile(
+      "{\n"
+      ".reg .pred p;\n"
+      "WAIT_%=:\n"
+      "mbarrier.try_wait.parity.shared::cta.b64 p, [%0], %1;\n"
+      "@!p bra WAIT_%=;\n"
+      "}\n" ::"r"(smem_u32(bar)),
+      "r"(parity)
+      : "memory");
+}
+__device__ __forceinline__ uint64_t policy_evict_first() {
+  uint64_t pol;
+  asm volatile("createpolicy.fractional.L2::evict_first.b64 %0, 1.0;" : "=l"(pol));
+  return pol;
+}
+__device__ __forceinline__ uint64_t policy_evict_last() {
+  uint64_t pol;
+  asm volatile("createpolicy.fractional.L2::evict_last.b64 %0, 1.0;" : "=l"(pol));
+  return pol;
+}
+__device__ __forceinline__ void bulk_g2s(void* dst, const void* src, uint32_t bytes,
+                                         uint64_t* bar, uint64_t pol) {
+  asm volatile(
+      "cp.async.bulk.shared::cluster.global.mbarrier::complete_tx::bytes.L2::cache_hint"
+      " [%0], [%1], %2, [%3], %4;" ::"r"(smem_u32(dst)),
+      "l"(src), "r"(bytes), "r"(smem_u32(bar)), "l"(pol)
+      : "memory");
+}
+__device__ __forceinline__ unsigned long long ld_slot(const unsigned long long* p, uint64_t pol) {
+  unsigned long long v;
+  asm volatile("ld.global.nc.L2::cache_hint.u64 %0, [%1], %2;" : "=l"(v) : "l"(p), "l"(pol));
+  return v;
+}
+__device__ __forceinline__ void consumer_sync() {
+  asm volatile("bar.sync 1, %0;" ::"n"(kConsumers) : "memory");
+}
+
+__device__ __forceinline__ long long measure(int op, int32_t a, int32_t b) {
+  if (op == HX_AGG_SUM_MUL) return (long long)a * (long long)b;
+  if (op == HX_AGG_SUM_SUB) return (long long)a - (long long)b;
+  return (long long)a;
+}
+
+// Per-thread view of the join tables (loaded once per CTA).
+struct JoinState {
+  const unsigned long long* slots;
+  int32_t c;
+  int32_t log2cap;
+  uint32_t mask;
+  int32_t jstride;
+};
+
+// Process the rows {ctid + k*kConsumers : k < R, row < rows_valid} of one staged tile whose
+// column c, row r is at sbase[c * stride + r].
+template <int NJ, bool GROUPED>
+__device__ __forceinline__ void process_tile(const K1Params& p, const JoinState (&js)[HX_MAX_JOINS],
+                                             const int32_t* sbase, int stride, int rows_valid,
+                                             int ctid, uint64_t pol_last, bool smem_table,
+                                             unsigned long long* s_sum, uint32_t* s_cnt,
+                                             long long& acc_sum, long long& acc_cnt) {
+  uint32_t alive = 0;
+#pragma unroll
+  for (int k = 0; k < kRowsPerThread; ++k)
+    alive |= (uint32_t)(ctid + k * kConsumers < rows_valid) << k;
+  // filter: predicates on lineorder columns
+  for (int q = 0; q < p.n_preds; ++q) {
+    const DevPred& pr = p.preds[q];
+    const int32_t* sc = sbase + pr.c * stride + ctid;
+#pragma unroll
+    for (int k = 0; k < kRowsPerThread; ++k)
+      if ((alive >> k) & 1u)
+        if (!pred_pass(pr, sc[k * kConsumers])) alive &= ~(1u << k);
+  }
+  int32_t gidx[kRowsPerThread];
+#pragma unroll
+  for (int k = 0; k < kRowsPerThread; ++k) gidx[k] = 0;
+  // probe x k: the R probes of a join are issued before any result is inspected
+#pragma unroll
+  for (int j = 0; j < NJ; ++j) {
+    if (!alive) break;
+    int32_t key[kRowsPerThread];
+    uint32_t h[kRowsPerThread];
+    const int32_t* sc = sbase + js[j].c * stride + ctid;
+#pragma unroll
+    for (int k = 0; k < kRowsPerThread; ++k) {
+      key[k] = ((alive >> k) & 1u) ? sc[k * kConsumers] : 0;
+      h[k] = ht_home(key[k], js[j].log2cap);
+    }
+    uint32_t pending = alive;
+    while (pending) {
+      unsigned long long v[kRowsPerThread];
+#pragma unroll
+      for (int k = 0; k < kRowsPerThread; ++k)
+        v[k] = ((pending >> k) & 1u) ? ld_slot(js[j].slots + h[k], pol_last) : 0ull;
+#pragma unroll
+      for (int k = 0; k < kRowsPerThread; ++k) {
+        if (!((pending >> k) & 1u)) continue;
+        if (v[k] == kEmptySlot) {  // miss: the row has no partner in this dimension
+          alive &= ~(1u << k);
+          pending &= ~(1u << k);
+        } else if ((int32_t)(uint32_t)v[k] == key[k]) {
+          gidx[k] += (int32_t)(v[k] >> 32) * js[j].jstride;
+          pending &= ~(1u << k);
+        } else {
+          h[k] = (h[k] + 1u) & js[j].mask;
+        }
+      }
+    }
+  }
+  // reduce
+  const int32_t* sa = sbase + p.agg_a * stride + ctid;
+  const int32_t* sb = sbase + p.agg_b * stride + ctid;
+#pragma unroll
+  for (int k = 0; k < kRowsPerThread; ++k) {
+    if (!((alive >> k) & 1u)) continue;
+    const long long m = measure(p.agg_op, sa[k * kConsumers], sb[k * kConsumers]);
+    if (GROUPED) {
+      if (smem_table) {
+        atomicAdd(s_sum + gidx[k], (unsigned long long)m);
+        atomicAdd(s_cnt + gidx[k], 1u);
+      } else {
+        atomicAdd(p.g_sum + gidx[k], (unsigned long long)m);
+        atomicAdd(p.g_cnt + gidx[k], 1ull);
+      }
+    } else {
+      acc_sum += m;
+      acc_cnt += 1;
+    }
+  }
+}
+
+template <int NJ, bool GROUPED>
+__global__ void __launch_bounds__(kThreads) k1_probe_agg(const __grid_constant__ K1Params p) {
+  extern __shared__ __align__(128) unsigned char smem[];
+  uint64_t* full = reinterpret_cast<uint64_t*>(smem);
+  uint64_t* empty = full + p.stages;
+  long long* red = reinterpret_cast<long long*>(smem + 128);                // 2 x 8 warps
+  int32_t* headbuf = reinterpret_cast<int32_t*>(smem + 128 + 256);           // 8 cols x 4
+  unsigned long long* s_sum = reinterpret_cast<unsigned long long*>(smem + 512);
+  uint32_t* s_cnt = reinterpret_cast<uint32_t*>(s_sum + p.smem_groups);
+  const size_t table_bytes = ((size_t)p.smem_groups * 12 + 127) & ~size_t(127);
+  int32_t* stage0 = reinterpret_cast<int32_t*>(smem + 512 + table_bytes);
+  const int stage_elems = p.n_cols * kTileRows;
+
+  const int tid = threadIdx.x;
+  const int warp = tid >> 5;
+  if (tid == kConsumers) {
+    for (int s = 0; s < p.stages; ++s) {
+      mbar_init(full + s, 1);
+      mbar_init(empty + s, kConsumerWarps);
+    }
+    asm volatile("fence.mbarrier_init.release.cluster;" ::: "memory");
+  }
+  __syncthreads();
+
+  if (warp == kConsumerWarps) {
+    // ---------------- producer warp: stream tiles HBM -> smem ring ----------------
+    if ((tid & 31) == 0) {
+      const uint64_t pol = policy_evict_first();
+      int64_t k = 0;
+      for (int64_t t = blockIdx.x; t < p.n_tiles; t += gridDim.x, ++k) {
+        const int s = (int)(k % p.stages);
+        if (k >= p.stages) mbar_wait(empty + s, (uint32_t)(((k / p.stages) - 1) & 1));
+        const int64_t r0 = t * kTileRows;
+        const int64_t rows = std::min<int64_t>(kTileRows, p.n_rows - r0);
+        const uint32_t bytes = (uint32_t)(rows & ~int64_t(3)) * 4u;
+        mbar_arrive_expect_tx(full + s, bytes * p.n_cols);
+        if (bytes) {
+          int32_t* dst = stage0 + (size_t)s * stage_elems;
+          for (int c = 0; c < p.n_cols; ++c)
+            bulk_g2s(dst + c * kTileRows, p.col[c] + r0, bytes, full + s, pol);
+        }
+      }
+    }
+    return;
+  }
+
+  // ---------------- consumer warps ----------------
+  const int ctid = tid;  // 0..255
+  const uint64_t pol_last = policy_evict_last();
+  JoinState js[HX_MAX_JOINS];
+#pragma unroll
+  for (int j = 0; j < HX_MAX_JOINS; ++j) {
+    if (j < NJ) {
+      js[j].slots = p.joins[j].slots;
+      js[j].c = p.joins[j].c;
+      js[j].log2cap = p.joins[j].hdr->log2cap;
+      js[j].mask = (1u << js[j].log2cap) - 1u;
+      js[j].jstride = GROUPED ? p.meta->jstride[j] : 0;
+    } else {
+      js[j] = JoinState{nullptr, 0, kMinLog2Cap, 0u, 0};
+    }
+  }
+  const long long n_groups = GROUPED ? p.meta->n_groups : 1;
+  const bool smem_table = GROUPED && n_groups <= p.smem_groups;
+  if (smem_table) {
+    for (int g = ctid; g < n_groups; g += kConsumers) {
+      s_sum[g] = 0;
+      s_cnt[g] = 0;
+    }
+  }
+  long long acc_sum = 0, acc_cnt = 0;
+  // misaligned head rows (views at a row offset): CTA 0 reads them directly
+  if (blockIdx.x == 0 && p.head_rows > 0) {
+    if (ctid < p.head_rows)
+      for (int c = 0; c < p.n_cols; ++c) headbuf[c * 4 + ctid] = p.head_col[c][ctid];
+    consumer_sync();
+    process_tile<NJ, GROUPED>(p, js, headbuf, 4, p.head_rows, ctid, pol_last, smem_table, s_sum,
+                              s_cnt, acc_sum, acc_cnt);
+  }
+  consumer_sync();
+
+  int64_t k = 0;
+  for (int64_t t = blockIdx.x; t < p.n_tiles; t += gridDim.x, ++k) {
+    const int s = (int)(k % p.stages);
+    mbar_wait(full + s, (uint32_t)((k / p.stages) & 1));
+    int32_t* st = stage0 + (size_t)s * stage_elems;
+    const int64_t r0 = t * kTileRows;
+    const int rows = (int)std::min<int64_t>(kTileRows, p.n_rows - r0);
+    const int copied = rows & ~3;
+    if (copied != rows) {  // ragged tail: the last <= 3 rows are not 16-byte multiples
+      if (ctid < rows - copied)
+        for (int c = 0; c < p.n_cols; ++c)
+          st[c * kTileRows + copied + ctid] = p.col[c][r0 + copied + ctid];
+      consumer_sync();
+    }
+    process_tile<NJ, GROUPED>(p, js, st, kTileRows, rows, ctid, pol_last, smem_table, s_sum, s_cnt,
+                              acc_sum, acc_cnt);
+    __syncwarp();
+    if ((tid & 31) == 0) mbar_arrive(empty + s);
+  }
+
+  // ---------------- flush the CTA's partial aggregate ----------------
+  if (GROUPED) {
+    if (smem_table) {
+      consumer_sync();
+      for (int g = ctid; g < n_groups; g += kConsumers) {
+        const uint32_t c = s_cnt[g];
+        if (c) {
+          atomicAdd(p.g_sum + g, s_sum[g]);
+          atomicAdd(p.g_cnt + g, (unsigned long long)c);
+        }
+      }
+    }
+  } else {
+    // neighbourhood reduce (warp shuffle, then the CTA) + one leader atomic (Listing 1 L27-29)
+#pragma unroll
+    for (int o = 16; o > 0; o >>= 1) {
+      acc_sum += __shfl_xor_sync(kFull, acc_sum, o);
+      acc_cnt += __shfl_xor_sync(kFull, acc_cnt, o);
+    }
+    if ((tid & 31) == 0) {
+      red[warp] = acc_sum;
+      red[kConsumerWarps + warp] = acc_cnt;
+    }
+    consumer_sync();
+    if (ctid == 0) {
+      long long s = 0, c = 0;
+      for (int w = 0; w < kConsumerWarps; ++w) {
+        s += red[w];
+        c += red[kConsumerWarps + w];
+      }
+      if (c) {
+        atomicAdd(p.g_sum, (unsigned long long)s);
+        atomicAdd(p.g_cnt, (unsigned long long)c);
+      }
+    }
+  }
+}
+
+// Group layout from the dimension ranks (device-side; no host round trip) and zeroing of
+// the group arrays. Every CTA computes n_groups; CTA 0 publishes the meta.
+__global__ void k1_prepare(AggMeta* meta, const HtHeader* g0, const HtHeader* g1,
+                           const HtHeader* g2, int n_gdims, int4 gdim_join,
+                           unsigned long long* sums, unsigned long long* cnts,
+                           long long cap_groups, int fresh) {
+  const HtHeader* hdrs[HX_MAX_GDIMS] = {g0, g1, g2};
+  const int gj[HX_MAX_GDIMS] = {gdim_join.x, gdim_join.y, gdim_join.z};
+  int32_t nr[HX_MAX_GDIMS] = {1, 1, 1};
+  long long n = 1;
+  for (int g = 0; g < n_gdims; ++g) {
+    nr[g] = hdrs[g]->n_ranks;
+    n *= nr[g];
+  }
+  const bool over = n > cap_groups;
+  if (over) n = cap_groups;
+  if (fresh) {
+    if (blockIdx.x == 0 && threadIdx.x == 0) {
+      AggMeta m{};
+      m.n_groups = n;
+      long long stride = 1;
+      for (int j = 0; j < HX_MAX_JOINS; ++j) m.jstride[j] = 0;
+      for (int g = n_gdims - 1; g >= 0; --g) {
+        m.jstride[gj[g]] = (int32_t)stride;
+        stride *= nr[g];
+      }
+      for (int g = 0; g < HX_MAX_GDIMS; ++g) m.n_ranks[g] = nr[g];
+      m.error = over ? HX_ECAPACITY : 0;
+      *meta = m;
+    }
+    for (long long i = blockIdx.x * (long long)blockDim.x + threadIdx.x; i < n;
+         i += (long long)gridDim.x * blockDim.x) {
+      sums[i] = 0;
+      cnts[i] = 0;
+    }
+  }
+}
+
+template <int NJ, bool G>
+void set_attrs() {
+  cudaFuncSetAttribute(k1_probe_agg<NJ, G>, cudaFuncAttributeMaxDynamicSharedMemorySize,
+                       200 * 1024);
+}
+
+using KernelFn = void (*)(K1Params);
+
+KernelFn pick_kernel(int nj, bool grouped) {
+  static const KernelFn table[2][HX_MAX_JOINS + 1] = {
+      {k1_probe_agg<0, false>, k1_probe_agg<1, false>, k1_probe_agg<2, false>,
+       k1_probe_agg<3, false>, k1_probe_agg<4, false>},
+      {k1_probe_agg<0, true>, k1_probe_agg<1, true>, k1_probe_agg<2, true>,
+       k1_probe_agg<3, true>, k1_probe_agg<4, true>}};
+  return table[grouped ? 1 : 0][nj];
+}
+
+size_t k1_smem_bytes(int n_cols, int stages, int smem_groups) {
+  const size_t table_bytes = ((size_t)smem_groups * 12 + 127) & ~size_t(127);
+  return 512 + table_bytes + (size_t)stages * n_cols * kTileRows * sizeof(int32_t);
+}
+
+int pick_stages(int n_cols) {
+  // ~96 KB of tiles in flight per CTA (2 CTAs per SM): 3 stages up to 4 columns, 2 beyond
+  const size_t stage = (size_t)n_cols * kTileRows * 4;
+  return std::max(2, std::min(4, (int)((96 * 1024) / stage)));
+}
+
+}  // namespace
+
+int k1_occupancy(hx_ctx* ctx) {
+  static bool attrs = false;
+  if (!attrs) {
+    set_attrs<0, false>(); set_attrs<1, false>(); set_attrs<2, false>(); set_attrs<3, false>();
+    set_attrs<4, false>(); set_attrs<0, true>(); set_attrs<1, true>(); set_attrs<2, true>();
+    set_attrs<3, true>(); set_attrs<4, true>();
+    attrs = true;
+  }
+  int occ = 0;
+  cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, k1_probe_agg<3, true>, kThreads,
+                                                k1_smem_bytes(4, pick_stages(4), kSmemGroups));
+  return occ;
+}
+
+int probe_agg(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht* const* hts,
+              int n_hts, hx_agg* agg, bool fresh) {
+  HX_REQUIRE(ctx && fact && sh && agg, HX_EINVAL, "hx_pipeline_probe_agg: null argument");
+  HX_REQUIRE(sh->n_preds >= 0 && sh->n_preds <= HX_MAX_PREDS && sh->n_joins >= 0 &&
+                 sh->n_joins <= HX_MAX_JOINS && sh->n_gdims >= 0 && sh->n_gdims <= HX_MAX_GDIMS &&
+                 sh->agg_op >= HX_AGG_SUM && sh->agg_op <= HX_AGG_SUM_SUB,
+             HX_EINVAL, "hx_pipeline_probe_agg: bad query shape");
+  HX_REQUIRE(fact->placement != HX_PLACE_HOST_PINNED, HX_EUNSUPPORTED,
+             "hx_pipeline_probe_agg: host-resident fact tables are not supported");
+  K1Params p{};
+  // distinct fact columns the shape references -> staged columns
+  int32_t ids[kMaxStageCols];
+  int n_cols = 0;
+  auto stage_of = [&](int32_t col_id) -> int {
+    for (int i = 0; i < n_cols; ++i)
+      if (ids[i] == col_id) return i;
+    if (n_cols == kMaxStageCols) return -2;
+    if (!table_has_col(fact, col_id)) return -1;
+    ids[n_cols] = col_id;
+    return n_cols++;
+  };
+  for (int q = 0; q < sh->n_preds; ++q) {
+    const hx_pred& pr = sh->preds[q];
+    int c = stage_of(pr.col_id);
+    HX_REQUIRE(c >= 0, HX_EINVAL, "hx_pipeline_probe_agg: predicate column not in fact table");
+    HX_REQUIRE(pr.kind == HX_PRED_RANGE || (pr.kind == HX_PRED_IN && pr.n_in >= 1 && pr.n_in <= 4),
+               HX_EINVAL, "hx_pipeline_probe_agg: bad predicate");
+    p.preds[q] = DevPred{c, pr.kind, pr.lo, pr.hi, pr.n_in, {pr.in[0], pr.in[1], pr.in[2], pr.in[3]}};
+  }
+  p.n_preds = sh->n_preds;
+  for (int j = 0; j < sh->n_joins; ++j) {
+    int c = stage_of(sh->join_fk_col[j]);
+    HX_REQUIRE(c >= 0, HX_EINVAL, "hx_pipeline_probe_agg: join FK column not in fact table");
+    HX_REQUIRE(sh->join_ht[j] >= 0 && sh->join_ht[j] < n_hts && hts && hts[sh->join_ht[j]],
+               HX_EINVAL, "hx_pipeline_probe_agg: bad join hash table index");
+    const hx_ht* ht = hts[sh->join_ht[j]];
+    p.joins[j] = JoinDev{c, ht->slots, ht->hdr};
+  }
+  p.agg_op = sh->agg_op;
+  p.agg_a = stage_of(sh->agg_a);
+  p.agg_b = sh->agg_op == HX_AGG_SUM ? p.agg_a : stage_of(sh->agg_b);
+  HX_REQUIRE(p.agg_a >= 0 && p.agg_b >= 0, HX_EINVAL,
+             "hx_pipeline_probe_agg: measure column not in fact table (or > 8 columns)");
+
+  // group layout: host-known upper bound for the arrays, exact count on the device
+  long long bound = 1;
+  for (int g = 0; g < sh->n_gdims; ++g) {
+    const int j = sh->gdim_join[g];
+    HX_REQUIRE(j >= 0 && j < sh->n_joins, HX_EINVAL, "hx_pipeline_probe_agg: bad gdim_join");
+    for (int g2 = 0; g2 < g; ++g2)
+      HX_REQUIRE(sh->gdim_join[g2] != j, HX_EINVAL, "hx_pipeline_probe_agg: repeated gdim_join");
+    const hx_ht* ht = hts[sh->join_ht[j]];
+    bound *= std::max<long long>(1, std::min<long long>(ht->domain, std::max<int64_t>(ht->dim_rows, 1)));
+    bound = std::min<long long>(bound, (long long)HX_MAX_GROUPS + 1);
+  }
+  if (fresh) {
+    HX_REQUIRE(bound <= HX_MAX_GROUPS, HX_ECAPACITY, "hx_pipeline_probe_agg: too many groups");
+    agg->cap_groups = bound;
+    agg->n_gdims = sh->n_gdims;
+    for (int g = 0; g < sh->n_gdims; ++g) agg->gdim_ht[g] = hts[sh->join_ht[sh->gdim_join[g]]];
+    const size_t bytes = 256 + 2 * (size_t)bound * sizeof(unsigned long long);
+    HX_CK(cudaMallocAsync(&agg->base, bytes, ctx->stream));
+    agg->meta = reinterpret_cast<AggMeta*>(agg->base);
+    agg->sums = reinterpret_cast<unsigned long long*>(static_cast<char*>(agg->base) + 256);
+    agg->cnts = agg->sums + bound;
+  } else {
+    HX_REQUIRE(agg->n_gdims == sh->n_gdims, HX_EINVAL,
+               "hx_pipeline_probe_agg_into: shape differs from the agg's");
+  }
+  for (int j = 0; j < sh->n_joins; ++j) agg->deps.push_back(hts[sh->join_ht[j]]);
+
+  {  // k1_prepare
+    const HtHeader* gh[HX_MAX_GDIMS] = {nullptr, nullptr, nullptr};
+    int4 gj = make_int4(0, 0, 0, 0);
+    int* gjp = &gj.x;
+    for (int g = 0; g < sh->n_gdims; ++g) {
+      gh[g] = hts[sh->join_ht[sh->gdim_join[g]]]->hdr;
+      gjp[g] = sh->gdim_join[g];
+    }
+    const int grid = (int)std::max<long long>(1, std::min<long long>((agg->cap_groups + 255) / 256,
+                                                                     (long long)ctx->n_sms * 4));
+    k1_prepare<<<grid, 256, 0, ctx->stream>>>(agg->meta, gh[0], gh[1], gh[2], sh->n_gdims, gj,
+                                             agg->sums, agg->cnts, agg->cap_groups, fresh ? 1 : 0);
+    HX_CK_LAUNCH("k1_prepare");
+  }
+
+  // tiles: the head rows up to 16-byte alignment are handled separately
+  const uintptr_t mis = reinterpret_cast<uintptr_t>(table_col(fact, ids[0])) & 15u;
+  for (int c = 0; c < n_cols; ++c)
+    HX_REQUIRE((reinterpret_cast<uintptr_t>(table_col(fact, ids[c])) & 15u) == mis &&
+                   (mis & 3u) == 0,
+               HX_EUNSUPPORTED, "hx_pipeline_probe_agg: columns with different alignment");
+  const int64_t head = std::min<int64_t>(fact->n_rows, mis ? (16 - (int64_t)mis) / 4 : 0);
+  p.n_cols = n_cols;
+  for (int c = 0; c < n_cols; ++c) {
+    p.head_col[c] = table_col(fact, ids[c]);
+    p.col[c] = p.head_col[c] + head;
+  }
+  p.head_rows = (int32_t)head;
+  p.n_rows = fact->n_rows - head;
+  p.n_tiles = (p.n_rows + kTileRows - 1) / kTileRows;
+  p.stages = pick_stages(n_cols);
+  p.meta = agg->meta;
+  p.g_sum = agg->sums;
+  p.g_cnt = agg->cnts;
+  const bool grouped = sh->n_gdims > 0;
+  p.smem_groups = grouped ? (int32_t)std::min<long long>(kSmemGroups, agg->cap_groups) : 0;
+  if (fact->n_rows == 0) return HX_OK;
+
+  if (!ctx->k1_ctas_per_sm) ctx->k1_ctas_per_sm = std::max(1, k1_occupancy(ctx));
+  KernelFn fn = pick_kernel(sh->n_joins, grouped);
+  const size_t smem = k1_smem_bytes(n_cols, p.stages, p.smem_groups);
+  int occ = 0;
+  HX_CK(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, fn, kThreads, smem));
+  occ = std::max(1, occ);
+  const int64_t grid = std::max<int64_t>(1, std::min<int64_t>(p.n_tiles, (int64_t)ctx->n_sms * occ));
+  cudaEvent_t e0 = nullptr, e1 = nullptr;
+  if (ctx->prof_on) {
+    e0 = pooled_event(ctx);
+    e1 = pooled_event(ctx);
+    HX_CK(cudaEventRecord(e0, ctx->stream));
+  }
+  fn<<<(unsigned)grid, kThreads, smem, ctx->stream>>>(p);
+  HX_CK_LAUNCH("k1_probe_agg");
+  if (ctx->prof_on) {
+    HX_CK(cudaEventRecord(e1, ctx->stream));
+    ctx->prof_events.push_back({e0, e1});
+    ctx->prof_launches += 1;
+    ctx->prof_bytes += fact->n_rows * 4 * n_cols;
+  }
+  return HX_OK;
+}
+
+}  // namespace hx

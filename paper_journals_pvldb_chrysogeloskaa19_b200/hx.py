@@ -1,0 +1,264 @@
+"""Thin Python binding of the libhx C-ABI with the same call names (include/hx.h).
+
+Argument marshalling only. Objects own their C handles and free them on close()/__del__.
+PyTorch, when used by a caller, only provides device memory (tensor data pointers) and
+streams (`torch.cuda.current_stream().cuda_stream`); nothing here imports torch.
+"""
+from __future__ import annotations
+
+import ctypes
+from typing import Dict, List, Optional, Sequence, Tuple
+
+import numpy as np
+
+from . import _hx
+from ._hx import call, hx_col, hx_query_shape, pred  # noqa: F401  (re-exported)
+
+
+class Context:
+    """hx_init / hx_finalize: one GPU, one stream (cudaStream_t as int, 0 = library-owned)."""
+
+    def __init__(self, device: int = 0, stream: int = 0):
+        h = ctypes.c_void_p()
+        call("hx_init", device, ctypes.c_void_p(stream or None), ctypes.byref(h))
+        self.h = h
+        self.device = device
+
+    @property
+    def stream(self) -> int:
+        s = ctypes.c_void_p()
+        call("hx_ctx_stream", self.h, ctypes.byref(s))
+        return s.value or 0
+
+    def info(self) -> Tuple[int, int]:
+        a, b = ctypes.c_int(), ctypes.c_int()
+        call("hx_ctx_info", self.h, ctypes.byref(a), ctypes.byref(b))
+        return a.value, b.value
+
+    def comm_init(self, nranks: int, rank: int, uid: bytes) -> None:
+        buf = ctypes.create_string_buffer(uid, 128)
+        call("hx_comm_init", self.h, nranks, rank, buf)
+
+    def profile_enable(self, on: bool = True) -> None:
+        call("hx_profile_enable", self.h, int(on))
+
+    def profile_read(self, reset: bool = True) -> Tuple[float, int, int]:
+        ms, n, b = ctypes.c_double(), ctypes.c_int64(), ctypes.c_int64()
+        call("hx_profile_read", self.h, ctypes.byref(ms), ctypes.byref(n), ctypes.byref(b),
+             int(reset))
+        return ms.value, n.value, b.value
+
+    def close(self) -> None:
+        if getattr(self, "h", None):
+            call("hx_finalize", self.h)
+            self.h = None
+
+    def __del__(self):
+        try:
+            self.close()
+        except Exception:
+            pass
+
+
+def comm_unique_id() -> bytes:
+    buf = ctypes.create_string_buffer(128)
+    call("hx_comm_unique_id", buf)
+    return buf.raw
+
+
+class Partition:
+    """hx_router_partition: block handles {row_begin, row_end, part}."""
+
+    def __init__(self, n_rows: int, n_parts: int, block_rows: int, policy: int = _hx.HX_POLICY_RANGE):
+        h = ctypes.c_void_p()
+        call("hx_router_partition", n_rows, n_parts, block_rows, policy, ctypes.byref(h))
+        self.h = h
+        self.n_parts = n_parts
+
+    def blocks(self) -> List[Tuple[int, int, int]]:
+        n = ctypes.c_int64()
+        ptr = ctypes.POINTER(_hx.hx_block)()
+        call("hx_partition_info", self.h, ctypes.byref(n), ctypes.byref(ptr))
+        return [(ptr[i].row_begin, ptr[i].row_end, ptr[i].part) for i in range(n.value)]
+
+    def rows(self, part: int) -> int:
+        n = ctypes.c_int64()
+        call("hx_partition_rows", self.h, part, ctypes.byref(n))
+        return n.value
+
+    def close(self):
+        if getattr(self, "h", None):
+            call("hx_partition_free", self.h)
+            self.h = None
+
+    def __del__(self):
+        try:
+            self.close()
+        except Exception:
+            pass
+
+
+def router_partition(n_rows: int, n_parts: int, block_rows: int,
+                     policy: int = _hx.HX_POLICY_RANGE) -> Partition:
+    return Partition(n_rows, n_parts, block_rows, policy)
+
+
+class Table:
+    def __init__(self, ctx: Context, h, keep=None, parent=None):
+        self.ctx, self.h, self._keep, self._parent = ctx, h, keep, parent
+
+    @property
+    def n_rows(self) -> int:
+        n, c = ctypes.c_int64(), ctypes.c_int()
+        call("hx_table_info", self.h, ctypes.byref(n), ctypes.byref(c))
+        return n.value
+
+    def slice(self, row_begin: int, row_end: int) -> "Table":
+        h = ctypes.c_void_p()
+        call("hx_table_slice", self.h, row_begin, row_end, ctypes.byref(h))
+        return Table(self.ctx, h, parent=self)
+
+    def close(self):
+        if getattr(self, "h", None):
+            call("hx_table_free", self.h)
+            self.h = None
+
+    def __del__(self):
+        try:
+            self.close()
+        except Exception:
+            pass
+
+
+def load_columns(ctx: Context, cols: Sequence[Tuple[int, int, int]],
+                 part: Optional[Partition] = None, part_index: int = 0,
+                 placement: int = _hx.HX_PLACE_COPY, keep=None) -> Table:
+    """cols: (col_id, data pointer (host or device), n_rows). `keep` holds the buffers
+    alive for views."""
+    arr = (hx_col * len(cols))()
+    for i, (cid, ptr, n) in enumerate(cols):
+        arr[i].col_id, arr[i].data, arr[i].n_rows = cid, ptr, n
+    h = ctypes.c_void_p()
+    call("hx_load_columns", ctx.h, arr, len(cols), part.h if part else None, part_index,
+         placement, ctypes.byref(h))
+    return Table(ctx, h, keep=keep)
+
+
+def load_numpy(ctx: Context, cols: Dict[int, np.ndarray], part: Optional[Partition] = None,
+               part_index: int = 0) -> Table:
+    """Copy host int32 numpy columns to the device (HX_PLACE_COPY, H2D on the ctx stream)."""
+    keep = {k: np.ascontiguousarray(v, dtype=np.int32) for k, v in cols.items()}
+    spec = [(k, v.ctypes.data if v.size else 0, v.size) for k, v in keep.items()]
+    t = load_columns(ctx, spec, part, part_index, _hx.HX_PLACE_COPY, keep=keep)
+    return t
+
+
+class HashTable:
+    def __init__(self, ctx: Context, h, dim: Table):
+        self.ctx, self.h, self._dim = ctx, h, dim
+
+    def info(self, with_codes: bool = False):
+        nk, ns, nr = ctypes.c_int64(), ctypes.c_int64(), ctypes.c_int32()
+        call("hx_ht_info", self.h, ctypes.byref(nk), ctypes.byref(ns), ctypes.byref(nr), None)
+        codes = None
+        if with_codes:
+            buf = (ctypes.c_int32 * max(1, nr.value))()
+            call("hx_ht_info", self.h, None, None, None, buf)
+            codes = list(buf)[: nr.value]
+        return {"n_keys": nk.value, "n_slots": ns.value, "n_ranks": nr.value, "rank_to_code": codes}
+
+    def broadcast(self, root: int = 0) -> None:
+        call("hx_ht_broadcast", self.ctx.h, self.h, root)
+
+    def close(self):
+        if getattr(self, "h", None):
+            call("hx_ht_free", self.h)
+            self.h = None
+
+    def __del__(self):
+        try:
+            self.close()
+        except Exception:
+            pass
+
+
+def build_dim_ht(ctx: Context, dim: Table, key_col: int, preds: Sequence[_hx.hx_pred] = (),
+                 group_col: int = -1, group_lo: int = 0, group_hi: int = 0) -> HashTable:
+    arr = (_hx.hx_pred * max(1, len(preds)))(*preds)
+    h = ctypes.c_void_p()
+    call("hx_build_dim_ht", ctx.h, dim.h, key_col, arr, len(preds), group_col, group_lo,
+         group_hi, ctypes.byref(h))
+    return HashTable(ctx, h, dim)
+
+
+def query_shape(preds=(), joins=(), agg_op=_hx.HX_AGG_SUM, agg_a=0, agg_b=0,
+                gdims=()) -> hx_query_shape:
+    """joins: sequence of (fk_col_id, ht_index) in probe order; gdims: join indices."""
+    s = hx_query_shape()
+    s.n_preds = len(preds)
+    for i, p in enumerate(preds):
+        s.preds[i] = p
+    s.n_joins = len(joins)
+    for i, (fk, ht) in enumerate(joins):
+        s.join_fk_col[i], s.join_ht[i] = fk, ht
+    s.agg_op, s.agg_a, s.agg_b = agg_op, agg_a, agg_b
+    s.n_gdims = len(gdims)
+    for i, g in enumerate(gdims):
+        s.gdim_join[i] = g
+    return s
+
+
+class Agg:
+    def __init__(self, ctx: Context, h, n_gdims: int, deps):
+        self.ctx, self.h, self.n_gdims, self._deps = ctx, h, n_gdims, deps
+
+    def close(self):
+        if getattr(self, "h", None):
+            call("hx_agg_free", self.h)
+            self.h = None
+
+    def __del__(self):
+        try:
+            self.close()
+        except Exception:
+            pass
+
+
+def _hts_array(hts: Sequence[HashTable]):
+    arr = (ctypes.c_void_p * max(1, len(hts)))()
+    for i, t in enumerate(hts):
+        arr[i] = t.h.value
+    return arr
+
+
+def pipeline_probe_agg(ctx: Context, fact: Table, shape: hx_query_shape,
+                       hts: Sequence[HashTable]) -> Agg:
+    h = ctypes.c_void_p()
+    call("hx_pipeline_probe_agg", ctx.h, fact.h, ctypes.byref(shape), _hts_array(hts), len(hts),
+         ctypes.byref(h))
+    return Agg(ctx, h, shape.n_gdims, (fact, list(hts)))
+
+
+def pipeline_probe_agg_into(ctx: Context, fact: Table, shape: hx_query_shape,
+                            hts: Sequence[HashTable], agg: Agg) -> None:
+    call("hx_pipeline_probe_agg_into", ctx.h, fact.h, ctypes.byref(shape), _hts_array(hts),
+         len(hts), agg.h)
+
+
+def merge_aggregates(ctx: Context, agg: Agg, root: int = -1, cap: int = 1 << 16):
+    """-> (keys int32[n, n_gdims], sums int64[n], counts int64[n]) for non-empty groups."""
+    while True:
+        sums = np.zeros(cap, np.int64)
+        cnts = np.zeros(cap, np.int64)
+        keys = np.zeros(cap * max(1, agg.n_gdims), np.int32)
+        n = ctypes.c_int64()
+        rc = getattr(_hx.lib(), "hx_merge_aggregates")(
+            ctx.h, agg.h, root, sums.ctypes.data_as(_hx._PI64), cnts.ctypes.data_as(_hx._PI64),
+            keys.ctypes.data_as(_hx._PI32), cap, ctypes.byref(n))
+        if rc == _hx.HX_ECAPACITY and n.value > cap:
+            cap = n.value
+            continue
+        if rc != _hx.HX_OK:
+            raise _hx.HxError(rc, "hx_merge_aggregates", _hx.lib().hx_last_error().decode())
+        k = n.value
+        return keys[: k * agg.n_gdims].reshape(k, agg.n_gdims), sums[:k], cnts[:k]

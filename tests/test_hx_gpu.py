@@ -1,0 +1,152 @@
+"""GPU parity of libhx against the oracle, through the C-ABI (ctypes binding).
+
+Bar: bit-exact — the set of (group codes, int64 SUM, int64 COUNT) rows
+and their ORDER BY order — for all 13 SSB queries. Inputs are seeded (ssbgen / ssb_tiny).
+"""
+import numpy as np
+import pytest
+
+import oracle
+import ssbgen
+from ssb_tiny import tiny_db
+
+pytestmark = pytest.mark.gpu
+
+torch = pytest.importorskip("torch")
+if not torch.cuda.is_available():
+    pytest.skip("needs a CUDA GPU", allow_module_level=True)
+
+from paper_journals_pvldb_chrysogeloskaa19_b200 import _hx, hx, ssb  # noqa: E402
+
+QUERIES = ssb.QUERIES
+C = ssbgen.COLS
+
+
+@pytest.fixture(scope="module")
+def ctx():
+    c = hx.Context(0)
+    yield c
+    c.close()
+
+
+def run_all(ctx, db, queries=QUERIES):
+    dims, fact = ssb.load_db_numpy(ctx, db)
+    eng = ssb.SsbEngine(ctx, dims, fact)
+    return {q: eng.run(q) for q in queries}
+
+
+# ---- small SSB databases: several tiles and a ragged tail ------------------------------
+@pytest.mark.parametrize("sf,seed", [(0.01, 42), (0.05, 7)])
+def test_parity_small_sf(ctx, sf, seed):
+    db = ssbgen.database(seed, ssbgen.sizes(sf))
+    got = run_all(ctx, db)
+    for q in QUERIES:
+        assert got[q] == oracle.run_query(q, db), q
+
+
+def test_parity_handcrafted(ctx, handcrafted):
+    db, expect = handcrafted
+    got = run_all(ctx, db)
+    for q in QUERIES:
+        assert got[q] == expect[q], q
+
+
+@pytest.mark.parametrize("seed", [1, 2, 3])
+def test_parity_tiny_skewed(ctx, seed):
+    """Missing FKs, boundary dates, dense group domains (every query non-empty)."""
+    db = tiny_db(seed, n_lo=20011)
+    got = run_all(ctx, db)
+    for q in QUERIES:
+        assert got[q] == oracle.run_query(q, db), q
+
+
+@pytest.mark.parametrize("n_lo", [0, 1, 3, 4, 5, 2047, 2048, 2049, 4096 * 3 + 1])
+def test_ragged_sizes(ctx, n_lo):
+    db = tiny_db(11, n_lo=max(n_lo, 1))
+    if n_lo == 0:
+        db["lineorder"] = {k: v[:0] for k, v in db["lineorder"].items()}
+    got = run_all(ctx, db)
+    for q in QUERIES:
+        assert got[q] == oracle.run_query(q, db), (q, n_lo)
+
+
+def test_duplicate_dimension_key_is_reported(ctx):
+    db = tiny_db(3, dup_keys=True)
+    dims, fact = ssb.load_db_numpy(ctx, db)
+    eng = ssb.SsbEngine(ctx, dims, fact)
+    with pytest.raises(_hx.HxError) as ei:
+        eng.run("q4.1")
+    assert ei.value.code == _hx.HX_EDUPKEY
+
+
+# ---- hash-table self-check (K2) ------------------------------------------------------------
+def test_hash_table_contents(ctx):
+    sz = ssbgen.sizes(0.1)
+    db = ssbgen.database(5, sz)
+    dims, _ = ssb.load_db_numpy(ctx, {**db, "lineorder": {k: v[:1] for k, v in db["lineorder"].items()}})
+    cust = db["customer"]
+    ht = hx.build_dim_ht(ctx, dims["customer"], C["c_custkey"],
+                         [hx.pred(C["c_region"], 1, 1)], C["c_nation"], 0, 24)
+    info = ht.info(with_codes=True)
+    passing = cust["c_region"] == 1
+    assert info["n_keys"] == int(passing.sum())
+    assert info["n_slots"] >= 2 * info["n_keys"] and info["n_slots"] & (info["n_slots"] - 1) == 0
+    assert info["rank_to_code"] == sorted(set(cust["c_nation"][passing].tolist()))
+    # probe every key through a one-join pipeline: COUNT per nation rank == dimension counts
+    keys = cust["c_custkey"]
+    fact = hx.load_numpy(ctx, {C["lo_custkey"]: keys, C["lo_revenue"]: np.ones_like(keys)})
+    shape = hx.query_shape(joins=[(C["lo_custkey"], 0)], agg_a=C["lo_revenue"], gdims=[0])
+    agg = hx.pipeline_probe_agg(ctx, fact, shape, [ht])
+    k, s, c = hx.merge_aggregates(ctx, agg)
+    want = {n: int((cust["c_nation"][passing] == n).sum()) for n in info["rank_to_code"]}
+    assert {int(a): int(b) for a, b in zip(k[:, 0], c)} == want
+    assert int(c.sum()) == int(passing.sum())  # every passing key hit, every other key missed
+
+
+# ---- router / partition invariance (fake multi-GPU on one device) ----------------------
+@pytest.mark.parametrize("n_parts,block_rows,policy", [(2, 4097, 0), (3, 1000, 1), (4, 1 << 22, 0)])
+def test_partition_invariance(ctx, n_parts, block_rows, policy):
+    db = ssbgen.database(9, ssbgen.sizes(0.02))
+    n = len(db["lineorder"]["lo_orderdate"])
+    part = hx.router_partition(n, n_parts, block_rows, policy)
+    blocks = part.blocks()
+    assert sum(e - b for b, e, _ in blocks) == n
+    assert sum(part.rows(i) for i in range(n_parts)) == n
+    dims, _ = ssb.load_db_numpy(ctx, {**db, "lineorder": {k: v[:1] for k, v in db["lineorder"].items()}})
+    facts = [hx.load_numpy(ctx, {C[c]: v for c, v in db["lineorder"].items()}, part, i)
+             for i in range(n_parts)]
+    eng = ssb.SsbEngine(ctx, dims, facts[0])
+    for q in QUERIES:
+        plan = ssb.PLANS[q]
+        hts = [eng.build(b) for _, b in plan.joins]
+        shape = eng.shape(plan)
+        agg = hx.pipeline_probe_agg(ctx, facts[0], shape, hts)
+        for f in facts[1:]:
+            hx.pipeline_probe_agg_into(ctx, f, shape, hts, agg)
+        keys, sums, cnts = hx.merge_aggregates(ctx, agg)
+        rows = ssb.order_by(plan, [tuple(int(x) for x in keys[i]) + (int(sums[i]), int(cnts[i]))
+                                   for i in range(len(sums))])
+        assert rows == oracle.run_query(q, db), (q, n_parts)
+
+
+@pytest.mark.parametrize("offset", [1, 2, 3, 5])
+def test_misaligned_views(ctx, offset):
+    """Slices at a row offset are not 16-byte aligned: head rows take the direct path."""
+    db = ssbgen.database(4, ssbgen.sizes(0.01))
+    dims, fact = ssb.load_db_numpy(ctx, db)
+    n = fact.n_rows
+    sl = fact.slice(offset, n - 7)
+    eng = ssb.SsbEngine(ctx, dims, sl)
+    for q in QUERIES:
+        assert eng.run(q) == oracle.run_query(q, db, offset, n - 7), q
+
+
+def test_device_generated_columns_match_host(ctx):
+    """ssbgen's device fill is bit-identical to the host fill (inputs for the bench)."""
+    sz = ssbgen.sizes(0.02)
+    for col in ("lo_orderdate", "lo_revenue", "lo_supplycost", "c_city", "p_brand1", "d_weeknuminyear"):
+        n = ssbgen.table_rows(sz, col)
+        t = torch.empty(n, dtype=torch.int32, device="cuda")
+        ssbgen.column_device(42, sz, col, t.data_ptr(), 0, n, torch.cuda.current_stream().cuda_stream)
+        torch.cuda.synchronize()
+        assert np.array_equal(t.cpu().numpy(), ssbgen.column(42, sz, col)), col
