@@ -1,0 +1,400 @@
+#!/usr/bin/env python
+"""Benchmark of the HetExchange SSB hot path on B200 (BASELINE.json metric).
+
+One STEP = all 13 SSB queries, each one pass of the whole hot path over this GPU's
+lineorder partition: filter + hash-table build of every joined dimension (K2), the fused
+scan -> filter -> probe x k -> aggregate pipeline (K1), and the union-router merge of the
+partial aggregates (NCCL allreduce when N > 1) with the result copied to the host.
+
+Workload (config.workload): SSB SF10 per GPU, HBM-resident (BASELINE.json configs[1] at
+N=1; weak scaling: N GPUs run SF 10*N with lineorder range-partitioned in 2^22-row router
+blocks and the dimensions replicated). Synthetic dbgen-shaped data from ssbgen (seed 42),
+generated directly in HBM outside the timed region. Each query scans 0.96-1.44 GB per GPU,
+larger than the 126 MB L2, so no L2 flush is needed between queries.
+
+    python bench.py [--gpus N] [--steps K] [--warmup W] [--sf SF_PER_GPU] [--impl reference]
+    python -m torch.distributed.run --nproc-per-node N ... bench.py --gpus N ...
+"""
+from __future__ import annotations
+
+import argparse
+import json
+import os
+import statistics
+import subprocess
+import sys
+import tempfile
+import time
+
+ROOT = os.path.dirname(os.path.abspath(__file__))
+sys.path.insert(0, ROOT)
+
+import numpy as np  # noqa: E402
+
+import ssbgen  # noqa: E402
+
+with open(os.path.join(ROOT, "BASELINE.json")) as _f:
+    METRIC = json.load(_f)["metric"]
+UNIT = "lineorder rows/s"
+SEED = 42
+BLOCK_ROWS = 1 << 22
+
+
+def parse():
+    ap = argparse.ArgumentParser()
+    ap.add_argument("--gpus", type=int, default=1)
+    ap.add_argument("--steps", type=int, default=10)
+    ap.add_argument("--warmup", type=int, default=3)
+    ap.add_argument("--sf", type=float, default=10.0, help="SSB scale factor per GPU")
+    ap.add_argument("--impl", default="hx", choices=["hx", "reference"])
+    ap.add_argument("--no-cpu-baseline", action="store_true")
+    ap.add_argument("--no-e2e", action="store_true")
+    ap.add_argument("--queries", default="all")
+    ap.add_argument("--no-graph", action="store_true", help="enqueue plans without a CUDA graph")
+    return ap.parse_args()
+
+
+def dist_env():
+    world = int(os.environ.get("WORLD_SIZE", "1"))
+    rank = int(os.environ.get("RANK", "0"))
+    local = int(os.environ.get("LOCAL_RANK", "0"))
+    return world, rank, local
+
+
+def peaks():
+    try:
+        with open(os.path.join(ROOT, "MEASURED_PEAKS.json")) as f:
+            m = json.load(f)
+        return float(m["hbm_gbs"]), "measured (MEASURED_PEAKS.json hbm_gbs)"
+    except Exception:
+        return 6650.0, "fallback (B200_PROFILING.md)"
+
+
+def workload_name(sf, world):
+    return f"SSB all 13 queries, SF{sf:g} per GPU (SF{sf * world:g} total), HBM-resident"
+
+
+def config(args, world, n_rows_gpu, queries):
+    return {"workload": workload_name(args.sf, world), "sf_per_gpu": args.sf,
+            "sf_total": args.sf * world, "queries": queries,
+            "lineorder_rows_per_gpu": n_rows_gpu, "router_block_rows": BLOCK_ROWS,
+            "parallelism": f"lineorder block-partitioned over {world} GPU(s); dims replicated; "
+                           "partials merged by NCCL allreduce" if world > 1 else "1 GPU",
+            "l2": "inputs larger than L2 (each query scans >= 0.96 GB/GPU vs 126 MB L2); no flush"}
+
+
+class Clocks:
+    """nvidia-smi sampling DURING the timed region (B200_PROFILING.md clocks line)."""
+
+    def __init__(self, index):
+        self.index, self.proc, self.path = index, None, None
+
+    def start(self):
+        try:
+            fd, self.path = tempfile.mkstemp(suffix=".csv")
+            os.close(fd)
+            self.proc = subprocess.Popen(
+                ["nvidia-smi", "-i", str(self.index), "--query-gpu=clocks.sm,clocks.max.sm,"
+                 "clocks_event_reasons.active,clocks_event_reasons.hw_slowdown,"
+                 "clocks_event_reasons.hw_thermal_slowdown,clocks_event_reasons.sw_thermal_slowdown,"
+                 "clocks_event_reasons.sw_power_cap", "--format=csv,noheader,nounits", "-lms", "100"],
+                stdout=open(self.path, "w"), stderr=subprocess.DEVNULL)
+        except Exception:
+            self.proc = None
+
+    def stop(self):
+        if not self.proc:
+            return None
+        time.sleep(0.25)
+        self.proc.terminate()
+        self.proc.wait()
+        sm, mx, reasons = [], 0, set()
+        names = ["hw_slowdown", "hw_thermal_slowdown", "sw_thermal_slowdown", "sw_power_cap"]
+        with open(self.path) as f:
+            for line in f:
+                parts = [p.strip() for p in line.split(",")]
+                if len(parts) < 7:
+                    continue
+                try:
+                    sm.append(float(parts[0]))
+                    mx = max(mx, float(parts[1]))
+                except ValueError:
+                    continue
+                for n, v in zip(names, parts[3:7]):
+                    if v.lower() == "active":
+                        reasons.add(n)
+        os.unlink(self.path)
+        if not sm:
+            return None
+        return {"sm_mhz": statistics.median(sm), "sm_max_mhz": mx, "reasons": sorted(reasons),
+                "samples": len(sm)}
+
+
+def ncu_traffic():
+    """DRAM bytes per K1 launch from the committed ncu --set full capture (or None)."""
+    p = os.path.join(ROOT, "profiles", "k1_traffic.json")
+    try:
+        with open(p) as f:
+            return json.load(f)
+    except Exception:
+        return None
+
+
+# ---------------------------------------------------------------------------------------
+def run_reference(args, world, rank):
+    """--impl reference: the oracle (the paper's method as a plain CPU program) as it stands,
+    on this box's host cores, over a bounded sample of the same workload per step."""
+    import oracle
+    if rank != 0:
+        return
+    sz = ssbgen.sizes(args.sf * world)
+    threads = os.cpu_count() or 1
+    sample = min(sz["n_lineorder"], 125_000 * threads)
+    db = ssbgen.database(SEED, sz, 0, sample)
+    queries = oracle.QUERIES if args.queries == "all" else args.queries.split(",")
+
+    def step():
+        for q in queries:
+            oracle.run_query_ranges(q, db, threads)
+
+    for _ in range(args.warmup):
+        step()
+    t0 = time.perf_counter()
+    for _ in range(args.steps):
+        step()
+    dt = (time.perf_counter() - t0) / args.steps
+    value = len(queries) * sample / dt
+    samp = f"lineorder rows [0, {sample}) of SF{args.sf * world:g} (dims full), {len(queries)} queries"
+    line = {"impl": "reference", "metric": METRIC, "value": value, "unit": UNIT, "n_gpus": world,
+            "steps": args.steps, "warmup": args.warmup, "ms_per_step": dt * 1e3,
+            "higher_is_better": True, "scaling": "weak", "vs_baseline": None, "dtype": "int64",
+            "data": f"synthetic (ssbgen dbgen-shaped SSB, seed {SEED})",
+            "config": config(args, world, sz["n_lineorder"] // world, queries),
+            "cpu_baseline": {"value": value, "unit": UNIT, "cores": threads, "kind": "oracle",
+                             "sample": samp},
+            "e2e": {"value": value, "unit": UNIT, "h2d_bytes_per_step": 0, "d2h_bytes_per_step": 0}}
+    print(json.dumps(line), flush=True)
+
+
+def cpu_baseline(args, world):
+    """The oracle, single-threaded as it stands, on a bounded sample (rank 0, N=1)."""
+    import oracle
+    sz = ssbgen.sizes(args.sf * world)
+    sample = min(sz["n_lineorder"], 2_000_000)
+    db = ssbgen.database(SEED, sz, 0, sample)
+    t0 = time.perf_counter()
+    for q in oracle.QUERIES:
+        oracle.run_query(q, db)
+    dt = time.perf_counter() - t0
+    return {"value": 13 * sample / dt, "unit": UNIT, "cores": 1, "kind": "oracle",
+            "sample": f"13 queries over lineorder rows [0, {sample}) of SF{args.sf * world:g} "
+                      f"(full dims), single-threaded, {dt:.1f} s"}
+
+
+def main():
+    args = parse()
+    world, rank, local = dist_env()
+    if args.impl == "reference":
+        run_reference(args, world, rank)
+        return
+
+    import torch
+    import torch.distributed as dist
+    from paper_journals_pvldb_chrysogeloskaa19_b200 import hx, ssb
+
+    torch.cuda.set_device(local)
+    if world > 1:
+        dist.init_process_group("nccl", device_id=torch.device("cuda", local))
+    stream = torch.cuda.current_stream()
+    ctx = hx.Context(local, stream.cuda_stream)
+    if world > 1:
+        uid = [hx.comm_unique_id() if rank == 0 else None]
+        dist.broadcast_object_list(uid, src=0)
+        ctx.comm_init(world, rank, uid[0])
+    queries = ssb.QUERIES if args.queries == "all" else args.queries.split(",")
+    C = ssbgen.COLS
+
+    # ---- data in HBM: this rank's router blocks of lineorder, full replicated dims -------
+    sz = ssbgen.sizes(args.sf * world)
+    part = hx.router_partition(sz["n_lineorder"], world, BLOCK_ROWS)
+    mine = [(b, e) for b, e, p in part.blocks() if p == rank]
+    r0, r1 = (mine[0][0], mine[-1][1]) if mine else (0, 0)
+    n_mine = r1 - r0
+    keep = []
+
+    def dev_table(cols, row_begin, n):
+        spec = []
+        for c in cols:
+            t = torch.empty(max(n, 1), dtype=torch.int32, device="cuda")
+            ssbgen.column_device(SEED, sz, c, t.data_ptr(), row_begin, n, stream.cuda_stream)
+            keep.append(t)
+            spec.append((C[c], t.data_ptr(), n))
+        return hx.load_columns(ctx, spec, placement=hx._hx.HX_PLACE_VIEW)
+
+    dims = {t: dev_table(ssbgen.TABLE_COLS[t], 0, ssbgen.table_rows(sz, ssbgen.TABLE_COLS[t][0]))
+            for t in ("date", "customer", "supplier", "part")}
+    fact = dev_table(ssbgen.TABLE_COLS["lineorder"], r0, n_mine)
+    torch.cuda.synchronize()
+    eng = ssb.SsbEngine(ctx, dims, fact)
+    # one prepared plan per query (HT + group buffers allocated once, builds sized once);
+    # the 13 executions are captured into ONE CUDA graph: a step is one graph launch plus
+    # the 13 host reads of the finalized results
+    plans = {q: eng.plan(q) for q in queries}
+    graph = None if args.no_graph else hx.capture(ctx, lambda: [plans[q].enqueue() for q in queries])
+    k1_acc = [0.0, 0, 0]
+
+    def step(timed=False):
+        if graph is not None:
+            graph.launch()
+        else:
+            for q in queries:
+                plans[q].enqueue()
+        out = [plans[q].rows() for q in queries]
+        if timed:
+            for q in queries:
+                ms_, b_ = plans[q].hp.k1_time()
+                k1_acc[0] += ms_
+                k1_acc[1] += 1
+                k1_acc[2] += b_
+        return out
+
+    # ---- warm-up, then exactly K timed steps ---------------------------------------------
+    for _ in range(args.warmup):
+        step()
+    ctx.stats(reset=True)
+    clocks = Clocks(local)
+    if world > 1:
+        dist.barrier()
+    torch.cuda.synchronize()
+    clocks.start()
+    e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+    e0.record(stream)
+    for _ in range(args.steps):
+        step(timed=True)
+    e1.record(stream)
+    torch.cuda.synchronize()
+    if world > 1:
+        dist.barrier()
+    clk = clocks.stop()
+    ms = e0.elapsed_time(e1)
+    k1_ms, k1_n, k1_bytes = k1_acc
+    launches, _, _ = ctx.stats(reset=True)
+    if world > 1:
+        t = torch.tensor([ms, float(launches)], device="cuda", dtype=torch.float64)
+        dist.all_reduce(t[:1], op=dist.ReduceOp.MAX)
+        dist.all_reduce(t[1:], op=dist.ReduceOp.SUM)
+        ms, launches = float(t[0]), int(t[1])
+    ms_step = ms / args.steps
+    total_rows = sz["n_lineorder"]
+    value = len(queries) * total_rows / (ms_step / 1e3)
+
+    peak, peak_src = peaks()
+    achieved = (k1_bytes / (k1_ms / 1e3)) / 1e9 if k1_ms > 0 else 0.0
+    tr = ncu_traffic()
+    roofline = {"bound": "hbm", "achieved": achieved, "peak": peak, "unit": "GB/s",
+                "frac": achieved / peak, "peak_source": peak_src,
+                "kernel": "k1_probe_agg (fused scan->filter->probe->aggregate), all 13 queries",
+                "algorithmic_bytes_per_launch": k1_bytes / max(k1_n, 1),
+                "k1_ms_per_launch": k1_ms / max(k1_n, 1),
+                "traffic": tr["dram_bytes_per_launch"] if tr else None,
+                "traffic_source": tr["source"] if tr else None}
+
+    # ---- per query (after the timed region): K1-only and whole-query time ---------------
+    per_query = {}
+    B = {q: 4 * len(ssb.FACT_COLS[q]) for q in queries}
+    for q in queries:
+        reps = 5
+        qe0, qe1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+        kms = 0.0
+        qe0.record(stream)
+        for _ in range(reps):
+            plans[q].enqueue()
+            plans[q].rows()
+            kms += plans[q].hp.k1_time()[0]
+        qe1.record(stream)
+        torch.cuda.synchronize()
+        qms = qe0.elapsed_time(qe1) / reps
+        kms /= reps
+        per_query[q] = {"query_ms": round(qms, 4), "k1_ms": round(kms, 4),
+                        "rows_per_s": n_mine / (qms / 1e3),
+                        "k1_hbm_gbps": n_mine * B[q] / (kms / 1e3) / 1e9 if kms else None,
+                        "k1_frac_of_peak": (n_mine * B[q] / (kms / 1e3) / 1e9) / peak if kms else None,
+                        "bytes_per_row": B[q]}
+
+    # ---- e2e through the C-ABI with HOST buffers (H2D + queries + D2H inside the clock) ---
+    e2e = None
+    if not args.no_e2e:
+        host = {}
+        for t in ("lineorder", "date", "customer", "supplier", "part"):
+            host[t] = {}
+            for c in ssbgen.TABLE_COLS[t]:
+                n = n_mine if t == "lineorder" else ssbgen.table_rows(sz, c)
+                buf = torch.empty(max(n, 1), dtype=torch.int32, pin_memory=True)
+                ssbgen.column(SEED, sz, c, r0 if t == "lineorder" else 0, n, out=buf.numpy())
+                host[t][c] = (buf, n)
+
+        def e2e_step():
+            def load(t):
+                return hx.load_columns(ctx, [(C[c], b.data_ptr(), n) for c, (b, n) in host[t].items()])
+            d = {t: load(t) for t in ("date", "customer", "supplier", "part")}
+            f = load("lineorder")
+            e = ssb.SsbEngine(ctx, d, f)
+            pend = [e.start(q) for q in queries]
+            out = [e.finish(p) for p in pend]
+            for tb in list(d.values()) + [f]:
+                tb.close()
+            return out
+
+        e2e_step()
+        ctx.stats(reset=True)
+        if world > 1:
+            dist.barrier()
+        torch.cuda.synchronize()
+        t0 = time.perf_counter()
+        for _ in range(args.steps):
+            e2e_step()
+        torch.cuda.synchronize()
+        dt = (time.perf_counter() - t0) / args.steps
+        _, h2d, d2h = ctx.stats(reset=True)
+        if world > 1:
+            t = torch.tensor([dt], device="cuda", dtype=torch.float64)
+            dist.all_reduce(t, op=dist.ReduceOp.MAX)
+            dt = float(t[0])
+        e2e = {"value": len(queries) * total_rows / dt, "unit": UNIT,
+               "h2d_bytes_per_step": h2d // args.steps, "d2h_bytes_per_step": d2h // args.steps,
+               "ms_per_step": dt * 1e3,
+               "path": "hx_load_columns(pinned host -> HBM) + 13 x (hx_build_dim_ht.. + "
+                       "hx_pipeline_probe_agg + hx_merge_aggregates -> host)"}
+
+    cpu = None
+    if rank == 0 and world == 1 and not args.no_cpu_baseline:
+        cpu = cpu_baseline(args, world)
+
+    if rank == 0:
+        n_sms, ctas = ctx.info()
+        line = {"metric": METRIC, "value": value, "unit": UNIT, "n_gpus": world,
+                "steps": args.steps, "warmup": args.warmup, "ms_per_step": ms_step,
+                "higher_is_better": True, "scaling": "weak", "vs_baseline": None,
+                "dtype": "int32 columns, int64 accumulate",
+                "data": f"synthetic (ssbgen dbgen-shaped SSB distributions, seed {SEED}), "
+                        "generated in HBM",
+                "config": config(args, world, n_mine, queries),
+                "hbm_gbps_per_gpu": sum(n_mine * B[q] for q in queries) / (ms_step / 1e3) / 1e9,
+                "roofline": roofline, "cpu_baseline": cpu, "e2e": e2e, "clocks": clk,
+                "gpu_launches": launches, "per_query": per_query,
+                "k1_ctas_per_sm": ctas, "n_sms": n_sms}
+        print(json.dumps(line), flush=True)
+    # release library objects before their context
+    if graph is not None:
+        graph.close()
+    for pl in plans.values():
+        pl.close()
+    for t in list(dims.values()) + [fact]:
+        t.close()
+    ctx.close()
+    if world > 1:
+        dist.destroy_process_group()
+
+
+if __name__ == "__main__":
+    main()

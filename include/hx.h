@@ -110,8 +110,8 @@ int hx_table_free(hx_table* t);
  * manager), PAPER.md:231-233 (build-phase atomics).
  * Rows of `dim` passing the AND of `preds` (range lo <= v <= hi, or v IN in[0..n_in)) are
  * inserted as key -> rank into an open-addressing table in HBM (linear probing, 8-byte
- * slots {int32 key, int32 rank}, capacity the power of two >= 2*n_pass, min 16), built
- * with warp-cooperative CAS inserts. If group_col >= 0 its values must lie in
+ * slots {int32 key, int32 rank} in 16-byte buckets, capacity the power of two >=
+ * 4*n_pass, min 16), built with warp-cooperative CAS inserts. Key -1 is reserved. If group_col >= 0 its values must lie in
  * [group_lo, group_hi]; rank = position of the row's group code among the DISTINCT codes
  * of the passing rows in ascending order (dense ranks; rank_to_code recovers the code).
  * group_col < 0: membership only, rank 0, one rank.
@@ -194,6 +194,47 @@ int hx_merge_aggregates(hx_ctx* ctx, hx_agg* agg, int root, int64_t* sums, int64
                         int32_t* keys, int64_t cap, int64_t* n_rows);
 int hx_agg_free(hx_agg* agg);
 
+/* ---- prepared plans and CUDA graphs (the native runtime around K1/K2) ----------------
+ * PAPER.md:769-790 §4.1 (pipelines are generated and compiled once per query, then run),
+ * PAPER.md:1043-1050 §4.3 (block arenas pre-allocated at initialisation: no allocation at
+ * query time). A plan bundles one query's dimension builds (builds[j] builds the table
+ * that shape->join_ht indexes: join_ht[j] is an index into builds[]), the fused pipeline
+ * over `fact`, the union-router merge (NCCL allreduce of the partial group arrays when the
+ * ctx has > 1 ranks) and the finalize step (a7: empty groups dropped, group codes decoded)
+ * ON THE DEVICE, with the result copied into pinned host memory. hx_plan_create allocates
+ * everything and runs the builds once, synchronously, to size the group arrays exactly;
+ * hx_plan_enqueue is asynchronous, allocation-free and free of host synchronisation, so a
+ * sequence of enqueues can be captured into a CUDA graph (hx_graph_*) and replayed. If the
+ * dimensions change so that the group count differs from the plan's, the execution reports
+ * HX_ECAPACITY (re-create the plan). The fact table and dims must outlive the plan. */
+typedef struct {
+  int32_t dim;                 /* index into the dims[] array of hx_plan_create   */
+  int32_t key_col;
+  int32_t n_preds;
+  hx_pred preds[HX_MAX_PREDS];
+  int32_t group_col;           /* -1: membership only                              */
+  int32_t group_lo, group_hi;
+} hx_build_spec;
+typedef struct hx_plan hx_plan;
+int hx_plan_create(hx_ctx* ctx, const hx_table* fact, hx_table* const* dims, int n_dims,
+                   const hx_build_spec* builds, int n_builds, const hx_query_shape* shape,
+                   hx_plan** out);
+int hx_plan_enqueue(hx_ctx* ctx, hx_plan* plan);
+/* Waits for the last enqueued execution; rows as hx_merge_aggregates (group-index order). */
+int hx_plan_result(hx_plan* plan, int64_t* sums, int64_t* counts, int32_t* keys, int64_t cap,
+                   int64_t* n_rows);
+/* K1 device time of the last execution (CUDA events around the launch) and its
+   algorithmic bytes (rows x 4 B x distinct fact columns). Waits for the execution. */
+int hx_plan_k1_time(hx_plan* plan, float* ms, int64_t* bytes);
+int hx_plan_info(hx_plan* plan, int64_t* n_groups, int* n_gdims);
+int hx_plan_free(hx_plan* plan);
+typedef struct hx_graph hx_graph;
+/* Capture every hx_plan_enqueue between begin and end on the ctx stream into a graph. */
+int hx_graph_begin(hx_ctx* ctx);
+int hx_graph_end(hx_ctx* ctx, hx_graph** out);
+int hx_graph_launch(hx_ctx* ctx, hx_graph* graph);
+int hx_graph_free(hx_graph* graph);
+
 /* ---- measurement ------------------------------------------------------------------
  * When enabled, CUDA events bracket every K1 launch on the ctx stream. hx_profile_read
  * synchronises and returns the summed K1 device time (ms), launch count and algorithmic
@@ -201,6 +242,9 @@ int hx_agg_free(hx_agg* agg);
 int hx_profile_enable(hx_ctx* ctx, int on);
 int hx_profile_read(hx_ctx* ctx, double* k1_ms, int64_t* k1_launches, int64_t* k1_bytes,
                     int reset);
+/* Counters since the last reset: kernels libhx launched, bytes it copied host->device
+   (hx_load_columns from host memory) and device->host (hx_merge_aggregates, hx_ht_info). */
+int hx_stats(hx_ctx* ctx, int64_t* launches, int64_t* h2d_bytes, int64_t* d2h_bytes, int reset);
 
 #ifdef __cplusplus
 }

@@ -54,6 +54,12 @@ class hx_query_shape(ctypes.Structure):
                 ("n_gdims", ctypes.c_int32), ("gdim_join", ctypes.c_int32 * HX_MAX_GDIMS)]
 
 
+class hx_build_spec(ctypes.Structure):
+    _fields_ = [("dim", ctypes.c_int32), ("key_col", ctypes.c_int32), ("n_preds", ctypes.c_int32),
+                ("preds", hx_pred * HX_MAX_PREDS), ("group_col", ctypes.c_int32),
+                ("group_lo", ctypes.c_int32), ("group_hi", ctypes.c_int32)]
+
+
 _P = ctypes.c_void_p
 _PP = ctypes.POINTER(ctypes.c_void_p)
 _I = ctypes.c_int
@@ -89,6 +95,18 @@ _SIGS = {
     "hx_agg_free": ([_P], _I),
     "hx_profile_enable": ([_P, _I], _I),
     "hx_profile_read": ([_P, ctypes.POINTER(ctypes.c_double), _PI64, _PI64, _I], _I),
+    "hx_stats": ([_P, _PI64, _PI64, _PI64, _I], _I),
+    "hx_plan_create": ([_P, _P, _PP, _I, ctypes.POINTER(hx_build_spec), _I,
+                        ctypes.POINTER(hx_query_shape), _PP], _I),
+    "hx_plan_enqueue": ([_P, _P], _I),
+    "hx_plan_result": ([_P, _PI64, _PI64, _PI32, _I64, _PI64], _I),
+    "hx_plan_k1_time": ([_P, ctypes.POINTER(ctypes.c_float), _PI64], _I),
+    "hx_plan_info": ([_P, _PI64, ctypes.POINTER(_I)], _I),
+    "hx_plan_free": ([_P], _I),
+    "hx_graph_begin": ([_P], _I),
+    "hx_graph_end": ([_P, _PP], _I),
+    "hx_graph_launch": ([_P, _P], _I),
+    "hx_graph_free": ([_P], _I),
 }
 EXPORTED = sorted(_SIGS)
 

@@ -253,6 +253,11 @@ int hx_load_columns(hx_ctx* ctx, const hx_col* cols, int n_cols, const hx_partit
     t->owned = true;
     for (int c = 0; c < n_cols; ++c) {
       t->dev[c] = nullptr;
+      cudaPointerAttributes pa{};
+      bool src_host = true;
+      if (n > 0 && cudaPointerGetAttributes(&pa, cols[c].data) == cudaSuccess)
+        src_host = pa.type != cudaMemoryTypeDevice && pa.type != cudaMemoryTypeManaged;
+      cudaGetLastError();
       if (n == 0) continue;
       cudaError_t e = cudaMallocAsync(&t->dev[c], ((size_t)n * 4 + 255) & ~size_t(255), ctx->stream);
       if (e != cudaSuccess) {
@@ -264,6 +269,7 @@ int hx_load_columns(hx_ctx* ctx, const hx_col* cols, int n_cols, const hx_partit
       for (auto& r : ranges) {
         HX_CK(cudaMemcpyAsync(t->dev[c] + off, cols[c].data + r.first,
                               (size_t)(r.second - r.first) * 4, cudaMemcpyDefault, ctx->stream));
+        if (src_host) ctx->h2d_bytes += (r.second - r.first) * 4;
         off += r.second - r.first;
       }
     }
@@ -376,8 +382,7 @@ int hx_ht_broadcast(hx_ctx* ctx, hx_ht* ht, int root) {
 int hx_ht_free(hx_ht* ht) {
   HX_REQUIRE(ht, HX_EINVAL, "hx_ht_free: null table");
   cudaSetDevice(ht->ctx->device);
-  if (ht->base) cudaFreeAsync(ht->base, ht->ctx->stream);
-  delete ht;
+  ht_destroy(ht);
   return HX_OK;
 }
 
@@ -455,6 +460,8 @@ int hx_merge_aggregates(hx_ctx* ctx, hx_agg* agg, int root, int64_t* sums, int64
                             cudaMemcpyDeviceToHost, ctx->stream));
   }
   HX_CK(cudaStreamSynchronize(ctx->stream));
+  ctx->d2h_bytes += (int64_t)sizeof(m) + 16 * ng;
+  for (int g = 0; g < agg->n_gdims; ++g) ctx->d2h_bytes += 4 * (int64_t)r2c[g].size();
   // finalize (a7): drop empty groups (an ungrouped query keeps its one row), decode codes
   int64_t rows = 0;
   for (int64_t i = 0; i < ng; ++i) {
@@ -516,6 +523,15 @@ int hx_profile_read(hx_ctx* ctx, double* k1_ms, int64_t* k1_launches, int64_t* k
     ctx->prof_launches = 0;
     ctx->prof_bytes = 0;
   }
+  return HX_OK;
+}
+
+int hx_stats(hx_ctx* ctx, int64_t* launches, int64_t* h2d_bytes, int64_t* d2h_bytes, int reset) {
+  HX_REQUIRE(ctx, HX_EINVAL, "hx_stats: null ctx");
+  if (launches) *launches = ctx->launches;
+  if (h2d_bytes) *h2d_bytes = ctx->h2d_bytes;
+  if (d2h_bytes) *d2h_bytes = ctx->d2h_bytes;
+  if (reset) ctx->launches = ctx->h2d_bytes = ctx->d2h_bytes = 0;
   return HX_OK;
 }
 

@@ -7,8 +7,9 @@
 // this is a B200-first design:
 //   * one HBM allocation per table (header, dense-rank maps, slot array) so the fused
 //     probe kernel sees one L2-friendly region;
-//   * 8-byte slots {int32 key, int32 rank} written with one 64-bit CAS, linear probing,
-//     capacity = next pow2 >= 2 * passing rows (load factor <= 0.5), Fibonacci hashing;
+//   * 8-byte slots {int32 key, int32 rank} written with one 64-bit CAS, linear probing from
+//     the first slot of a 16-byte bucket (one 128-bit load per probe step), capacity = next
+//     pow2 >= 4 * passing rows (load factor <= 0.25), Fibonacci hashing;
 //   * sizing happens ON THE DEVICE (count kernel -> rank kernel writes log2cap), so a query
 //     enqueues build -> probe -> merge with no host round trip (CUDA-graph capturable);
 //   * inserts are warp-cooperative: the warp takes one pending key at a time and inspects
@@ -52,6 +53,7 @@ __global__ void k2_filter_mark(BuildParams p) {
   for (int64_t i = (int64_t)blockIdx.x * blockDim.x + threadIdx.x; i < p.n_rows; i += stride) {
     if (!row_pass(p, i)) continue;
     ++local;
+    if (__ldg(p.key + i) == kEmptyKey) atomicExch(&p.hdr->error, HX_EINVAL);  // reserved key
     if (p.group) {
       int32_t code = __ldg(p.group + i) - p.group_lo;
       if (code < 0 || code >= p.domain)
@@ -92,7 +94,7 @@ __global__ void k2_rank(BuildParams p) {
   if (threadIdx.x == 0) {
     int n = p.hdr->n_keys;
     int lg = kMinLog2Cap;
-    while (lg < p.max_log2cap && (1ll << lg) < 2ll * n) ++lg;
+    while (lg < p.max_log2cap && (1ll << lg) < (long long)kLoadInv * n) ++lg;
     p.hdr->log2cap = lg;
     p.hdr->n_ranks = p.group ? running : 1;
     p.hdr->max_log2cap = p.max_log2cap;
@@ -177,9 +179,9 @@ int ceil_log2(int64_t x) {
 
 }  // namespace
 
-int build_dim_ht(hx_ctx* ctx, const hx_table* dim, int32_t key_col, const hx_pred* preds,
-                 int n_preds, int32_t group_col, int32_t group_lo, int32_t group_hi,
-                 hx_ht** out) {
+// Validate a build and allocate its table (no kernels launched).
+int ht_create(hx_ctx* ctx, const hx_table* dim, int32_t key_col, const hx_pred* preds,
+              int n_preds, int32_t group_col, int32_t group_lo, int32_t group_hi, hx_ht** out) {
   HX_REQUIRE(ctx && dim && out, HX_EINVAL, "hx_build_dim_ht: null argument");
   HX_REQUIRE(n_preds >= 0 && n_preds <= HX_MAX_PREDS && (n_preds == 0 || preds), HX_EINVAL,
              "hx_build_dim_ht: bad predicate list");
@@ -210,7 +212,7 @@ int build_dim_ht(hx_ctx* ctx, const hx_table* dim, int32_t key_col, const hx_pre
   p.n_rows = dim->n_rows;
   p.group_lo = group_lo;
   p.domain = (int32_t)domain;
-  p.max_log2cap = std::max(kMinLog2Cap, ceil_log2(2 * std::max<int64_t>(dim->n_rows, 1)));
+  p.max_log2cap = std::max(kMinLog2Cap, ceil_log2(kLoadInv * std::max<int64_t>(dim->n_rows, 1)));
 
   hx_ht* ht = new hx_ht();
   ht->ctx = ctx;
@@ -234,10 +236,17 @@ int build_dim_ht(hx_ctx* ctx, const hx_table* dim, int32_t key_col, const hx_pre
   p.c2r = ht->code_to_rank;
   p.r2c = ht->rank_to_code;
   p.slots = ht->slots;
+  ht->build = new BuildParams(p);
   *out = ht;
+  return HX_OK;
+}
 
-  HX_CK(cudaMemsetAsync(ht->base, 0, sizeof(HtHeader) + domain * sizeof(int32_t), ctx->stream));
-  const int64_t want = (dim->n_rows + 255) / 256;
+// Enqueue the four build kernels (asynchronous; CUDA-graph capturable). Re-running a build
+// on the same table rebuilds it from scratch.
+int ht_enqueue_build(hx_ctx* ctx, hx_ht* ht) {
+  const BuildParams& p = *static_cast<const BuildParams*>(ht->build);
+  HX_CK(cudaMemsetAsync(ht->base, 0, sizeof(HtHeader) + p.domain * sizeof(int32_t), ctx->stream));
+  const int64_t want = (p.n_rows + 255) / 256;
   const int grid = (int)std::max<int64_t>(1, std::min<int64_t>(want, (int64_t)ctx->n_sms * 8));
   k2_filter_mark<<<grid, 256, 0, ctx->stream>>>(p);
   HX_CK_LAUNCH("k2_filter_mark");
@@ -249,6 +258,28 @@ int build_dim_ht(hx_ctx* ctx, const hx_table* dim, int32_t key_col, const hx_pre
   HX_CK_LAUNCH("k2_clear");
   k2_insert<<<grid, 256, 0, ctx->stream>>>(p);
   HX_CK_LAUNCH("k2_insert");
+  ctx->launches += 4;
+  return HX_OK;
+}
+
+void ht_destroy(hx_ht* ht) {
+  if (ht->base) cudaFreeAsync(ht->base, ht->ctx->stream);
+  delete static_cast<BuildParams*>(ht->build);
+  delete ht;
+}
+
+int build_dim_ht(hx_ctx* ctx, const hx_table* dim, int32_t key_col, const hx_pred* preds,
+                 int n_preds, int32_t group_col, int32_t group_lo, int32_t group_hi,
+                 hx_ht** out) {
+  hx_ht* ht = nullptr;
+  int rc = ht_create(ctx, dim, key_col, preds, n_preds, group_col, group_lo, group_hi, &ht);
+  if (rc != HX_OK) return rc;
+  rc = ht_enqueue_build(ctx, ht);
+  if (rc != HX_OK) {
+    ht_destroy(ht);
+    return rc;
+  }
+  *out = ht;
   return HX_OK;
 }
 

@@ -43,9 +43,20 @@ struct HtHeader {
   int32_t n_inserted;
 };
 
-// Multiplicative (Fibonacci) hashing: the top log2cap bits of key * 2^32/phi.
+// Slots are grouped in 16-byte buckets of kBucketSlots = 2 (one 128-bit load per probe
+// step). A key's home is the first slot of its bucket; linear probing proceeds slot by
+// slot from there, so within a bucket slot 1 is filled only after slot 0 and "slot 1 of the
+// bucket is empty" proves a miss. Load factor <= 1/kLoadInv.
+constexpr int kBucketSlots = 2;
+constexpr int kLoadInv = 4;
+constexpr int32_t kEmptyKey = -1;  // keys must differ from -1 (checked by the build)
+
+// Multiplicative (Fibonacci) hashing: the top log2(cap/2) bits of key * 2^32/phi.
+__host__ __device__ __forceinline__ uint32_t ht_bucket(int32_t key, int log2cap) {
+  return ((uint32_t)key * 2654435769u) >> (33 - log2cap);
+}
 __host__ __device__ __forceinline__ uint32_t ht_home(int32_t key, int log2cap) {
-  return ((uint32_t)key * 2654435769u) >> (32 - log2cap);
+  return ht_bucket(key, log2cap) << 1;
 }
 
 // Device-side predicate (a copy of hx_pred with the column resolved to a pointer or a
@@ -83,6 +94,9 @@ struct hx_ctx {
   std::vector<cudaEvent_t> event_pool;
   int64_t prof_launches = 0, prof_bytes = 0;
   double prof_ms = 0.0;
+  // hx_stats counters
+  int64_t launches = 0, h2d_bytes = 0, d2h_bytes = 0;
+  int64_t capture_launches = 0, capture_d2h = 0;  // counters at hx_graph_begin
 };
 
 struct hx_partition {
@@ -115,6 +129,7 @@ struct hx_ht {
   int32_t group_lo = 0;
   bool has_group = false;
   int64_t dim_rows = 0;
+  void* build = nullptr;           // hx::BuildParams (hx_build.cu): re-enqueueable build
 };
 
 struct hx_agg {
@@ -143,10 +158,33 @@ namespace hx {
 int build_dim_ht(hx_ctx* ctx, const hx_table* dim, int32_t key_col, const hx_pred* preds,
                  int n_preds, int32_t group_col, int32_t group_lo, int32_t group_hi,
                  hx_ht** out);
+int ht_create(hx_ctx* ctx, const hx_table* dim, int32_t key_col, const hx_pred* preds,
+              int n_preds, int32_t group_col, int32_t group_lo, int32_t group_hi, hx_ht** out);
+int ht_enqueue_build(hx_ctx* ctx, hx_ht* ht);
+void ht_destroy(hx_ht* ht);
 int probe_agg(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* shape,
               hx_ht* const* hts, int n_hts, hx_agg* agg, bool fresh);
 int k1_occupancy(hx_ctx* ctx);
+struct K1Prepared;  // a resolved K1 launch (hx_probe.cu)
+long long k1_group_bound(const hx_query_shape* sh, hx_ht* const* hts, int n_hts);
+int agg_alloc(hx_ctx* ctx, hx_agg* agg, long long cap_groups, const hx_query_shape* sh,
+              hx_ht* const* hts);
+int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht* const* hts,
+             int n_hts, const hx_agg* agg, K1Prepared** out);
+int k1_enqueue(hx_ctx* ctx, const K1Prepared* k, bool fresh, cudaEvent_t e0, cudaEvent_t e1);
+void k1_free(K1Prepared* k);
+int64_t k1_bytes(const K1Prepared* k);
 const int32_t* table_col(const hx_table* t, int32_t col_id);
 bool table_has_col(const hx_table* t, int32_t col_id);
 cudaEvent_t pooled_event(hx_ctx* ctx);
+
+// Record `e` on `s`; under stream capture it becomes an external event-record node of the
+// graph (so the host can wait on / time each replay), otherwise a plain record.
+inline cudaError_t record_event(cudaEvent_t e, cudaStream_t s) {
+  cudaStreamCaptureStatus st = cudaStreamCaptureStatusNone;
+  cudaError_t r = cudaStreamIsCapturing(s, &st);
+  if (r != cudaSuccess) return r;
+  return st == cudaStreamCaptureStatusActive ? cudaEventRecordWithFlags(e, s, cudaEventRecordExternal)
+                                             : cudaEventRecord(e, s);
+}
 }  // namespace hx

@@ -1,0 +1,361 @@
+// hx_plan.cu — prepared query plans and CUDA-graph capture (the native runtime around K1/K2).
+//
+// PAPER.md:769-790 §4.1: a query is split into pipelines that are compiled once and then
+// executed; §4.2: parallelism and affinity are fixed when the pipeline
+// instances are created; §4.3: memory is pre-allocated at initialisation
+// so that query execution does not allocate. A plan is that for one SSB query on one GPU:
+// creation validates the shape, allocates every buffer (hash tables, group arrays, result
+// buffer in pinned host memory) and runs the builds once to size the group arrays exactly;
+// execution (hx_plan_enqueue) is then one asynchronous, allocation-free, sync-free sequence
+//   K2 builds -> K1 prepare -> K1 -> [NCCL allreduce of the partials] -> finalize -> D2H
+// that a CUDA graph can capture, so a whole SSB step replays with one launch.
+#include <cub/block/block_scan.cuh>
+
+#include <algorithm>
+#include <cstring>
+
+#include "hx_internal.cuh"
+
+namespace hx {
+namespace {
+
+constexpr int kOutInline = 4096;  // result rows copied to the host by every execution
+
+struct OutHeader {
+  long long n_rows;
+  long long n_groups;
+  int32_t error;
+  int32_t n_gdims;
+  int32_t pad[10];
+};
+static_assert(sizeof(OutHeader) == 64, "OutHeader is 64 bytes");
+
+struct OutRow {
+  long long sum;
+  long long cnt;
+  int32_t key[HX_MAX_GDIMS];
+  int32_t pad;
+};
+static_assert(sizeof(OutRow) == 32, "OutRow is 32 bytes");
+
+struct FinalizeArgs {
+  const AggMeta* meta;
+  const unsigned long long* sums;
+  const unsigned long long* cnts;
+  int32_t n_gdims;
+  const int32_t* r2c[HX_MAX_GDIMS];       // nullptr: membership-only dimension (code 0)
+  const HtHeader* deps[HX_MAX_JOINS];
+  int32_t n_deps;
+  long long expect_groups;                 // the plan's group count (-1: any)
+  OutHeader* hdr;
+  OutRow* rows;
+  long long out_cap;
+};
+
+// a7 Finalize on the device: ordered compaction of the non-empty groups (a query without
+// GROUP BY keeps its one row) and decoding of each group index into dictionary codes.
+__global__ void k1_finalize(FinalizeArgs a) {
+  using Scan = cub::BlockScan<int, 1024>;
+  __shared__ typename Scan::TempStorage tmp;
+  __shared__ long long running;
+  const long long n = a.meta->n_groups;
+  int err = a.meta->error;
+  for (int d = 0; d < a.n_deps && !err; ++d) err = a.deps[d]->error;
+  if (!err && a.expect_groups >= 0 && n != a.expect_groups) err = HX_ECAPACITY;
+  if (threadIdx.x == 0) running = 0;
+  __syncthreads();
+  if (!err) {
+    for (long long base = 0; base < n; base += 1024) {
+      const long long g = base + threadIdx.x;
+      const int flag = g < n && (a.n_gdims == 0 || a.cnts[g] > 0);
+      int excl, total;
+      Scan(tmp).ExclusiveSum(flag, excl, total);
+      const long long pos = running + excl;
+      if (flag && pos < a.out_cap) {
+        OutRow r{};
+        r.sum = (long long)a.sums[g];
+        r.cnt = (long long)a.cnts[g];
+        long long rem = g;
+        for (int d = a.n_gdims - 1; d >= 0; --d) {
+          const long long nr = a.meta->n_ranks[d] > 0 ? a.meta->n_ranks[d] : 1;
+          const int rank = (int)(rem % nr);
+          rem /= nr;
+          r.key[d] = a.r2c[d] ? a.r2c[d][rank] : 0;
+        }
+        a.rows[pos] = r;
+      }
+      __syncthreads();
+      if (threadIdx.x == 0) running += total;
+      __syncthreads();
+    }
+  }
+  if (threadIdx.x == 0) {
+    OutHeader h{};
+    h.n_rows = err ? 0 : running;
+    h.n_groups = n;
+    h.error = err;
+    h.n_gdims = a.n_gdims;
+    *a.hdr = h;
+  }
+}
+
+}  // namespace
+}  // namespace hx
+
+using namespace hx;
+
+struct hx_plan {
+  hx_ctx* ctx = nullptr;
+  std::vector<hx_ht*> hts;
+  hx_agg agg;
+  K1Prepared* k1 = nullptr;
+  long long n_groups = 1;
+  FinalizeArgs fin{};
+  void* d_out = nullptr;
+  void* h_out = nullptr;       // pinned
+  size_t out_bytes = 0, inline_bytes = 0;
+  cudaEvent_t done = nullptr, k1_e0 = nullptr, k1_e1 = nullptr;
+  bool enqueued = false;
+};
+
+struct hx_graph {
+  hx_ctx* ctx = nullptr;
+  cudaGraph_t graph = nullptr;
+  cudaGraphExec_t exec = nullptr;
+  int64_t launches = 0;
+  int64_t d2h = 0;
+};
+
+static void plan_destroy(hx_plan* pl) {
+  if (!pl) return;
+  cudaSetDevice(pl->ctx->device);
+  cudaStreamSynchronize(pl->ctx->stream);
+  for (hx_ht* t : pl->hts) ht_destroy(t);
+  if (pl->agg.base) cudaFreeAsync(pl->agg.base, pl->ctx->stream);
+  if (pl->k1) k1_free(pl->k1);
+  if (pl->d_out) cudaFreeAsync(pl->d_out, pl->ctx->stream);
+  if (pl->h_out) cudaFreeHost(pl->h_out);
+  for (cudaEvent_t e : {pl->done, pl->k1_e0, pl->k1_e1})
+    if (e) cudaEventDestroy(e);
+  delete pl;
+}
+
+extern "C" {
+
+int hx_plan_create(hx_ctx* ctx, const hx_table* fact, hx_table* const* dims, int n_dims,
+                   const hx_build_spec* builds, int n_builds, const hx_query_shape* shape,
+                   hx_plan** out) {
+  HX_REQUIRE(ctx && fact && shape && out && (n_builds == 0 || (builds && dims)), HX_EINVAL,
+             "hx_plan_create: null argument");
+  HX_REQUIRE(n_builds >= 0 && n_builds <= HX_MAX_JOINS, HX_EINVAL, "hx_plan_create: bad n_builds");
+  HX_CK(cudaSetDevice(ctx->device));
+  hx_plan* pl = new hx_plan();
+  pl->ctx = ctx;
+  pl->agg.ctx = ctx;
+  auto bail = [&](int rc) {
+    plan_destroy(pl);
+    return rc;
+  };
+  // 1) hash tables: allocate, build once
+  for (int b = 0; b < n_builds; ++b) {
+    const hx_build_spec& s = builds[b];
+    if (s.dim < 0 || s.dim >= n_dims || !dims[s.dim] || s.n_preds < 0 || s.n_preds > HX_MAX_PREDS)
+      return bail(fail(HX_EINVAL, "hx_plan_create: bad build spec"));
+    hx_ht* ht = nullptr;
+    int rc = ht_create(ctx, dims[s.dim], s.key_col, s.preds, s.n_preds, s.group_col, s.group_lo,
+                       s.group_hi, &ht);
+    if (rc != HX_OK) return bail(rc);
+    pl->hts.push_back(ht);
+    rc = ht_enqueue_build(ctx, ht);
+    if (rc != HX_OK) return bail(rc);
+  }
+  // 2) exact group count from the built tables (the plan's one synchronisation)
+  const long long bound = k1_group_bound(shape, pl->hts.data(), n_builds);
+  if (bound < 1 || shape->n_joins > HX_MAX_JOINS || shape->n_gdims > HX_MAX_GDIMS)
+    return bail(fail(HX_EINVAL, "hx_plan_create: bad gdim_join / join_ht"));
+  std::vector<HtHeader> hh(n_builds);
+  for (int b = 0; b < n_builds; ++b) {
+    cudaError_t e = cudaMemcpyAsync(&hh[b], pl->hts[b]->hdr, sizeof(HtHeader),
+                                    cudaMemcpyDeviceToHost, ctx->stream);
+    if (e != cudaSuccess) return bail(cuda_fail(e, "cudaMemcpyAsync", __FILE__, __LINE__));
+  }
+  {
+    cudaError_t e = cudaStreamSynchronize(ctx->stream);
+    if (e != cudaSuccess) return bail(cuda_fail(e, "cudaStreamSynchronize", __FILE__, __LINE__));
+  }
+  for (int b = 0; b < n_builds; ++b) {
+    if (hh[b].error == HX_EDUPKEY) return bail(fail(HX_EDUPKEY, "dimension build: duplicate primary key"));
+    if (hh[b].error) return bail(fail(HX_EINVAL, "dimension build: bad key or group code"));
+  }
+  long long ng = 1;
+  for (int g = 0; g < shape->n_gdims; ++g) ng *= std::max(1, hh[shape->join_ht[shape->gdim_join[g]]].n_ranks);
+  if (ng > HX_MAX_GROUPS) return bail(fail(HX_ECAPACITY, "hx_plan_create: too many groups"));
+  pl->n_groups = ng;
+  int rc = agg_alloc(ctx, &pl->agg, ng, shape, pl->hts.data());
+  if (rc != HX_OK) return bail(rc);
+  for (int j = 0; j < shape->n_joins; ++j) pl->agg.deps.push_back(pl->hts[shape->join_ht[j]]);
+  // 3) the K1 launch
+  rc = k1_setup(ctx, fact, shape, pl->hts.data(), n_builds, &pl->agg, &pl->k1);
+  if (rc != HX_OK) return bail(rc);
+  // 4) result buffers
+  pl->out_bytes = sizeof(OutHeader) + (size_t)ng * sizeof(OutRow);
+  pl->inline_bytes = sizeof(OutHeader) + (size_t)std::min<long long>(ng, kOutInline) * sizeof(OutRow);
+  HX_CK(cudaMallocAsync(&pl->d_out, pl->out_bytes, ctx->stream));
+  {
+    cudaError_t e = cudaMallocHost(&pl->h_out, pl->inline_bytes);
+    if (e != cudaSuccess) return bail(cuda_fail(e, "cudaMallocHost", __FILE__, __LINE__));
+  }
+  FinalizeArgs& f = pl->fin;
+  f.meta = pl->agg.meta;
+  f.sums = pl->agg.sums;
+  f.cnts = pl->agg.cnts;
+  f.n_gdims = shape->n_gdims;
+  for (int g = 0; g < shape->n_gdims; ++g) {
+    const hx_ht* ht = pl->agg.gdim_ht[g];
+    f.r2c[g] = ht->has_group ? ht->rank_to_code : nullptr;
+  }
+  f.n_deps = (int)pl->agg.deps.size();
+  for (int d = 0; d < f.n_deps; ++d) f.deps[d] = pl->agg.deps[d]->hdr;
+  f.expect_groups = ng;
+  f.hdr = static_cast<OutHeader*>(pl->d_out);
+  f.rows = reinterpret_cast<OutRow*>(f.hdr + 1);
+  f.out_cap = ng;
+  for (cudaEvent_t* e : {&pl->done, &pl->k1_e0, &pl->k1_e1}) {
+    cudaError_t err = cudaEventCreate(e);
+    if (err != cudaSuccess) return bail(cuda_fail(err, "cudaEventCreate", __FILE__, __LINE__));
+  }
+  *out = pl;
+  return HX_OK;
+}
+
+int hx_plan_enqueue(hx_ctx* ctx, hx_plan* pl) {
+  HX_REQUIRE(ctx && pl && pl->ctx == ctx, HX_EINVAL, "hx_plan_enqueue: bad argument");
+  HX_CK(cudaSetDevice(ctx->device));
+  for (hx_ht* ht : pl->hts) {
+    int rc = ht_enqueue_build(ctx, ht);
+    if (rc != HX_OK) return rc;
+  }
+  int rc = k1_enqueue(ctx, pl->k1, true, pl->k1_e0, pl->k1_e1);
+  if (rc != HX_OK) return rc;
+  if (ctx->comm && ctx->nranks > 1) {
+    // union router: partial {sum,cnt} arrays are adjacent, one allreduce over NVLink
+    ncclResult_t r = ncclAllReduce(pl->agg.sums, pl->agg.sums, 2 * (size_t)pl->n_groups,
+                                   ncclUint64, ncclSum, ctx->comm, ctx->stream);
+    HX_REQUIRE(r == ncclSuccess, HX_ENCCL, std::string("ncclAllReduce: ") + ncclGetErrorString(r));
+  }
+  k1_finalize<<<1, 1024, 0, ctx->stream>>>(pl->fin);
+  HX_CK_LAUNCH("k1_finalize");
+  ctx->launches += 1;
+  HX_CK(cudaMemcpyAsync(pl->h_out, pl->d_out, pl->inline_bytes, cudaMemcpyDeviceToHost, ctx->stream));
+  ctx->d2h_bytes += (int64_t)pl->inline_bytes;
+  HX_CK(record_event(pl->done, ctx->stream));
+  pl->enqueued = true;
+  return HX_OK;
+}
+
+int hx_plan_result(hx_plan* pl, int64_t* sums, int64_t* counts, int32_t* keys, int64_t cap,
+                   int64_t* n_rows) {
+  HX_REQUIRE(pl && n_rows && cap >= 0 && (cap == 0 || (sums && counts)), HX_EINVAL,
+             "hx_plan_result: bad argument");
+  HX_REQUIRE(pl->enqueued, HX_EINVAL, "hx_plan_result: plan never executed");
+  HX_CK(cudaSetDevice(pl->ctx->device));
+  HX_CK(cudaEventSynchronize(pl->done));
+  const OutHeader* h = static_cast<const OutHeader*>(pl->h_out);
+  *n_rows = 0;
+  if (h->error == HX_EDUPKEY) return fail(HX_EDUPKEY, "dimension build: duplicate primary key");
+  if (h->error == HX_ECAPACITY)
+    return fail(HX_ECAPACITY, "hx_plan: group count changed since the plan was created");
+  if (h->error) return fail(HX_EINVAL, "dimension build: bad key or group code");
+  const int64_t n = h->n_rows;
+  *n_rows = n;
+  if (n > cap) return fail(HX_ECAPACITY, "hx_plan_result: output buffer too small");
+  const OutRow* rows = reinterpret_cast<const OutRow*>(h + 1);
+  std::vector<OutRow> rest;
+  if (n > kOutInline) {  // large results: the rows beyond the inline block
+    rest.resize(n - kOutInline);
+    HX_CK(cudaMemcpy(rest.data(), pl->fin.rows + kOutInline, rest.size() * sizeof(OutRow),
+                     cudaMemcpyDeviceToHost));
+  }
+  const int nd = pl->fin.n_gdims;
+  for (int64_t i = 0; i < n; ++i) {
+    const OutRow& r = i < kOutInline ? rows[i] : rest[i - kOutInline];
+    sums[i] = r.sum;
+    counts[i] = r.cnt;
+    for (int d = 0; d < nd; ++d) keys[i * nd + d] = r.key[d];
+  }
+  return HX_OK;
+}
+
+int hx_plan_k1_time(hx_plan* pl, float* ms, int64_t* bytes) {
+  HX_REQUIRE(pl && pl->enqueued, HX_EINVAL, "hx_plan_k1_time: plan never executed");
+  HX_CK(cudaEventSynchronize(pl->done));
+  if (ms) {
+    *ms = 0.f;
+    if (pl->k1_e0 && k1_bytes(pl->k1) > 0) HX_CK(cudaEventElapsedTime(ms, pl->k1_e0, pl->k1_e1));
+  }
+  if (bytes) *bytes = k1_bytes(pl->k1);
+  return HX_OK;
+}
+
+int hx_plan_info(hx_plan* pl, int64_t* n_groups, int* n_gdims) {
+  HX_REQUIRE(pl, HX_EINVAL, "hx_plan_info: null plan");
+  if (n_groups) *n_groups = pl->n_groups;
+  if (n_gdims) *n_gdims = pl->fin.n_gdims;
+  return HX_OK;
+}
+
+int hx_plan_free(hx_plan* pl) {
+  HX_REQUIRE(pl, HX_EINVAL, "hx_plan_free: null plan");
+  plan_destroy(pl);
+  return HX_OK;
+}
+
+// ---- CUDA graphs ---------------------------------------------------------------------------
+int hx_graph_begin(hx_ctx* ctx) {
+  HX_REQUIRE(ctx, HX_EINVAL, "hx_graph_begin: null ctx");
+  HX_CK(cudaSetDevice(ctx->device));
+  ctx->capture_launches = ctx->launches;
+  ctx->capture_d2h = ctx->d2h_bytes;
+  HX_CK(cudaStreamBeginCapture(ctx->stream, cudaStreamCaptureModeThreadLocal));
+  return HX_OK;
+}
+
+int hx_graph_end(hx_ctx* ctx, hx_graph** out) {
+  HX_REQUIRE(ctx && out, HX_EINVAL, "hx_graph_end: null argument");
+  HX_CK(cudaSetDevice(ctx->device));
+  hx_graph* g = new hx_graph();
+  g->ctx = ctx;
+  cudaError_t e = cudaStreamEndCapture(ctx->stream, &g->graph);
+  if (e == cudaSuccess) e = cudaGraphInstantiate(&g->exec, g->graph, 0);
+  g->launches = ctx->launches - ctx->capture_launches;
+  ctx->launches = ctx->capture_launches;  // captured, not executed
+  g->d2h = ctx->d2h_bytes - ctx->capture_d2h;
+  ctx->d2h_bytes = ctx->capture_d2h;
+  if (e != cudaSuccess) {
+    if (g->graph) cudaGraphDestroy(g->graph);
+    delete g;
+    return cuda_fail(e, "cudaStreamEndCapture/cudaGraphInstantiate", __FILE__, __LINE__);
+  }
+  *out = g;
+  return HX_OK;
+}
+
+int hx_graph_launch(hx_ctx* ctx, hx_graph* g) {
+  HX_REQUIRE(ctx && g && g->ctx == ctx, HX_EINVAL, "hx_graph_launch: bad argument");
+  HX_CK(cudaSetDevice(ctx->device));
+  HX_CK(cudaGraphLaunch(g->exec, ctx->stream));
+  ctx->launches += g->launches;
+  ctx->d2h_bytes += g->d2h;
+  return HX_OK;
+}
+
+int hx_graph_free(hx_graph* g) {
+  HX_REQUIRE(g, HX_EINVAL, "hx_graph_free: null graph");
+  cudaSetDevice(g->ctx->device);
+  if (g->exec) cudaGraphExecDestroy(g->exec);
+  if (g->graph) cudaGraphDestroy(g->graph);
+  delete g;
+  return HX_OK;
+}
+
+}  // extern "C"

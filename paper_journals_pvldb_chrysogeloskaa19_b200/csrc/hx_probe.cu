@@ -35,10 +35,14 @@ constexpr unsigned kFull = 0xFFFFFFFFu;
 constexpr int kConsumerWarps = 8;
 constexpr int kConsumers = kConsumerWarps * 32;
 constexpr int kThreads = kConsumers + 32;  // + one producer warp
-constexpr int kRowsPerThread = 8;          // R
-constexpr int kTileRows = kConsumers * kRowsPerThread;  // T = 2048
+constexpr int kRowsPerThread = 4;          // R
+constexpr int kTileRows = kConsumers * kRowsPerThread;  // T = 1024
+constexpr int kCtasPerSm = 3;             // target residency (registers, smem budget)
 constexpr int kMaxStageCols = 8;
 constexpr int kSmemGroups = 1024;          // per-CTA group table capacity
+// dynamic smem: [barriers 128 | reduce 256 | head 128 | queues 8 x 256 x (1+4) B | groups | tiles]
+constexpr int kSmemQueueOff = 512;
+constexpr int kSmemFixed = kSmemQueueOff + kConsumers * kRowsPerThread * 5;
 
 struct JoinDev {
   int32_t c;                               // staged column of the FK
@@ -123,109 +127,257 @@ __device__ __forceinline__ long long measure(int op, int32_t a, int32_t b) {
   return (long long)a;
 }
 
-// Per-thread view of the join tables (loaded once per CTA).
+// Per-warp view of one join's hash table (loaded once per CTA).
 struct JoinState {
-  const unsigned long long* slots;
-  int32_t c;
-  int32_t log2cap;
-  uint32_t mask;
-  int32_t jstride;
+  const ulonglong2* buckets;  // 16-byte buckets of two {key, rank} slots
+  int32_t c;                  // staged column of the FK
+  int32_t shift;              // 33 - log2cap (bucket hash)
+  uint32_t bmask;             // n_buckets - 1
+  int32_t jstride;            // weight of this join's rank in the group index
 };
 
-// Process the rows {ctid + k*kConsumers : k < R, row < rows_valid} of one staged tile whose
-// column c, row r is at sbase[c * stride + r].
+__device__ __forceinline__ uint32_t bucket_of(int32_t key, int shift) {
+  return ((uint32_t)key * 2654435769u) >> shift;
+}
+
+// One probe step for one row: hit (rank returned), miss, or continue at the next bucket.
+// Within a bucket slot 1 is filled only after slot 0, so an empty slot 1 proves a miss.
+__device__ __forceinline__ void probe_step(const ulonglong2 v, int32_t key, bool& hit, bool& miss,
+                                           int32_t& rank) {
+  const bool h0 = (int32_t)(uint32_t)v.x == key;
+  const bool h1 = (int32_t)(uint32_t)v.y == key;
+  hit = h0 || h1;
+  miss = !hit && (int32_t)(uint32_t)v.y == kEmptyKey;
+  rank = (int32_t)((h0 ? v.x : v.y) >> 32);
+}
+
+// Full probe of one row (loops over buckets until hit or miss).
+__device__ __forceinline__ bool probe_row(const JoinState& j, int32_t key, int32_t& rank) {
+  uint32_t b = bucket_of(key, j.shift);
+  while (true) {
+    bool hit, miss;
+    probe_step(__ldg(j.buckets + b), key, hit, miss, rank);
+    if (hit) return true;
+    if (miss) return false;
+    b = (b + 1) & j.bmask;
+  }
+}
+
+template <bool GROUPED>
+__device__ __forceinline__ void accumulate(const K1Params& p, bool smem_table,
+                                           unsigned long long* s_sum, uint32_t* s_cnt,
+                                           int32_t g, long long m, long long& acc_sum,
+                                           long long& acc_cnt) {
+  if (GROUPED) {
+    if (smem_table) {
+      atomicAdd(s_sum + g, (unsigned long long)m);
+      atomicAdd(s_cnt + g, 1u);
+    } else {
+      atomicAdd(p.g_sum + g, (unsigned long long)m);
+      atomicAdd(p.g_cnt + g, 1ull);
+    }
+  } else {
+    acc_sum += m;
+    acc_cnt += 1;
+  }
+}
+
+// Process one staged tile. Warp w owns rows [w*256, w*256+256) of the tile; lane l holds
+// rows w*256 + k*32 + l (k < 8): conflict-free shared-memory reads. Column c, row r of the
+// tile is at sbase[c * stride + r].
+//   stage A  predicates on lineorder columns, branch-free, for the 8 rows of each lane;
+//   stage B  (no predicates) the first join is probed in place for all 8 rows at once —
+//            8 independent 128-bit L2 loads in flight per lane;
+//   compact  survivors are appended to a per-warp queue with ballot + popc (the GPU
+//            "selection vector"), so the remaining joins and the aggregate run with every
+//            lane busy instead of mostly-masked lanes;
+//   stage C  remaining probes + measure + group-table atomics, two queued rows per lane.
 template <int NJ, bool GROUPED>
 __device__ __forceinline__ void process_tile(const K1Params& p, const JoinState (&js)[HX_MAX_JOINS],
                                              const int32_t* sbase, int stride, int rows_valid,
-                                             int ctid, uint64_t pol_last, bool smem_table,
+                                             int warp, int lane, bool smem_table,
                                              unsigned long long* s_sum, uint32_t* s_cnt,
+                                             uint8_t* q_row, int32_t* q_g,
                                              long long& acc_sum, long long& acc_cnt) {
-  uint32_t alive = 0;
+  const int wbase = warp * (32 * kRowsPerThread);
+  const int32_t* tb = sbase + wbase + lane;
+  uint32_t m = 0;
 #pragma unroll
-  for (int k = 0; k < kRowsPerThread; ++k)
-    alive |= (uint32_t)(ctid + k * kConsumers < rows_valid) << k;
-  // filter: predicates on lineorder columns
+  for (int k = 0; k < kRowsPerThread; ++k) m |= (uint32_t)(wbase + k * 32 + lane < rows_valid) << k;
+  if (__ballot_sync(kFull, m) == 0) return;
+
+  // stage A: lineorder predicates (kind is uniform: one branch per predicate, not per row)
   for (int q = 0; q < p.n_preds; ++q) {
     const DevPred& pr = p.preds[q];
-    const int32_t* sc = sbase + pr.c * stride + ctid;
-#pragma unroll
-    for (int k = 0; k < kRowsPerThread; ++k)
-      if ((alive >> k) & 1u)
-        if (!pred_pass(pr, sc[k * kConsumers])) alive &= ~(1u << k);
-  }
-  int32_t gidx[kRowsPerThread];
-#pragma unroll
-  for (int k = 0; k < kRowsPerThread; ++k) gidx[k] = 0;
-  // probe x k: the R probes of a join are issued before any result is inspected
-#pragma unroll
-  for (int j = 0; j < NJ; ++j) {
-    if (!alive) break;
-    int32_t key[kRowsPerThread];
-    uint32_t h[kRowsPerThread];
-    const int32_t* sc = sbase + js[j].c * stride + ctid;
-#pragma unroll
-    for (int k = 0; k < kRowsPerThread; ++k) {
-      key[k] = ((alive >> k) & 1u) ? sc[k * kConsumers] : 0;
-      h[k] = ht_home(key[k], js[j].log2cap);
-    }
-    uint32_t pending = alive;
-    while (pending) {
-      unsigned long long v[kRowsPerThread];
+    const int32_t* col = tb + pr.c * stride;
+    if (pr.kind == HX_PRED_RANGE) {
+      const uint32_t lo = (uint32_t)pr.lo, span = (uint32_t)pr.hi - (uint32_t)pr.lo;
 #pragma unroll
       for (int k = 0; k < kRowsPerThread; ++k)
-        v[k] = ((pending >> k) & 1u) ? ld_slot(js[j].slots + h[k], pol_last) : 0ull;
+        m &= ~((uint32_t)(((uint32_t)col[k * 32] - lo) > span) << k);
+    } else {
 #pragma unroll
       for (int k = 0; k < kRowsPerThread; ++k) {
-        if (!((pending >> k) & 1u)) continue;
-        if (v[k] == kEmptySlot) {  // miss: the row has no partner in this dimension
-          alive &= ~(1u << k);
-          pending &= ~(1u << k);
-        } else if ((int32_t)(uint32_t)v[k] == key[k]) {
-          gidx[k] += (int32_t)(v[k] >> 32) * js[j].jstride;
-          pending &= ~(1u << k);
+        const int32_t v = col[k * 32];
+        bool ok = false;
+#pragma unroll
+        for (int i = 0; i < 4; ++i) ok |= (i < pr.n_in) && v == pr.in[i];
+        m &= ~((uint32_t)(!ok) << k);
+      }
+    }
+  }
+
+  int32_t g[kRowsPerThread];
+#pragma unroll
+  for (int k = 0; k < kRowsPerThread; ++k) g[k] = 0;
+  int j0 = 0;
+  if (NJ > 0 && p.n_preds == 0) {
+    // stage B: ONE probe step of the first join for all R rows of the lane (R independent
+    // 128-bit loads in flight). Rows whose bucket was full without a verdict (rare at load
+    // factor 1/4) are queued with ~next_bucket in place of the group index and finish in
+    // stage C, so the warp never waits on its longest probe chain here.
+    const JoinState& j = js[0];
+    const int32_t* col = tb + j.c * stride;
+    ulonglong2 v[kRowsPerThread];
+    int32_t key[kRowsPerThread];
+    uint32_t b[kRowsPerThread];
+#pragma unroll
+    for (int k = 0; k < kRowsPerThread; ++k) {
+      key[k] = col[k * 32];
+      b[k] = bucket_of(key[k], j.shift);
+      if ((m >> k) & 1u) v[k] = __ldg(j.buckets + b[k]);
+    }
+#pragma unroll
+    for (int k = 0; k < kRowsPerThread; ++k) {
+      if (!((m >> k) & 1u)) continue;
+      bool hit, miss;
+      int32_t rank;
+      probe_step(v[k], key[k], hit, miss, rank);
+      g[k] = hit ? rank * j.jstride : (int32_t)~((b[k] + 1) & j.bmask);
+      m &= ~((uint32_t)miss << k);
+    }
+    j0 = 1;
+  }
+
+  if (NJ == 0) {
+    const int32_t* ca = tb + p.agg_a * stride;
+    const int32_t* cb = tb + p.agg_b * stride;
+#pragma unroll
+    for (int k = 0; k < kRowsPerThread; ++k)
+      if ((m >> k) & 1u)
+        accumulate<GROUPED>(p, smem_table, s_sum, s_cnt, g[k],
+                            measure(p.agg_op, ca[k * 32], cb[k * 32]), acc_sum, acc_cnt);
+    return;
+  }
+
+  // compaction: append this warp's survivors to its queue
+  int qn = 0;
+  const uint32_t lt = (1u << lane) - 1u;
+#pragma unroll
+  for (int k = 0; k < kRowsPerThread; ++k) {
+    const bool a = (m >> k) & 1u;
+    const uint32_t bal = __ballot_sync(kFull, a);
+    if (a) {
+      const int pos = qn + __popc(bal & lt);
+      q_row[pos] = (uint8_t)(k * 32 + lane);
+      q_g[pos] = g[k];
+    }
+    qn += __popc(bal);
+  }
+  __syncwarp();
+
+  // stage C: (deferred first-join probes), remaining joins and the aggregate over the
+  // queue, two rows per lane
+  const int32_t* wcol = sbase + wbase;
+  for (int i = lane; i < qn; i += 64) {
+    const bool two = i + 32 < qn;
+    int r[2] = {q_row[i], two ? q_row[i + 32] : q_row[i]};
+    int32_t gg[2] = {q_g[i], two ? q_g[i + 32] : 0};
+    bool alive[2] = {true, two};
+#pragma unroll
+    for (int jx = 0; jx < NJ; ++jx) {
+      const JoinState& j = js[jx];
+      const int32_t* col = wcol + j.c * stride;
+      int32_t key[2] = {col[r[0]], col[r[1]]};
+      uint32_t b[2];
+      bool pend[2];
+#pragma unroll
+      for (int u = 0; u < 2; ++u) {
+        if (jx < j0) {  // resume a deferred probe of the first join
+          pend[u] = alive[u] && gg[u] < 0;
+          b[u] = pend[u] ? ~(uint32_t)gg[u] : 0u;
+          if (pend[u]) gg[u] = 0;
         } else {
-          h[k] = (h[k] + 1u) & js[j].mask;
+          pend[u] = alive[u];
+          b[u] = bucket_of(key[u], j.shift);
+        }
+      }
+      while (pend[0] || pend[1]) {
+        ulonglong2 v[2];
+#pragma unroll
+        for (int u = 0; u < 2; ++u)
+          if (pend[u]) v[u] = __ldg(j.buckets + b[u]);
+#pragma unroll
+        for (int u = 0; u < 2; ++u) {
+          if (!pend[u]) continue;
+          bool hit, miss;
+          int32_t rank;
+          probe_step(v[u], key[u], hit, miss, rank);
+          if (hit) gg[u] += rank * j.jstride;
+          if (miss) alive[u] = false;
+          pend[u] = !(hit || miss);
+          b[u] = (b[u] + 1) & j.bmask;
         }
       }
     }
-  }
-  // reduce
-  const int32_t* sa = sbase + p.agg_a * stride + ctid;
-  const int32_t* sb = sbase + p.agg_b * stride + ctid;
+    const int32_t* ca = wcol + p.agg_a * stride;
+    const int32_t* cb = wcol + p.agg_b * stride;
 #pragma unroll
-  for (int k = 0; k < kRowsPerThread; ++k) {
-    if (!((alive >> k) & 1u)) continue;
-    const long long m = measure(p.agg_op, sa[k * kConsumers], sb[k * kConsumers]);
-    if (GROUPED) {
-      if (smem_table) {
-        atomicAdd(s_sum + gidx[k], (unsigned long long)m);
-        atomicAdd(s_cnt + gidx[k], 1u);
-      } else {
-        atomicAdd(p.g_sum + gidx[k], (unsigned long long)m);
-        atomicAdd(p.g_cnt + gidx[k], 1ull);
-      }
-    } else {
-      acc_sum += m;
-      acc_cnt += 1;
-    }
+    for (int u = 0; u < 2; ++u)
+      if (alive[u])
+        accumulate<GROUPED>(p, smem_table, s_sum, s_cnt, gg[u],
+                            measure(p.agg_op, ca[r[u]], cb[r[u]]), acc_sum, acc_cnt);
+  }
+  __syncwarp();  // the queue is reused by the next tile
+}
+
+__device__ __forceinline__ void mbar_wait_sleep(uint64_t* bar, uint32_t parity) {
+  uint32_t ok = 0;
+  while (true) {
+    asm volatile(
+        "{\n"
+        ".reg .pred p;\n"
+        "mbarrier.try_wait.parity.shared::cta.b64 p, [%1], %2;\n"
+        "selp.u32 %0, 1, 0, p;\n"
+        "}\n"
+        : "=r"(ok)
+        : "r"(smem_u32(bar)), "r"(parity)
+        : "memory");
+    if (ok) return;
+    __nanosleep(128);
   }
 }
 
 template <int NJ, bool GROUPED>
-__global__ void __launch_bounds__(kThreads) k1_probe_agg(const __grid_constant__ K1Params p) {
+__global__ void __launch_bounds__(kThreads, kCtasPerSm) k1_probe_agg(const __grid_constant__ K1Params p) {
   extern __shared__ __align__(128) unsigned char smem[];
   uint64_t* full = reinterpret_cast<uint64_t*>(smem);
   uint64_t* empty = full + p.stages;
   long long* red = reinterpret_cast<long long*>(smem + 128);                // 2 x 8 warps
   int32_t* headbuf = reinterpret_cast<int32_t*>(smem + 128 + 256);           // 8 cols x 4
-  unsigned long long* s_sum = reinterpret_cast<unsigned long long*>(smem + 512);
+  uint8_t* q_rows = smem + kSmemQueueOff;                                    // 8 x 256 B
+  int32_t* q_gs = reinterpret_cast<int32_t*>(smem + kSmemQueueOff + kConsumers * kRowsPerThread);
+  unsigned long long* s_sum = reinterpret_cast<unsigned long long*>(smem + kSmemFixed);
   uint32_t* s_cnt = reinterpret_cast<uint32_t*>(s_sum + p.smem_groups);
   const size_t table_bytes = ((size_t)p.smem_groups * 12 + 127) & ~size_t(127);
-  int32_t* stage0 = reinterpret_cast<int32_t*>(smem + 512 + table_bytes);
+  int32_t* stage0 = reinterpret_cast<int32_t*>(smem + kSmemFixed + table_bytes);
   const int stage_elems = p.n_cols * kTileRows;
 
+  // a failed group layout (capacity, or a plan whose dimensions changed) disables the pass
+  if (GROUPED && p.meta->error) return;
   const int tid = threadIdx.x;
   const int warp = tid >> 5;
+  const int lane = tid & 31;
   if (tid == kConsumers) {
     for (int s = 0; s < p.stages; ++s) {
       mbar_init(full + s, 1);
@@ -237,12 +389,12 @@ __global__ void __launch_bounds__(kThreads) k1_probe_agg(const __grid_constant__
 
   if (warp == kConsumerWarps) {
     // ---------------- producer warp: stream tiles HBM -> smem ring ----------------
-    if ((tid & 31) == 0) {
+    if (lane == 0) {
       const uint64_t pol = policy_evict_first();
       int64_t k = 0;
       for (int64_t t = blockIdx.x; t < p.n_tiles; t += gridDim.x, ++k) {
         const int s = (int)(k % p.stages);
-        if (k >= p.stages) mbar_wait(empty + s, (uint32_t)(((k / p.stages) - 1) & 1));
+        if (k >= p.stages) mbar_wait_sleep(empty + s, (uint32_t)(((k / p.stages) - 1) & 1));
         const int64_t r0 = t * kTileRows;
         const int64_t rows = std::min<int64_t>(kTileRows, p.n_rows - r0);
         const uint32_t bytes = (uint32_t)(rows & ~int64_t(3)) * 4u;
@@ -259,18 +411,20 @@ __global__ void __launch_bounds__(kThreads) k1_probe_agg(const __grid_constant__
 
   // ---------------- consumer warps ----------------
   const int ctid = tid;  // 0..255
-  const uint64_t pol_last = policy_evict_last();
+  uint8_t* q_row = q_rows + warp * (32 * kRowsPerThread);
+  int32_t* q_g = q_gs + warp * (32 * kRowsPerThread);
   JoinState js[HX_MAX_JOINS];
 #pragma unroll
   for (int j = 0; j < HX_MAX_JOINS; ++j) {
     if (j < NJ) {
-      js[j].slots = p.joins[j].slots;
+      const int lg = p.joins[j].hdr->log2cap;
+      js[j].buckets = reinterpret_cast<const ulonglong2*>(p.joins[j].slots);
       js[j].c = p.joins[j].c;
-      js[j].log2cap = p.joins[j].hdr->log2cap;
-      js[j].mask = (1u << js[j].log2cap) - 1u;
+      js[j].shift = 33 - lg;
+      js[j].bmask = (1u << (lg - 1)) - 1u;
       js[j].jstride = GROUPED ? p.meta->jstride[j] : 0;
     } else {
-      js[j] = JoinState{nullptr, 0, kMinLog2Cap, 0u, 0};
+      js[j] = JoinState{nullptr, 0, 32, 0u, 0};
     }
   }
   const long long n_groups = GROUPED ? p.meta->n_groups : 1;
@@ -287,8 +441,8 @@ __global__ void __launch_bounds__(kThreads) k1_probe_agg(const __grid_constant__
     if (ctid < p.head_rows)
       for (int c = 0; c < p.n_cols; ++c) headbuf[c * 4 + ctid] = p.head_col[c][ctid];
     consumer_sync();
-    process_tile<NJ, GROUPED>(p, js, headbuf, 4, p.head_rows, ctid, pol_last, smem_table, s_sum,
-                              s_cnt, acc_sum, acc_cnt);
+    process_tile<NJ, GROUPED>(p, js, headbuf, 4, p.head_rows, warp, lane, smem_table, s_sum,
+                              s_cnt, q_row, q_g, acc_sum, acc_cnt);
   }
   consumer_sync();
 
@@ -306,10 +460,10 @@ __global__ void __launch_bounds__(kThreads) k1_probe_agg(const __grid_constant__
           st[c * kTileRows + copied + ctid] = p.col[c][r0 + copied + ctid];
       consumer_sync();
     }
-    process_tile<NJ, GROUPED>(p, js, st, kTileRows, rows, ctid, pol_last, smem_table, s_sum, s_cnt,
-                              acc_sum, acc_cnt);
+    process_tile<NJ, GROUPED>(p, js, st, kTileRows, rows, warp, lane, smem_table, s_sum, s_cnt,
+                              q_row, q_g, acc_sum, acc_cnt);
     __syncwarp();
-    if ((tid & 31) == 0) mbar_arrive(empty + s);
+    if (lane == 0) mbar_arrive(empty + s);
   }
 
   // ---------------- flush the CTA's partial aggregate ----------------
@@ -331,7 +485,7 @@ __global__ void __launch_bounds__(kThreads) k1_probe_agg(const __grid_constant__
       acc_sum += __shfl_xor_sync(kFull, acc_sum, o);
       acc_cnt += __shfl_xor_sync(kFull, acc_cnt, o);
     }
-    if ((tid & 31) == 0) {
+    if (lane == 0) {
       red[warp] = acc_sum;
       red[kConsumerWarps + warp] = acc_cnt;
     }
@@ -361,7 +515,7 @@ __global__ void k1_prepare(AggMeta* meta, const HtHeader* g0, const HtHeader* g1
   int32_t nr[HX_MAX_GDIMS] = {1, 1, 1};
   long long n = 1;
   for (int g = 0; g < n_gdims; ++g) {
-    nr[g] = hdrs[g]->n_ranks;
+    nr[g] = max(1, hdrs[g]->n_ranks);  // an empty dimension still gives one (empty) rank
     n *= nr[g];
   }
   const bool over = n > cap_groups;
@@ -407,13 +561,17 @@ KernelFn pick_kernel(int nj, bool grouped) {
 
 size_t k1_smem_bytes(int n_cols, int stages, int smem_groups) {
   const size_t table_bytes = ((size_t)smem_groups * 12 + 127) & ~size_t(127);
-  return 512 + table_bytes + (size_t)stages * n_cols * kTileRows * sizeof(int32_t);
+  return kSmemFixed + table_bytes + (size_t)stages * n_cols * kTileRows * sizeof(int32_t);
 }
 
-int pick_stages(int n_cols) {
-  // ~96 KB of tiles in flight per CTA (2 CTAs per SM): 3 stages up to 4 columns, 2 beyond
+int pick_stages(int n_cols, int smem_groups) {
+  // as many tile stages as fit next to kCtasPerSm CTAs per SM (228 KB SM, 1 KB reserved
+  // per CTA), at least double buffering
+  const size_t budget = (228 * 1024) / kCtasPerSm - 1024;
+  const size_t fixed = kSmemFixed + (((size_t)smem_groups * 12 + 127) & ~size_t(127));
   const size_t stage = (size_t)n_cols * kTileRows * 4;
-  return std::max(2, std::min(4, (int)((96 * 1024) / stage)));
+  const int s = budget > fixed ? (int)((budget - fixed) / stage) : 0;
+  return std::max(2, std::min(4, s));
 }
 
 }  // namespace
@@ -428,20 +586,68 @@ int k1_occupancy(hx_ctx* ctx) {
   }
   int occ = 0;
   cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, k1_probe_agg<3, true>, kThreads,
-                                                k1_smem_bytes(4, pick_stages(4), kSmemGroups));
+                                                k1_smem_bytes(4, pick_stages(4, kSmemGroups), kSmemGroups));
   return occ;
 }
 
-int probe_agg(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht* const* hts,
-              int n_hts, hx_agg* agg, bool fresh) {
-  HX_REQUIRE(ctx && fact && sh && agg, HX_EINVAL, "hx_pipeline_probe_agg: null argument");
+// A fully resolved K1 launch (kernel, parameters, grid, prepare-kernel arguments): built once
+// on the host, enqueued any number of times (hx_pipeline_probe_agg, plans, CUDA graphs).
+struct K1Prepared {
+  K1Params p;
+  KernelFn fn = nullptr;
+  size_t smem = 0;
+  int grid = 0;
+  const HtHeader* gh[HX_MAX_GDIMS] = {nullptr, nullptr, nullptr};
+  int4 gj = make_int4(0, 0, 0, 0);
+  int n_gdims = 0;
+  int prep_grid = 1;
+  long long cap_groups = 1;
+  int64_t rows = 0;
+  int n_cols = 0;
+};
+
+long long k1_group_bound(const hx_query_shape* sh, hx_ht* const* hts, int n_hts) {
+  long long bound = 1;
+  for (int g = 0; g < sh->n_gdims; ++g) {
+    const int j = sh->gdim_join[g];
+    if (j < 0 || j >= sh->n_joins || sh->join_ht[j] < 0 || sh->join_ht[j] >= n_hts) return -1;
+    for (int g2 = 0; g2 < g; ++g2)
+      if (sh->gdim_join[g2] == j) return -1;
+    const hx_ht* ht = hts[sh->join_ht[j]];
+    bound *= std::max<long long>(1, std::min<long long>(ht->domain, std::max<int64_t>(ht->dim_rows, 1)));
+    bound = std::min<long long>(bound, (long long)HX_MAX_GROUPS + 1);
+  }
+  return bound;
+}
+
+int agg_alloc(hx_ctx* ctx, hx_agg* agg, long long cap_groups, const hx_query_shape* sh,
+              hx_ht* const* hts) {
+  HX_REQUIRE(cap_groups >= 1 && cap_groups <= HX_MAX_GROUPS, HX_ECAPACITY,
+             "hx_pipeline_probe_agg: too many groups");
+  agg->cap_groups = cap_groups;
+  agg->n_gdims = sh->n_gdims;
+  for (int g = 0; g < sh->n_gdims; ++g) agg->gdim_ht[g] = hts[sh->join_ht[sh->gdim_join[g]]];
+  const size_t bytes = 256 + 2 * (size_t)cap_groups * sizeof(unsigned long long);
+  HX_CK(cudaMallocAsync(&agg->base, bytes, ctx->stream));
+  agg->meta = reinterpret_cast<AggMeta*>(agg->base);
+  agg->sums = reinterpret_cast<unsigned long long*>(static_cast<char*>(agg->base) + 256);
+  agg->cnts = agg->sums + cap_groups;
+  return HX_OK;
+}
+
+int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht* const* hts,
+             int n_hts, const hx_agg* agg, K1Prepared** out) {
+  HX_REQUIRE(ctx && fact && sh && agg && out, HX_EINVAL, "hx_pipeline_probe_agg: null argument");
   HX_REQUIRE(sh->n_preds >= 0 && sh->n_preds <= HX_MAX_PREDS && sh->n_joins >= 0 &&
                  sh->n_joins <= HX_MAX_JOINS && sh->n_gdims >= 0 && sh->n_gdims <= HX_MAX_GDIMS &&
                  sh->agg_op >= HX_AGG_SUM && sh->agg_op <= HX_AGG_SUM_SUB,
              HX_EINVAL, "hx_pipeline_probe_agg: bad query shape");
   HX_REQUIRE(fact->placement != HX_PLACE_HOST_PINNED, HX_EUNSUPPORTED,
              "hx_pipeline_probe_agg: host-resident fact tables are not supported");
-  K1Params p{};
+  HX_REQUIRE(agg->n_gdims == sh->n_gdims, HX_EINVAL,
+             "hx_pipeline_probe_agg: shape differs from the agg's");
+  K1Prepared k{};
+  K1Params& p = k.p;
   // distinct fact columns the shape references -> staged columns
   int32_t ids[kMaxStageCols];
   int n_cols = 0;
@@ -475,49 +681,15 @@ int probe_agg(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht
   p.agg_b = sh->agg_op == HX_AGG_SUM ? p.agg_a : stage_of(sh->agg_b);
   HX_REQUIRE(p.agg_a >= 0 && p.agg_b >= 0, HX_EINVAL,
              "hx_pipeline_probe_agg: measure column not in fact table (or > 8 columns)");
-
-  // group layout: host-known upper bound for the arrays, exact count on the device
-  long long bound = 1;
+  HX_REQUIRE(k1_group_bound(sh, hts, n_hts) >= 1, HX_EINVAL, "hx_pipeline_probe_agg: bad gdim_join");
   for (int g = 0; g < sh->n_gdims; ++g) {
-    const int j = sh->gdim_join[g];
-    HX_REQUIRE(j >= 0 && j < sh->n_joins, HX_EINVAL, "hx_pipeline_probe_agg: bad gdim_join");
-    for (int g2 = 0; g2 < g; ++g2)
-      HX_REQUIRE(sh->gdim_join[g2] != j, HX_EINVAL, "hx_pipeline_probe_agg: repeated gdim_join");
-    const hx_ht* ht = hts[sh->join_ht[j]];
-    bound *= std::max<long long>(1, std::min<long long>(ht->domain, std::max<int64_t>(ht->dim_rows, 1)));
-    bound = std::min<long long>(bound, (long long)HX_MAX_GROUPS + 1);
+    k.gh[g] = hts[sh->join_ht[sh->gdim_join[g]]]->hdr;
+    (&k.gj.x)[g] = sh->gdim_join[g];
   }
-  if (fresh) {
-    HX_REQUIRE(bound <= HX_MAX_GROUPS, HX_ECAPACITY, "hx_pipeline_probe_agg: too many groups");
-    agg->cap_groups = bound;
-    agg->n_gdims = sh->n_gdims;
-    for (int g = 0; g < sh->n_gdims; ++g) agg->gdim_ht[g] = hts[sh->join_ht[sh->gdim_join[g]]];
-    const size_t bytes = 256 + 2 * (size_t)bound * sizeof(unsigned long long);
-    HX_CK(cudaMallocAsync(&agg->base, bytes, ctx->stream));
-    agg->meta = reinterpret_cast<AggMeta*>(agg->base);
-    agg->sums = reinterpret_cast<unsigned long long*>(static_cast<char*>(agg->base) + 256);
-    agg->cnts = agg->sums + bound;
-  } else {
-    HX_REQUIRE(agg->n_gdims == sh->n_gdims, HX_EINVAL,
-               "hx_pipeline_probe_agg_into: shape differs from the agg's");
-  }
-  for (int j = 0; j < sh->n_joins; ++j) agg->deps.push_back(hts[sh->join_ht[j]]);
-
-  {  // k1_prepare
-    const HtHeader* gh[HX_MAX_GDIMS] = {nullptr, nullptr, nullptr};
-    int4 gj = make_int4(0, 0, 0, 0);
-    int* gjp = &gj.x;
-    for (int g = 0; g < sh->n_gdims; ++g) {
-      gh[g] = hts[sh->join_ht[sh->gdim_join[g]]]->hdr;
-      gjp[g] = sh->gdim_join[g];
-    }
-    const int grid = (int)std::max<long long>(1, std::min<long long>((agg->cap_groups + 255) / 256,
-                                                                     (long long)ctx->n_sms * 4));
-    k1_prepare<<<grid, 256, 0, ctx->stream>>>(agg->meta, gh[0], gh[1], gh[2], sh->n_gdims, gj,
-                                             agg->sums, agg->cnts, agg->cap_groups, fresh ? 1 : 0);
-    HX_CK_LAUNCH("k1_prepare");
-  }
-
+  k.n_gdims = sh->n_gdims;
+  k.cap_groups = agg->cap_groups;
+  k.prep_grid = (int)std::max<long long>(1, std::min<long long>((agg->cap_groups + 255) / 256,
+                                                                (long long)ctx->n_sms * 4));
   // tiles: the head rows up to 16-byte alignment are handled separately
   const uintptr_t mis = reinterpret_cast<uintptr_t>(table_col(fact, ids[0])) & 15u;
   for (int c = 0; c < n_cols; ++c)
@@ -533,36 +705,71 @@ int probe_agg(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht
   p.head_rows = (int32_t)head;
   p.n_rows = fact->n_rows - head;
   p.n_tiles = (p.n_rows + kTileRows - 1) / kTileRows;
-  p.stages = pick_stages(n_cols);
   p.meta = agg->meta;
   p.g_sum = agg->sums;
   p.g_cnt = agg->cnts;
   const bool grouped = sh->n_gdims > 0;
   p.smem_groups = grouped ? (int32_t)std::min<long long>(kSmemGroups, agg->cap_groups) : 0;
-  if (fact->n_rows == 0) return HX_OK;
-
-  if (!ctx->k1_ctas_per_sm) ctx->k1_ctas_per_sm = std::max(1, k1_occupancy(ctx));
-  KernelFn fn = pick_kernel(sh->n_joins, grouped);
-  const size_t smem = k1_smem_bytes(n_cols, p.stages, p.smem_groups);
+  p.stages = pick_stages(n_cols, p.smem_groups);
+  k.fn = pick_kernel(sh->n_joins, grouped);
+  k.smem = k1_smem_bytes(n_cols, p.stages, p.smem_groups);
   int occ = 0;
-  HX_CK(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, fn, kThreads, smem));
+  HX_CK(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, k.fn, kThreads, k.smem));
   occ = std::max(1, occ);
-  const int64_t grid = std::max<int64_t>(1, std::min<int64_t>(p.n_tiles, (int64_t)ctx->n_sms * occ));
+  k.grid = (int)std::max<int64_t>(1, std::min<int64_t>(p.n_tiles, (int64_t)ctx->n_sms * occ));
+  k.rows = fact->n_rows;
+  k.n_cols = n_cols;
+  *out = new K1Prepared(k);
+  return HX_OK;
+}
+
+// prepare (group layout + zeroing when `fresh`) then K1; optional timing events around K1.
+int k1_enqueue(hx_ctx* ctx, const K1Prepared* k, bool fresh, cudaEvent_t e0, cudaEvent_t e1) {
+  const K1Params& p = k->p;
+  k1_prepare<<<k->prep_grid, 256, 0, ctx->stream>>>(const_cast<AggMeta*>(p.meta), k->gh[0], k->gh[1], k->gh[2],
+                                                    k->n_gdims, k->gj, p.g_sum, p.g_cnt,
+                                                    k->cap_groups, fresh ? 1 : 0);
+  HX_CK_LAUNCH("k1_prepare");
+  ctx->launches += 1;
+  if (k->rows == 0) return HX_OK;
+  if (e0) HX_CK(record_event(e0, ctx->stream));
+  k->fn<<<(unsigned)k->grid, kThreads, k->smem, ctx->stream>>>(p);
+  HX_CK_LAUNCH("k1_probe_agg");
+  ctx->launches += 1;
+  if (e1) HX_CK(record_event(e1, ctx->stream));
+  return HX_OK;
+}
+
+void k1_free(K1Prepared* k) { delete k; }
+int64_t k1_bytes(const K1Prepared* k) { return k->rows * 4 * k->n_cols; }
+
+int probe_agg(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht* const* hts,
+              int n_hts, hx_agg* agg, bool fresh) {
+  HX_REQUIRE(ctx && fact && sh && agg, HX_EINVAL, "hx_pipeline_probe_agg: null argument");
+  if (fresh) {
+    const long long bound = k1_group_bound(sh, hts, n_hts);
+    HX_REQUIRE(bound >= 1 && sh->n_joins <= HX_MAX_JOINS && sh->n_gdims <= HX_MAX_GDIMS,
+               HX_EINVAL, "hx_pipeline_probe_agg: bad gdim_join / join_ht");
+    int rc = agg_alloc(ctx, agg, bound, sh, hts);
+    if (rc != HX_OK) return rc;
+  }
+  K1Prepared* k = nullptr;
+  int rc = k1_setup(ctx, fact, sh, hts, n_hts, agg, &k);
+  if (rc != HX_OK) return rc;
+  for (int j = 0; j < sh->n_joins; ++j) agg->deps.push_back(hts[sh->join_ht[j]]);
   cudaEvent_t e0 = nullptr, e1 = nullptr;
-  if (ctx->prof_on) {
+  if (ctx->prof_on && k->rows > 0) {
     e0 = pooled_event(ctx);
     e1 = pooled_event(ctx);
-    HX_CK(cudaEventRecord(e0, ctx->stream));
   }
-  fn<<<(unsigned)grid, kThreads, smem, ctx->stream>>>(p);
-  HX_CK_LAUNCH("k1_probe_agg");
-  if (ctx->prof_on) {
-    HX_CK(cudaEventRecord(e1, ctx->stream));
+  rc = k1_enqueue(ctx, k, fresh, e0, e1);
+  if (rc == HX_OK && e0) {
     ctx->prof_events.push_back({e0, e1});
     ctx->prof_launches += 1;
-    ctx->prof_bytes += fact->n_rows * 4 * n_cols;
+    ctx->prof_bytes += k1_bytes(k);
   }
-  return HX_OK;
+  k1_free(k);
+  return rc;
 }
 
 }  // namespace hx

@@ -7,6 +7,7 @@ streams (`torch.cuda.current_stream().cuda_stream`); nothing here imports torch.
 from __future__ import annotations
 
 import ctypes
+import weakref
 from typing import Dict, List, Optional, Sequence, Tuple
 
 import numpy as np
@@ -48,8 +49,21 @@ class Context:
              int(reset))
         return ms.value, n.value, b.value
 
+    def stats(self, reset: bool = False) -> Tuple[int, int, int]:
+        """(kernels launched, H2D bytes, D2H bytes) since the last reset."""
+        a, b, c = ctypes.c_int64(), ctypes.c_int64(), ctypes.c_int64()
+        call("hx_stats", self.h, ctypes.byref(a), ctypes.byref(b), ctypes.byref(c), int(reset))
+        return a.value, b.value, c.value
+
     def close(self) -> None:
         if getattr(self, "h", None):
+            # free every live library object of this context first (graphs before the plans
+            # they replay, plans / aggs before the tables they reference)
+            kids = list(getattr(self, "_children", ()))
+            for cls in (Graph, Plan, Agg, HashTable, Table):
+                for k in kids:
+                    if isinstance(k, cls):
+                        k.close()
             call("hx_finalize", self.h)
             self.h = None
 
@@ -58,6 +72,12 @@ class Context:
             self.close()
         except Exception:
             pass
+
+
+def _adopt(ctx: Context, obj) -> None:
+    if not hasattr(ctx, "_children"):
+        ctx._children = weakref.WeakSet()
+    ctx._children.add(obj)
 
 
 def comm_unique_id() -> bytes:
@@ -106,6 +126,7 @@ def router_partition(n_rows: int, n_parts: int, block_rows: int,
 class Table:
     def __init__(self, ctx: Context, h, keep=None, parent=None):
         self.ctx, self.h, self._keep, self._parent = ctx, h, keep, parent
+        _adopt(ctx, self)
 
     @property
     def n_rows(self) -> int:
@@ -156,6 +177,7 @@ def load_numpy(ctx: Context, cols: Dict[int, np.ndarray], part: Optional[Partiti
 class HashTable:
     def __init__(self, ctx: Context, h, dim: Table):
         self.ctx, self.h, self._dim = ctx, h, dim
+        _adopt(ctx, self)
 
     def info(self, with_codes: bool = False):
         nk, ns, nr = ctypes.c_int64(), ctypes.c_int64(), ctypes.c_int32()
@@ -211,6 +233,7 @@ def query_shape(preds=(), joins=(), agg_op=_hx.HX_AGG_SUM, agg_a=0, agg_b=0,
 class Agg:
     def __init__(self, ctx: Context, h, n_gdims: int, deps):
         self.ctx, self.h, self.n_gdims, self._deps = ctx, h, n_gdims, deps
+        _adopt(ctx, self)
 
     def close(self):
         if getattr(self, "h", None):
@@ -245,7 +268,99 @@ def pipeline_probe_agg_into(ctx: Context, fact: Table, shape: hx_query_shape,
          len(hts), agg.h)
 
 
-def merge_aggregates(ctx: Context, agg: Agg, root: int = -1, cap: int = 1 << 16):
+class Plan:
+    """hx_plan_*: one prepared query (builds + fused pipeline + merge + finalize)."""
+
+    def __init__(self, ctx: Context, fact: Table, dims: Sequence[Table], builds, shape):
+        dim_arr = (ctypes.c_void_p * max(1, len(dims)))(*[d.h.value for d in dims])
+        b_arr = (_hx.hx_build_spec * max(1, len(builds)))(*builds)
+        h = ctypes.c_void_p()
+        call("hx_plan_create", ctx.h, fact.h, dim_arr, len(dims), b_arr, len(builds),
+             ctypes.byref(shape), ctypes.byref(h))
+        self.ctx, self.h, self._keep = ctx, h, (fact, list(dims))
+        _adopt(ctx, self)
+        ng, nd = ctypes.c_int64(), ctypes.c_int()
+        call("hx_plan_info", h, ctypes.byref(ng), ctypes.byref(nd))
+        self.n_groups, self.n_gdims = ng.value, nd.value
+        cap = max(1, self.n_groups)
+        self._sums = np.zeros(cap, np.int64)
+        self._cnts = np.zeros(cap, np.int64)
+        self._keys = np.zeros(cap * max(1, self.n_gdims), np.int32)
+
+    def enqueue(self) -> None:
+        call("hx_plan_enqueue", self.ctx.h, self.h)
+
+    def result(self):
+        """-> (keys int32[n, n_gdims], sums int64[n], counts int64[n]) of the last run."""
+        n = ctypes.c_int64()
+        call("hx_plan_result", self.h, self._sums.ctypes.data_as(_hx._PI64),
+             self._cnts.ctypes.data_as(_hx._PI64), self._keys.ctypes.data_as(_hx._PI32),
+             len(self._sums), ctypes.byref(n))
+        k = n.value
+        return (self._keys[: k * self.n_gdims].reshape(k, self.n_gdims).copy(),
+                self._sums[:k].copy(), self._cnts[:k].copy())
+
+    def k1_time(self) -> Tuple[float, int]:
+        ms, b = ctypes.c_float(), ctypes.c_int64()
+        call("hx_plan_k1_time", self.h, ctypes.byref(ms), ctypes.byref(b))
+        return ms.value, b.value
+
+    def close(self):
+        if getattr(self, "h", None):
+            call("hx_plan_free", self.h)
+            self.h = None
+
+    def __del__(self):
+        try:
+            self.close()
+        except Exception:
+            pass
+
+
+def build_spec(dim: int, key_col: int, preds=(), group_col: int = -1, group_lo: int = 0,
+               group_hi: int = 0) -> _hx.hx_build_spec:
+    s = _hx.hx_build_spec()
+    s.dim, s.key_col, s.n_preds = dim, key_col, len(preds)
+    for i, p in enumerate(preds):
+        s.preds[i] = p
+    s.group_col, s.group_lo, s.group_hi = group_col, group_lo, group_hi
+    return s
+
+
+class Graph:
+    """hx_graph_*: CUDA graph of the plan executions enqueued inside `with capture(ctx)`."""
+
+    def __init__(self, ctx: Context, h):
+        self.ctx, self.h = ctx, h
+        _adopt(ctx, self)
+
+    def launch(self) -> None:
+        call("hx_graph_launch", self.ctx.h, self.h)
+
+    def close(self):
+        if getattr(self, "h", None):
+            call("hx_graph_free", self.h)
+            self.h = None
+
+    def __del__(self):
+        try:
+            self.close()
+        except Exception:
+            pass
+
+
+def capture(ctx: Context, fn) -> Graph:
+    """Run fn() (plan enqueues) under stream capture and return the instantiated graph."""
+    call("hx_graph_begin", ctx.h)
+    try:
+        fn()
+    finally:
+        h = ctypes.c_void_p()
+        call("hx_graph_end", ctx.h, ctypes.byref(h))
+    return Graph(ctx, h)
+
+
+def merge_aggregates(ctx: Context, agg: Agg, root: int = -1, cap: int = 4096):
     """-> (keys int32[n, n_gdims], sums int64[n], counts int64[n]) for non-empty groups."""
     while True:
         sums = np.zeros(cap, np.int64)

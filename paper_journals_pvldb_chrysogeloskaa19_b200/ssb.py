@@ -181,6 +181,45 @@ class SsbEngine:
     def run(self, q: str) -> List[Tuple]:
         return self.finish(self.start(q))
 
+    # ---- prepared plans (allocation- and sync-free executions, graph capturable) ----------
+    DIM_ORDER = ("date", "customer", "supplier", "part")
+
+    def plan(self, q: str, fact: Optional[hx.Table] = None) -> "QueryPlan":
+        plan = PLANS[q]
+        dims = [self.dims[t] for t in self.DIM_ORDER]
+        builds = []
+        for _, b in plan.joins:
+            g = b.group
+            builds.append(hx.build_spec(self.DIM_ORDER.index(b.table), C[b.key],
+                                        [_hx_pred(t) for t in b.preds],
+                                        C[g[0]] if g else -1, g[1] if g else 0, g[2] if g else 0))
+        return QueryPlan(plan, hx.Plan(self.ctx, fact or self.fact, dims, builds, self.shape(plan)))
+
+
+class QueryPlan:
+    """A prepared SSB query: enqueue() runs builds -> K1 -> merge -> finalize on the device;
+    rows() waits and returns the result in ORDER BY order."""
+
+    def __init__(self, plan: Plan, hp: hx.Plan):
+        self.plan, self.hp = plan, hp
+
+    def enqueue(self) -> None:
+        self.hp.enqueue()
+
+    def rows(self) -> List[Tuple]:
+        keys, sums, cnts = self.hp.result()
+        # the device finalize emits groups in group-index order = the group codes ascending in
+        # SELECT order (dense ranks preserve code order), which already is the ORDER BY of
+        # Q2.x / Q4.x; Q3.x re-sorts by (d_year asc, revenue desc, codes asc)
+        if self.plan.order_q3 and len(sums) > 1:
+            idx = np.lexsort(tuple(keys[:, c] for c in range(keys.shape[1] - 1, -1, -1))
+                             + (-sums, keys[:, 2]))
+            keys, sums, cnts = keys[idx], sums[idx], cnts[idx]
+        return [tuple(k) + (s, c) for k, s, c in zip(keys.tolist(), sums.tolist(), cnts.tolist())]
+
+    def close(self) -> None:
+        self.hp.close()
+
 
 def order_by(plan: Plan, rows: List[Tuple]) -> List[Tuple]:
     """SSB ORDER BY: the group keys ascending (Q2, Q4), or d_year asc, revenue desc (Q3;

@@ -1,0 +1,142 @@
+"""CPU-side checks of the product library (no GPU needed):
+
+  * libhx.so loads and exports every entry point include/hx.h declares;
+  * the router (hx_router_partition, host-only) produces disjoint block handles covering
+    [0, n_rows), contiguous and balanced for RANGE, block b -> b % P for ROUND_ROBIN;
+  * without a GPU the library fails loudly (HX_ECUDA) — there is no CPU fallback;
+  * the multi-GPU data path (router partition -> per-rank partial aggregate -> union-router
+    sum) is exercised with world_size 2 over torch.distributed gloo.
+"""
+import os
+import re
+
+import numpy as np
+import pytest
+
+ROOT = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
+
+from paper_journals_pvldb_chrysogeloskaa19_b200 import _hx, hx  # noqa: E402
+
+
+def header_functions():
+    src = open(os.path.join(ROOT, "include", "hx.h")).read()
+    src = re.sub(r"/\*.*?\*/", "", src, flags=re.S)
+    return sorted(set(re.findall(r"\b(hx_[a-z0-9_]+)\s*\(", src)))
+
+
+def test_header_symbols_exported():
+    names = header_functions()
+    assert "hx_pipeline_probe_agg" in names and "hx_merge_aggregates" in names
+    lib = _hx.lib()
+    for n in names:
+        assert hasattr(lib, n), f"libhx.so does not export {n}"
+    assert set(names) == set(_hx.EXPORTED), set(names) ^ set(_hx.EXPORTED)
+
+
+def test_boundary_calls_named_in_north_star():
+    names = header_functions()
+    for n in ("hx_load_columns", "hx_build_dim_ht", "hx_pipeline_probe_agg",
+              "hx_router_partition", "hx_merge_aggregates"):
+        assert n in names
+
+
+@pytest.mark.parametrize("n_rows,parts,block", [(0, 3, 5), (10, 3, 3), (1, 4, 1 << 22),
+                                                (1000, 7, 64), (4097, 2, 4096)])
+@pytest.mark.parametrize("policy", [_hx.HX_POLICY_RANGE, _hx.HX_POLICY_ROUND_ROBIN])
+def test_router_partition(n_rows, parts, block, policy):
+    p = hx.router_partition(n_rows, parts, block, policy)
+    blocks = p.blocks()
+    assert len(blocks) == (n_rows + block - 1) // block
+    cover = np.zeros(n_rows, np.int32)
+    for b, (r0, r1, part) in enumerate(blocks):
+        assert r0 == b * block and r1 == min(n_rows, (b + 1) * block)
+        assert 0 <= part < parts
+        cover[r0:r1] += 1
+        if policy == _hx.HX_POLICY_ROUND_ROBIN:
+            assert part == b % parts
+    assert (cover == 1).all()  # disjoint, union = [0, n_rows)
+    assert sum(p.rows(i) for i in range(parts)) == n_rows
+    if policy == _hx.HX_POLICY_RANGE:
+        owners = [part for _, _, part in blocks]
+        assert owners == sorted(owners)  # contiguous runs of whole blocks
+        counts = np.bincount(owners, minlength=parts) if owners else np.zeros(parts)
+        assert counts.max() - counts.min() <= 1  # balanced to within one block
+
+
+def test_router_rejects_bad_arguments():
+    with pytest.raises(_hx.HxError) as e:
+        hx.router_partition(-1, 2, 10)
+    assert e.value.code == _hx.HX_EINVAL
+    with pytest.raises(_hx.HxError):
+        hx.router_partition(10, 0, 10)
+    with pytest.raises(_hx.HxError):
+        hx.router_partition(10, 2, 0)
+
+
+def test_no_gpu_fails_loudly():
+    import torch
+    if torch.cuda.is_available():
+        pytest.skip("a GPU is present")
+    with pytest.raises(_hx.HxError) as e:
+        hx.Context(0)
+    assert e.value.code in (_hx.HX_ECUDA, _hx.HX_EINVAL)
+
+
+# ---- world_size 2 over gloo: router partition -> partials -> union-router merge -------------
+def _rank_main(rank, world, port, out):
+    import torch
+    import torch.distributed as dist
+
+    import oracle
+    from ssb_tiny import tiny_db
+
+    os.environ.update(MASTER_ADDR="127.0.0.1", MASTER_PORT=str(port))
+    dist.init_process_group("gloo", rank=rank, world_size=world)
+    db = tiny_db(17, n_lo=12007)
+    n = len(db["lineorder"]["lo_orderdate"])
+    part = hx.router_partition(n, world, 1000, _hx.HX_POLICY_ROUND_ROBIN)
+    mine = [(b, e) for b, e, p in part.blocks() if p == rank]
+    results = {}
+    for q in ("q2.1", "q3.1", "q4.2"):
+        partial = {}
+        for b, e in mine:
+            for k, (s, c) in oracle.as_dict(oracle.run_query(q, db, b, e)).items():
+                s0, c0 = partial.get(k, (0, 0))
+                partial[k] = (s0 + s, c0 + c)
+        # dense group arrays over the union of keys (as the device arrays are dense)
+        keys = sorted(set().union(*[set(oracle.as_dict(oracle.run_query(q, db)).keys())]))
+        arr = torch.tensor([[partial.get(k, (0, 0))[0], partial.get(k, (0, 0))[1]] for k in keys],
+                           dtype=torch.int64)
+        dist.all_reduce(arr)  # the union router's global aggregation
+        results[q] = {k: (int(arr[i, 0]), int(arr[i, 1])) for i, k in enumerate(keys)}
+    out.put((rank, results))
+    dist.destroy_process_group()
+
+
+def test_two_rank_partition_merge_gloo():
+    import multiprocessing as mp
+    import socket
+    import sys
+
+    sys.path.insert(0, os.path.join(ROOT, "tests"))
+    import oracle
+    from ssb_tiny import tiny_db
+
+    s = socket.socket()
+    s.bind(("127.0.0.1", 0))
+    port = s.getsockname()[1]
+    s.close()
+    ctx = mp.get_context("spawn")
+    q = ctx.Queue()
+    procs = [ctx.Process(target=_rank_main, args=(r, 2, port, q)) for r in range(2)]
+    for p in procs:
+        p.start()
+    got = [q.get(timeout=240) for _ in procs]
+    for p in procs:
+        p.join(timeout=60)
+        assert p.exitcode == 0
+    db = tiny_db(17, n_lo=12007)
+    for rank, res in got:
+        for qq, merged in res.items():
+            want = oracle.as_dict(oracle.run_query(qq, db))
+            assert {k: v for k, v in merged.items() if v[1] > 0} == want, (rank, qq)

@@ -141,6 +141,30 @@ def test_misaligned_views(ctx, offset):
         assert eng.run(q) == oracle.run_query(q, db, offset, n - 7), q
 
 
+@pytest.mark.parametrize("seed", [3, 8])
+def test_plans_and_graph_replay(ctx, seed):
+    """Prepared plans (device finalize) and a CUDA graph of all 13 executions, replayed
+    twice, give the oracle's rows every time."""
+    db = tiny_db(seed, n_lo=30001)
+    dims, fact = ssb.load_db_numpy(ctx, db)
+    eng = ssb.SsbEngine(ctx, dims, fact)
+    plans = {q: eng.plan(q) for q in QUERIES}
+    want = {q: oracle.run_query(q, db) for q in QUERIES}
+    for q, pl in plans.items():  # plain enqueue
+        pl.enqueue()
+        assert pl.rows() == want[q], q
+    graph = hx.capture(ctx, lambda: [pl.enqueue() for pl in plans.values()])
+    for _ in range(2):
+        graph.launch()
+        for q, pl in plans.items():
+            assert pl.rows() == want[q], q
+    ms, nbytes = plans["q2.1"].hp.k1_time()
+    assert ms > 0 and nbytes == 30001 * 16
+    graph.close()
+    for pl in plans.values():
+        pl.close()
+
+
 def test_device_generated_columns_match_host(ctx):
     """ssbgen's device fill is bit-identical to the host fill (inputs for the bench)."""
     sz = ssbgen.sizes(0.02)

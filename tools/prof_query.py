@@ -1,0 +1,54 @@
+"""Run selected SSB queries on device-generated SF data (for ncu / nsight captures).
+
+    python tools/prof_query.py --sf 10 --queries q1.1,q2.1 --reps 2
+"""
+import argparse
+import os
+import sys
+
+ROOT = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
+sys.path.insert(0, ROOT)
+
+import torch  # noqa: E402
+
+import ssbgen  # noqa: E402
+from paper_journals_pvldb_chrysogeloskaa19_b200 import _hx, hx, ssb  # noqa: E402
+
+
+def device_db(ctx, sz, seed=42):
+    keep, stream = [], torch.cuda.current_stream().cuda_stream
+
+    def table(cols, n):
+        spec = []
+        for c in cols:
+            t = torch.empty(max(n, 1), dtype=torch.int32, device="cuda")
+            ssbgen.column_device(seed, sz, c, t.data_ptr(), 0, n, stream)
+            keep.append(t)
+            spec.append((ssbgen.COLS[c], t.data_ptr(), n))
+        return hx.load_columns(ctx, spec, placement=_hx.HX_PLACE_VIEW, keep=keep)
+
+    dims = {t: table(ssbgen.TABLE_COLS[t], ssbgen.table_rows(sz, ssbgen.TABLE_COLS[t][0]))
+            for t in ("date", "customer", "supplier", "part")}
+    fact = table(ssbgen.TABLE_COLS["lineorder"], sz["n_lineorder"])
+    torch.cuda.synchronize()
+    return dims, fact
+
+
+def main():
+    ap = argparse.ArgumentParser()
+    ap.add_argument("--sf", type=float, default=10)
+    ap.add_argument("--queries", default="q1.1,q2.1,q3.1,q4.1")
+    ap.add_argument("--reps", type=int, default=2)
+    a = ap.parse_args()
+    ctx = hx.Context(0, torch.cuda.current_stream().cuda_stream)
+    dims, fact = device_db(ctx, ssbgen.sizes(a.sf))
+    eng = ssb.SsbEngine(ctx, dims, fact)
+    for _ in range(a.reps):
+        for q in a.queries.split(","):
+            eng.run(q)
+    torch.cuda.synchronize()
+    print("ok")
+
+
+if __name__ == "__main__":
+    main()
