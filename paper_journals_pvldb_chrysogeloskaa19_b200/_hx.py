@@ -11,7 +11,7 @@ import ctypes
 import os
 
 _HERE = os.path.dirname(os.path.abspath(__file__))
-LIB_PATH = os.path.join(_HERE, "libhx.so")
+LIB_PATH = os.environ.get("HX_LIB", os.path.join(_HERE, "libhx.so"))  # HX_LIB: tuning builds
 
 HX_OK, HX_EINVAL, HX_ECUDA, HX_ENCCL, HX_ENOMEM, HX_ECAPACITY, HX_EDUPKEY, HX_EUNSUPPORTED = (
     0, -1, -2, -3, -4, -5, -6, -7)

@@ -96,6 +96,11 @@ int hx_init(int device, void* stream, hx_ctx** out) {
     cudaMemPoolSetAttribute(pool, cudaMemPoolAttrReleaseThreshold, &thr);
   }
   ctx->k1_ctas_per_sm = std::max(1, k1_occupancy(ctx));
+  for (int a = 0; a < hx_ctx::kAux; ++a) {
+    HX_CK(cudaStreamCreateWithFlags(&ctx->aux[a], cudaStreamNonBlocking));
+    HX_CK(cudaEventCreateWithFlags(&ctx->join_ev[a], cudaEventDisableTiming));
+  }
+  HX_CK(cudaEventCreateWithFlags(&ctx->fork_ev, cudaEventDisableTiming));
   *out = ctx;
   return HX_OK;
 }
@@ -109,6 +114,14 @@ int hx_finalize(hx_ctx* ctx) {
     cudaEventDestroy(pr.second);
   }
   for (auto e : ctx->event_pool) cudaEventDestroy(e);
+  for (int a = 0; a < hx_ctx::kAux; ++a) {
+    if (ctx->aux[a]) {
+      cudaStreamSynchronize(ctx->aux[a]);
+      cudaStreamDestroy(ctx->aux[a]);
+    }
+    if (ctx->join_ev[a]) cudaEventDestroy(ctx->join_ev[a]);
+  }
+  if (ctx->fork_ev) cudaEventDestroy(ctx->fork_ev);
   if (ctx->comm) ncclCommDestroy(ctx->comm);
   if (ctx->own_stream) cudaStreamDestroy(ctx->stream);
   delete ctx;
@@ -375,6 +388,10 @@ int hx_ht_broadcast(hx_ctx* ctx, hx_ht* ht, int root) {
   HX_REQUIRE(h.log2cap <= ht->max_log2cap, HX_EINVAL,
              "hx_ht_broadcast: tables differ in size across ranks");
   HX_NCCL(ncclBroadcast(ht->slots, ht->slots, (size_t(1) << h.log2cap) * 8, ncclUint8, root,
+                        ctx->comm, ctx->stream));
+  HX_REQUIRE(h.bloom_log2w <= ht->max_bloom_log2w, HX_EINVAL,
+             "hx_ht_broadcast: tables differ in size across ranks");
+  HX_NCCL(ncclBroadcast(ht->bloom, ht->bloom, (size_t(1) << h.bloom_log2w) * 4, ncclUint8, root,
                         ctx->comm, ctx->stream));
   return HX_OK;
 }

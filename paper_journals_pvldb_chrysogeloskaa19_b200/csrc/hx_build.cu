@@ -35,7 +35,8 @@ struct BuildParams {
   int32_t* c2r;
   int32_t* r2c;
   unsigned long long* slots;
-  int32_t group_lo, domain, max_log2cap;
+  uint32_t* bloom;
+  int32_t group_lo, domain, max_log2cap, max_bloom_log2w;
 };
 
 __device__ __forceinline__ bool row_pass(const BuildParams& p, int64_t i) {
@@ -96,6 +97,7 @@ __global__ void k2_rank(BuildParams p) {
     int lg = kMinLog2Cap;
     while (lg < p.max_log2cap && (1ll << lg) < (long long)kLoadInv * n) ++lg;
     p.hdr->log2cap = lg;
+    p.hdr->bloom_log2w = min(p.max_bloom_log2w, bloom_log2w_for(n));
     p.hdr->n_ranks = p.group ? running : 1;
     p.hdr->max_log2cap = p.max_log2cap;
     p.hdr->group_lo = p.group_lo;
@@ -103,18 +105,22 @@ __global__ void k2_rank(BuildParams p) {
   }
 }
 
-// Empty the slots in use (the capacity is only known on the device).
+// Empty the slots and Bloom words in use (their sizes are only known on the device).
 __global__ void k2_clear(BuildParams p) {
   const int64_t cap = 1ll << p.hdr->log2cap;
+  const int64_t words = 1ll << p.hdr->bloom_log2w;
   const int64_t stride = (int64_t)gridDim.x * blockDim.x;
-  for (int64_t i = (int64_t)blockIdx.x * blockDim.x + threadIdx.x; i < cap; i += stride)
+  for (int64_t i = (int64_t)blockIdx.x * blockDim.x + threadIdx.x; i < cap; i += stride) {
     p.slots[i] = kEmptySlot;
+    if (i < words) p.bloom[i] = 0u;
+  }
 }
 
 // Warp-cooperative linear-probing insert of every passing row.
 __global__ void k2_insert(BuildParams p) {
   const int lane = threadIdx.x & 31;
   const int log2cap = p.hdr->log2cap;
+  const int blw = p.hdr->bloom_log2w;
   const uint32_t mask = (1u << log2cap) - 1u;
   const int64_t stride = (int64_t)gridDim.x * blockDim.x;
   for (int64_t base = (int64_t)blockIdx.x * blockDim.x + (threadIdx.x & ~31); base < p.n_rows;
@@ -128,6 +134,21 @@ __global__ void k2_insert(BuildParams p) {
         int32_t code = __ldg(p.group + i) - p.group_lo;
         has = code >= 0 && code < p.domain;  // out-of-range codes were flagged by the filter
         if (has) rank = p.c2r[code];
+      }
+      if (has) atomicOr(p.bloom + bloom_word(key, blw), bloom_mask(key));
+    }
+    // optimistic pass: every lane CASes its key into its home slot at once (at load factor
+    // <= 1/4 most succeed in one round trip); only keys whose home slot was taken enter the
+    // warp-cooperative probe below
+    if (has) {
+      const unsigned long long packed =
+          ((unsigned long long)(uint32_t)rank << 32) | (unsigned long long)(uint32_t)key;
+      const unsigned long long old = atomicCAS(p.slots + ht_home(key, log2cap), kEmptySlot, packed);
+      if (old == kEmptySlot) {
+        has = false;
+      } else if ((int32_t)(uint32_t)old == key) {
+        atomicExch(&p.hdr->error, HX_EDUPKEY);
+        has = false;
       }
     }
     unsigned pending = __ballot_sync(kFull, has);
@@ -221,8 +242,11 @@ int ht_create(hx_ctx* ctx, const hx_table* dim, int32_t key_col, const hx_pred* 
   ht->has_group = group_col >= 0;
   ht->max_log2cap = p.max_log2cap;
   ht->dim_rows = dim->n_rows;
+  p.max_bloom_log2w = bloom_log2w_for(std::max<int64_t>(dim->n_rows, 1));
+  ht->max_bloom_log2w = p.max_bloom_log2w;
   const size_t maps = (sizeof(HtHeader) + 2 * domain * sizeof(int32_t) + 255) & ~size_t(255);
-  ht->bytes = maps + (size_t(1) << p.max_log2cap) * sizeof(unsigned long long);
+  const size_t slot_bytes = (size_t(1) << p.max_log2cap) * sizeof(unsigned long long);
+  ht->bytes = maps + slot_bytes + (size_t(1) << p.max_bloom_log2w) * sizeof(uint32_t);
   cudaError_t e = cudaMallocAsync(&ht->base, ht->bytes, ctx->stream);
   if (e != cudaSuccess) {
     delete ht;
@@ -236,6 +260,8 @@ int ht_create(hx_ctx* ctx, const hx_table* dim, int32_t key_col, const hx_pred* 
   p.c2r = ht->code_to_rank;
   p.r2c = ht->rank_to_code;
   p.slots = ht->slots;
+  ht->bloom = reinterpret_cast<uint32_t*>(static_cast<char*>(ht->base) + maps + slot_bytes);
+  p.bloom = ht->bloom;
   ht->build = new BuildParams(p);
   *out = ht;
   return HX_OK;
@@ -243,20 +269,21 @@ int ht_create(hx_ctx* ctx, const hx_table* dim, int32_t key_col, const hx_pred* 
 
 // Enqueue the four build kernels (asynchronous; CUDA-graph capturable). Re-running a build
 // on the same table rebuilds it from scratch.
-int ht_enqueue_build(hx_ctx* ctx, hx_ht* ht) {
+int ht_enqueue_build(hx_ctx* ctx, hx_ht* ht, cudaStream_t stream) {
   const BuildParams& p = *static_cast<const BuildParams*>(ht->build);
-  HX_CK(cudaMemsetAsync(ht->base, 0, sizeof(HtHeader) + p.domain * sizeof(int32_t), ctx->stream));
+  cudaStream_t s = stream ? stream : ctx->stream;
+  HX_CK(cudaMemsetAsync(ht->base, 0, sizeof(HtHeader) + p.domain * sizeof(int32_t), s));
   const int64_t want = (p.n_rows + 255) / 256;
   const int grid = (int)std::max<int64_t>(1, std::min<int64_t>(want, (int64_t)ctx->n_sms * 8));
-  k2_filter_mark<<<grid, 256, 0, ctx->stream>>>(p);
+  k2_filter_mark<<<grid, 256, 0, s>>>(p);
   HX_CK_LAUNCH("k2_filter_mark");
-  k2_rank<<<1, 1024, 0, ctx->stream>>>(p);
+  k2_rank<<<1, 1024, 0, s>>>(p);
   HX_CK_LAUNCH("k2_rank");
   const int64_t slots_max = int64_t(1) << p.max_log2cap;
   const int cgrid = (int)std::min<int64_t>((slots_max + 255) / 256, (int64_t)ctx->n_sms * 16);
-  k2_clear<<<cgrid, 256, 0, ctx->stream>>>(p);
+  k2_clear<<<cgrid, 256, 0, s>>>(p);
   HX_CK_LAUNCH("k2_clear");
-  k2_insert<<<grid, 256, 0, ctx->stream>>>(p);
+  k2_insert<<<grid, 256, 0, s>>>(p);
   HX_CK_LAUNCH("k2_insert");
   ctx->launches += 4;
   return HX_OK;

@@ -40,8 +40,26 @@ struct HtHeader {
   int32_t max_log2cap;
   int32_t group_lo;
   int32_t domain;
-  int32_t n_inserted;
+  int32_t bloom_log2w;  // log2 of the Bloom filter's 32-bit words in use (device-written)
 };
+
+// Blocked Bloom filter over the passing keys (one 32-bit word per key, two bits set), built
+// with the table. K1 stages it in shared memory to drop most non-matching rows before any
+// L2 probe (semi-join reduction). kBloomBitsPerKey bits per key: false positives ~5%.
+constexpr int kBloomBitsPerKey = 8;
+__host__ __device__ __forceinline__ int bloom_log2w_for(long long n_keys) {
+  long long bits = n_keys * kBloomBitsPerKey;
+  int l = 5;
+  while ((1ll << l) < bits) ++l;
+  return l - 5;
+}
+__host__ __device__ __forceinline__ uint32_t bloom_word(int32_t key, int log2w) {
+  return log2w == 0 ? 0u : ((uint32_t)key * 0x85EBCA6Bu) >> (32 - log2w);
+}
+__host__ __device__ __forceinline__ uint32_t bloom_mask(int32_t key) {
+  const uint32_t h = (uint32_t)key * 0xC2B2AE35u;
+  return (1u << (h >> 27)) | (1u << ((h >> 22) & 31u));
+}
 
 // Slots are grouped in 16-byte buckets of kBucketSlots = 2 (one 128-bit load per probe
 // step). A key's home is the first slot of its bucket; linear probing proceeds slot by
@@ -97,6 +115,11 @@ struct hx_ctx {
   // hx_stats counters
   int64_t launches = 0, h2d_bytes = 0, d2h_bytes = 0;
   int64_t capture_launches = 0, capture_d2h = 0;  // counters at hx_graph_begin
+  // fork/join of the independent dimension builds of a plan (parallel graph branches)
+  static constexpr int kAux = 4;
+  cudaStream_t aux[kAux] = {nullptr, nullptr, nullptr, nullptr};
+  cudaEvent_t fork_ev = nullptr;
+  cudaEvent_t join_ev[kAux] = {nullptr, nullptr, nullptr, nullptr};
 };
 
 struct hx_partition {
@@ -130,6 +153,9 @@ struct hx_ht {
   bool has_group = false;
   int64_t dim_rows = 0;
   void* build = nullptr;           // hx::BuildParams (hx_build.cu): re-enqueueable build
+  uint32_t* bloom = nullptr;       // Bloom filter words (after the slots)
+  int32_t max_bloom_log2w = 0;
+  int64_t known_keys = -1;         // passing keys, when a plan has observed them (else -1)
 };
 
 struct hx_agg {
@@ -160,7 +186,7 @@ int build_dim_ht(hx_ctx* ctx, const hx_table* dim, int32_t key_col, const hx_pre
                  hx_ht** out);
 int ht_create(hx_ctx* ctx, const hx_table* dim, int32_t key_col, const hx_pred* preds,
               int n_preds, int32_t group_col, int32_t group_lo, int32_t group_hi, hx_ht** out);
-int ht_enqueue_build(hx_ctx* ctx, hx_ht* ht);
+int ht_enqueue_build(hx_ctx* ctx, hx_ht* ht, cudaStream_t stream = nullptr);
 void ht_destroy(hx_ht* ht);
 int probe_agg(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* shape,
               hx_ht* const* hts, int n_hts, hx_agg* agg, bool fresh);

@@ -186,6 +186,7 @@ int hx_plan_create(hx_ctx* ctx, const hx_table* fact, hx_table* const* dims, int
   for (int b = 0; b < n_builds; ++b) {
     if (hh[b].error == HX_EDUPKEY) return bail(fail(HX_EDUPKEY, "dimension build: duplicate primary key"));
     if (hh[b].error) return bail(fail(HX_EINVAL, "dimension build: bad key or group code"));
+    pl->hts[b]->known_keys = hh[b].n_keys;  // lets K1 reserve shared memory for its filter
   }
   long long ng = 1;
   for (int g = 0; g < shape->n_gdims; ++g) ng *= std::max(1, hh[shape->join_ht[shape->gdim_join[g]]].n_ranks);
@@ -231,9 +232,26 @@ int hx_plan_create(hx_ctx* ctx, const hx_table* fact, hx_table* const* dims, int
 int hx_plan_enqueue(hx_ctx* ctx, hx_plan* pl) {
   HX_REQUIRE(ctx && pl && pl->ctx == ctx, HX_EINVAL, "hx_plan_enqueue: bad argument");
   HX_CK(cudaSetDevice(ctx->device));
-  for (hx_ht* ht : pl->hts) {
-    int rc = ht_enqueue_build(ctx, ht);
-    if (rc != HX_OK) return rc;
+  // the dimension builds are independent: fork them onto the auxiliary streams (parallel
+  // branches of a captured graph) and join before K1
+  const int nb = (int)pl->hts.size();
+  if (nb > 1 && ctx->aux[0]) {
+    HX_CK(cudaEventRecord(ctx->fork_ev, ctx->stream));
+    const int used = std::min(nb, (int)hx_ctx::kAux);
+    for (int a = 0; a < used; ++a) HX_CK(cudaStreamWaitEvent(ctx->aux[a], ctx->fork_ev, 0));
+    for (int b = 0; b < nb; ++b) {
+      int rc = ht_enqueue_build(ctx, pl->hts[b], ctx->aux[b % hx_ctx::kAux]);
+      if (rc != HX_OK) return rc;
+    }
+    for (int a = 0; a < used; ++a) {
+      HX_CK(cudaEventRecord(ctx->join_ev[a], ctx->aux[a]));
+      HX_CK(cudaStreamWaitEvent(ctx->stream, ctx->join_ev[a], 0));
+    }
+  } else {
+    for (hx_ht* ht : pl->hts) {
+      int rc = ht_enqueue_build(ctx, ht);
+      if (rc != HX_OK) return rc;
+    }
   }
   int rc = k1_enqueue(ctx, pl->k1, true, pl->k1_e0, pl->k1_e1);
   if (rc != HX_OK) return rc;

@@ -32,12 +32,19 @@ namespace hx {
 namespace {
 
 constexpr unsigned kFull = 0xFFFFFFFFu;
-constexpr int kConsumerWarps = 8;
+#ifndef HX_K1_WARPS
+#define HX_K1_WARPS 16  // consumer warps per CTA (tuned: tools/variants/run.sh)
+#endif
+#ifndef HX_K1_CTAS
+#define HX_K1_CTAS 1    // resident CTAs per SM the launch bounds / smem budget target
+                        // (one CTA per SM shares one copy of the Bloom filters)
+#endif
+constexpr int kConsumerWarps = HX_K1_WARPS;
 constexpr int kConsumers = kConsumerWarps * 32;
 constexpr int kThreads = kConsumers + 32;  // + one producer warp
 constexpr int kRowsPerThread = 4;          // R
 constexpr int kTileRows = kConsumers * kRowsPerThread;  // T = 1024
-constexpr int kCtasPerSm = 3;             // target residency (registers, smem budget)
+constexpr int kCtasPerSm = HX_K1_CTAS;    // target residency (registers, smem budget)
 constexpr int kMaxStageCols = 8;
 constexpr int kSmemGroups = 1024;          // per-CTA group table capacity
 // dynamic smem: [barriers 128 | reduce 256 | head 128 | queues 8 x 256 x (1+4) B | groups | tiles]
@@ -48,6 +55,8 @@ struct JoinDev {
   int32_t c;                               // staged column of the FK
   const unsigned long long* slots;
   const HtHeader* hdr;
+  const uint32_t* bloom;                   // the table's Bloom filter (global)
+  int32_t bloom_words;                     // shared-memory words reserved for it (0: none)
 };
 
 struct K1Params {
@@ -66,6 +75,7 @@ struct K1Params {
   unsigned long long* g_sum;
   unsigned long long* g_cnt;
   int32_t smem_groups;                     // 0 for ungrouped instances
+  int32_t filter_words;                    // sum of joins[].bloom_words
 };
 
 // ---- PTX helpers: mbarrier, bulk copy, cache policies -------------------------------------
@@ -134,7 +144,14 @@ struct JoinState {
   int32_t shift;              // 33 - log2cap (bucket hash)
   uint32_t bmask;             // n_buckets - 1
   int32_t jstride;            // weight of this join's rank in the group index
+  const uint32_t* sbloom;     // Bloom filter staged in shared memory (nullptr: none)
+  int32_t blw;                // its log2 word count
 };
+
+__device__ __forceinline__ bool bloom_pass(const JoinState& j, int32_t key) {
+  const uint32_t m = bloom_mask(key);
+  return (j.sbloom[bloom_word(key, j.blw)] & m) == m;
+}
 
 __device__ __forceinline__ uint32_t bucket_of(int32_t key, int shift) {
   return ((uint32_t)key * 2654435769u) >> shift;
@@ -182,16 +199,19 @@ __device__ __forceinline__ void accumulate(const K1Params& p, bool smem_table,
   }
 }
 
-// Process one staged tile. Warp w owns rows [w*256, w*256+256) of the tile; lane l holds
-// rows w*256 + k*32 + l (k < 8): conflict-free shared-memory reads. Column c, row r of the
-// tile is at sbase[c * stride + r].
-//   stage A  predicates on lineorder columns, branch-free, for the 8 rows of each lane;
-//   stage B  (no predicates) the first join is probed in place for all 8 rows at once —
-//            8 independent 128-bit L2 loads in flight per lane;
+// Process one staged tile. Warp w owns rows [w*128, w*128+128) of the tile; lane l holds the
+// 4 consecutive rows w*128 + 4l .. +3, read with one 128-bit shared-memory load per column
+// (512 contiguous bytes per warp: conflict-free). Column c, row r of the tile is at
+// sbase[c * stride + r].
+//   stage A  predicates on lineorder columns, branch-free, for the 4 rows of each lane;
+//   stage B  (no predicates) the first join is probed in place for all 4 rows at once —
+//            4 independent 128-bit L2 loads in flight per lane;
 //   compact  survivors are appended to a per-warp queue with ballot + popc (the GPU
 //            "selection vector"), so the remaining joins and the aggregate run with every
 //            lane busy instead of mostly-masked lanes;
-//   stage C  remaining probes + measure + group-table atomics, two queued rows per lane.
+//   stage C  one queued row per lane: the probes of ALL remaining joins are issued together
+//            (independent keys, so one L2 round trip instead of one per join), then the
+//            measure and the group-table atomic.
 template <int NJ, bool GROUPED>
 __device__ __forceinline__ void process_tile(const K1Params& p, const JoinState (&js)[HX_MAX_JOINS],
                                              const int32_t* sbase, int stride, int rows_valid,
@@ -200,50 +220,61 @@ __device__ __forceinline__ void process_tile(const K1Params& p, const JoinState 
                                              uint8_t* q_row, int32_t* q_g,
                                              long long& acc_sum, long long& acc_cnt) {
   const int wbase = warp * (32 * kRowsPerThread);
-  const int32_t* tb = sbase + wbase + lane;
+  const int r0 = wbase + lane * kRowsPerThread;
+  const int32_t* tb = sbase + r0;
   uint32_t m = 0;
 #pragma unroll
-  for (int k = 0; k < kRowsPerThread; ++k) m |= (uint32_t)(wbase + k * 32 + lane < rows_valid) << k;
+  for (int k = 0; k < kRowsPerThread; ++k) m |= (uint32_t)(r0 + k < rows_valid) << k;
   if (__ballot_sync(kFull, m) == 0) return;
 
   // stage A: lineorder predicates (kind is uniform: one branch per predicate, not per row)
   for (int q = 0; q < p.n_preds; ++q) {
     const DevPred& pr = p.preds[q];
-    const int32_t* col = tb + pr.c * stride;
+    const int4 v = *reinterpret_cast<const int4*>(tb + pr.c * stride);
+    const int32_t vv[4] = {v.x, v.y, v.z, v.w};
     if (pr.kind == HX_PRED_RANGE) {
       const uint32_t lo = (uint32_t)pr.lo, span = (uint32_t)pr.hi - (uint32_t)pr.lo;
 #pragma unroll
       for (int k = 0; k < kRowsPerThread; ++k)
-        m &= ~((uint32_t)(((uint32_t)col[k * 32] - lo) > span) << k);
+        m &= ~((uint32_t)(((uint32_t)vv[k] - lo) > span) << k);
     } else {
 #pragma unroll
       for (int k = 0; k < kRowsPerThread; ++k) {
-        const int32_t v = col[k * 32];
         bool ok = false;
 #pragma unroll
-        for (int i = 0; i < 4; ++i) ok |= (i < pr.n_in) && v == pr.in[i];
+        for (int i = 0; i < 4; ++i) ok |= (i < pr.n_in) && vv[k] == pr.in[i];
         m &= ~((uint32_t)(!ok) << k);
       }
     }
+  }
+
+  // stage F: semi-join reduction with the shared-memory Bloom filters of the joins that have
+  // one (no false negatives; ~5% false positives are removed by the exact probe in stage C)
+#pragma unroll
+  for (int jx = 0; jx < NJ; ++jx) {
+    if (!js[jx].sbloom) continue;
+    const int4 kv = *reinterpret_cast<const int4*>(tb + js[jx].c * stride);
+    const int32_t key[4] = {kv.x, kv.y, kv.z, kv.w};
+#pragma unroll
+    for (int k = 0; k < kRowsPerThread; ++k) m &= ~((uint32_t)!bloom_pass(js[jx], key[k]) << k);
   }
 
   int32_t g[kRowsPerThread];
 #pragma unroll
   for (int k = 0; k < kRowsPerThread; ++k) g[k] = 0;
   int j0 = 0;
-  if (NJ > 0 && p.n_preds == 0) {
-    // stage B: ONE probe step of the first join for all R rows of the lane (R independent
+  if (NJ > 0 && p.n_preds == 0 && !js[0].sbloom) {
+    // stage B: ONE probe step of the first join for the lane's 4 rows (4 independent
     // 128-bit loads in flight). Rows whose bucket was full without a verdict (rare at load
     // factor 1/4) are queued with ~next_bucket in place of the group index and finish in
     // stage C, so the warp never waits on its longest probe chain here.
     const JoinState& j = js[0];
-    const int32_t* col = tb + j.c * stride;
+    const int4 kv = *reinterpret_cast<const int4*>(tb + j.c * stride);
+    const int32_t key[4] = {kv.x, kv.y, kv.z, kv.w};
     ulonglong2 v[kRowsPerThread];
-    int32_t key[kRowsPerThread];
     uint32_t b[kRowsPerThread];
 #pragma unroll
     for (int k = 0; k < kRowsPerThread; ++k) {
-      key[k] = col[k * 32];
       b[k] = bucket_of(key[k], j.shift);
       if ((m >> k) & 1u) v[k] = __ldg(j.buckets + b[k]);
     }
@@ -260,13 +291,14 @@ __device__ __forceinline__ void process_tile(const K1Params& p, const JoinState 
   }
 
   if (NJ == 0) {
-    const int32_t* ca = tb + p.agg_a * stride;
-    const int32_t* cb = tb + p.agg_b * stride;
+    const int4 va = *reinterpret_cast<const int4*>(tb + p.agg_a * stride);
+    const int4 vb = *reinterpret_cast<const int4*>(tb + p.agg_b * stride);
+    const int32_t a4[4] = {va.x, va.y, va.z, va.w}, b4[4] = {vb.x, vb.y, vb.z, vb.w};
 #pragma unroll
     for (int k = 0; k < kRowsPerThread; ++k)
       if ((m >> k) & 1u)
-        accumulate<GROUPED>(p, smem_table, s_sum, s_cnt, g[k],
-                            measure(p.agg_op, ca[k * 32], cb[k * 32]), acc_sum, acc_cnt);
+        accumulate<GROUPED>(p, smem_table, s_sum, s_cnt, g[k], measure(p.agg_op, a4[k], b4[k]),
+                            acc_sum, acc_cnt);
     return;
   }
 
@@ -279,64 +311,58 @@ __device__ __forceinline__ void process_tile(const K1Params& p, const JoinState 
     const uint32_t bal = __ballot_sync(kFull, a);
     if (a) {
       const int pos = qn + __popc(bal & lt);
-      q_row[pos] = (uint8_t)(k * 32 + lane);
+      q_row[pos] = (uint8_t)(lane * kRowsPerThread + k);
       q_g[pos] = g[k];
     }
     qn += __popc(bal);
   }
   __syncwarp();
 
-  // stage C: (deferred first-join probes), remaining joins and the aggregate over the
-  // queue, two rows per lane
+  // stage C: one queued row per lane; every remaining join (and a deferred first-join probe)
+  // is probed concurrently
   const int32_t* wcol = sbase + wbase;
-  for (int i = lane; i < qn; i += 64) {
-    const bool two = i + 32 < qn;
-    int r[2] = {q_row[i], two ? q_row[i + 32] : q_row[i]};
-    int32_t gg[2] = {q_g[i], two ? q_g[i + 32] : 0};
-    bool alive[2] = {true, two};
+  for (int i = lane; i < qn; i += 32) {
+    const int r = q_row[i];
+    int32_t gg = q_g[i];
+    bool alive = true;
+    int32_t key[NJ > 0 ? NJ : 1];
+    uint32_t b[NJ > 0 ? NJ : 1];
+    uint32_t pend = 0;
 #pragma unroll
     for (int jx = 0; jx < NJ; ++jx) {
-      const JoinState& j = js[jx];
-      const int32_t* col = wcol + j.c * stride;
-      int32_t key[2] = {col[r[0]], col[r[1]]};
-      uint32_t b[2];
-      bool pend[2];
-#pragma unroll
-      for (int u = 0; u < 2; ++u) {
-        if (jx < j0) {  // resume a deferred probe of the first join
-          pend[u] = alive[u] && gg[u] < 0;
-          b[u] = pend[u] ? ~(uint32_t)gg[u] : 0u;
-          if (pend[u]) gg[u] = 0;
-        } else {
-          pend[u] = alive[u];
-          b[u] = bucket_of(key[u], j.shift);
-        }
-      }
-      while (pend[0] || pend[1]) {
-        ulonglong2 v[2];
-#pragma unroll
-        for (int u = 0; u < 2; ++u)
-          if (pend[u]) v[u] = __ldg(j.buckets + b[u]);
-#pragma unroll
-        for (int u = 0; u < 2; ++u) {
-          if (!pend[u]) continue;
-          bool hit, miss;
-          int32_t rank;
-          probe_step(v[u], key[u], hit, miss, rank);
-          if (hit) gg[u] += rank * j.jstride;
-          if (miss) alive[u] = false;
-          pend[u] = !(hit || miss);
-          b[u] = (b[u] + 1) & j.bmask;
-        }
+      key[jx] = wcol[js[jx].c * stride + r];
+      if (jx < j0) {  // resume a deferred probe of the first join
+        const bool deferred = gg < 0;
+        b[jx] = deferred ? ~(uint32_t)gg : 0u;
+        pend |= (uint32_t)deferred << jx;
+      } else {
+        b[jx] = bucket_of(key[jx], js[jx].shift);
+        pend |= 1u << jx;
       }
     }
-    const int32_t* ca = wcol + p.agg_a * stride;
-    const int32_t* cb = wcol + p.agg_b * stride;
+    if (gg < 0) gg = 0;
+    while (pend) {
+      ulonglong2 v[NJ > 0 ? NJ : 1];
 #pragma unroll
-    for (int u = 0; u < 2; ++u)
-      if (alive[u])
-        accumulate<GROUPED>(p, smem_table, s_sum, s_cnt, gg[u],
-                            measure(p.agg_op, ca[r[u]], cb[r[u]]), acc_sum, acc_cnt);
+      for (int jx = 0; jx < NJ; ++jx)
+        if ((pend >> jx) & 1u) v[jx] = __ldg(js[jx].buckets + b[jx]);
+#pragma unroll
+      for (int jx = 0; jx < NJ; ++jx) {
+        if (!((pend >> jx) & 1u)) continue;
+        bool hit, miss;
+        int32_t rank;
+        probe_step(v[jx], key[jx], hit, miss, rank);
+        if (hit) gg += rank * js[jx].jstride;
+        alive = alive && !miss;
+        pend &= ~((uint32_t)(hit || miss) << jx);
+        b[jx] = (b[jx] + 1) & js[jx].bmask;
+      }
+      if (!alive) pend = 0;
+    }
+    if (alive)
+      accumulate<GROUPED>(p, smem_table, s_sum, s_cnt, gg,
+                          measure(p.agg_op, wcol[p.agg_a * stride + r], wcol[p.agg_b * stride + r]),
+                          acc_sum, acc_cnt);
   }
   __syncwarp();  // the queue is reused by the next tile
 }
@@ -370,7 +396,9 @@ __global__ void __launch_bounds__(kThreads, kCtasPerSm) k1_probe_agg(const __gri
   unsigned long long* s_sum = reinterpret_cast<unsigned long long*>(smem + kSmemFixed);
   uint32_t* s_cnt = reinterpret_cast<uint32_t*>(s_sum + p.smem_groups);
   const size_t table_bytes = ((size_t)p.smem_groups * 12 + 127) & ~size_t(127);
-  int32_t* stage0 = reinterpret_cast<int32_t*>(smem + kSmemFixed + table_bytes);
+  uint32_t* s_filters = reinterpret_cast<uint32_t*>(smem + kSmemFixed + table_bytes);
+  const size_t filter_bytes = ((size_t)p.filter_words * 4 + 127) & ~size_t(127);
+  int32_t* stage0 = reinterpret_cast<int32_t*>(smem + kSmemFixed + table_bytes + filter_bytes);
   const int stage_elems = p.n_cols * kTileRows;
 
   // a failed group layout (capacity, or a plan whose dimensions changed) disables the pass
@@ -391,10 +419,11 @@ __global__ void __launch_bounds__(kThreads, kCtasPerSm) k1_probe_agg(const __gri
     // ---------------- producer warp: stream tiles HBM -> smem ring ----------------
     if (lane == 0) {
       const uint64_t pol = policy_evict_first();
-      int64_t k = 0;
-      for (int64_t t = blockIdx.x; t < p.n_tiles; t += gridDim.x, ++k) {
-        const int s = (int)(k % p.stages);
-        if (k >= p.stages) mbar_wait_sleep(empty + s, (uint32_t)(((k / p.stages) - 1) & 1));
+      int s = 0;
+      uint32_t ph = 0;
+      bool wrapped = false;
+      for (int64_t t = blockIdx.x; t < p.n_tiles; t += gridDim.x) {
+        if (wrapped) mbar_wait_sleep(empty + s, ph ^ 1u);
         const int64_t r0 = t * kTileRows;
         const int64_t rows = std::min<int64_t>(kTileRows, p.n_rows - r0);
         const uint32_t bytes = (uint32_t)(rows & ~int64_t(3)) * 4u;
@@ -403,6 +432,11 @@ __global__ void __launch_bounds__(kThreads, kCtasPerSm) k1_probe_agg(const __gri
           int32_t* dst = stage0 + (size_t)s * stage_elems;
           for (int c = 0; c < p.n_cols; ++c)
             bulk_g2s(dst + c * kTileRows, p.col[c] + r0, bytes, full + s, pol);
+        }
+        if (++s == p.stages) {
+          s = 0;
+          ph ^= 1u;
+          wrapped = true;
         }
       }
     }
@@ -423,8 +457,32 @@ __global__ void __launch_bounds__(kThreads, kCtasPerSm) k1_probe_agg(const __gri
       js[j].shift = 33 - lg;
       js[j].bmask = (1u << (lg - 1)) - 1u;
       js[j].jstride = GROUPED ? p.meta->jstride[j] : 0;
+      js[j].sbloom = nullptr;
+      js[j].blw = 0;
     } else {
-      js[j] = JoinState{nullptr, 0, 32, 0u, 0};
+      js[j] = JoinState{nullptr, 0, 32, 0u, 0, nullptr, 0};
+    }
+  }
+  // stage the Bloom filters that fit their reservation into shared memory (once per CTA)
+  {
+    uint32_t* dst = s_filters;
+#pragma unroll
+    for (int j = 0; j < NJ; ++j) {
+      const int reserved = p.joins[j].bloom_words;
+      if (reserved == 0) continue;
+      const int lw = p.joins[j].hdr->bloom_log2w;
+      if ((1 << lw) <= reserved) {
+        const uint4* src = reinterpret_cast<const uint4*>(p.joins[j].bloom);
+        if (lw >= 2) {
+          for (int i = ctid; i < (1 << lw) / 4; i += kConsumers)
+            reinterpret_cast<uint4*>(dst)[i] = __ldg(src + i);
+        } else if (ctid < (1 << lw)) {
+          dst[ctid] = __ldg(p.joins[j].bloom + ctid);
+        }
+        js[j].sbloom = dst;
+        js[j].blw = lw;
+      }
+      dst += reserved;
     }
   }
   const long long n_groups = GROUPED ? p.meta->n_groups : 1;
@@ -446,10 +504,10 @@ __global__ void __launch_bounds__(kThreads, kCtasPerSm) k1_probe_agg(const __gri
   }
   consumer_sync();
 
-  int64_t k = 0;
-  for (int64_t t = blockIdx.x; t < p.n_tiles; t += gridDim.x, ++k) {
-    const int s = (int)(k % p.stages);
-    mbar_wait(full + s, (uint32_t)((k / p.stages) & 1));
+  int s = 0;
+  uint32_t ph = 0;
+  for (int64_t t = blockIdx.x; t < p.n_tiles; t += gridDim.x) {
+    mbar_wait(full + s, ph);
     int32_t* st = stage0 + (size_t)s * stage_elems;
     const int64_t r0 = t * kTileRows;
     const int rows = (int)std::min<int64_t>(kTileRows, p.n_rows - r0);
@@ -464,6 +522,10 @@ __global__ void __launch_bounds__(kThreads, kCtasPerSm) k1_probe_agg(const __gri
                               q_row, q_g, acc_sum, acc_cnt);
     __syncwarp();
     if (lane == 0) mbar_arrive(empty + s);
+    if (++s == p.stages) {
+      s = 0;
+      ph ^= 1u;
+    }
   }
 
   // ---------------- flush the CTA's partial aggregate ----------------
@@ -545,7 +607,7 @@ __global__ void k1_prepare(AggMeta* meta, const HtHeader* g0, const HtHeader* g1
 template <int NJ, bool G>
 void set_attrs() {
   cudaFuncSetAttribute(k1_probe_agg<NJ, G>, cudaFuncAttributeMaxDynamicSharedMemorySize,
-                       200 * 1024);
+                       227 * 1024);
 }
 
 using KernelFn = void (*)(K1Params);
@@ -559,15 +621,20 @@ KernelFn pick_kernel(int nj, bool grouped) {
   return table[grouped ? 1 : 0][nj];
 }
 
-size_t k1_smem_bytes(int n_cols, int stages, int smem_groups) {
+size_t k1_smem_bytes(int n_cols, int stages, int smem_groups, int filter_words = 0) {
   const size_t table_bytes = ((size_t)smem_groups * 12 + 127) & ~size_t(127);
-  return kSmemFixed + table_bytes + (size_t)stages * n_cols * kTileRows * sizeof(int32_t);
+  const size_t filter_bytes = ((size_t)filter_words * 4 + 127) & ~size_t(127);
+  return kSmemFixed + table_bytes + filter_bytes +
+         (size_t)stages * n_cols * kTileRows * sizeof(int32_t);
 }
 
+// Per-CTA shared memory for `ctas` resident CTAs per SM (228 KB per SM, 1 KB reserved each).
+constexpr size_t smem_budget(int ctas) { return (228 * 1024) / ctas - 1024; }
+
 int pick_stages(int n_cols, int smem_groups) {
-  // as many tile stages as fit next to kCtasPerSm CTAs per SM (228 KB SM, 1 KB reserved
-  // per CTA), at least double buffering
-  const size_t budget = (228 * 1024) / kCtasPerSm - 1024;
+  // as many tile stages as fit next to kCtasPerSm CTAs per SM, at least double buffering
+  // (at most ~96 KB of tiles per CTA: the rest of a large CTA is left for Bloom filters)
+  const size_t budget = std::min<size_t>(smem_budget(kCtasPerSm), 96 * 1024 + 24 * 1024);
   const size_t fixed = kSmemFixed + (((size_t)smem_groups * 12 + 127) & ~size_t(127));
   const size_t stage = (size_t)n_cols * kTileRows * 4;
   const int s = budget > fixed ? (int)((budget - fixed) / stage) : 0;
@@ -674,7 +741,7 @@ int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht*
     HX_REQUIRE(sh->join_ht[j] >= 0 && sh->join_ht[j] < n_hts && hts && hts[sh->join_ht[j]],
                HX_EINVAL, "hx_pipeline_probe_agg: bad join hash table index");
     const hx_ht* ht = hts[sh->join_ht[j]];
-    p.joins[j] = JoinDev{c, ht->slots, ht->hdr};
+    p.joins[j] = JoinDev{c, ht->slots, ht->hdr, ht->bloom, 0};
   }
   p.agg_op = sh->agg_op;
   p.agg_a = stage_of(sh->agg_a);
@@ -711,8 +778,22 @@ int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht*
   const bool grouped = sh->n_gdims > 0;
   p.smem_groups = grouped ? (int32_t)std::min<long long>(kSmemGroups, agg->cap_groups) : 0;
   p.stages = pick_stages(n_cols, p.smem_groups);
+  // shared-memory Bloom filters (semi-join reduction) for the joins whose passing key count
+  // is known (a plan observed it) and selective (at most half the dimension passes), in
+  // probe order, while the CTA still fits twice per SM
+  p.filter_words = 0;
+  for (int j = 0; j < sh->n_joins; ++j) {
+    const hx_ht* ht = hts[sh->join_ht[j]];
+    if (ht->known_keys < 0 || 2 * ht->known_keys > ht->dim_rows) continue;
+    const int words = std::max(4, 1 << std::min(ht->max_bloom_log2w, bloom_log2w_for(ht->known_keys)));
+    if (k1_smem_bytes(n_cols, p.stages, p.smem_groups, p.filter_words + words) >
+        smem_budget(std::min(kCtasPerSm, 2)))
+      continue;
+    p.joins[j].bloom_words = words;
+    p.filter_words += words;
+  }
   k.fn = pick_kernel(sh->n_joins, grouped);
-  k.smem = k1_smem_bytes(n_cols, p.stages, p.smem_groups);
+  k.smem = k1_smem_bytes(n_cols, p.stages, p.smem_groups, p.filter_words);
   int occ = 0;
   HX_CK(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, k.fn, kThreads, k.smem));
   occ = std::max(1, occ);
