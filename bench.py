@@ -43,7 +43,7 @@ BLOCK_ROWS = 1 << 22
 def parse():
     ap = argparse.ArgumentParser()
     ap.add_argument("--gpus", type=int, default=1)
-    ap.add_argument("--steps", type=int, default=10)
+    ap.add_argument("--steps", type=int, default=50)
     ap.add_argument("--warmup", type=int, default=3)
     ap.add_argument("--sf", type=float, default=10.0, help="SSB scale factor per GPU")
     ap.add_argument("--impl", default="hx", choices=["hx", "reference"])
@@ -97,7 +97,7 @@ class Clocks:
                 ["nvidia-smi", "-i", str(self.index), "--query-gpu=clocks.sm,clocks.max.sm,"
                  "clocks_event_reasons.active,clocks_event_reasons.hw_slowdown,"
                  "clocks_event_reasons.hw_thermal_slowdown,clocks_event_reasons.sw_thermal_slowdown,"
-                 "clocks_event_reasons.sw_power_cap", "--format=csv,noheader,nounits", "-lms", "100"],
+                 "clocks_event_reasons.sw_power_cap", "--format=csv,noheader,nounits", "-lms", "20"],
                 stdout=open(self.path, "w"), stderr=subprocess.DEVNULL)
         except Exception:
             self.proc = None
@@ -240,15 +240,15 @@ def main():
     # the 13 executions are captured into ONE CUDA graph: a step is one graph launch plus
     # the 13 host reads of the finalized results
     plans = {q: eng.plan(q) for q in queries}
-    graph = None if args.no_graph else hx.capture(ctx, lambda: [plans[q].enqueue() for q in queries])
+    order = [plans[q].hp for q in queries]
+    graph = None if args.no_graph else hx.capture(ctx, lambda: hx.plans_enqueue(ctx, order))
     k1_acc = [0.0, 0, 0]
 
     def step(timed=False):
         if graph is not None:
             graph.launch()
         else:
-            for q in queries:
-                plans[q].enqueue()
+            hx.plans_enqueue(ctx, order)
         out = [plans[q].rows() for q in queries]
         if timed:
             for q in queries:

@@ -220,6 +220,11 @@ int hx_plan_create(hx_ctx* ctx, const hx_table* fact, hx_table* const* dims, int
                    const hx_build_spec* builds, int n_builds, const hx_query_shape* shape,
                    hx_plan** out);
 int hx_plan_enqueue(hx_ctx* ctx, hx_plan* plan);
+/* Enqueue several plans as one step: every plan's builds first (on auxiliary streams, so
+   they overlap the pipelines of the plans before them), then each plan's pipeline, merge and
+   finalize in order, each waiting only for its own builds. Same results as n x
+   hx_plan_enqueue; capturable. */
+int hx_plans_enqueue(hx_ctx* ctx, hx_plan* const* plans, int n);
 /* Waits for the last enqueued execution; rows as hx_merge_aggregates (group-index order). */
 int hx_plan_result(hx_plan* plan, int64_t* sums, int64_t* counts, int32_t* keys, int64_t cap,
                    int64_t* n_rows);

@@ -99,6 +99,7 @@ _SIGS = {
     "hx_plan_create": ([_P, _P, _PP, _I, ctypes.POINTER(hx_build_spec), _I,
                         ctypes.POINTER(hx_query_shape), _PP], _I),
     "hx_plan_enqueue": ([_P, _P], _I),
+    "hx_plans_enqueue": ([_P, _PP, _I], _I),
     "hx_plan_result": ([_P, _PI64, _PI64, _PI32, _I64, _PI64], _I),
     "hx_plan_k1_time": ([_P, ctypes.POINTER(ctypes.c_float), _PI64], _I),
     "hx_plan_info": ([_P, _PI64, ctypes.POINTER(_I)], _I),

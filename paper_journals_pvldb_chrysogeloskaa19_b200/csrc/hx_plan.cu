@@ -115,6 +115,7 @@ struct hx_plan {
   void* h_out = nullptr;       // pinned
   size_t out_bytes = 0, inline_bytes = 0;
   cudaEvent_t done = nullptr, k1_e0 = nullptr, k1_e1 = nullptr;
+  cudaEvent_t built_ev[hx_ctx::kAux] = {nullptr, nullptr, nullptr, nullptr};
   bool enqueued = false;
 };
 
@@ -126,6 +127,9 @@ struct hx_graph {
   int64_t d2h = 0;
 };
 
+static int plan_enqueue_builds(hx_ctx* ctx, hx_plan* pl);
+static int plan_enqueue_probe(hx_ctx* ctx, hx_plan* pl);
+
 static void plan_destroy(hx_plan* pl) {
   if (!pl) return;
   cudaSetDevice(pl->ctx->device);
@@ -136,6 +140,8 @@ static void plan_destroy(hx_plan* pl) {
   if (pl->d_out) cudaFreeAsync(pl->d_out, pl->ctx->stream);
   if (pl->h_out) cudaFreeHost(pl->h_out);
   for (cudaEvent_t e : {pl->done, pl->k1_e0, pl->k1_e1})
+    if (e) cudaEventDestroy(e);
+  for (cudaEvent_t e : pl->built_ev)
     if (e) cudaEventDestroy(e);
   delete pl;
 }
@@ -225,6 +231,10 @@ int hx_plan_create(hx_ctx* ctx, const hx_table* fact, hx_table* const* dims, int
     cudaError_t err = cudaEventCreate(e);
     if (err != cudaSuccess) return bail(cuda_fail(err, "cudaEventCreate", __FILE__, __LINE__));
   }
+  for (cudaEvent_t& e : pl->built_ev) {
+    cudaError_t err = cudaEventCreateWithFlags(&e, cudaEventDisableTiming);
+    if (err != cudaSuccess) return bail(cuda_fail(err, "cudaEventCreate", __FILE__, __LINE__));
+  }
   *out = pl;
   return HX_OK;
 }
@@ -232,27 +242,53 @@ int hx_plan_create(hx_ctx* ctx, const hx_table* fact, hx_table* const* dims, int
 int hx_plan_enqueue(hx_ctx* ctx, hx_plan* pl) {
   HX_REQUIRE(ctx && pl && pl->ctx == ctx, HX_EINVAL, "hx_plan_enqueue: bad argument");
   HX_CK(cudaSetDevice(ctx->device));
-  // the dimension builds are independent: fork them onto the auxiliary streams (parallel
-  // branches of a captured graph) and join before K1
-  const int nb = (int)pl->hts.size();
-  if (nb > 1 && ctx->aux[0]) {
-    HX_CK(cudaEventRecord(ctx->fork_ev, ctx->stream));
-    const int used = std::min(nb, (int)hx_ctx::kAux);
-    for (int a = 0; a < used; ++a) HX_CK(cudaStreamWaitEvent(ctx->aux[a], ctx->fork_ev, 0));
-    for (int b = 0; b < nb; ++b) {
-      int rc = ht_enqueue_build(ctx, pl->hts[b], ctx->aux[b % hx_ctx::kAux]);
-      if (rc != HX_OK) return rc;
-    }
-    for (int a = 0; a < used; ++a) {
-      HX_CK(cudaEventRecord(ctx->join_ev[a], ctx->aux[a]));
-      HX_CK(cudaStreamWaitEvent(ctx->stream, ctx->join_ev[a], 0));
-    }
-  } else {
-    for (hx_ht* ht : pl->hts) {
-      int rc = ht_enqueue_build(ctx, ht);
-      if (rc != HX_OK) return rc;
-    }
+  HX_CK(cudaEventRecord(ctx->fork_ev, ctx->stream));
+  for (int a = 0; a < hx_ctx::kAux; ++a) HX_CK(cudaStreamWaitEvent(ctx->aux[a], ctx->fork_ev, 0));
+  int rc = plan_enqueue_builds(ctx, pl);
+  if (rc != HX_OK) return rc;
+  return plan_enqueue_probe(ctx, pl);
+}
+
+int hx_plans_enqueue(hx_ctx* ctx, hx_plan* const* plans, int n) {
+  HX_REQUIRE(ctx && (n == 0 || plans) && n >= 0, HX_EINVAL, "hx_plans_enqueue: bad argument");
+  for (int i = 0; i < n; ++i)
+    HX_REQUIRE(plans[i] && plans[i]->ctx == ctx, HX_EINVAL, "hx_plans_enqueue: bad plan");
+  HX_CK(cudaSetDevice(ctx->device));
+  // every build of every plan first (forked from one point: they overlap the pipelines of
+  // the earlier plans), then the pipelines in order, each waiting only for its own builds
+  HX_CK(cudaEventRecord(ctx->fork_ev, ctx->stream));
+  for (int a = 0; a < hx_ctx::kAux; ++a) HX_CK(cudaStreamWaitEvent(ctx->aux[a], ctx->fork_ev, 0));
+  for (int i = 0; i < n; ++i) {
+    int rc = plan_enqueue_builds(ctx, plans[i]);
+    if (rc != HX_OK) return rc;
   }
+  for (int i = 0; i < n; ++i) {
+    int rc = plan_enqueue_probe(ctx, plans[i]);
+    if (rc != HX_OK) return rc;
+  }
+  return HX_OK;
+}
+
+}  // extern "C"
+
+// builds of one plan on the auxiliary streams (which must already follow the main stream's
+// fork point); records the plan's per-stream completion events
+static int plan_enqueue_builds(hx_ctx* ctx, hx_plan* pl) {
+  const int nb = (int)pl->hts.size();
+  for (int b = 0; b < nb; ++b) {
+    int rc = ht_enqueue_build(ctx, pl->hts[b], ctx->aux[b % hx_ctx::kAux]);
+    if (rc != HX_OK) return rc;
+  }
+  for (int a = 0; a < std::min(nb, (int)hx_ctx::kAux); ++a)
+    HX_CK(cudaEventRecord(pl->built_ev[a], ctx->aux[a]));
+  return HX_OK;
+}
+
+// K1 (after the plan's builds) -> merge -> finalize -> D2H on the main stream
+static int plan_enqueue_probe(hx_ctx* ctx, hx_plan* pl) {
+  const int nb = (int)pl->hts.size();
+  for (int a = 0; a < std::min(nb, (int)hx_ctx::kAux); ++a)
+    HX_CK(cudaStreamWaitEvent(ctx->stream, pl->built_ev[a], 0));
   int rc = k1_enqueue(ctx, pl->k1, true, pl->k1_e0, pl->k1_e1);
   if (rc != HX_OK) return rc;
   if (ctx->comm && ctx->nranks > 1) {
@@ -270,6 +306,8 @@ int hx_plan_enqueue(hx_ctx* ctx, hx_plan* pl) {
   pl->enqueued = true;
   return HX_OK;
 }
+
+extern "C" {
 
 int hx_plan_result(hx_plan* pl, int64_t* sums, int64_t* counts, int32_t* keys, int64_t cap,
                    int64_t* n_rows) {

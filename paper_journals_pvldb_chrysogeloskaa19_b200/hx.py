@@ -317,6 +317,12 @@ class Plan:
             pass
 
 
+def plans_enqueue(ctx: Context, plans: Sequence["Plan"]) -> None:
+    """hx_plans_enqueue: all builds first (overlapping earlier pipelines), then pipelines."""
+    arr = (ctypes.c_void_p * max(1, len(plans)))(*[p.h.value for p in plans])
+    call("hx_plans_enqueue", ctx.h, arr, len(plans))
+
+
 def build_spec(dim: int, key_col: int, preds=(), group_col: int = -1, group_lo: int = 0,
                group_hi: int = 0) -> _hx.hx_build_spec:
     s = _hx.hx_build_spec()

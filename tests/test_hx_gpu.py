@@ -158,6 +158,16 @@ def test_plans_and_graph_replay(ctx, seed):
         graph.launch()
         for q, pl in plans.items():
             assert pl.rows() == want[q], q
+    # one step: every build first (overlapping earlier pipelines), then the pipelines
+    ordered = [pl.hp for pl in plans.values()]
+    hx.plans_enqueue(ctx, ordered)
+    for q, pl in plans.items():
+        assert pl.rows() == want[q], q
+    graph2 = hx.capture(ctx, lambda: hx.plans_enqueue(ctx, ordered))
+    graph2.launch()
+    for q, pl in plans.items():
+        assert pl.rows() == want[q], q
+    graph2.close()
     ms, nbytes = plans["q2.1"].hp.k1_time()
     assert ms > 0 and nbytes == 30001 * 16
     graph.close()
