@@ -53,12 +53,17 @@ __host__ __device__ __forceinline__ int bloom_log2w_for(long long n_keys) {
   while ((1ll << l) < bits) ++l;
   return l - 5;
 }
+// One multiply: the word is the top log2w bits of h, the two bit positions are h[6..10] and
+// h[11..15] (disjoint from the word bits while log2w <= 16, i.e. filters up to 256 KB).
+__host__ __device__ __forceinline__ uint32_t bloom_hash(int32_t key) {
+  return (uint32_t)key * 0x85EBCA6Bu;
+}
 __host__ __device__ __forceinline__ uint32_t bloom_word(int32_t key, int log2w) {
-  return log2w == 0 ? 0u : ((uint32_t)key * 0x85EBCA6Bu) >> (32 - log2w);
+  return log2w == 0 ? 0u : bloom_hash(key) >> (32 - log2w);
 }
 __host__ __device__ __forceinline__ uint32_t bloom_mask(int32_t key) {
-  const uint32_t h = (uint32_t)key * 0xC2B2AE35u;
-  return (1u << (h >> 27)) | (1u << ((h >> 22) & 31u));
+  const uint32_t h = bloom_hash(key);
+  return (1u << ((h >> 6) & 31u)) | (1u << ((h >> 11) & 31u));
 }
 
 // Slots are grouped in 16-byte buckets of kBucketSlots = 2 (one 128-bit load per probe

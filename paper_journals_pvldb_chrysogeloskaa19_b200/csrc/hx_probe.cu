@@ -49,7 +49,9 @@ constexpr int kMaxStageCols = 8;
 constexpr int kSmemGroups = 1024;          // per-CTA group table capacity
 // dynamic smem: [barriers 128 | reduce 256 | head 128 | queues 8 x 256 x (1+4) B | groups | tiles]
 constexpr int kSmemQueueOff = 512;
-constexpr int kSmemFixed = kSmemQueueOff + kConsumers * kRowsPerThread * 5;
+constexpr int kCarryBytes = (HX_MAX_JOINS + 3) * 32 * 4;  // one CarryBuf per consumer warp
+constexpr int kSmemCarryOff = kSmemQueueOff + kConsumers * kRowsPerThread * 5;
+constexpr int kSmemFixed = kSmemCarryOff + kConsumerWarps * kCarryBytes;
 
 struct JoinDev {
   int32_t c;                               // staged column of the FK
@@ -148,9 +150,12 @@ struct JoinState {
   int32_t blw;                // its log2 word count
 };
 
+// Same test as (word & bloom_mask(key)) == bloom_mask(key), in fewer instructions: the two
+// bit positions are tested with rotates (shf.r.wrap takes the shift modulo 32). blw >= 1.
 __device__ __forceinline__ bool bloom_pass(const JoinState& j, int32_t key) {
-  const uint32_t m = bloom_mask(key);
-  return (j.sbloom[bloom_word(key, j.blw)] & m) == m;
+  const uint32_t h = bloom_hash(key);
+  const uint32_t w = j.sbloom[h >> (32 - j.blw)];
+  return (__funnelshift_r(w, w, h >> 6) & __funnelshift_r(w, w, h >> 11)) & 1u;
 }
 
 __device__ __forceinline__ uint32_t bucket_of(int32_t key, int shift) {
@@ -187,7 +192,16 @@ __device__ __forceinline__ void accumulate(const K1Params& p, bool smem_table,
                                            long long& acc_cnt) {
   if (GROUPED) {
     if (smem_table) {
-      atomicAdd(s_sum + g, (unsigned long long)m);
+      // the shared-memory SUM is kept as two 32-bit words (sm_100 has no native 64-bit
+      // shared atomic add): add the low word, carry into the high word on wrap-around —
+      // exact modulo 2^64 like the int64 sum
+      uint32_t* s_lo = reinterpret_cast<uint32_t*>(s_sum);
+      uint32_t* s_hi = s_lo + p.smem_groups;
+      const unsigned long long um = (unsigned long long)m;
+      const uint32_t lo = (uint32_t)um, hi = (uint32_t)(um >> 32);
+      const uint32_t old = atomicAdd(s_lo + g, lo);
+      const uint32_t up = hi + (uint32_t)(old + lo < old);
+      if (up) atomicAdd(s_hi + g, up);
       atomicAdd(s_cnt + g, 1u);
     } else {
       atomicAdd(p.g_sum + g, (unsigned long long)m);
@@ -197,6 +211,108 @@ __device__ __forceinline__ void accumulate(const K1Params& p, bool smem_table,
     acc_sum += m;
     acc_cnt += 1;
   }
+}
+
+// A queued row for stage C, by value: the FK of every join, the measure operands, and the
+// group-index part known so far (or ~next_bucket of a deferred first-join probe).
+struct CarryEntry {
+  int32_t key[HX_MAX_JOINS];
+  int32_t a, b, g;
+};
+// Per-warp buffer of the (< 32) queued rows carried to the next tile (SoA, one slot per lane).
+struct CarryBuf {
+  int32_t key[HX_MAX_JOINS][32];
+  int32_t a[32], b[32], g[32];
+};
+
+// Entry idx of the combined sequence [carried rows..., this tile's queue...].
+template <int NJ>
+__device__ __forceinline__ CarryEntry load_entry(const K1Params& p,
+                                                 const JoinState (&js)[HX_MAX_JOINS],
+                                                 const CarryBuf* cb, int n_carry,
+                                                 const uint8_t* q_row, const int32_t* q_g, int j0,
+                                                 const int32_t* wcol, int stride, int idx) {
+  CarryEntry e;
+  if (idx < n_carry) {
+#pragma unroll
+    for (int jx = 0; jx < NJ; ++jx) e.key[jx] = cb->key[jx][idx];
+    e.a = cb->a[idx];
+    e.b = cb->b[idx];
+    e.g = cb->g[idx];
+  } else {
+    const int i = idx - n_carry;
+    const int r = q_row[i];
+#pragma unroll
+    for (int jx = 0; jx < NJ; ++jx) e.key[jx] = wcol[js[jx].c * stride + r];
+    e.a = wcol[p.agg_a * stride + r];
+    e.b = wcol[p.agg_b * stride + r];
+    e.g = j0 ? q_g[i] : 0;
+  }
+  return e;
+}
+
+// Stage C for one row: the remaining shared-memory filters, then the probes of every join
+// not yet resolved issued together (one L2 round trip), then measure + group atomic.
+template <int NJ, bool GROUPED>
+__device__ __forceinline__ void stage_c_row(const K1Params& p, const JoinState (&js)[HX_MAX_JOINS],
+                                            const CarryEntry& e, int j0, int jf, bool smem_table,
+                                            unsigned long long* s_sum, uint32_t* s_cnt,
+                                            long long& acc_sum, long long& acc_cnt) {
+  int32_t gg = e.g;
+  bool alive = true;
+  uint32_t b[NJ > 0 ? NJ : 1];
+  uint32_t pend = 0;
+#pragma unroll
+  for (int jx = 0; jx < NJ; ++jx) {
+    if (jx < j0) {  // resume a deferred probe of the first join
+      const bool deferred = gg < 0;
+      b[jx] = deferred ? ~(uint32_t)gg : 0u;
+      pend |= (uint32_t)deferred << jx;
+    } else {
+      b[jx] = bucket_of(e.key[jx], js[jx].shift);
+      pend |= 1u << jx;
+      if (jx != jf && js[jx].sbloom) alive = alive && bloom_pass(js[jx], e.key[jx]);
+    }
+  }
+  if (!alive) pend = 0;
+  if (gg < 0) gg = 0;
+  while (pend) {
+    ulonglong2 v[NJ > 0 ? NJ : 1];
+#pragma unroll
+    for (int jx = 0; jx < NJ; ++jx)
+      if ((pend >> jx) & 1u) v[jx] = __ldg(js[jx].buckets + b[jx]);
+#pragma unroll
+    for (int jx = 0; jx < NJ; ++jx) {
+      if (!((pend >> jx) & 1u)) continue;
+      bool hit, miss;
+      int32_t rank;
+      probe_step(v[jx], e.key[jx], hit, miss, rank);
+      if (hit) gg += rank * js[jx].jstride;
+      alive = alive && !miss;
+      pend &= ~((uint32_t)(hit || miss) << jx);
+      b[jx] = (b[jx] + 1) & js[jx].bmask;
+    }
+    if (!alive) pend = 0;
+  }
+  if (alive)
+    accumulate<GROUPED>(p, smem_table, s_sum, s_cnt, gg, measure(p.agg_op, e.a, e.b), acc_sum,
+                        acc_cnt);
+}
+
+// Join whose filter runs on every row (first filtered join in probe order), or -1.
+template <int NJ>
+__device__ __forceinline__ int first_filter(const JoinState (&js)[HX_MAX_JOINS]) {
+  int jf = -1;
+#pragma unroll
+  for (int jx = NJ - 1; jx >= 0; --jx)
+    if (js[jx].sbloom) jf = jx;
+  return jf;
+}
+// 1 when stage B probes the first join in place (no lineorder predicate, no filter on it).
+template <int NJ>
+__device__ __forceinline__ int first_join_in_place(const K1Params& p,
+                                                   const JoinState (&js)[HX_MAX_JOINS]) {
+  return (NJ > 0 && p.n_preds == 0 && !js[0].sbloom) ? 1 : 0;
 }
 
 // Process one staged tile. Warp w owns rows [w*128, w*128+128) of the tile; lane l holds the
@@ -217,8 +333,9 @@ __device__ __forceinline__ void process_tile(const K1Params& p, const JoinState 
                                              const int32_t* sbase, int stride, int rows_valid,
                                              int warp, int lane, bool smem_table,
                                              unsigned long long* s_sum, uint32_t* s_cnt,
-                                             uint8_t* q_row, int32_t* q_g,
-                                             long long& acc_sum, long long& acc_cnt) {
+                                             uint8_t* q_row, int32_t* q_g, CarryBuf* cb,
+                                             int& n_carry, long long& acc_sum,
+                                             long long& acc_cnt) {
   const int wbase = warp * (32 * kRowsPerThread);
   const int r0 = wbase + lane * kRowsPerThread;
   const int32_t* tb = sbase + r0;
@@ -248,11 +365,14 @@ __device__ __forceinline__ void process_tile(const K1Params& p, const JoinState 
     }
   }
 
-  // stage F: semi-join reduction with the shared-memory Bloom filters of the joins that have
-  // one (no false negatives; ~5% false positives are removed by the exact probe in stage C)
+  // stage F: semi-join reduction with the shared-memory Bloom filter of the first filtered
+  // join (the most selective: joins are in ascending pass fraction) on every row; the other
+  // joins' filters are applied to the few survivors in stage C. No false negatives; the
+  // ~5% false positives are removed by the exact probe.
+  const int jf = first_filter<NJ>(js);
 #pragma unroll
   for (int jx = 0; jx < NJ; ++jx) {
-    if (!js[jx].sbloom) continue;
+    if (jx != jf) continue;
     const int4 kv = *reinterpret_cast<const int4*>(tb + js[jx].c * stride);
     const int32_t key[4] = {kv.x, kv.y, kv.z, kv.w};
 #pragma unroll
@@ -262,8 +382,8 @@ __device__ __forceinline__ void process_tile(const K1Params& p, const JoinState 
   int32_t g[kRowsPerThread];
 #pragma unroll
   for (int k = 0; k < kRowsPerThread; ++k) g[k] = 0;
-  int j0 = 0;
-  if (NJ > 0 && p.n_preds == 0 && !js[0].sbloom) {
+  const int j0 = first_join_in_place<NJ>(p, js);
+  if (j0) {
     // stage B: ONE probe step of the first join for the lane's 4 rows (4 independent
     // 128-bit loads in flight). Rows whose bucket was full without a verdict (rare at load
     // factor 1/4) are queued with ~next_bucket in place of the group index and finish in
@@ -287,7 +407,6 @@ __device__ __forceinline__ void process_tile(const K1Params& p, const JoinState 
       g[k] = hit ? rank * j.jstride : (int32_t)~((b[k] + 1) & j.bmask);
       m &= ~((uint32_t)miss << k);
     }
-    j0 = 1;
   }
 
   if (NJ == 0) {
@@ -302,69 +421,73 @@ __device__ __forceinline__ void process_tile(const K1Params& p, const JoinState 
     return;
   }
 
-  // compaction: append this warp's survivors to its queue
-  int qn = 0;
-  const uint32_t lt = (1u << lane) - 1u;
+  // compaction: append this warp's survivors to its queue — a warp prefix sum of the lanes'
+  // survivor counts gives each lane its slots; a lane then writes only its surviving rows
+  const int cnt = __popc(m);
+  int incl = cnt;
 #pragma unroll
-  for (int k = 0; k < kRowsPerThread; ++k) {
-    const bool a = (m >> k) & 1u;
-    const uint32_t bal = __ballot_sync(kFull, a);
-    if (a) {
-      const int pos = qn + __popc(bal & lt);
-      q_row[pos] = (uint8_t)(lane * kRowsPerThread + k);
-      q_g[pos] = g[k];
+  for (int o = 1; o < 32; o <<= 1) {
+    const int t = __shfl_up_sync(kFull, incl, o);
+    if (lane >= o) incl += t;
+  }
+  const int qn = __shfl_sync(kFull, incl, 31);
+  int pos = incl - cnt;
+  for (uint32_t bits = m; bits; bits &= bits - 1u, ++pos) {
+    const int k = __ffs(bits) - 1;
+    q_row[pos] = (uint8_t)(lane * kRowsPerThread + k);
+    if (j0) {
+      int32_t gv = 0;
+#pragma unroll
+      for (int kk = 0; kk < kRowsPerThread; ++kk) gv = kk == k ? g[kk] : gv;
+      q_g[pos] = gv;
     }
-    qn += __popc(bal);
   }
   __syncwarp();
 
-  // stage C: one queued row per lane; every remaining join (and a deferred first-join probe)
-  // is probed concurrently
+  // stage C in full batches of 32: the warp's queue of this tile is appended to the rows
+  // carried over from earlier tiles; every complete batch of 32 is processed now (one row per
+  // lane, all lanes busy), the < 32 left over are copied (as values) into the carry buffer,
+  // so the tile's shared-memory stage can be released.
   const int32_t* wcol = sbase + wbase;
-  for (int i = lane; i < qn; i += 32) {
-    const int r = q_row[i];
-    int32_t gg = q_g[i];
-    bool alive = true;
-    int32_t key[NJ > 0 ? NJ : 1];
-    uint32_t b[NJ > 0 ? NJ : 1];
-    uint32_t pend = 0;
-#pragma unroll
-    for (int jx = 0; jx < NJ; ++jx) {
-      key[jx] = wcol[js[jx].c * stride + r];
-      if (jx < j0) {  // resume a deferred probe of the first join
-        const bool deferred = gg < 0;
-        b[jx] = deferred ? ~(uint32_t)gg : 0u;
-        pend |= (uint32_t)deferred << jx;
-      } else {
-        b[jx] = bucket_of(key[jx], js[jx].shift);
-        pend |= 1u << jx;
-      }
-    }
-    if (gg < 0) gg = 0;
-    while (pend) {
-      ulonglong2 v[NJ > 0 ? NJ : 1];
-#pragma unroll
-      for (int jx = 0; jx < NJ; ++jx)
-        if ((pend >> jx) & 1u) v[jx] = __ldg(js[jx].buckets + b[jx]);
-#pragma unroll
-      for (int jx = 0; jx < NJ; ++jx) {
-        if (!((pend >> jx) & 1u)) continue;
-        bool hit, miss;
-        int32_t rank;
-        probe_step(v[jx], key[jx], hit, miss, rank);
-        if (hit) gg += rank * js[jx].jstride;
-        alive = alive && !miss;
-        pend &= ~((uint32_t)(hit || miss) << jx);
-        b[jx] = (b[jx] + 1) & js[jx].bmask;
-      }
-      if (!alive) pend = 0;
-    }
-    if (alive)
-      accumulate<GROUPED>(p, smem_table, s_sum, s_cnt, gg,
-                          measure(p.agg_op, wcol[p.agg_a * stride + r], wcol[p.agg_b * stride + r]),
-                          acc_sum, acc_cnt);
+  const int total = n_carry + qn;
+  const int full_end = total & ~31;
+  for (int base = 0; base < full_end; base += 32) {
+    CarryEntry e = load_entry<NJ>(p, js, cb, n_carry, q_row, q_g, j0, wcol, stride, base + lane);
+    stage_c_row<NJ, GROUPED>(p, js, e, j0, jf, smem_table, s_sum, s_cnt, acc_sum, acc_cnt);
   }
-  __syncwarp();  // the queue is reused by the next tile
+  {
+    const int idx = full_end + lane;
+    const bool has = idx < total;
+    CarryEntry e{};
+    if (has) e = load_entry<NJ>(p, js, cb, n_carry, q_row, q_g, j0, wcol, stride, idx);
+    __syncwarp();
+    if (has) {
+#pragma unroll
+      for (int jx = 0; jx < NJ; ++jx) cb->key[jx][lane] = e.key[jx];
+      cb->a[lane] = e.a;
+      cb->b[lane] = e.b;
+      cb->g[lane] = e.g;
+    }
+    n_carry = total - full_end;
+  }
+  __syncwarp();  // the queue and the carry buffer are reused by the next tile
+}
+
+// The rows still carried by a warp after its last tile (fewer than 32).
+template <int NJ, bool GROUPED>
+__device__ __forceinline__ void drain_carry(const K1Params& p, const JoinState (&js)[HX_MAX_JOINS],
+                                            const CarryBuf* cb, int n_carry, int lane, int j0,
+                                            int jf, bool smem_table, unsigned long long* s_sum,
+                                            uint32_t* s_cnt, long long& acc_sum,
+                                            long long& acc_cnt) {
+  if (lane >= n_carry) return;
+  CarryEntry e;
+#pragma unroll
+  for (int jx = 0; jx < NJ; ++jx) e.key[jx] = cb->key[jx][lane];
+  e.a = cb->a[lane];
+  e.b = cb->b[lane];
+  e.g = cb->g[lane];
+  stage_c_row<NJ, GROUPED>(p, js, e, j0, jf, smem_table, s_sum, s_cnt, acc_sum, acc_cnt);
 }
 
 __device__ __forceinline__ void mbar_wait_sleep(uint64_t* bar, uint32_t parity) {
@@ -447,6 +570,8 @@ __global__ void __launch_bounds__(kThreads, kCtasPerSm) k1_probe_agg(const __gri
   const int ctid = tid;  // 0..255
   uint8_t* q_row = q_rows + warp * (32 * kRowsPerThread);
   int32_t* q_g = q_gs + warp * (32 * kRowsPerThread);
+  CarryBuf* cb = reinterpret_cast<CarryBuf*>(smem + kSmemCarryOff + warp * kCarryBytes);
+  int n_carry = 0;
   JoinState js[HX_MAX_JOINS];
 #pragma unroll
   for (int j = 0; j < HX_MAX_JOINS; ++j) {
@@ -476,11 +601,11 @@ __global__ void __launch_bounds__(kThreads, kCtasPerSm) k1_probe_agg(const __gri
         if (lw >= 2) {
           for (int i = ctid; i < (1 << lw) / 4; i += kConsumers)
             reinterpret_cast<uint4*>(dst)[i] = __ldg(src + i);
-        } else if (ctid < (1 << lw)) {
-          dst[ctid] = __ldg(p.joins[j].bloom + ctid);
+        } else if (ctid < 2) {  // 1-2 words: replicate to two so that blw >= 1
+          dst[ctid] = __ldg(p.joins[j].bloom + (lw == 0 ? 0 : ctid));
         }
         js[j].sbloom = dst;
-        js[j].blw = lw;
+        js[j].blw = lw == 0 ? 1 : lw;
       }
       dst += reserved;
     }
@@ -488,8 +613,10 @@ __global__ void __launch_bounds__(kThreads, kCtasPerSm) k1_probe_agg(const __gri
   const long long n_groups = GROUPED ? p.meta->n_groups : 1;
   const bool smem_table = GROUPED && n_groups <= p.smem_groups;
   if (smem_table) {
+    uint32_t* s_lo = reinterpret_cast<uint32_t*>(s_sum);
     for (int g = ctid; g < n_groups; g += kConsumers) {
-      s_sum[g] = 0;
+      s_lo[g] = 0;
+      s_lo[p.smem_groups + g] = 0;
       s_cnt[g] = 0;
     }
   }
@@ -500,7 +627,7 @@ __global__ void __launch_bounds__(kThreads, kCtasPerSm) k1_probe_agg(const __gri
       for (int c = 0; c < p.n_cols; ++c) headbuf[c * 4 + ctid] = p.head_col[c][ctid];
     consumer_sync();
     process_tile<NJ, GROUPED>(p, js, headbuf, 4, p.head_rows, warp, lane, smem_table, s_sum,
-                              s_cnt, q_row, q_g, acc_sum, acc_cnt);
+                              s_cnt, q_row, q_g, cb, n_carry, acc_sum, acc_cnt);
   }
   consumer_sync();
 
@@ -519,7 +646,7 @@ __global__ void __launch_bounds__(kThreads, kCtasPerSm) k1_probe_agg(const __gri
       consumer_sync();
     }
     process_tile<NJ, GROUPED>(p, js, st, kTileRows, rows, warp, lane, smem_table, s_sum, s_cnt,
-                              q_row, q_g, acc_sum, acc_cnt);
+                              q_row, q_g, cb, n_carry, acc_sum, acc_cnt);
     __syncwarp();
     if (lane == 0) mbar_arrive(empty + s);
     if (++s == p.stages) {
@@ -528,14 +655,22 @@ __global__ void __launch_bounds__(kThreads, kCtasPerSm) k1_probe_agg(const __gri
     }
   }
 
+  // the rows this warp still carries
+  if (NJ > 0)
+    drain_carry<NJ, GROUPED>(p, js, cb, n_carry, lane, first_join_in_place<NJ>(p, js),
+                             first_filter<NJ>(js), smem_table, s_sum, s_cnt, acc_sum, acc_cnt);
+  __syncwarp();
+
   // ---------------- flush the CTA's partial aggregate ----------------
   if (GROUPED) {
     if (smem_table) {
       consumer_sync();
+      const uint32_t* s_lo = reinterpret_cast<const uint32_t*>(s_sum);
       for (int g = ctid; g < n_groups; g += kConsumers) {
         const uint32_t c = s_cnt[g];
         if (c) {
-          atomicAdd(p.g_sum + g, s_sum[g]);
+          atomicAdd(p.g_sum + g,
+                    ((unsigned long long)s_lo[p.smem_groups + g] << 32) | s_lo[g]);
           atomicAdd(p.g_cnt + g, (unsigned long long)c);
         }
       }
@@ -634,8 +769,8 @@ constexpr size_t smem_budget(int ctas) { return (228 * 1024) / ctas - 1024; }
 int pick_stages(int n_cols, int smem_groups) {
   // as many tile stages as fit next to kCtasPerSm CTAs per SM, at least double buffering
   // (at most ~96 KB of tiles per CTA: the rest of a large CTA is left for Bloom filters)
-  const size_t budget = std::min<size_t>(smem_budget(kCtasPerSm), 96 * 1024 + 24 * 1024);
   const size_t fixed = kSmemFixed + (((size_t)smem_groups * 12 + 127) & ~size_t(127));
+  const size_t budget = std::min<size_t>(smem_budget(kCtasPerSm), fixed + 96 * 1024);
   const size_t stage = (size_t)n_cols * kTileRows * 4;
   const int s = budget > fixed ? (int)((budget - fixed) / stage) : 0;
   return std::max(2, std::min(4, s));
