@@ -35,6 +35,9 @@ constexpr unsigned kFull = 0xFFFFFFFFu;
 #ifndef HX_K1_WARPS
 #define HX_K1_WARPS 16  // consumer warps per CTA (tuned: tools/variants/run.sh)
 #endif
+#ifndef HX_K1_STAGE_KB
+#define HX_K1_STAGE_KB 160  // max shared memory for the tile ring (the rest: Bloom filters)
+#endif
 #ifndef HX_K1_CTAS
 #define HX_K1_CTAS 1    // resident CTAs per SM the launch bounds / smem budget target
                         // (one CTA per SM shares one copy of the Bloom filters)
@@ -770,7 +773,7 @@ int pick_stages(int n_cols, int smem_groups) {
   // as many tile stages as fit next to kCtasPerSm CTAs per SM, at least double buffering
   // (at most ~96 KB of tiles per CTA: the rest of a large CTA is left for Bloom filters)
   const size_t fixed = kSmemFixed + (((size_t)smem_groups * 12 + 127) & ~size_t(127));
-  const size_t budget = std::min<size_t>(smem_budget(kCtasPerSm), fixed + 96 * 1024);
+  const size_t budget = std::min<size_t>(smem_budget(kCtasPerSm), fixed + HX_K1_STAGE_KB * 1024);
   const size_t stage = (size_t)n_cols * kTileRows * 4;
   const int s = budget > fixed ? (int)((budget - fixed) / stage) : 0;
   return std::max(2, std::min(4, s));
