@@ -51,6 +51,8 @@ def parse():
     ap.add_argument("--no-e2e", action="store_true")
     ap.add_argument("--queries", default="all")
     ap.add_argument("--no-graph", action="store_true", help="enqueue plans without a CUDA graph")
+    ap.add_argument("--variant", default="hbm", choices=["hbm", "host"],
+                    help="host: lineorder in pinned host memory streamed over PCIe (config 5)")
     return ap.parse_args()
 
 
@@ -70,12 +72,16 @@ def peaks():
         return 6650.0, "fallback (B200_PROFILING.md)"
 
 
-def workload_name(sf, world):
+def workload_name(sf, world, variant="hbm", queries=None):
+    if variant == "host":
+        return (f"SSB {'/'.join(q.upper() for q in queries)}, SF{sf:g} per GPU (SF{sf * world:g} "
+                "total), lineorder host-resident in pinned memory, streamed over PCIe (mem-move)")
     return f"SSB all 13 queries, SF{sf:g} per GPU (SF{sf * world:g} total), HBM-resident"
 
 
 def config(args, world, n_rows_gpu, queries):
-    return {"workload": workload_name(args.sf, world), "sf_per_gpu": args.sf,
+    return {"workload": workload_name(args.sf, world, getattr(args, "variant", "hbm"), queries),
+            "sf_per_gpu": args.sf,
             "sf_total": args.sf * world, "queries": queries,
             "lineorder_rows_per_gpu": n_rows_gpu, "router_block_rows": BLOCK_ROWS,
             "parallelism": f"lineorder block-partitioned over {world} GPU(s); dims replicated; "
@@ -211,7 +217,10 @@ def main():
         uid = [hx.comm_unique_id() if rank == 0 else None]
         dist.broadcast_object_list(uid, src=0)
         ctx.comm_init(world, rank, uid[0])
-    queries = ssb.QUERIES if args.queries == "all" else args.queries.split(",")
+    if args.queries == "all":
+        queries = ["q2.1", "q3.1", "q4.1"] if args.variant == "host" else ssb.QUERIES
+    else:
+        queries = args.queries.split(",")
     C = ssbgen.COLS
 
     # ---- data in HBM: this rank's router blocks of lineorder, full replicated dims -------
@@ -233,7 +242,17 @@ def main():
 
     dims = {t: dev_table(ssbgen.TABLE_COLS[t], 0, ssbgen.table_rows(sz, ssbgen.TABLE_COLS[t][0]))
             for t in ("date", "customer", "supplier", "part")}
-    fact = dev_table(ssbgen.TABLE_COLS["lineorder"], r0, n_mine)
+    if args.variant == "host":
+        # §8(a) a8: lineorder stays in page-locked host memory; K1 streams it over PCIe
+        spec = []
+        for c in ssbgen.TABLE_COLS["lineorder"]:
+            buf = torch.empty(max(n_mine, 1), dtype=torch.int32, pin_memory=True)
+            ssbgen.column(SEED, sz, c, r0, n_mine, out=buf.numpy())
+            keep.append(buf)
+            spec.append((C[c], buf.data_ptr(), n_mine))
+        fact = hx.load_columns(ctx, spec, placement=hx._hx.HX_PLACE_HOST_PINNED)
+    else:
+        fact = dev_table(ssbgen.TABLE_COLS["lineorder"], r0, n_mine)
     torch.cuda.synchronize()
     eng = ssb.SsbEngine(ctx, dims, fact)
     # one prepared plan per query (HT + group buffers allocated once, builds sized once);
@@ -278,7 +297,7 @@ def main():
     clk = clocks.stop()
     ms = e0.elapsed_time(e1)
     k1_ms, k1_n, k1_bytes = k1_acc
-    launches, _, _ = ctx.stats(reset=True)
+    launches, step_h2d, step_d2h = ctx.stats(reset=True)
     if world > 1:
         t = torch.tensor([ms, float(launches)], device="cuda", dtype=torch.float64)
         dist.all_reduce(t[:1], op=dist.ReduceOp.MAX)
@@ -293,11 +312,30 @@ def main():
     tr = ncu_traffic()
     roofline = {"bound": "hbm", "achieved": achieved, "peak": peak, "unit": "GB/s",
                 "frac": achieved / peak, "peak_source": peak_src,
-                "kernel": "k1_probe_agg (fused scan->filter->probe->aggregate), all 13 queries",
+                "kernel": f"k1_probe_agg (fused scan->filter->probe->aggregate), {len(queries)} queries",
                 "algorithmic_bytes_per_launch": k1_bytes / max(k1_n, 1),
                 "k1_ms_per_launch": k1_ms / max(k1_n, 1),
                 "traffic": tr["dram_bytes_per_launch"] if tr else None,
                 "traffic_source": tr["source"] if tr else None}
+    if args.variant == "host":
+        # the streamed pipeline (H2D copies overlapped with K1) is bound by the host link:
+        # peak = this run's own pinned H2D copy bandwidth (1 GiB, best of 3)
+        hb = torch.empty(1 << 28, dtype=torch.int32, pin_memory=True)
+        db_ = torch.empty(1 << 28, dtype=torch.int32, device="cuda")
+        best = 0.0
+        for _ in range(3):
+            c0, c1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+            c0.record(stream)
+            db_.copy_(hb, non_blocking=True)
+            c1.record(stream)
+            torch.cuda.synchronize()
+            best = max(best, hb.numel() * 4 / (c0.elapsed_time(c1) / 1e3) / 1e9)
+        del hb, db_
+        roofline.update({"bound": "pcie", "peak": best, "frac": achieved / best,
+                         "peak_source": "measured in this run: pinned H2D cudaMemcpyAsync, 1 GiB, best of 3",
+                         "kernel": "mem-move H2D ring + k1_probe_agg per block (achieved = streamed "
+                                   "referenced-column bytes / span of the query's K1 launches)",
+                         "traffic": None, "traffic_source": None})
 
     # ---- per query (after the timed region): K1-only and whole-query time ---------------
     per_query = {}
@@ -323,7 +361,14 @@ def main():
 
     # ---- e2e through the C-ABI with HOST buffers (H2D + queries + D2H inside the clock) ---
     e2e = None
-    if not args.no_e2e:
+    if args.variant == "host":
+        # the timed step already moves every input from pinned host memory (H2D ring) and
+        # reads the results back: it IS the end-to-end measurement
+        e2e = {"value": value, "unit": UNIT, "h2d_bytes_per_step": step_h2d // args.steps,
+               "d2h_bytes_per_step": step_d2h // args.steps, "ms_per_step": ms_step,
+               "path": "plans over a HX_PLACE_HOST_PINNED fact table: H2D staging ring + K1 "
+                       "per block + merge + finalize + D2H, one CUDA graph per step"}
+    elif not args.no_e2e:
         host = {}
         for t in ("lineorder", "date", "customer", "supplier", "part"):
             host[t] = {}

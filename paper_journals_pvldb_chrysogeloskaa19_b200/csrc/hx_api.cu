@@ -101,6 +101,7 @@ int hx_init(int device, void* stream, hx_ctx** out) {
     HX_CK(cudaEventCreateWithFlags(&ctx->join_ev[a], cudaEventDisableTiming));
   }
   HX_CK(cudaEventCreateWithFlags(&ctx->fork_ev, cudaEventDisableTiming));
+  HX_CK(cudaStreamCreateWithFlags(&ctx->copy_stream, cudaStreamNonBlocking));
   *out = ctx;
   return HX_OK;
 }
@@ -122,6 +123,10 @@ int hx_finalize(hx_ctx* ctx) {
     if (ctx->join_ev[a]) cudaEventDestroy(ctx->join_ev[a]);
   }
   if (ctx->fork_ev) cudaEventDestroy(ctx->fork_ev);
+  if (ctx->copy_stream) {
+    cudaStreamSynchronize(ctx->copy_stream);
+    cudaStreamDestroy(ctx->copy_stream);
+  }
   if (ctx->comm) ncclCommDestroy(ctx->comm);
   if (ctx->own_stream) cudaStreamDestroy(ctx->stream);
   delete ctx;

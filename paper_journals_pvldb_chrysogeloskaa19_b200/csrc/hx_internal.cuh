@@ -119,12 +119,13 @@ struct hx_ctx {
   double prof_ms = 0.0;
   // hx_stats counters
   int64_t launches = 0, h2d_bytes = 0, d2h_bytes = 0;
-  int64_t capture_launches = 0, capture_d2h = 0;  // counters at hx_graph_begin
+  int64_t capture_launches = 0, capture_d2h = 0, capture_h2d = 0;  // at hx_graph_begin
   // fork/join of the independent dimension builds of a plan (parallel graph branches)
   static constexpr int kAux = 4;
   cudaStream_t aux[kAux] = {nullptr, nullptr, nullptr, nullptr};
   cudaEvent_t fork_ev = nullptr;
   cudaEvent_t join_ev[kAux] = {nullptr, nullptr, nullptr, nullptr};
+  cudaStream_t copy_stream = nullptr;  // mem-move H2D copies of host-resident blocks
 };
 
 struct hx_partition {
@@ -202,7 +203,13 @@ int agg_alloc(hx_ctx* ctx, hx_agg* agg, long long cap_groups, const hx_query_sha
               hx_ht* const* hts);
 int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht* const* hts,
              int n_hts, const hx_agg* agg, K1Prepared** out);
-int k1_enqueue(hx_ctx* ctx, const K1Prepared* k, bool fresh, cudaEvent_t e0, cudaEvent_t e1);
+struct StageRing;   // device staging ring for host-resident fact tables (hx_probe.cu)
+constexpr int64_t kHostBlockRows = int64_t(1) << 21;  // mem-move block: 8 MB per int32 column
+int k1_enqueue(hx_ctx* ctx, const K1Prepared* k, bool fresh, cudaEvent_t e0, cudaEvent_t e1,
+               StageRing* ring = nullptr);
+bool k1_is_host(const K1Prepared* k);
+int ring_create(hx_ctx* ctx, const K1Prepared* k, int64_t block_rows, StageRing** out);
+void ring_destroy(hx_ctx* ctx, StageRing* r);
 void k1_free(K1Prepared* k);
 int64_t k1_bytes(const K1Prepared* k);
 const int32_t* table_col(const hx_table* t, int32_t col_id);

@@ -116,6 +116,7 @@ struct hx_plan {
   size_t out_bytes = 0, inline_bytes = 0;
   cudaEvent_t done = nullptr, k1_e0 = nullptr, k1_e1 = nullptr;
   cudaEvent_t built_ev[hx_ctx::kAux] = {nullptr, nullptr, nullptr, nullptr};
+  StageRing* ring = nullptr;   // host-resident fact table: the mem-move staging ring
   bool enqueued = false;
 };
 
@@ -124,7 +125,7 @@ struct hx_graph {
   cudaGraph_t graph = nullptr;
   cudaGraphExec_t exec = nullptr;
   int64_t launches = 0;
-  int64_t d2h = 0;
+  int64_t d2h = 0, h2d = 0;
 };
 
 static int plan_enqueue_builds(hx_ctx* ctx, hx_plan* pl);
@@ -137,6 +138,7 @@ static void plan_destroy(hx_plan* pl) {
   for (hx_ht* t : pl->hts) ht_destroy(t);
   if (pl->agg.base) cudaFreeAsync(pl->agg.base, pl->ctx->stream);
   if (pl->k1) k1_free(pl->k1);
+  ring_destroy(pl->ctx, pl->ring);
   if (pl->d_out) cudaFreeAsync(pl->d_out, pl->ctx->stream);
   if (pl->h_out) cudaFreeHost(pl->h_out);
   for (cudaEvent_t e : {pl->done, pl->k1_e0, pl->k1_e1})
@@ -204,6 +206,10 @@ int hx_plan_create(hx_ctx* ctx, const hx_table* fact, hx_table* const* dims, int
   // 3) the K1 launch
   rc = k1_setup(ctx, fact, shape, pl->hts.data(), n_builds, &pl->agg, &pl->k1);
   if (rc != HX_OK) return bail(rc);
+  if (k1_is_host(pl->k1) && fact->n_rows > 0) {
+    rc = ring_create(ctx, pl->k1, kHostBlockRows, &pl->ring);
+    if (rc != HX_OK) return bail(rc);
+  }
   // 4) result buffers
   pl->out_bytes = sizeof(OutHeader) + (size_t)ng * sizeof(OutRow);
   pl->inline_bytes = sizeof(OutHeader) + (size_t)std::min<long long>(ng, kOutInline) * sizeof(OutRow);
@@ -289,7 +295,7 @@ static int plan_enqueue_probe(hx_ctx* ctx, hx_plan* pl) {
   const int nb = (int)pl->hts.size();
   for (int a = 0; a < std::min(nb, (int)hx_ctx::kAux); ++a)
     HX_CK(cudaStreamWaitEvent(ctx->stream, pl->built_ev[a], 0));
-  int rc = k1_enqueue(ctx, pl->k1, true, pl->k1_e0, pl->k1_e1);
+  int rc = k1_enqueue(ctx, pl->k1, true, pl->k1_e0, pl->k1_e1, pl->ring);
   if (rc != HX_OK) return rc;
   if (ctx->comm && ctx->nranks > 1) {
     // union router: partial {sum,cnt} arrays are adjacent, one allreduce over NVLink
@@ -372,6 +378,7 @@ int hx_graph_begin(hx_ctx* ctx) {
   HX_CK(cudaSetDevice(ctx->device));
   ctx->capture_launches = ctx->launches;
   ctx->capture_d2h = ctx->d2h_bytes;
+  ctx->capture_h2d = ctx->h2d_bytes;
   HX_CK(cudaStreamBeginCapture(ctx->stream, cudaStreamCaptureModeThreadLocal));
   return HX_OK;
 }
@@ -387,6 +394,8 @@ int hx_graph_end(hx_ctx* ctx, hx_graph** out) {
   ctx->launches = ctx->capture_launches;  // captured, not executed
   g->d2h = ctx->d2h_bytes - ctx->capture_d2h;
   ctx->d2h_bytes = ctx->capture_d2h;
+  g->h2d = ctx->h2d_bytes - ctx->capture_h2d;
+  ctx->h2d_bytes = ctx->capture_h2d;
   if (e != cudaSuccess) {
     if (g->graph) cudaGraphDestroy(g->graph);
     delete g;
@@ -402,6 +411,7 @@ int hx_graph_launch(hx_ctx* ctx, hx_graph* g) {
   HX_CK(cudaGraphLaunch(g->exec, ctx->stream));
   ctx->launches += g->launches;
   ctx->d2h_bytes += g->d2h;
+  ctx->h2d_bytes += g->h2d;
   return HX_OK;
 }
 

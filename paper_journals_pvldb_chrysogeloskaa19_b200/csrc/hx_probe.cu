@@ -809,6 +809,23 @@ struct K1Prepared {
   long long cap_groups = 1;
   int64_t rows = 0;
   int n_cols = 0;
+  // host-resident fact table (§8(a) a8): the staged columns live in pinned host memory and
+  // are streamed block by block through a device staging ring (mem-move)
+  bool host = false;
+  const int32_t* host_col[kMaxStageCols] = {};
+  int occ = 1;
+};
+
+// Device staging ring of the mem-move for a host-resident fact table: kRingStages buffers of
+// block_rows rows x the staged columns, filled by H2D copies on the ctx's copy stream while K1
+// consumes the previous block on the compute stream (Listing 1 L7-19).
+constexpr int kRingStages = 3;
+struct StageRing {
+  int64_t block_rows = 0;
+  int n_cols = 0;
+  void* base = nullptr;
+  int32_t* buf[kRingStages][kMaxStageCols] = {};
+  cudaEvent_t full[kRingStages] = {}, freed[kRingStages] = {};
 };
 
 long long k1_group_bound(const hx_query_shape* sh, hx_ht* const* hts, int n_hts) {
@@ -847,8 +864,6 @@ int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht*
                  sh->n_joins <= HX_MAX_JOINS && sh->n_gdims >= 0 && sh->n_gdims <= HX_MAX_GDIMS &&
                  sh->agg_op >= HX_AGG_SUM && sh->agg_op <= HX_AGG_SUM_SUB,
              HX_EINVAL, "hx_pipeline_probe_agg: bad query shape");
-  HX_REQUIRE(fact->placement != HX_PLACE_HOST_PINNED, HX_EUNSUPPORTED,
-             "hx_pipeline_probe_agg: host-resident fact tables are not supported");
   HX_REQUIRE(agg->n_gdims == sh->n_gdims, HX_EINVAL,
              "hx_pipeline_probe_agg: shape differs from the agg's");
   K1Prepared k{};
@@ -895,12 +910,15 @@ int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht*
   k.cap_groups = agg->cap_groups;
   k.prep_grid = (int)std::max<long long>(1, std::min<long long>((agg->cap_groups + 255) / 256,
                                                                 (long long)ctx->n_sms * 4));
-  // tiles: the head rows up to 16-byte alignment are handled separately
-  const uintptr_t mis = reinterpret_cast<uintptr_t>(table_col(fact, ids[0])) & 15u;
-  for (int c = 0; c < n_cols; ++c)
+  // tiles: the head rows up to 16-byte alignment are handled separately (device tables; a
+  // host-resident table is staged block by block into aligned device buffers instead)
+  k.host = fact->placement == HX_PLACE_HOST_PINNED;
+  const uintptr_t mis = k.host ? 0 : reinterpret_cast<uintptr_t>(table_col(fact, ids[0])) & 15u;
+  for (int c = 0; c < n_cols && !k.host; ++c)
     HX_REQUIRE((reinterpret_cast<uintptr_t>(table_col(fact, ids[c])) & 15u) == mis &&
                    (mis & 3u) == 0,
                HX_EUNSUPPORTED, "hx_pipeline_probe_agg: columns with different alignment");
+  for (int c = 0; c < n_cols && k.host; ++c) k.host_col[c] = table_col(fact, ids[c]);
   const int64_t head = std::min<int64_t>(fact->n_rows, mis ? (16 - (int64_t)mis) / 4 : 0);
   p.n_cols = n_cols;
   for (int c = 0; c < n_cols; ++c) {
@@ -935,6 +953,7 @@ int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht*
   int occ = 0;
   HX_CK(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, k.fn, kThreads, k.smem));
   occ = std::max(1, occ);
+  k.occ = occ;
   k.grid = (int)std::max<int64_t>(1, std::min<int64_t>(p.n_tiles, (int64_t)ctx->n_sms * occ));
   k.rows = fact->n_rows;
   k.n_cols = n_cols;
@@ -942,8 +961,82 @@ int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht*
   return HX_OK;
 }
 
+bool k1_is_host(const K1Prepared* k) { return k->host; }
+
+int ring_create(hx_ctx* ctx, const K1Prepared* k, int64_t block_rows, StageRing** out) {
+  HX_REQUIRE(block_rows > 0 && block_rows % 4 == 0, HX_EINVAL, "staging block must be a multiple of 4 rows");
+  StageRing* r = new StageRing();
+  r->block_rows = std::min<int64_t>(block_rows, std::max<int64_t>(4, (k->rows + 3) & ~int64_t(3)));
+  r->n_cols = k->n_cols;
+  const size_t col_bytes = ((size_t)r->block_rows * 4 + 255) & ~size_t(255);
+  cudaError_t e = cudaMallocAsync(&r->base, col_bytes * r->n_cols * kRingStages, ctx->stream);
+  if (e != cudaSuccess) {
+    delete r;
+    return cuda_fail(e, "cudaMallocAsync(staging ring)", __FILE__, __LINE__);
+  }
+  for (int s = 0; s < kRingStages; ++s) {
+    for (int c = 0; c < r->n_cols; ++c)
+      r->buf[s][c] = reinterpret_cast<int32_t*>(static_cast<char*>(r->base) +
+                                                col_bytes * (s * r->n_cols + c));
+    cudaEventCreateWithFlags(&r->full[s], cudaEventDisableTiming);
+    cudaEventCreateWithFlags(&r->freed[s], cudaEventDisableTiming);
+  }
+  *out = r;
+  return HX_OK;
+}
+
+void ring_destroy(hx_ctx* ctx, StageRing* r) {
+  if (!r) return;
+  if (r->base) cudaFreeAsync(r->base, ctx->stream);
+  for (int s = 0; s < kRingStages; ++s) {
+    if (r->full[s]) cudaEventDestroy(r->full[s]);
+    if (r->freed[s]) cudaEventDestroy(r->freed[s]);
+  }
+  delete r;
+}
+
+// K1 over a host-resident fact table: block b is copied H2D into ring slot b % 3 on the copy
+// stream (after K1 released that slot), K1 runs on it on the compute stream and accumulates
+// into the same group arrays. Copies of the next blocks overlap the current K1.
+static int k1_enqueue_host(hx_ctx* ctx, const K1Prepared* k, StageRing* ring, cudaEvent_t e0,
+                           cudaEvent_t e1) {
+  HX_REQUIRE(ring && ring->n_cols == k->n_cols, HX_EINVAL, "host-resident K1 needs a staging ring");
+  const int64_t B = ring->block_rows;
+  const int64_t nb = (k->rows + B - 1) / B;
+  if (e0) HX_CK(record_event(e0, ctx->stream));
+  HX_CK(cudaEventRecord(ctx->fork_ev, ctx->stream));
+  HX_CK(cudaStreamWaitEvent(ctx->copy_stream, ctx->fork_ev, 0));
+  for (int64_t b = 0; b < nb; ++b) {
+    const int s = (int)(b % kRingStages);
+    const int64_t r0 = b * B, rows = std::min<int64_t>(B, k->rows - r0);
+    if (b >= kRingStages) HX_CK(cudaStreamWaitEvent(ctx->copy_stream, ring->freed[s], 0));
+    for (int c = 0; c < k->n_cols; ++c)
+      HX_CK(cudaMemcpyAsync(ring->buf[s][c], k->host_col[c] + r0, (size_t)rows * 4,
+                            cudaMemcpyHostToDevice, ctx->copy_stream));
+    ctx->h2d_bytes += rows * 4 * k->n_cols;
+    HX_CK(cudaEventRecord(ring->full[s], ctx->copy_stream));
+    HX_CK(cudaStreamWaitEvent(ctx->stream, ring->full[s], 0));
+    K1Params p = k->p;
+    for (int c = 0; c < k->n_cols; ++c) p.col[c] = p.head_col[c] = ring->buf[s][c];
+    p.head_rows = 0;
+    p.n_rows = rows;
+    p.n_tiles = (rows + kTileRows - 1) / kTileRows;
+    const int grid = (int)std::max<int64_t>(1, std::min<int64_t>(p.n_tiles, (int64_t)ctx->n_sms * k->occ));
+    k->fn<<<(unsigned)grid, kThreads, k->smem, ctx->stream>>>(p);
+    HX_CK_LAUNCH("k1_probe_agg");
+    ctx->launches += 1;
+    HX_CK(cudaEventRecord(ring->freed[s], ctx->stream));
+  }
+  // the copy stream rejoins the compute stream (required under graph capture)
+  HX_CK(cudaEventRecord(ctx->fork_ev, ctx->copy_stream));
+  HX_CK(cudaStreamWaitEvent(ctx->stream, ctx->fork_ev, 0));
+  if (e1) HX_CK(record_event(e1, ctx->stream));
+  return HX_OK;
+}
+
 // prepare (group layout + zeroing when `fresh`) then K1; optional timing events around K1.
-int k1_enqueue(hx_ctx* ctx, const K1Prepared* k, bool fresh, cudaEvent_t e0, cudaEvent_t e1) {
+int k1_enqueue(hx_ctx* ctx, const K1Prepared* k, bool fresh, cudaEvent_t e0, cudaEvent_t e1,
+               StageRing* ring) {
   const K1Params& p = k->p;
   k1_prepare<<<k->prep_grid, 256, 0, ctx->stream>>>(const_cast<AggMeta*>(p.meta), k->gh[0], k->gh[1], k->gh[2],
                                                     k->n_gdims, k->gj, p.g_sum, p.g_cnt,
@@ -951,6 +1044,7 @@ int k1_enqueue(hx_ctx* ctx, const K1Prepared* k, bool fresh, cudaEvent_t e0, cud
   HX_CK_LAUNCH("k1_prepare");
   ctx->launches += 1;
   if (k->rows == 0) return HX_OK;
+  if (k->host) return k1_enqueue_host(ctx, k, ring, e0, e1);
   if (e0) HX_CK(record_event(e0, ctx->stream));
   k->fn<<<(unsigned)k->grid, kThreads, k->smem, ctx->stream>>>(p);
   HX_CK_LAUNCH("k1_probe_agg");
@@ -981,12 +1075,21 @@ int probe_agg(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht
     e0 = pooled_event(ctx);
     e1 = pooled_event(ctx);
   }
-  rc = k1_enqueue(ctx, k, fresh, e0, e1);
+  StageRing* ring = nullptr;
+  if (k->host && k->rows > 0) {
+    rc = ring_create(ctx, k, kHostBlockRows, &ring);
+    if (rc != HX_OK) {
+      k1_free(k);
+      return rc;
+    }
+  }
+  rc = k1_enqueue(ctx, k, fresh, e0, e1, ring);
   if (rc == HX_OK && e0) {
     ctx->prof_events.push_back({e0, e1});
     ctx->prof_launches += 1;
     ctx->prof_bytes += k1_bytes(k);
   }
+  ring_destroy(ctx, ring);  // stream-ordered free: after the K1 launches that use it
   k1_free(k);
   return rc;
 }

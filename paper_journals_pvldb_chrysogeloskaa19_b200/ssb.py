@@ -238,3 +238,21 @@ def load_db_numpy(ctx: hx.Context, db: Dict[str, Dict[str, np.ndarray]],
             for t in ("date", "customer", "supplier", "part")}
     fact = hx.load_numpy(ctx, {C[c]: v for c, v in db["lineorder"].items()}, part, part_index)
     return dims, fact
+
+
+def load_db_host_resident(ctx: hx.Context, db: Dict[str, Dict[str, np.ndarray]], pin):
+    """Dimensions to the device; lineorder stays in page-locked host memory
+    (HX_PLACE_HOST_PINNED): K1 streams it block by block over PCIe (mem-move, §8(a) a8).
+    `pin(n)` returns a page-locked int32 buffer of n values with .ctypes / data_ptr access
+    (e.g. lambda n: torch.empty(n, dtype=torch.int32, pin_memory=True))."""
+    dims = {t: hx.load_numpy(ctx, {C[c]: v for c, v in db[t].items()})
+            for t in ("date", "customer", "supplier", "part")}
+    keep, spec = [], []
+    for c, v in db["lineorder"].items():
+        buf = pin(max(1, len(v)))
+        arr = buf.numpy() if hasattr(buf, "numpy") else buf
+        arr[: len(v)] = v
+        keep.append(buf)
+        spec.append((C[c], arr.ctypes.data, len(v)))
+    fact = hx.load_columns(ctx, spec, placement=_hx.HX_PLACE_HOST_PINNED, keep=keep)
+    return dims, fact

@@ -175,6 +175,25 @@ def test_plans_and_graph_replay(ctx, seed):
         pl.close()
 
 
+@pytest.mark.parametrize("sf", [0.002, 0.4])
+def test_host_resident_streaming(ctx, sf):
+    """§8(a) a8: lineorder in pinned host memory, streamed over PCIe in 2^21-row blocks
+    (SF0.4 = 2.4 M rows: two blocks, the second partial), plain and planned paths."""
+    db = ssbgen.database(13, ssbgen.sizes(sf))
+    pin = lambda n: torch.empty(n, dtype=torch.int32, pin_memory=True)
+    dims, fact = ssb.load_db_host_resident(ctx, db, pin)
+    eng = ssb.SsbEngine(ctx, dims, fact)
+    for q in ("q1.1", "q2.1", "q3.1", "q4.1", "q4.3"):
+        want = oracle.run_query(q, db)
+        assert eng.run(q) == want, q
+        pl = eng.plan(q)
+        pl.enqueue()
+        assert pl.rows() == want, q
+        pl.enqueue()  # re-execution reuses the staging ring
+        assert pl.rows() == want, q
+        pl.close()
+
+
 def test_device_generated_columns_match_host(ctx):
     """ssbgen's device fill is bit-identical to the host fill (inputs for the bench)."""
     sz = ssbgen.sizes(0.02)
