@@ -18,8 +18,11 @@ all: ssbgen/libssbgen.so ssbgen/libssbgen_cuda.so oracle/liboracle.so $(if $(wil
 ssbgen/libssbgen.so: ssbgen/ssbgen_host.c ssbgen/ssbgen.h
 	gcc -O2 -fopenmp -shared -fPIC -Wall -o $@ ssbgen/ssbgen_host.c
 
+# -Xptxas -O1: ptxas 12.9 -O3 miscompiles two inlined splitmix64 chains in one expression for
+# sm_100a (wrong values, reproduced by tools/dbg_gen.cu); -O1 is exact (tests compare every
+# device-generated column with the host fill)
 ssbgen/libssbgen_cuda.so: ssbgen/ssbgen_cuda.cu ssbgen/ssbgen.h
-	$(NVCC) $(NVFLAGS) -shared -o $@ ssbgen/ssbgen_cuda.cu
+	$(NVCC) $(NVFLAGS) -Xptxas -O1 -shared -o $@ ssbgen/ssbgen_cuda.cu
 
 oracle/liboracle.so: oracle/ssb_oracle.cpp
 	g++ -O2 -std=c++17 -shared -fPIC -Wall -o $@ oracle/ssb_oracle.cpp

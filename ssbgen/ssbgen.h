@@ -94,10 +94,15 @@ SSBGEN_FN void ssbgen_civil(int64_t z, int32_t* y, int32_t* m, int32_t* d) {
 
 SSBGEN_FN int ssbgen_is_leap(int32_t y) { return (y % 4 == 0 && y % 100 != 0) || y % 400 == 0; }
 
+/* Days before month m (1-based) in a non-leap year, without a lookup table (device code
+   keeps no local arrays): 0,31,59,90,120,151,181,212,243,273,304,334. */
+SSBGEN_FN int32_t ssbgen_days_before_month(int32_t m) {
+  return m <= 2 ? (m - 1) * 31 : (153 * (m - 3) + 2) / 5 + 59;
+}
+
 /* 1-based day number within the year. */
 SSBGEN_FN int32_t ssbgen_daynuminyear(int32_t y, int32_t m, int32_t d) {
-  const int32_t cum[12] = {0, 31, 59, 90, 120, 151, 181, 212, 243, 273, 304, 334};
-  return cum[m - 1] + d + ((m > 2 && ssbgen_is_leap(y)) ? 1 : 0);
+  return ssbgen_days_before_month(m) + d + ((m > 2 && ssbgen_is_leap(y)) ? 1 : 0);
 }
 
 /* yyyymmdd of day index `day` counted from 1992-01-01. */
@@ -112,16 +117,36 @@ SSBGEN_FN int32_t ssbgen_retail(int64_t pk) {
   return (int32_t)(90000 + ((pk / 10) % 20001) + 100 * (pk % 1000));
 }
 
-/* Region of each nation code (nations alphabetical, regions alphabetical; TPC-H map). */
+/* Region of each nation code (nations alphabetical, regions alphabetical; TPC-H map):
+   ALGERIA ARGENTINA BRAZIL CANADA CHINA EGYPT ETHIOPIA FRANCE GERMANY INDIA INDONESIA
+   IRAN IRAQ JAPAN JORDAN KENYA MOROCCO MOZAMBIQUE PERU ROMANIA RUSSIA SAUDI ARABIA
+   UNITED KINGDOM UNITED STATES VIETNAM -> 0111240332244200011334312, packed 3 bits/nation. */
 SSBGEN_FN int32_t ssbgen_nation_region(int32_t nation) {
-  /* ALGERIA ARGENTINA BRAZIL CANADA CHINA EGYPT ETHIOPIA FRANCE GERMANY INDIA INDONESIA
-     IRAN IRAQ JAPAN JORDAN KENYA MOROCCO MOZAMBIQUE PERU ROMANIA RUSSIA SAUDI ARABIA
-     UNITED KINGDOM UNITED STATES VIETNAM */
-  const int8_t r[25] = {0, 1, 1, 1, 2, 4, 0, 3, 3, 2, 2, 4, 4, 2, 4, 0, 0, 0, 1, 3, 3, 4, 3, 1, 2};
-  return r[nation];
+  const uint64_t lo = 0ull | 0ull << 0 | 1ull << 3 | 1ull << 6 | 1ull << 9 | 2ull << 12 |
+                      4ull << 15 | 0ull << 18 | 3ull << 21 | 3ull << 24 | 2ull << 27 | 2ull << 30 |
+                      4ull << 33 | 4ull << 36 | 2ull << 39 | 4ull << 42 | 0ull << 45 | 0ull << 48 |
+                      0ull << 51 | 1ull << 54 | 3ull << 57 | 3ull << 60;  /* nations 0..20 */
+  const uint64_t hi = 4ull << 0 | 3ull << 3 | 1ull << 6 | 2ull << 9;        /* nations 21..24 */
+  return nation < 21 ? (int32_t)((lo >> (3 * nation)) & 7u) : (int32_t)((hi >> (3 * (nation - 21))) & 7u);
 }
 
-/* Value of column `col` at row `row` (0-based). Returns 0 for an unknown column. */
+/* The independent random variables, each a pure function of (seed, row). */
+SSBGEN_FN int32_t ssbgen_lo_partkey(uint64_t seed, const ssbgen_sizes* sz, int64_t row) {
+  return 1 + (int32_t)ssbgen_uniform(seed, SSBGEN_ST_PARTKEY, row, (uint32_t)sz->n_part);
+}
+SSBGEN_FN int32_t ssbgen_lo_quantity(uint64_t seed, int64_t row) {
+  return 1 + (int32_t)ssbgen_uniform(seed, SSBGEN_ST_QUANTITY, row, 50);
+}
+SSBGEN_FN int32_t ssbgen_lo_discount(uint64_t seed, int64_t row) {
+  return (int32_t)ssbgen_uniform(seed, SSBGEN_ST_DISCOUNT, row, 11);
+}
+SSBGEN_FN int32_t ssbgen_p_category(uint64_t seed, int64_t row) {
+  return (int32_t)ssbgen_uniform(seed, SSBGEN_ST_P_MFGR, row, 5) * 5 +
+         (int32_t)ssbgen_uniform(seed, SSBGEN_ST_P_CAT, row, 5);
+}
+
+/* Value of column `col` at row `row` (0-based). Returns 0 for an unknown column.
+   (No recursion and no local arrays: identical code runs on the host and the device.) */
 SSBGEN_FN int32_t ssbgen_value(uint64_t seed, const ssbgen_sizes* sz, int col, int64_t row) {
   switch (col) {
     case SSB_LO_ORDERDATE:
@@ -129,22 +154,21 @@ SSBGEN_FN int32_t ssbgen_value(uint64_t seed, const ssbgen_sizes* sz, int col, i
     case SSB_LO_CUSTKEY:
       return 1 + (int32_t)ssbgen_uniform(seed, SSBGEN_ST_CUSTKEY, row, (uint32_t)sz->n_customer);
     case SSB_LO_PARTKEY:
-      return 1 + (int32_t)ssbgen_uniform(seed, SSBGEN_ST_PARTKEY, row, (uint32_t)sz->n_part);
+      return ssbgen_lo_partkey(seed, sz, row);
     case SSB_LO_SUPPKEY:
       return 1 + (int32_t)ssbgen_uniform(seed, SSBGEN_ST_SUPPKEY, row, (uint32_t)sz->n_supplier);
     case SSB_LO_QUANTITY:
-      return 1 + (int32_t)ssbgen_uniform(seed, SSBGEN_ST_QUANTITY, row, 50);
+      return ssbgen_lo_quantity(seed, row);
     case SSB_LO_DISCOUNT:
-      return (int32_t)ssbgen_uniform(seed, SSBGEN_ST_DISCOUNT, row, 11);
+      return ssbgen_lo_discount(seed, row);
     case SSB_LO_EXTENDEDPRICE:
     case SSB_LO_REVENUE:
     case SSB_LO_SUPPLYCOST: {
-      int64_t pk = ssbgen_value(seed, sz, SSB_LO_PARTKEY, row);
-      int64_t retail = ssbgen_retail(pk);
+      const int64_t retail = ssbgen_retail(ssbgen_lo_partkey(seed, sz, row));
       if (col == SSB_LO_SUPPLYCOST) return (int32_t)(6 * retail / 10);
-      int64_t ext = (int64_t)ssbgen_value(seed, sz, SSB_LO_QUANTITY, row) * retail;
+      const int64_t ext = (int64_t)ssbgen_lo_quantity(seed, row) * retail;
       if (col == SSB_LO_EXTENDEDPRICE) return (int32_t)ext;
-      return (int32_t)(ext * (100 - ssbgen_value(seed, sz, SSB_LO_DISCOUNT, row)) / 100);
+      return (int32_t)(ext * (100 - ssbgen_lo_discount(seed, row)) / 100);
     }
     case SSB_D_DATEKEY: return ssbgen_datekey(row);
     case SSB_D_YEAR: return ssbgen_datekey(row) / 10000;
@@ -154,27 +178,27 @@ SSBGEN_FN int32_t ssbgen_value(uint64_t seed, const ssbgen_sizes* sz, int col, i
     case SSB_D_WEEKNUMINYEAR: {
       int32_t y, m, d;
       ssbgen_civil(SSBGEN_EPOCH_1992 + row, &y, &m, &d);
-      int32_t dn = ssbgen_daynuminyear(y, m, d);
+      const int32_t dn = ssbgen_daynuminyear(y, m, d);
       return col == SSB_D_DAYNUMINYEAR ? dn : dn / 7 + 1;
     }
     case SSB_C_CUSTKEY: case SSB_S_SUPPKEY: case SSB_P_PARTKEY:
       return (int32_t)(row + 1);
     case SSB_C_NATION: return (int32_t)ssbgen_uniform(seed, SSBGEN_ST_C_NATION, row, 25);
-    case SSB_C_REGION: return ssbgen_nation_region(ssbgen_value(seed, sz, SSB_C_NATION, row));
+    case SSB_C_REGION:
+      return ssbgen_nation_region((int32_t)ssbgen_uniform(seed, SSBGEN_ST_C_NATION, row, 25));
     case SSB_C_CITY:
-      return ssbgen_value(seed, sz, SSB_C_NATION, row) * 10 +
+      return (int32_t)ssbgen_uniform(seed, SSBGEN_ST_C_NATION, row, 25) * 10 +
              (int32_t)ssbgen_uniform(seed, SSBGEN_ST_C_CITY, row, 10);
     case SSB_S_NATION: return (int32_t)ssbgen_uniform(seed, SSBGEN_ST_S_NATION, row, 25);
-    case SSB_S_REGION: return ssbgen_nation_region(ssbgen_value(seed, sz, SSB_S_NATION, row));
+    case SSB_S_REGION:
+      return ssbgen_nation_region((int32_t)ssbgen_uniform(seed, SSBGEN_ST_S_NATION, row, 25));
     case SSB_S_CITY:
-      return ssbgen_value(seed, sz, SSB_S_NATION, row) * 10 +
+      return (int32_t)ssbgen_uniform(seed, SSBGEN_ST_S_NATION, row, 25) * 10 +
              (int32_t)ssbgen_uniform(seed, SSBGEN_ST_S_CITY, row, 10);
     case SSB_P_MFGR: return (int32_t)ssbgen_uniform(seed, SSBGEN_ST_P_MFGR, row, 5);
-    case SSB_P_CATEGORY:
-      return ssbgen_value(seed, sz, SSB_P_MFGR, row) * 5 +
-             (int32_t)ssbgen_uniform(seed, SSBGEN_ST_P_CAT, row, 5);
+    case SSB_P_CATEGORY: return ssbgen_p_category(seed, row);
     case SSB_P_BRAND1:
-      return ssbgen_value(seed, sz, SSB_P_CATEGORY, row) * 40 +
+      return ssbgen_p_category(seed, row) * 40 +
              (int32_t)ssbgen_uniform(seed, SSBGEN_ST_P_BRAND, row, 40);
     default: return 0;
   }

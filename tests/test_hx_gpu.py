@@ -194,12 +194,57 @@ def test_host_resident_streaming(ctx, sf):
         pl.close()
 
 
-def test_device_generated_columns_match_host(ctx):
-    """ssbgen's device fill is bit-identical to the host fill (inputs for the bench)."""
-    sz = ssbgen.sizes(0.02)
-    for col in ("lo_orderdate", "lo_revenue", "lo_supplycost", "c_city", "p_brand1", "d_weeknuminyear"):
-        n = ssbgen.table_rows(sz, col)
+@pytest.mark.parametrize("sf", [10, 100])
+def test_parity_full_size_bench_configuration(ctx, sf):
+    """BASELINE.json configs[1] (SF10, 60 M lineorder rows) and configs[2]'s 1-GPU leg (SF100,
+    600 M rows) at full size in the launch configuration bench.py times: columns generated in
+    HBM, prepared plans, one CUDA graph for the 13 queries (hx_plans_enqueue). Bit-exact
+    against the oracle run over the host's cores in row ranges merged by summation (the
+    union-router merge)."""
+    import os
+    sz = ssbgen.sizes(sf)
+    stream = torch.cuda.current_stream().cuda_stream
+    keep = []
+
+    def table(cols, n):
+        spec = []
+        for c in cols:
+            t = torch.empty(n, dtype=torch.int32, device="cuda")
+            ssbgen.column_device(42, sz, c, t.data_ptr(), 0, n, stream)
+            keep.append(t)
+            spec.append((C[c], t.data_ptr(), n))
+        return hx.load_columns(ctx, spec, placement=_hx.HX_PLACE_VIEW, keep=keep)
+
+    dims = {t: table(ssbgen.TABLE_COLS[t], ssbgen.table_rows(sz, ssbgen.TABLE_COLS[t][0]))
+            for t in ("date", "customer", "supplier", "part")}
+    fact = table(ssbgen.TABLE_COLS["lineorder"], sz["n_lineorder"])
+    torch.cuda.synchronize()
+    eng = ssb.SsbEngine(ctx, dims, fact)
+    plans = {q: eng.plan(q) for q in QUERIES}
+    order = [plans[q].hp for q in QUERIES]
+    graph = hx.capture(ctx, lambda: hx.plans_enqueue(ctx, order))
+    graph.launch()
+    got = {q: plans[q].rows() for q in QUERIES}
+    db = ssbgen.database(42, sz)
+    for q in QUERIES:
+        want = oracle.run_query_ranges(q, db, os.cpu_count() or 8)
+        assert {tuple(r[:-2]): (r[-2], r[-1]) for r in got[q]} == want, q
+        plan = ssb.PLANS[q]
+        assert got[q] == ssb.order_by(plan, got[q]), q  # ORDER BY holds
+    graph.close()
+    for pl in plans.values():
+        pl.close()
+
+
+@pytest.mark.parametrize("sf", [0.02, 100])
+def test_device_generated_columns_match_host(ctx, sf):
+    """ssbgen's device fill is bit-identical to the host fill (the bench's inputs): every
+    column of every dimension, and a 4 M-row slice of every lineorder column."""
+    sz = ssbgen.sizes(sf)
+    for col in ssbgen.COLS:
+        n = min(ssbgen.table_rows(sz, col), 4_000_000)
+        r0 = ssbgen.table_rows(sz, col) - n  # the tail of the table (largest row counters)
         t = torch.empty(n, dtype=torch.int32, device="cuda")
-        ssbgen.column_device(42, sz, col, t.data_ptr(), 0, n, torch.cuda.current_stream().cuda_stream)
+        ssbgen.column_device(42, sz, col, t.data_ptr(), r0, n, torch.cuda.current_stream().cuda_stream)
         torch.cuda.synchronize()
-        assert np.array_equal(t.cpu().numpy(), ssbgen.column(42, sz, col)), col
+        assert np.array_equal(t.cpu().numpy(), ssbgen.column(42, sz, col, r0, n)), col
