@@ -24,6 +24,8 @@
 //     mixed radix of the probed dimensions' dense ranks, flushed with one global atomic per
 //     non-empty group per CTA; ungrouped queries reduce warp -> CTA -> one global atomic.
 #include <algorithm>
+#include <cstdio>
+#include <cstdlib>
 
 #include "hx_internal.cuh"
 
@@ -933,20 +935,45 @@ int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht*
   p.g_cnt = agg->cnts;
   const bool grouped = sh->n_gdims > 0;
   p.smem_groups = grouped ? (int32_t)std::min<long long>(kSmemGroups, agg->cap_groups) : 0;
-  p.stages = pick_stages(n_cols, p.smem_groups);
-  // shared-memory Bloom filters (semi-join reduction) for the joins whose passing key count
-  // is known (a plan observed it) and selective (at most half the dimension passes), in
-  // probe order, while the CTA still fits twice per SM
-  p.filter_words = 0;
+  // Shared-memory plan: the tile ring (pick_stages) and the Bloom filters (semi-join
+  // reduction) of the joins whose passing key count is known (a plan observed it) and that
+  // are selective (at most half the dimension passes). Filters are taken greedily in probe
+  // order in the shared memory the ring leaves free.
+  int want[HX_MAX_JOINS] = {0, 0, 0, 0};
   for (int j = 0; j < sh->n_joins; ++j) {
     const hx_ht* ht = hts[sh->join_ht[j]];
     if (ht->known_keys < 0 || 2 * ht->known_keys > ht->dim_rows) continue;
-    const int words = std::max(4, 1 << std::min(ht->max_bloom_log2w, bloom_log2w_for(ht->known_keys)));
-    if (k1_smem_bytes(n_cols, p.stages, p.smem_groups, p.filter_words + words) >
-        smem_budget(std::min(kCtasPerSm, 2)))
-      continue;
-    p.joins[j].bloom_words = words;
-    p.filter_words += words;
+    want[j] = std::max(4, 1 << std::min(ht->max_bloom_log2w, bloom_log2w_for(ht->known_keys)));
+  }
+  auto fit_filters = [&](int stages, int* words_out) {
+    int used = 0, n = 0;
+    for (int j = 0; j < sh->n_joins; ++j) {
+      words_out[j] = 0;
+      if (!want[j]) continue;
+      if (k1_smem_bytes(n_cols, stages, p.smem_groups, used + want[j]) >
+          smem_budget(std::min(kCtasPerSm, 2)))
+        continue;
+      words_out[j] = want[j];
+      used += want[j];
+      ++n;
+    }
+    return n;
+  };
+  // (measured: shrinking the ring to 2 stages to fit more filters lost 6% at SF100 and gained
+  // nothing at SF10, so the ring keeps pick_stages' depth and filters take what is left)
+  int chosen[HX_MAX_JOINS];
+  p.stages = pick_stages(n_cols, p.smem_groups);
+  fit_filters(p.stages, chosen);
+  p.filter_words = 0;
+  for (int j = 0; j < sh->n_joins; ++j) {
+    p.joins[j].bloom_words = chosen[j];
+    p.filter_words += chosen[j];
+  }
+  if (std::getenv("HX_DEBUG")) {  // launch plan of this K1 (tuning aid)
+    std::fprintf(stderr, "[hx] K1 joins=%d cols=%d stages=%d groups=%d filters:", sh->n_joins,
+                 n_cols, p.stages, p.smem_groups);
+    for (int j = 0; j < sh->n_joins; ++j) std::fprintf(stderr, " %d", p.joins[j].bloom_words);
+    std::fprintf(stderr, " smem=%zu\n", k1_smem_bytes(n_cols, p.stages, p.smem_groups, p.filter_words));
   }
   k.fn = pick_kernel(sh->n_joins, grouped);
   k.smem = k1_smem_bytes(n_cols, p.stages, p.smem_groups, p.filter_words);
