@@ -231,6 +231,10 @@ int hx_plan_result(hx_plan* plan, int64_t* sums, int64_t* counts, int32_t* keys,
 /* K1 device time of the last execution (CUDA events around the launch) and its
    algorithmic bytes (rows x 4 B x distinct fact columns). Waits for the execution. */
 int hx_plan_k1_time(hx_plan* plan, float* ms, int64_t* bytes);
+/* Device time from the start of `first`'s K1 to the end of `last`'s K1 in their last
+   executions (meaningful when both ran in one hx_plans_enqueue / graph launch, `first` before
+   `last`): the span of the pipelines, including the gaps between them. Waits for `last`. */
+int hx_plan_k1_span(hx_plan* first, hx_plan* last, float* ms);
 int hx_plan_info(hx_plan* plan, int64_t* n_groups, int* n_gdims);
 int hx_plan_free(hx_plan* plan);
 typedef struct hx_graph hx_graph;

@@ -102,6 +102,7 @@ _SIGS = {
     "hx_plans_enqueue": ([_P, _PP, _I], _I),
     "hx_plan_result": ([_P, _PI64, _PI64, _PI32, _I64, _PI64], _I),
     "hx_plan_k1_time": ([_P, ctypes.POINTER(ctypes.c_float), _PI64], _I),
+    "hx_plan_k1_span": ([_P, _P, ctypes.POINTER(ctypes.c_float)], _I),
     "hx_plan_info": ([_P, _PI64, ctypes.POINTER(_I)], _I),
     "hx_plan_free": ([_P], _I),
     "hx_graph_begin": ([_P], _I),

@@ -102,6 +102,8 @@ int hx_init(int device, void* stream, hx_ctx** out) {
   }
   HX_CK(cudaEventCreateWithFlags(&ctx->fork_ev, cudaEventDisableTiming));
   HX_CK(cudaStreamCreateWithFlags(&ctx->copy_stream, cudaStreamNonBlocking));
+  HX_CK(cudaStreamCreateWithFlags(&ctx->fin_stream, cudaStreamNonBlocking));
+  HX_CK(cudaEventCreateWithFlags(&ctx->fin_join_ev, cudaEventDisableTiming));
   *out = ctx;
   return HX_OK;
 }
@@ -127,6 +129,11 @@ int hx_finalize(hx_ctx* ctx) {
     cudaStreamSynchronize(ctx->copy_stream);
     cudaStreamDestroy(ctx->copy_stream);
   }
+  if (ctx->fin_stream) {
+    cudaStreamSynchronize(ctx->fin_stream);
+    cudaStreamDestroy(ctx->fin_stream);
+  }
+  if (ctx->fin_join_ev) cudaEventDestroy(ctx->fin_join_ev);
   if (ctx->comm) ncclCommDestroy(ctx->comm);
   if (ctx->own_stream) cudaStreamDestroy(ctx->stream);
   delete ctx;

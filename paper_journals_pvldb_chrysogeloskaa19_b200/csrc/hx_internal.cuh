@@ -126,6 +126,10 @@ struct hx_ctx {
   cudaEvent_t fork_ev = nullptr;
   cudaEvent_t join_ev[kAux] = {nullptr, nullptr, nullptr, nullptr};
   cudaStream_t copy_stream = nullptr;  // mem-move H2D copies of host-resident blocks
+  // finalize + D2H of each plan run off the main stream so the next pipeline's K1 does not
+  // wait for them; joined back into the main stream at the end of every enqueue call
+  cudaStream_t fin_stream = nullptr;
+  cudaEvent_t fin_join_ev = nullptr;
 };
 
 struct hx_partition {
@@ -205,8 +209,11 @@ int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht*
              int n_hts, const hx_agg* agg, K1Prepared** out);
 struct StageRing;   // device staging ring for host-resident fact tables (hx_probe.cu)
 constexpr int64_t kHostBlockRows = int64_t(1) << 21;  // mem-move block: 8 MB per int32 column
+// k1_prepare (clears the group arrays, publishes the group-space shape) on stream s
+int k1_enqueue_prepare(hx_ctx* ctx, const K1Prepared* k, bool fresh, cudaStream_t s);
+// [prepare on the main stream if `prepare`] then K1 on the main stream
 int k1_enqueue(hx_ctx* ctx, const K1Prepared* k, bool fresh, cudaEvent_t e0, cudaEvent_t e1,
-               StageRing* ring = nullptr);
+               StageRing* ring = nullptr, bool prepare = true);
 bool k1_is_host(const K1Prepared* k);
 int ring_create(hx_ctx* ctx, const K1Prepared* k, int64_t block_rows, StageRing** out);
 void ring_destroy(hx_ctx* ctx, StageRing* r);

@@ -115,6 +115,7 @@ struct hx_plan {
   void* h_out = nullptr;       // pinned
   size_t out_bytes = 0, inline_bytes = 0;
   cudaEvent_t done = nullptr, k1_e0 = nullptr, k1_e1 = nullptr;
+  cudaEvent_t probed = nullptr;  // K1 (+ merge) complete: the finalize branch forks here
   cudaEvent_t built_ev[hx_ctx::kAux] = {nullptr, nullptr, nullptr, nullptr};
   StageRing* ring = nullptr;   // host-resident fact table: the mem-move staging ring
   bool enqueued = false;
@@ -130,6 +131,7 @@ struct hx_graph {
 
 static int plan_enqueue_builds(hx_ctx* ctx, hx_plan* pl);
 static int plan_enqueue_probe(hx_ctx* ctx, hx_plan* pl);
+static int join_fin(hx_ctx* ctx);
 
 static void plan_destroy(hx_plan* pl) {
   if (!pl) return;
@@ -141,7 +143,7 @@ static void plan_destroy(hx_plan* pl) {
   ring_destroy(pl->ctx, pl->ring);
   if (pl->d_out) cudaFreeAsync(pl->d_out, pl->ctx->stream);
   if (pl->h_out) cudaFreeHost(pl->h_out);
-  for (cudaEvent_t e : {pl->done, pl->k1_e0, pl->k1_e1})
+  for (cudaEvent_t e : {pl->done, pl->k1_e0, pl->k1_e1, pl->probed})
     if (e) cudaEventDestroy(e);
   for (cudaEvent_t e : pl->built_ev)
     if (e) cudaEventDestroy(e);
@@ -241,6 +243,10 @@ int hx_plan_create(hx_ctx* ctx, const hx_table* fact, hx_table* const* dims, int
     cudaError_t err = cudaEventCreateWithFlags(&e, cudaEventDisableTiming);
     if (err != cudaSuccess) return bail(cuda_fail(err, "cudaEventCreate", __FILE__, __LINE__));
   }
+  {
+    cudaError_t err = cudaEventCreateWithFlags(&pl->probed, cudaEventDisableTiming);
+    if (err != cudaSuccess) return bail(cuda_fail(err, "cudaEventCreate", __FILE__, __LINE__));
+  }
   *out = pl;
   return HX_OK;
 }
@@ -252,7 +258,9 @@ int hx_plan_enqueue(hx_ctx* ctx, hx_plan* pl) {
   for (int a = 0; a < hx_ctx::kAux; ++a) HX_CK(cudaStreamWaitEvent(ctx->aux[a], ctx->fork_ev, 0));
   int rc = plan_enqueue_builds(ctx, pl);
   if (rc != HX_OK) return rc;
-  return plan_enqueue_probe(ctx, pl);
+  rc = plan_enqueue_probe(ctx, pl);
+  if (rc != HX_OK) return rc;
+  return join_fin(ctx);
 }
 
 int hx_plans_enqueue(hx_ctx* ctx, hx_plan* const* plans, int n) {
@@ -272,30 +280,35 @@ int hx_plans_enqueue(hx_ctx* ctx, hx_plan* const* plans, int n) {
     int rc = plan_enqueue_probe(ctx, plans[i]);
     if (rc != HX_OK) return rc;
   }
-  return HX_OK;
+  return n > 0 ? join_fin(ctx) : HX_OK;
 }
 
 }  // extern "C"
 
 // builds of one plan on the auxiliary streams (which must already follow the main stream's
-// fork point); records the plan's per-stream completion events
+// fork point), then K1's prepare on aux[0] once all of them are done: built_ev[0] marks the
+// plan ready for its K1, and none of this sits on the main stream between two K1 launches
 static int plan_enqueue_builds(hx_ctx* ctx, hx_plan* pl) {
   const int nb = (int)pl->hts.size();
   for (int b = 0; b < nb; ++b) {
     int rc = ht_enqueue_build(ctx, pl->hts[b], ctx->aux[b % hx_ctx::kAux]);
     if (rc != HX_OK) return rc;
   }
-  for (int a = 0; a < std::min(nb, (int)hx_ctx::kAux); ++a)
+  for (int a = 1; a < std::min(nb, (int)hx_ctx::kAux); ++a) {
     HX_CK(cudaEventRecord(pl->built_ev[a], ctx->aux[a]));
+    HX_CK(cudaStreamWaitEvent(ctx->aux[0], pl->built_ev[a], 0));
+  }
+  int rc = k1_enqueue_prepare(ctx, pl->k1, true, ctx->aux[0]);
+  if (rc != HX_OK) return rc;
+  HX_CK(cudaEventRecord(pl->built_ev[0], ctx->aux[0]));
   return HX_OK;
 }
 
-// K1 (after the plan's builds) -> merge -> finalize -> D2H on the main stream
+// K1 (after the plan's builds) -> merge on the main stream; finalize -> D2H on the finalize
+// stream, so the next plan's K1 starts as soon as this one's merge is done
 static int plan_enqueue_probe(hx_ctx* ctx, hx_plan* pl) {
-  const int nb = (int)pl->hts.size();
-  for (int a = 0; a < std::min(nb, (int)hx_ctx::kAux); ++a)
-    HX_CK(cudaStreamWaitEvent(ctx->stream, pl->built_ev[a], 0));
-  int rc = k1_enqueue(ctx, pl->k1, true, pl->k1_e0, pl->k1_e1, pl->ring);
+  HX_CK(cudaStreamWaitEvent(ctx->stream, pl->built_ev[0], 0));
+  int rc = k1_enqueue(ctx, pl->k1, true, pl->k1_e0, pl->k1_e1, pl->ring, /*prepare=*/false);
   if (rc != HX_OK) return rc;
   if (ctx->comm && ctx->nranks > 1) {
     // union router: partial {sum,cnt} arrays are adjacent, one allreduce over NVLink
@@ -303,13 +316,24 @@ static int plan_enqueue_probe(hx_ctx* ctx, hx_plan* pl) {
                                    ncclUint64, ncclSum, ctx->comm, ctx->stream);
     HX_REQUIRE(r == ncclSuccess, HX_ENCCL, std::string("ncclAllReduce: ") + ncclGetErrorString(r));
   }
-  k1_finalize<<<1, 1024, 0, ctx->stream>>>(pl->fin);
+  HX_CK(cudaEventRecord(pl->probed, ctx->stream));
+  HX_CK(cudaStreamWaitEvent(ctx->fin_stream, pl->probed, 0));
+  k1_finalize<<<1, 1024, 0, ctx->fin_stream>>>(pl->fin);
   HX_CK_LAUNCH("k1_finalize");
   ctx->launches += 1;
-  HX_CK(cudaMemcpyAsync(pl->h_out, pl->d_out, pl->inline_bytes, cudaMemcpyDeviceToHost, ctx->stream));
+  HX_CK(cudaMemcpyAsync(pl->h_out, pl->d_out, pl->inline_bytes, cudaMemcpyDeviceToHost,
+                        ctx->fin_stream));
   ctx->d2h_bytes += (int64_t)pl->inline_bytes;
-  HX_CK(record_event(pl->done, ctx->stream));
+  HX_CK(record_event(pl->done, ctx->fin_stream));
   pl->enqueued = true;
+  return HX_OK;
+}
+
+// the main stream waits for every finalize enqueued so far (a later execution of the same
+// plan must not overwrite its group arrays before they are read; graph capture needs the join)
+static int join_fin(hx_ctx* ctx) {
+  HX_CK(cudaEventRecord(ctx->fin_join_ev, ctx->fin_stream));
+  HX_CK(cudaStreamWaitEvent(ctx->stream, ctx->fin_join_ev, 0));
   return HX_OK;
 }
 
@@ -356,6 +380,16 @@ int hx_plan_k1_time(hx_plan* pl, float* ms, int64_t* bytes) {
     if (pl->k1_e0 && k1_bytes(pl->k1) > 0) HX_CK(cudaEventElapsedTime(ms, pl->k1_e0, pl->k1_e1));
   }
   if (bytes) *bytes = k1_bytes(pl->k1);
+  return HX_OK;
+}
+
+int hx_plan_k1_span(hx_plan* first, hx_plan* last, float* ms) {
+  HX_REQUIRE(first && last && ms && first->enqueued && last->enqueued && first->ctx == last->ctx,
+             HX_EINVAL, "hx_plan_k1_span: bad argument");
+  HX_REQUIRE(k1_bytes(first->k1) > 0 && k1_bytes(last->k1) > 0, HX_EINVAL,
+             "hx_plan_k1_span: a plan without K1 launch");
+  HX_CK(cudaEventSynchronize(last->done));
+  HX_CK(cudaEventElapsedTime(ms, first->k1_e0, last->k1_e1));
   return HX_OK;
 }
 

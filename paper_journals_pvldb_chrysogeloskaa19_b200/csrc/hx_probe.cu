@@ -1062,14 +1062,23 @@ static int k1_enqueue_host(hx_ctx* ctx, const K1Prepared* k, StageRing* ring, cu
 }
 
 // prepare (group layout + zeroing when `fresh`) then K1; optional timing events around K1.
-int k1_enqueue(hx_ctx* ctx, const K1Prepared* k, bool fresh, cudaEvent_t e0, cudaEvent_t e1,
-               StageRing* ring) {
+int k1_enqueue_prepare(hx_ctx* ctx, const K1Prepared* k, bool fresh, cudaStream_t s) {
   const K1Params& p = k->p;
-  k1_prepare<<<k->prep_grid, 256, 0, ctx->stream>>>(const_cast<AggMeta*>(p.meta), k->gh[0], k->gh[1], k->gh[2],
-                                                    k->n_gdims, k->gj, p.g_sum, p.g_cnt,
-                                                    k->cap_groups, fresh ? 1 : 0);
+  k1_prepare<<<k->prep_grid, 256, 0, s>>>(const_cast<AggMeta*>(p.meta), k->gh[0], k->gh[1],
+                                          k->gh[2], k->n_gdims, k->gj, p.g_sum, p.g_cnt,
+                                          k->cap_groups, fresh ? 1 : 0);
   HX_CK_LAUNCH("k1_prepare");
   ctx->launches += 1;
+  return HX_OK;
+}
+
+int k1_enqueue(hx_ctx* ctx, const K1Prepared* k, bool fresh, cudaEvent_t e0, cudaEvent_t e1,
+               StageRing* ring, bool prepare) {
+  const K1Params& p = k->p;
+  if (prepare) {
+    int rc = k1_enqueue_prepare(ctx, k, fresh, ctx->stream);
+    if (rc != HX_OK) return rc;
+  }
   if (k->rows == 0) return HX_OK;
   if (k->host) return k1_enqueue_host(ctx, k, ring, e0, e1);
   if (e0) HX_CK(record_event(e0, ctx->stream));

@@ -305,6 +305,12 @@ class Plan:
         call("hx_plan_k1_time", self.h, ctypes.byref(ms), ctypes.byref(b))
         return ms.value, b.value
 
+    def k1_span(self, last: "Plan") -> float:
+        """ms from this plan's K1 start to `last`'s K1 end (same enqueue)."""
+        ms = ctypes.c_float()
+        call("hx_plan_k1_span", self.h, last.h, ctypes.byref(ms))
+        return ms.value
+
     def close(self):
         if getattr(self, "h", None):
             call("hx_plan_free", self.h)
