@@ -51,6 +51,8 @@ def parse():
     ap.add_argument("--no-e2e", action="store_true")
     ap.add_argument("--queries", default="all")
     ap.add_argument("--no-graph", action="store_true", help="enqueue plans without a CUDA graph")
+    ap.add_argument("--no-pipeline", action="store_true",
+                    help="one plan set: the host reads a step's results before the next starts")
     ap.add_argument("--variant", default="hbm", choices=["hbm", "host"],
                     help="host: lineorder in pinned host memory streamed over PCIe (config 5)")
     return ap.parse_args()
@@ -261,30 +263,52 @@ def main():
     eng = ssb.SsbEngine(ctx, dims, fact)
     # one prepared plan per query (HT + group buffers allocated once, builds sized once);
     # the 13 executions are captured into ONE CUDA graph: a step is one graph launch plus
-    # the 13 host reads of the finalized results
-    plans = {q: eng.plan(q) for q in queries}
-    order = [plans[q].hp for q in queries]
-    graph = None if args.no_graph else hx.capture(ctx, lambda: hx.plans_enqueue(ctx, order))
+    # the 13 host reads of the finalized results. Two such plan sets alternate (steps i and
+    # i+1 use different buffers), so the host reads step i's results while the device
+    # already runs step i+1 — every step still builds, probes, merges and reads everything.
+    n_sets = 1 if (args.no_graph or args.no_pipeline) else 2
+    sets = []
+    for _ in range(n_sets):
+        pl_ = {q: eng.plan(q) for q in queries}
+        od_ = [pl_[q].hp for q in queries]
+        gr_ = None if args.no_graph else hx.capture(ctx, lambda od_=od_: hx.plans_enqueue(ctx, od_))
+        sets.append((pl_, od_, gr_))
+    plans, order, graph = sets[0]
     k1_acc = [0.0, 0, 0, 0.0]
 
-    def step(timed=False):
-        if graph is not None:
-            graph.launch()
+    def launch(st):
+        if st[2] is not None:
+            st[2].launch()
         else:
-            hx.plans_enqueue(ctx, order)
-        out = [plans[q].rows() for q in queries]
+            hx.plans_enqueue(ctx, st[1])
+
+    def collect(st, timed):
+        out = [st[0][q].rows() for q in queries]
         if timed:
-            k1_acc[3] += order[0].k1_span(order[-1])
+            k1_acc[3] += st[1][0].k1_span(st[1][-1])
             for q in queries:
-                ms_, b_ = plans[q].hp.k1_time()
+                ms_, b_ = st[0][q].hp.k1_time()
                 k1_acc[0] += ms_
                 k1_acc[1] += 1
                 k1_acc[2] += b_
         return out
 
+    def run_steps(n, timed=False):
+        prev = None
+        for i in range(n):
+            cur = sets[i % n_sets]
+            launch(cur)
+            if n_sets == 1:
+                collect(cur, timed)
+                continue
+            if prev is not None:
+                collect(prev, timed)
+            prev = cur
+        if prev is not None:
+            collect(prev, timed)
+
     # ---- warm-up, then exactly K timed steps ---------------------------------------------
-    for _ in range(args.warmup):
-        step()
+    run_steps(args.warmup)
     ctx.stats(reset=True)
     clocks = Clocks(local)
     if world > 1:
@@ -293,8 +317,7 @@ def main():
     clocks.start()
     e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
     e0.record(stream)
-    for _ in range(args.steps):
-        step(timed=True)
+    run_steps(args.steps, timed=True)
     e1.record(stream)
     torch.cuda.synchronize()
     if world > 1:
@@ -430,17 +453,20 @@ def main():
                 "dtype": "int32 columns, int64 accumulate",
                 "data": f"synthetic (ssbgen dbgen-shaped SSB distributions, seed {SEED}), "
                         "generated in HBM",
-                "config": config(args, world, n_mine, queries),
+                "config": dict(config(args, world, n_mine, queries), plan_sets=n_sets,
+                               step_overlap="host reads step i's results while the device runs "
+                                            "step i+1" if n_sets == 2 else "none"),
                 "hbm_gbps_per_gpu": sum(n_mine * B[q] for q in queries) / (ms_step / 1e3) / 1e9,
                 "roofline": roofline, "cpu_baseline": cpu, "e2e": e2e, "clocks": clk,
                 "gpu_launches": launches, "per_query": per_query,
                 "k1_ctas_per_sm": ctas, "n_sms": n_sms}
         print(json.dumps(line), flush=True)
     # release library objects before their context
-    if graph is not None:
-        graph.close()
-    for pl in plans.values():
-        pl.close()
+    for pl_, _, gr_ in sets:
+        if gr_ is not None:
+            gr_.close()
+        for pl in pl_.values():
+            pl.close()
     for t in list(dims.values()) + [fact]:
         t.close()
     ctx.close()

@@ -37,6 +37,14 @@ struct BuildParams {
   unsigned long long* slots;
   uint32_t* bloom;
   int32_t group_lo, domain, max_log2cap, max_bloom_log2w;
+  // direct map (nullptr: hash table)
+  uint32_t* dm;
+  int64_t dm_words;
+  uint32_t* dm_bm;  // membership bitmap over the same keys (nullptr when the map is 1-bit)
+  int64_t bm_words;
+  int32_t dm_kmin;
+  uint32_t dm_span;
+  int32_t dm_lw;
 };
 
 __device__ __forceinline__ bool row_pass(const BuildParams& p, int64_t i) {
@@ -47,14 +55,18 @@ __device__ __forceinline__ bool row_pass(const BuildParams& p, int64_t i) {
   return ok;
 }
 
-// Count passing rows; flag the group codes present among them.
+// Count passing rows and their key range; flag the group codes present among them.
 __global__ void k2_filter_mark(BuildParams p) {
   int local = 0;
+  uint32_t emin = 0xFFFFFFFFu, emax = 0u;
   const int64_t stride = (int64_t)gridDim.x * blockDim.x;
   for (int64_t i = (int64_t)blockIdx.x * blockDim.x + threadIdx.x; i < p.n_rows; i += stride) {
     if (!row_pass(p, i)) continue;
     ++local;
-    if (__ldg(p.key + i) == kEmptyKey) atomicExch(&p.hdr->error, HX_EINVAL);  // reserved key
+    const int32_t key = __ldg(p.key + i);
+    if (key == kEmptyKey) atomicExch(&p.hdr->error, HX_EINVAL);  // reserved key
+    emin = min(emin, key_enc(key));
+    emax = max(emax, key_enc(key));
     if (p.group) {
       int32_t code = __ldg(p.group + i) - p.group_lo;
       if (code < 0 || code >= p.domain)
@@ -65,7 +77,13 @@ __global__ void k2_filter_mark(BuildParams p) {
   }
 #pragma unroll
   for (int o = 16; o > 0; o >>= 1) local += __shfl_xor_sync(kFull, local, o);
-  if ((threadIdx.x & 31) == 0 && local) atomicAdd(&p.hdr->n_keys, local);
+  emin = __reduce_min_sync(kFull, emin);
+  emax = __reduce_max_sync(kFull, emax);
+  if ((threadIdx.x & 31) == 0 && local) {
+    atomicAdd(&p.hdr->n_keys, local);
+    atomicMax(&p.hdr->kmin_inv, ~emin);
+    atomicMax(&p.hdr->kmax_enc, emax);
+  }
 }
 
 // One CTA: dense ranks of the present group codes (exclusive scan of the flags), rank->code
@@ -192,6 +210,46 @@ __global__ void k2_insert(BuildParams p) {
   }
 }
 
+// Empty the Bloom words in use (direct-map builds have no slots to clear).
+__global__ void k2_clear_bloom(BuildParams p) {
+  const int64_t words = 1ll << p.hdr->bloom_log2w;
+  for (int64_t i = (int64_t)blockIdx.x * blockDim.x + threadIdx.x; i < words;
+       i += (int64_t)gridDim.x * blockDim.x)
+    p.bloom[i] = 0u;
+}
+
+// Direct-map build: entry (key - kmin) |= rank + 1 for every passing row, plus the key's
+// bit in the membership bitmap and the Bloom filter (K1 stages whichever of the three fits
+// its shared memory). A key outside the map (the dimension changed since the plan sized it)
+// or a rank too wide for the entry sets HX_ECAPACITY; a key already present sets
+// HX_EDUPKEY (the entries are non-zero).
+__global__ void k2_dm_insert(BuildParams p) {
+  const uint32_t vmask = dm_vmask(p.dm_lw);
+  const int blw = p.hdr->bloom_log2w;
+  const int64_t stride = (int64_t)gridDim.x * blockDim.x;
+  for (int64_t i = (int64_t)blockIdx.x * blockDim.x + threadIdx.x; i < p.n_rows; i += stride) {
+    if (!row_pass(p, i)) continue;
+    const int32_t key = __ldg(p.key + i);
+    uint32_t rank = 0;
+    if (p.group) {
+      const int32_t code = __ldg(p.group + i) - p.group_lo;
+      if (code < 0 || code >= p.domain) continue;  // flagged by the filter kernel
+      rank = (uint32_t)p.c2r[code];
+    }
+    const uint32_t u = (uint32_t)key - (uint32_t)p.dm_kmin;
+    if (u >= p.dm_span || rank + 1u > vmask) {
+      atomicExch(&p.hdr->error, HX_ECAPACITY);
+      continue;
+    }
+    const uint64_t bit = (uint64_t)u << p.dm_lw;
+    const uint32_t sh = (uint32_t)bit & 31u;
+    const uint32_t old = atomicOr(p.dm + (bit >> 5), (rank + 1u) << sh);
+    if ((old >> sh) & vmask) atomicExch(&p.hdr->error, HX_EDUPKEY);
+    if (p.dm_bm) atomicOr(p.dm_bm + (u >> 5), 1u << (u & 31u));
+    atomicOr(p.bloom + bloom_word(key, blw), bloom_mask(key));
+  }
+}
+
 int ceil_log2(int64_t x) {
   int l = 0;
   while ((1ll << l) < x) ++l;
@@ -279,6 +337,17 @@ int ht_enqueue_build(hx_ctx* ctx, hx_ht* ht, cudaStream_t stream) {
   HX_CK_LAUNCH("k2_filter_mark");
   k2_rank<<<1, 1024, 0, s>>>(p);
   HX_CK_LAUNCH("k2_rank");
+  if (p.dm) {  // direct map (+ bitmap, Bloom filter) instead of slots
+    HX_CK(cudaMemsetAsync(p.dm, 0, (size_t)(p.dm_words + p.bm_words) * sizeof(uint32_t), s));
+    const int bgrid = (int)std::min<int64_t>(((int64_t(1) << p.max_bloom_log2w) + 255) / 256,
+                                             (int64_t)ctx->n_sms * 4);
+    k2_clear_bloom<<<bgrid, 256, 0, s>>>(p);
+    HX_CK_LAUNCH("k2_clear_bloom");
+    k2_dm_insert<<<grid, 256, 0, s>>>(p);
+    HX_CK_LAUNCH("k2_dm_insert");
+    ctx->launches += 4;
+    return HX_OK;
+  }
   const int64_t slots_max = int64_t(1) << p.max_log2cap;
   const int cgrid = (int)std::min<int64_t>((slots_max + 255) / 256, (int64_t)ctx->n_sms * 16);
   k2_clear<<<cgrid, 256, 0, s>>>(p);
@@ -289,7 +358,33 @@ int ht_enqueue_build(hx_ctx* ctx, hx_ht* ht, cudaStream_t stream) {
   return HX_OK;
 }
 
+int ht_enable_direct(hx_ctx* ctx, hx_ht* ht, int32_t kmin, uint32_t span, int lw) {
+  HX_REQUIRE(lw >= 0 && lw <= 5 && ((uint64_t)span << lw) < (uint64_t(1) << 32), HX_EINVAL,
+             "direct map: bad width or span");
+  BuildParams& p = *static_cast<BuildParams*>(ht->build);
+  const int64_t words = dm_words_for(span, lw);
+  const int64_t bm_words = lw > 0 ? dm_words_for(span, 0) : 0;
+  if (ht->dm) cudaFreeAsync(ht->dm, ctx->stream);
+  ht->dm = nullptr;
+  HX_CK(cudaMallocAsync(&ht->dm, (size_t)(words + bm_words) * sizeof(uint32_t), ctx->stream));
+  ht->dm_words = words;
+  ht->dm_bm = lw > 0 ? ht->dm + words : ht->dm;
+  ht->bm_words = lw > 0 ? bm_words : words;
+  p.dm_bm = lw > 0 ? ht->dm + words : nullptr;
+  p.bm_words = bm_words;
+  ht->dm_kmin = kmin;
+  ht->dm_span = span;
+  ht->dm_lw = lw;
+  p.dm = ht->dm;
+  p.dm_words = words;
+  p.dm_kmin = kmin;
+  p.dm_span = span;
+  p.dm_lw = lw;
+  return HX_OK;
+}
+
 void ht_destroy(hx_ht* ht) {
+  if (ht->dm) cudaFreeAsync(ht->dm, ht->ctx->stream);
   if (ht->base) cudaFreeAsync(ht->base, ht->ctx->stream);
   delete static_cast<BuildParams*>(ht->build);
   delete ht;

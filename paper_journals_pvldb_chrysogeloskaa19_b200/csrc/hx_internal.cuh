@@ -41,7 +41,24 @@ struct HtHeader {
   int32_t group_lo;
   int32_t domain;
   int32_t bloom_log2w;  // log2 of the Bloom filter's 32-bit words in use (device-written)
+  // range of the passing keys, order-preserving encoded (key ^ 0x80000000): the filter kernel
+  // keeps ~min and max with atomicMax so that a zeroed header is the neutral element
+  uint32_t kmin_inv;
+  uint32_t kmax_enc;
 };
+__host__ __device__ __forceinline__ uint32_t key_enc(int32_t k) { return (uint32_t)k ^ 0x80000000u; }
+__host__ __device__ __forceinline__ int32_t key_dec(uint32_t e) { return (int32_t)(e ^ 0x80000000u); }
+
+// Direct map of a dense-key dimension (R20): entry (key - kmin), 2^lw bits wide,
+// holds rank + 1 of the passing row with that key (0: no passing row). With surrogate keys
+// 1..N (SSB) this is the hash table with the identity hash: one load, no probe chain, exact.
+__host__ __device__ __forceinline__ uint32_t dm_vmask(int lw) {
+  return lw >= 5 ? 0xFFFFFFFFu : ((1u << (1u << lw)) - 1u);
+}
+__host__ __device__ __forceinline__ int64_t dm_words_for(int64_t span, int lw) {
+  const int64_t w = ((((span << lw) + 31) >> 5) + 3) & ~int64_t(3);  // whole 16-byte units
+  return w < 4 ? 4 : w;
+}
 
 // Blocked Bloom filter over the passing keys (one 32-bit word per key, two bits set), built
 // with the table. K1 stages it in shared memory to drop most non-matching rows before any
@@ -166,6 +183,14 @@ struct hx_ht {
   uint32_t* bloom = nullptr;       // Bloom filter words (after the slots)
   int32_t max_bloom_log2w = 0;
   int64_t known_keys = -1;         // passing keys, when a plan has observed them (else -1)
+  // direct map (plans over dense keys; nullptr: hash-table build and probe)
+  uint32_t* dm = nullptr;
+  int64_t dm_words = 0;
+  uint32_t* dm_bm = nullptr;       // membership bitmap (== dm for a 1-bit map)
+  int64_t bm_words = 0;
+  int32_t dm_kmin = 0;
+  uint32_t dm_span = 0;
+  int32_t dm_lw = 0;
 };
 
 struct hx_agg {
@@ -198,6 +223,8 @@ int ht_create(hx_ctx* ctx, const hx_table* dim, int32_t key_col, const hx_pred* 
               int n_preds, int32_t group_col, int32_t group_lo, int32_t group_hi, hx_ht** out);
 int ht_enqueue_build(hx_ctx* ctx, hx_ht* ht, cudaStream_t stream = nullptr);
 void ht_destroy(hx_ht* ht);
+// switch a table's builds to a direct map over keys [kmin, kmin + span) with 2^lw-bit entries
+int ht_enable_direct(hx_ctx* ctx, hx_ht* ht, int32_t kmin, uint32_t span, int lw);
 int probe_agg(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* shape,
               hx_ht* const* hts, int n_hts, hx_agg* agg, bool fresh);
 int k1_occupancy(hx_ctx* ctx);

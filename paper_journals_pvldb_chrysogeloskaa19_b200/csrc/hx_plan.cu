@@ -12,6 +12,7 @@
 #include <cub/block/block_scan.cuh>
 
 #include <algorithm>
+#include <cstdlib>
 #include <cstring>
 
 #include "hx_internal.cuh"
@@ -20,6 +21,7 @@ namespace hx {
 namespace {
 
 constexpr int kOutInline = 4096;  // result rows copied to the host by every execution
+constexpr int64_t kDirectMaxBytes = int64_t(16) << 20;  // direct maps up to 16 MB (L2: 126 MB)
 
 struct OutHeader {
   long long n_rows;
@@ -197,6 +199,37 @@ int hx_plan_create(hx_ctx* ctx, const hx_table* fact, hx_table* const* dims, int
     if (hh[b].error == HX_EDUPKEY) return bail(fail(HX_EDUPKEY, "dimension build: duplicate primary key"));
     if (hh[b].error) return bail(fail(HX_EINVAL, "dimension build: bad key or group code"));
     pl->hts[b]->known_keys = hh[b].n_keys;  // lets K1 reserve shared memory for its filter
+  }
+  // dense keys (R20): the plan's builds produce direct maps over the passing-key
+  // range instead of hash tables when the map is no larger than kDirectMaxBytes (or than
+  // twice the hash table); HX_NO_DM=1 keeps hash tables (A/B measurements, tests)
+  // (all builds or none: one K1 instance probes either kind)
+  bool use_dm = std::getenv("HX_NO_DM") == nullptr;
+  int32_t dm_kmin[HX_MAX_JOINS] = {0, 0, 0, 0};
+  int64_t dm_span[HX_MAX_JOINS] = {0, 0, 0, 0};
+  int dm_lw[HX_MAX_JOINS] = {0, 0, 0, 0};
+  for (int b = 0; b < n_builds && use_dm; ++b) {
+    hx_ht* ht = pl->hts[b];
+    const HtHeader& h = hh[b];
+    int64_t kmin = 0, span = 0;
+    if (h.n_keys > 0) {
+      kmin = key_dec(~h.kmin_inv);
+      span = (int64_t)key_dec(h.kmax_enc) - kmin + 1;
+    }
+    const int64_t values = ht->has_group ? std::max(1, h.n_ranks) : 1;
+    int lw = 0;
+    while (lw < 5 && (int64_t)dm_vmask(lw) < values) ++lw;
+    const int64_t dm_bytes = dm_words_for(span, lw) * 4;
+    const int64_t ht_bytes = (int64_t(1) << h.log2cap) * 8;
+    if (span >= (int64_t(1) << 27) || dm_bytes > std::max<int64_t>(kDirectMaxBytes, 2 * ht_bytes))
+      use_dm = false;
+    dm_kmin[b] = (int32_t)kmin;
+    dm_span[b] = span;
+    dm_lw[b] = lw;
+  }
+  for (int b = 0; b < n_builds && use_dm; ++b) {
+    int rc = ht_enable_direct(ctx, pl->hts[b], dm_kmin[b], (uint32_t)dm_span[b], dm_lw[b]);
+    if (rc != HX_OK) return bail(rc);
   }
   long long ng = 1;
   for (int g = 0; g < shape->n_gdims; ++g) ng *= std::max(1, hh[shape->join_ht[shape->gdim_join[g]]].n_ranks);

@@ -64,6 +64,18 @@ struct JoinDev {
   const HtHeader* hdr;
   const uint32_t* bloom;                   // the table's Bloom filter (global)
   int32_t bloom_words;                     // shared-memory words reserved for it (0: none)
+  // direct map (dense keys; hx_internal.cuh): nullptr -> hash-table join
+  const uint32_t* dm;
+  int32_t dm_kmin;
+  uint32_t dm_span;
+  int32_t dm_lw;
+  uint32_t dm_vmask;
+  int32_t dm_words;
+  int32_t dm_smem;                         // byte offset of its copy in the DM smem region (-1: L2)
+  const uint32_t* bm;                      // its membership bitmap (1 bit per key of the range)
+  int32_t bm_words;
+  int32_t bm_smem;                         // byte offset of a staged bitmap (-1: none)
+  int32_t in_s;                            // 1: its shared-memory structure runs in stage S
 };
 
 struct K1Params {
@@ -83,7 +95,38 @@ struct K1Params {
   unsigned long long* g_cnt;
   int32_t smem_groups;                     // 0 for ungrouped instances
   int32_t filter_words;                    // sum of joins[].bloom_words
+  int32_t dm_bytes;                        // shared memory of the staged direct maps
+  // per-join bit masks (bit j = join j) of the shared-memory plan, tested with one
+  // instruction against the constant bank instead of re-reading the join descriptors
+  uint32_t m_dm;                           // direct-map join
+  uint32_t m_dmsm;                         // its full map is staged in shared memory
+  uint32_t m_bm;                           // its bitmap is staged in shared memory
+  uint32_t m_ins;                          // its shared-memory structure runs in stage S
 };
+
+// join kinds (uniform per launch: read from the kernel parameters)
+// (DM: the kernel instance whose joins are all direct maps; hash-table instances have none)
+__device__ __forceinline__ bool jbit(uint32_t m, int jx) { return (m >> jx) & 1u; }
+template <bool DM>
+__device__ __forceinline__ bool dm_smem(const K1Params& p, int jx) { return DM && jbit(p.m_dmsm, jx); }
+template <bool DM>
+__device__ __forceinline__ bool resolved_in_s(const K1Params& p, int jx) {
+  return DM && jbit(p.m_dmsm & p.m_ins, jx);
+}
+template <bool DM>
+__device__ __forceinline__ bool dm_l2(const K1Params& p, int jx) {
+  return DM && !jbit(p.m_dmsm, jx);
+}
+// Direct-map entry (rank + 1, or 0) of a key from the map's 32-bit word array
+__device__ __forceinline__ uint32_t dm_bit(const JoinDev& d, int32_t key) {
+  return ((uint32_t)key - (uint32_t)d.dm_kmin) << d.dm_lw;
+}
+__device__ __forceinline__ bool dm_in(const JoinDev& d, int32_t key) {
+  return (uint32_t)key - (uint32_t)d.dm_kmin < d.dm_span;
+}
+__device__ __forceinline__ uint32_t dm_entry(const JoinDev& d, uint32_t word, uint32_t bit) {
+  return __funnelshift_r(word, word, bit) & d.dm_vmask;  // shf.r.wrap: bit mod 32
+}
 
 // ---- PTX helpers: mbarrier, bulk copy, cache policies -------------------------------------
 __device__ __forceinline__ uint32_t smem_u32(const void* p) {
@@ -218,6 +261,38 @@ __device__ __forceinline__ void accumulate(const K1Params& p, bool smem_table,
   }
 }
 
+// Hash-table join whose Bloom filter runs on every row (the first filtered one in probe
+// order), or -1. (Direct-map joins apply their shared-memory filters in stage S.)
+template <int NJ, bool DM>
+__device__ __forceinline__ int first_filter(const JoinState (&js)[HX_MAX_JOINS]) {
+  int jf = -1;
+#pragma unroll
+  for (int jx = NJ - 1; jx >= 0; --jx)
+    if (!DM && js[jx].sbloom) jf = jx;
+  return jf;
+}
+template <int NJ, bool DM>
+__device__ __forceinline__ bool all_resolved_in_s(const K1Params& p) {
+  return DM && (p.m_dmsm & p.m_ins & ((1u << NJ) - 1u)) == ((1u << NJ) - 1u);
+}
+// 1 when stage B probes the first join in place (hash-table joins, no lineorder predicate,
+// no filter on the first join).
+template <int NJ, bool DM>
+__device__ __forceinline__ int first_join_in_place(const K1Params& p,
+                                                   const JoinState (&js)[HX_MAX_JOINS]) {
+  return (!DM && NJ > 0 && p.n_preds == 0 && !js[0].sbloom) ? 1 : 0;
+}
+// Group-index origin: a direct map yields rank + 1, so each join contributes one extra
+// stride, subtracted once up front.
+template <int NJ, bool GROUPED, bool DM>
+__device__ __forceinline__ int32_t group_origin(const JoinState (&js)[HX_MAX_JOINS]) {
+  int32_t g = 0;
+#pragma unroll
+  for (int jx = 0; jx < NJ; ++jx)
+    if (GROUPED && DM) g -= js[jx].jstride;
+  return g;
+}
+
 // A queued row for stage C, by value: the FK of every join, the measure operands, and the
 // group-index part known so far (or ~next_bucket of a deferred first-join probe).
 struct CarryEntry {
@@ -231,12 +306,13 @@ struct CarryBuf {
 };
 
 // Entry idx of the combined sequence [carried rows..., this tile's queue...].
-template <int NJ>
+template <int NJ, bool DM>
 __device__ __forceinline__ CarryEntry load_entry(const K1Params& p,
                                                  const JoinState (&js)[HX_MAX_JOINS],
                                                  const CarryBuf* cb, int n_carry,
-                                                 const uint8_t* q_row, const int32_t* q_g, int j0,
-                                                 const int32_t* wcol, int stride, int idx) {
+                                                 const uint8_t* q_row, const int32_t* q_g,
+                                                 bool carry_g, const int32_t* wcol, int stride,
+                                                 int idx) {
   CarryEntry e;
   if (idx < n_carry) {
 #pragma unroll
@@ -248,28 +324,66 @@ __device__ __forceinline__ CarryEntry load_entry(const K1Params& p,
     const int i = idx - n_carry;
     const int r = q_row[i];
 #pragma unroll
-    for (int jx = 0; jx < NJ; ++jx) e.key[jx] = wcol[js[jx].c * stride + r];
+    for (int jx = 0; jx < NJ; ++jx)
+      e.key[jx] = wcol[js[jx].c * stride + r];
     e.a = wcol[p.agg_a * stride + r];
     e.b = wcol[p.agg_b * stride + r];
-    e.g = j0 ? q_g[i] : 0;
+    e.g = carry_g ? q_g[i] : 0;
   }
   return e;
 }
 
 // Stage C for one row: the remaining shared-memory filters, then the probes of every join
 // not yet resolved issued together (one L2 round trip), then measure + group atomic.
-template <int NJ, bool GROUPED>
+template <int NJ, bool GROUPED, bool DM>
 __device__ __forceinline__ void stage_c_row(const K1Params& p, const JoinState (&js)[HX_MAX_JOINS],
-                                            const CarryEntry& e, int j0, int jf, bool smem_table,
+                                            const unsigned char* sdm, const CarryEntry& e,
+                                            int j0, int jf, bool smem_table,
                                             unsigned long long* s_sum, uint32_t* s_cnt,
                                             long long& acc_sum, long long& acc_cnt) {
-  int32_t gg = e.g;
+  // (direct maps: the group index is computed here from scratch; stage S only filtered)
+  int32_t gg = DM ? group_origin<NJ, GROUPED, DM>(js) : e.g;
   bool alive = true;
   uint32_t b[NJ > 0 ? NJ : 1];
+  uint32_t wdm[NJ > 0 ? NJ : 1];
   uint32_t pend = 0;
+  // direct-map joins not resolved in stage S: their shared-memory structures first (a full
+  // map resolves the join, a bitmap or Bloom filter only drops rows) ...
 #pragma unroll
   for (int jx = 0; jx < NJ; ++jx) {
-    if (jx < j0) {  // resume a deferred probe of the first join
+    const JoinDev& d = p.joins[jx];
+    if (!DM) continue;
+    // the stage-S join: its filter already ran; a full map is read again for the rank
+    if (jbit(p.m_ins, jx) && !(GROUPED && dm_smem<DM>(p, jx))) continue;
+    const int32_t key = e.key[jx];
+    if (dm_smem<DM>(p, jx)) {
+      const uint32_t bit = dm_bit(d, key);
+      const uint32_t* w = reinterpret_cast<const uint32_t*>(sdm + d.dm_smem);
+      const uint32_t v = dm_entry(d, dm_in(d, key) ? w[bit >> 5] : 0u, bit);
+      alive = alive && v != 0u;
+      if (GROUPED) gg += (int32_t)v * js[jx].jstride;
+    } else if (jbit(p.m_bm, jx)) {
+      const uint32_t u = (uint32_t)key - (uint32_t)d.dm_kmin;
+      const uint32_t* w = reinterpret_cast<const uint32_t*>(sdm + d.bm_smem);
+      alive = alive && u < d.dm_span && ((w[u >> 5] >> (u & 31u)) & 1u);
+    } else if (js[jx].sbloom) {
+      alive = alive && bloom_pass(js[jx], key);
+    }
+  }
+  // ... then the maps read from L2 (one 32-bit load each, only for rows still alive), issued
+  // together with the hash probes below
+#pragma unroll
+  for (int jx = 0; jx < NJ; ++jx) {
+    const JoinDev& d = p.joins[jx];
+    wdm[jx] = 0u;
+    if (dm_l2<DM>(p, jx) && alive && dm_in(d, e.key[jx]))
+      wdm[jx] = __ldg(d.dm + (dm_bit(d, e.key[jx]) >> 5));
+  }
+#pragma unroll
+  for (int jx = 0; jx < NJ; ++jx) {
+    if (DM) {  // direct map: resolved above or in stage S
+      b[jx] = 0u;
+    } else if (jx < j0) {  // resume a deferred probe of the first join
       const bool deferred = gg < 0;
       b[jx] = deferred ? ~(uint32_t)gg : 0u;
       pend |= (uint32_t)deferred << jx;
@@ -279,8 +393,16 @@ __device__ __forceinline__ void stage_c_row(const K1Params& p, const JoinState (
       if (jx != jf && js[jx].sbloom) alive = alive && bloom_pass(js[jx], e.key[jx]);
     }
   }
+  if (j0 && gg < 0) gg = 0;  // deferred-probe encoding (stage B runs only without direct maps)
+#pragma unroll
+  for (int jx = 0; jx < NJ; ++jx) {
+    const JoinDev& d = p.joins[jx];
+    if (!dm_l2<DM>(p, jx)) continue;
+    const uint32_t v = dm_entry(d, wdm[jx], dm_bit(d, e.key[jx]));
+    alive = alive && v != 0u;
+    if (GROUPED) gg += (int32_t)v * js[jx].jstride;
+  }
   if (!alive) pend = 0;
-  if (gg < 0) gg = 0;
   while (pend) {
     ulonglong2 v[NJ > 0 ? NJ : 1];
 #pragma unroll
@@ -304,22 +426,6 @@ __device__ __forceinline__ void stage_c_row(const K1Params& p, const JoinState (
                         acc_cnt);
 }
 
-// Join whose filter runs on every row (first filtered join in probe order), or -1.
-template <int NJ>
-__device__ __forceinline__ int first_filter(const JoinState (&js)[HX_MAX_JOINS]) {
-  int jf = -1;
-#pragma unroll
-  for (int jx = NJ - 1; jx >= 0; --jx)
-    if (js[jx].sbloom) jf = jx;
-  return jf;
-}
-// 1 when stage B probes the first join in place (no lineorder predicate, no filter on it).
-template <int NJ>
-__device__ __forceinline__ int first_join_in_place(const K1Params& p,
-                                                   const JoinState (&js)[HX_MAX_JOINS]) {
-  return (NJ > 0 && p.n_preds == 0 && !js[0].sbloom) ? 1 : 0;
-}
-
 // Process one staged tile. Warp w owns rows [w*128, w*128+128) of the tile; lane l holds the
 // 4 consecutive rows w*128 + 4l .. +3, read with one 128-bit shared-memory load per column
 // (512 contiguous bytes per warp: conflict-free). Column c, row r of the tile is at
@@ -333,10 +439,11 @@ __device__ __forceinline__ int first_join_in_place(const K1Params& p,
 //   stage C  one queued row per lane: the probes of ALL remaining joins are issued together
 //            (independent keys, so one L2 round trip instead of one per join), then the
 //            measure and the group-table atomic.
-template <int NJ, bool GROUPED>
+template <int NJ, bool GROUPED, bool DM>
 __device__ __forceinline__ void process_tile(const K1Params& p, const JoinState (&js)[HX_MAX_JOINS],
-                                             const int32_t* sbase, int stride, int rows_valid,
-                                             int warp, int lane, bool smem_table,
+                                             const unsigned char* sdm, const int32_t* sbase,
+                                             int stride, int rows_valid, int warp, int lane,
+                                             bool smem_table,
                                              unsigned long long* s_sum, uint32_t* s_cnt,
                                              uint8_t* q_row, int32_t* q_g, CarryBuf* cb,
                                              int& n_carry, long long& acc_sum,
@@ -374,7 +481,7 @@ __device__ __forceinline__ void process_tile(const K1Params& p, const JoinState 
   // join (the most selective: joins are in ascending pass fraction) on every row; the other
   // joins' filters are applied to the few survivors in stage C. No false negatives; the
   // ~5% false positives are removed by the exact probe.
-  const int jf = first_filter<NJ>(js);
+  const int jf = first_filter<NJ, DM>(js);
 #pragma unroll
   for (int jx = 0; jx < NJ; ++jx) {
     if (jx != jf) continue;
@@ -384,10 +491,43 @@ __device__ __forceinline__ void process_tile(const K1Params& p, const JoinState 
     for (int k = 0; k < kRowsPerThread; ++k) m &= ~((uint32_t)!bloom_pass(js[jx], key[k]) << k);
   }
 
+  // stage S: the shared-memory structure of the most selective direct-map join, on every row
+  // (branch-free): a full map clears a missing row and adds (rank + 1) * stride to the group
+  // index of a hit; a bitmap or Bloom filter only clears rows
   int32_t g[kRowsPerThread];
+  const int32_t g0 = group_origin<NJ, GROUPED, DM>(js);
 #pragma unroll
-  for (int k = 0; k < kRowsPerThread; ++k) g[k] = 0;
-  const int j0 = first_join_in_place<NJ>(p, js);
+  for (int k = 0; k < kRowsPerThread; ++k) g[k] = g0;
+#pragma unroll
+  for (int jx = 0; jx < NJ; ++jx) {
+    const JoinDev& d = p.joins[jx];
+    if (!DM || !jbit(p.m_ins, jx)) continue;
+    const int4 kv = *reinterpret_cast<const int4*>(tb + d.c * stride);
+    const int32_t key[4] = {kv.x, kv.y, kv.z, kv.w};
+    if (dm_smem<DM>(p, jx)) {  // the full map: exact verdict and rank
+      const uint32_t* w = reinterpret_cast<const uint32_t*>(sdm + d.dm_smem);
+#pragma unroll
+      for (int k = 0; k < kRowsPerThread; ++k) {
+        const uint32_t bit = dm_bit(d, key[k]);
+        const uint32_t word = dm_in(d, key[k]) ? w[bit >> 5] : 0u;
+        const uint32_t v = dm_entry(d, word, bit);
+        m &= ~((uint32_t)(v == 0u) << k);
+        if (GROUPED && all_resolved_in_s<NJ, DM>(p)) g[k] += (int32_t)v * js[jx].jstride;
+      }
+    } else if (jbit(p.m_bm, jx)) {  // its membership bitmap: exact verdict (rank from L2)
+      const uint32_t* w = reinterpret_cast<const uint32_t*>(sdm + d.bm_smem);
+#pragma unroll
+      for (int k = 0; k < kRowsPerThread; ++k) {
+        const uint32_t u = (uint32_t)key[k] - (uint32_t)d.dm_kmin;
+        const uint32_t word = u < d.dm_span ? w[u >> 5] : 0u;
+        m &= ~((uint32_t)(((word >> (u & 31u)) & 1u) == 0u) << k);
+      }
+    } else {  // its Bloom filter: no false negatives
+#pragma unroll
+      for (int k = 0; k < kRowsPerThread; ++k) m &= ~((uint32_t)!bloom_pass(js[jx], key[k]) << k);
+    }
+  }
+  const int j0 = first_join_in_place<NJ, DM>(p, js);
   if (j0) {
     // stage B: ONE probe step of the first join for the lane's 4 rows (4 independent
     // 128-bit loads in flight). Rows whose bucket was full without a verdict (rare at load
@@ -414,7 +554,7 @@ __device__ __forceinline__ void process_tile(const K1Params& p, const JoinState 
     }
   }
 
-  if (NJ == 0) {
+  if (NJ == 0 || all_resolved_in_s<NJ, DM>(p)) {  // every join resolved: aggregate in place
     const int4 va = *reinterpret_cast<const int4*>(tb + p.agg_a * stride);
     const int4 vb = *reinterpret_cast<const int4*>(tb + p.agg_b * stride);
     const int32_t a4[4] = {va.x, va.y, va.z, va.w}, b4[4] = {vb.x, vb.y, vb.z, vb.w};
@@ -437,10 +577,11 @@ __device__ __forceinline__ void process_tile(const K1Params& p, const JoinState 
   }
   const int qn = __shfl_sync(kFull, incl, 31);
   int pos = incl - cnt;
+  const bool carry_g = j0;
   for (uint32_t bits = m; bits; bits &= bits - 1u, ++pos) {
     const int k = __ffs(bits) - 1;
     q_row[pos] = (uint8_t)(lane * kRowsPerThread + k);
-    if (j0) {
+    if (carry_g) {
       int32_t gv = 0;
 #pragma unroll
       for (int kk = 0; kk < kRowsPerThread; ++kk) gv = kk == k ? g[kk] : gv;
@@ -457,14 +598,14 @@ __device__ __forceinline__ void process_tile(const K1Params& p, const JoinState 
   const int total = n_carry + qn;
   const int full_end = total & ~31;
   for (int base = 0; base < full_end; base += 32) {
-    CarryEntry e = load_entry<NJ>(p, js, cb, n_carry, q_row, q_g, j0, wcol, stride, base + lane);
-    stage_c_row<NJ, GROUPED>(p, js, e, j0, jf, smem_table, s_sum, s_cnt, acc_sum, acc_cnt);
+    CarryEntry e = load_entry<NJ, DM>(p, js, cb, n_carry, q_row, q_g, carry_g, wcol, stride, base + lane);
+    stage_c_row<NJ, GROUPED, DM>(p, js, sdm, e, j0, jf, smem_table, s_sum, s_cnt, acc_sum, acc_cnt);
   }
   {
     const int idx = full_end + lane;
     const bool has = idx < total;
     CarryEntry e{};
-    if (has) e = load_entry<NJ>(p, js, cb, n_carry, q_row, q_g, j0, wcol, stride, idx);
+    if (has) e = load_entry<NJ, DM>(p, js, cb, n_carry, q_row, q_g, carry_g, wcol, stride, idx);
     __syncwarp();
     if (has) {
 #pragma unroll
@@ -479,9 +620,10 @@ __device__ __forceinline__ void process_tile(const K1Params& p, const JoinState 
 }
 
 // The rows still carried by a warp after its last tile (fewer than 32).
-template <int NJ, bool GROUPED>
+template <int NJ, bool GROUPED, bool DM>
 __device__ __forceinline__ void drain_carry(const K1Params& p, const JoinState (&js)[HX_MAX_JOINS],
-                                            const CarryBuf* cb, int n_carry, int lane, int j0,
+                                            const unsigned char* sdm, const CarryBuf* cb,
+                                            int n_carry, int lane, int j0,
                                             int jf, bool smem_table, unsigned long long* s_sum,
                                             uint32_t* s_cnt, long long& acc_sum,
                                             long long& acc_cnt) {
@@ -492,7 +634,7 @@ __device__ __forceinline__ void drain_carry(const K1Params& p, const JoinState (
   e.a = cb->a[lane];
   e.b = cb->b[lane];
   e.g = cb->g[lane];
-  stage_c_row<NJ, GROUPED>(p, js, e, j0, jf, smem_table, s_sum, s_cnt, acc_sum, acc_cnt);
+  stage_c_row<NJ, GROUPED, DM>(p, js, sdm, e, j0, jf, smem_table, s_sum, s_cnt, acc_sum, acc_cnt);
 }
 
 __device__ __forceinline__ void mbar_wait_sleep(uint64_t* bar, uint32_t parity) {
@@ -512,7 +654,7 @@ __device__ __forceinline__ void mbar_wait_sleep(uint64_t* bar, uint32_t parity) 
   }
 }
 
-template <int NJ, bool GROUPED>
+template <int NJ, bool GROUPED, bool DM>
 __global__ void __launch_bounds__(kThreads, kCtasPerSm) k1_probe_agg(const __grid_constant__ K1Params p) {
   extern __shared__ __align__(128) unsigned char smem[];
   uint64_t* full = reinterpret_cast<uint64_t*>(smem);
@@ -526,7 +668,8 @@ __global__ void __launch_bounds__(kThreads, kCtasPerSm) k1_probe_agg(const __gri
   const size_t table_bytes = ((size_t)p.smem_groups * 12 + 127) & ~size_t(127);
   uint32_t* s_filters = reinterpret_cast<uint32_t*>(smem + kSmemFixed + table_bytes);
   const size_t filter_bytes = ((size_t)p.filter_words * 4 + 127) & ~size_t(127);
-  int32_t* stage0 = reinterpret_cast<int32_t*>(smem + kSmemFixed + table_bytes + filter_bytes);
+  unsigned char* sdm = smem + kSmemFixed + table_bytes + filter_bytes;  // staged direct maps
+  int32_t* stage0 = reinterpret_cast<int32_t*>(sdm + p.dm_bytes);
   const int stage_elems = p.n_cols * kTileRows;
 
   // a failed group layout (capacity, or a plan whose dimensions changed) disables the pass
@@ -615,6 +758,21 @@ __global__ void __launch_bounds__(kThreads, kCtasPerSm) k1_probe_agg(const __gri
       dst += reserved;
     }
   }
+  // stage the direct maps planned into shared memory (once per CTA)
+#pragma unroll
+  for (int j = 0; j < NJ; ++j) {
+    if (!dm_smem<DM>(p, j)) continue;
+    const uint4* src = reinterpret_cast<const uint4*>(p.joins[j].dm);
+    uint4* dst = reinterpret_cast<uint4*>(sdm + p.joins[j].dm_smem);
+    for (int i = ctid; i < p.joins[j].dm_words / 4; i += kConsumers) dst[i] = __ldg(src + i);
+  }
+#pragma unroll
+  for (int j = 0; j < NJ; ++j) {
+    if (!DM || !jbit(p.m_bm, j)) continue;
+    const uint4* src = reinterpret_cast<const uint4*>(p.joins[j].bm);
+    uint4* dst = reinterpret_cast<uint4*>(sdm + p.joins[j].bm_smem);
+    for (int i = ctid; i < p.joins[j].bm_words / 4; i += kConsumers) dst[i] = __ldg(src + i);
+  }
   const long long n_groups = GROUPED ? p.meta->n_groups : 1;
   const bool smem_table = GROUPED && n_groups <= p.smem_groups;
   if (smem_table) {
@@ -631,7 +789,7 @@ __global__ void __launch_bounds__(kThreads, kCtasPerSm) k1_probe_agg(const __gri
     if (ctid < p.head_rows)
       for (int c = 0; c < p.n_cols; ++c) headbuf[c * 4 + ctid] = p.head_col[c][ctid];
     consumer_sync();
-    process_tile<NJ, GROUPED>(p, js, headbuf, 4, p.head_rows, warp, lane, smem_table, s_sum,
+    process_tile<NJ, GROUPED, DM>(p, js, sdm, headbuf, 4, p.head_rows, warp, lane, smem_table, s_sum,
                               s_cnt, q_row, q_g, cb, n_carry, acc_sum, acc_cnt);
   }
   consumer_sync();
@@ -650,7 +808,7 @@ __global__ void __launch_bounds__(kThreads, kCtasPerSm) k1_probe_agg(const __gri
           st[c * kTileRows + copied + ctid] = p.col[c][r0 + copied + ctid];
       consumer_sync();
     }
-    process_tile<NJ, GROUPED>(p, js, st, kTileRows, rows, warp, lane, smem_table, s_sum, s_cnt,
+    process_tile<NJ, GROUPED, DM>(p, js, sdm, st, kTileRows, rows, warp, lane, smem_table, s_sum, s_cnt,
                               q_row, q_g, cb, n_carry, acc_sum, acc_cnt);
     __syncwarp();
     if (lane == 0) mbar_arrive(empty + s);
@@ -662,8 +820,8 @@ __global__ void __launch_bounds__(kThreads, kCtasPerSm) k1_probe_agg(const __gri
 
   // the rows this warp still carries
   if (NJ > 0)
-    drain_carry<NJ, GROUPED>(p, js, cb, n_carry, lane, first_join_in_place<NJ>(p, js),
-                             first_filter<NJ>(js), smem_table, s_sum, s_cnt, acc_sum, acc_cnt);
+    drain_carry<NJ, GROUPED, DM>(p, js, sdm, cb, n_carry, lane, first_join_in_place<NJ, DM>(p, js),
+                             first_filter<NJ, DM>(js), smem_table, s_sum, s_cnt, acc_sum, acc_cnt);
   __syncwarp();
 
   // ---------------- flush the CTA's partial aggregate ----------------
@@ -744,27 +902,28 @@ __global__ void k1_prepare(AggMeta* meta, const HtHeader* g0, const HtHeader* g1
   }
 }
 
-template <int NJ, bool G>
-void set_attrs() {
-  cudaFuncSetAttribute(k1_probe_agg<NJ, G>, cudaFuncAttributeMaxDynamicSharedMemorySize,
-                       227 * 1024);
-}
-
 using KernelFn = void (*)(K1Params);
 
-KernelFn pick_kernel(int nj, bool grouped) {
-  static const KernelFn table[2][HX_MAX_JOINS + 1] = {
-      {k1_probe_agg<0, false>, k1_probe_agg<1, false>, k1_probe_agg<2, false>,
-       k1_probe_agg<3, false>, k1_probe_agg<4, false>},
-      {k1_probe_agg<0, true>, k1_probe_agg<1, true>, k1_probe_agg<2, true>,
-       k1_probe_agg<3, true>, k1_probe_agg<4, true>}};
-  return table[grouped ? 1 : 0][nj];
+// [direct maps][grouped][joins]; join-less pipelines use the hash-table instances
+const KernelFn kKernels[2][2][HX_MAX_JOINS + 1] = {
+    {{k1_probe_agg<0, false, false>, k1_probe_agg<1, false, false>, k1_probe_agg<2, false, false>,
+      k1_probe_agg<3, false, false>, k1_probe_agg<4, false, false>},
+     {k1_probe_agg<0, true, false>, k1_probe_agg<1, true, false>, k1_probe_agg<2, true, false>,
+      k1_probe_agg<3, true, false>, k1_probe_agg<4, true, false>}},
+    {{k1_probe_agg<0, false, false>, k1_probe_agg<1, false, true>, k1_probe_agg<2, false, true>,
+      k1_probe_agg<3, false, true>, k1_probe_agg<4, false, true>},
+     {k1_probe_agg<0, true, false>, k1_probe_agg<1, true, true>, k1_probe_agg<2, true, true>,
+      k1_probe_agg<3, true, true>, k1_probe_agg<4, true, true>}}};
+
+KernelFn pick_kernel(int nj, bool grouped, bool dm) {
+  return kKernels[dm ? 1 : 0][grouped ? 1 : 0][nj];
 }
 
-size_t k1_smem_bytes(int n_cols, int stages, int smem_groups, int filter_words = 0) {
+size_t k1_smem_bytes(int n_cols, int stages, int smem_groups, int filter_words = 0,
+                     int dm_bytes = 0) {
   const size_t table_bytes = ((size_t)smem_groups * 12 + 127) & ~size_t(127);
   const size_t filter_bytes = ((size_t)filter_words * 4 + 127) & ~size_t(127);
-  return kSmemFixed + table_bytes + filter_bytes +
+  return kSmemFixed + table_bytes + filter_bytes + (size_t)dm_bytes +
          (size_t)stages * n_cols * kTileRows * sizeof(int32_t);
 }
 
@@ -786,13 +945,15 @@ int pick_stages(int n_cols, int smem_groups) {
 int k1_occupancy(hx_ctx* ctx) {
   static bool attrs = false;
   if (!attrs) {
-    set_attrs<0, false>(); set_attrs<1, false>(); set_attrs<2, false>(); set_attrs<3, false>();
-    set_attrs<4, false>(); set_attrs<0, true>(); set_attrs<1, true>(); set_attrs<2, true>();
-    set_attrs<3, true>(); set_attrs<4, true>();
+    for (int d = 0; d < 2; ++d)
+      for (int g = 0; g < 2; ++g)
+        for (int j = 0; j <= HX_MAX_JOINS; ++j)
+          cudaFuncSetAttribute(kKernels[d][g][j], cudaFuncAttributeMaxDynamicSharedMemorySize,
+                               227 * 1024);
     attrs = true;
   }
   int occ = 0;
-  cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, k1_probe_agg<3, true>, kThreads,
+  cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, k1_probe_agg<3, true, false>, kThreads,
                                                 k1_smem_bytes(4, pick_stages(4, kSmemGroups), kSmemGroups));
   return occ;
 }
@@ -896,7 +1057,30 @@ int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht*
     HX_REQUIRE(sh->join_ht[j] >= 0 && sh->join_ht[j] < n_hts && hts && hts[sh->join_ht[j]],
                HX_EINVAL, "hx_pipeline_probe_agg: bad join hash table index");
     const hx_ht* ht = hts[sh->join_ht[j]];
-    p.joins[j] = JoinDev{c, ht->slots, ht->hdr, ht->bloom, 0};
+    JoinDev d{};
+    d.c = c;
+    d.slots = ht->slots;
+    d.hdr = ht->hdr;
+    d.bloom = ht->bloom;
+    d.dm_smem = -1;
+    if (ht->dm) {
+      d.dm = ht->dm;
+      d.dm_kmin = ht->dm_kmin;
+      d.dm_span = ht->dm_span;
+      d.dm_lw = ht->dm_lw;
+      d.dm_vmask = dm_vmask(ht->dm_lw);
+      d.dm_words = (int32_t)ht->dm_words;
+      d.bm = ht->dm_bm;
+      d.bm_words = (int32_t)ht->bm_words;
+    }
+    d.bm_smem = -1;
+    p.joins[j] = d;
+  }
+  {
+    int n_dm = 0;
+    for (int j = 0; j < sh->n_joins; ++j) n_dm += p.joins[j].dm != nullptr;
+    HX_REQUIRE(n_dm == 0 || n_dm == sh->n_joins, HX_EINVAL,
+               "hx_pipeline_probe_agg: direct-map and hash-table joins in one pipeline");
   }
   p.agg_op = sh->agg_op;
   p.agg_a = stage_of(sh->agg_a);
@@ -935,48 +1119,113 @@ int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht*
   p.g_cnt = agg->cnts;
   const bool grouped = sh->n_gdims > 0;
   p.smem_groups = grouped ? (int32_t)std::min<long long>(kSmemGroups, agg->cap_groups) : 0;
-  // Shared-memory plan: the tile ring (pick_stages) and the Bloom filters (semi-join
-  // reduction) of the joins whose passing key count is known (a plan observed it) and that
-  // are selective (at most half the dimension passes). Filters are taken greedily in probe
-  // order in the shared memory the ring leaves free.
-  int want[HX_MAX_JOINS] = {0, 0, 0, 0};
+  // Shared-memory plan. The tile ring keeps pick_stages' depth (measured: shrinking it to fit
+  // more filters lost 6% at SF100); the rest of the CTA's shared memory is given out in two
+  // passes over the joins whose passing key count a plan observed:
+  //   1. selective joins (at most half the dimension passes), most selective first, get a
+  //      filter that runs on every row: a direct-map join its full map (exact, also resolves
+  //      the rank) if that is at most twice its smallest filter, else the smaller of its
+  //      membership bitmap (exact) and its Bloom filter; a hash-table join its Bloom filter;
+  //   2. the direct maps still read from L2 are then staged in full, smallest first (each
+  //      saves one L2 lookup per surviving row), replacing their filter.
+  p.stages = pick_stages(n_cols, p.smem_groups);
+  enum { kNone = 0, kFull, kBitmap, kBloom };
+  int kind[HX_MAX_JOINS] = {kNone, kNone, kNone, kNone};
+  int bloom_w[HX_MAX_JOINS] = {0, 0, 0, 0};
+  double pass[HX_MAX_JOINS] = {1, 1, 1, 1};
+  int ord[HX_MAX_JOINS] = {0, 1, 2, 3};
   for (int j = 0; j < sh->n_joins; ++j) {
     const hx_ht* ht = hts[sh->join_ht[j]];
-    if (ht->known_keys < 0 || 2 * ht->known_keys > ht->dim_rows) continue;
-    want[j] = std::max(4, 1 << std::min(ht->max_bloom_log2w, bloom_log2w_for(ht->known_keys)));
+    if (ht->known_keys < 0) continue;
+    pass[j] = (double)ht->known_keys / (double)std::max<int64_t>(1, ht->dim_rows);
+    bloom_w[j] = std::max(4, 1 << std::min(ht->max_bloom_log2w, bloom_log2w_for(ht->known_keys)));
   }
-  auto fit_filters = [&](int stages, int* words_out) {
-    int used = 0, n = 0;
-    for (int j = 0; j < sh->n_joins; ++j) {
-      words_out[j] = 0;
-      if (!want[j]) continue;
-      if (k1_smem_bytes(n_cols, stages, p.smem_groups, used + want[j]) >
-          smem_budget(std::min(kCtasPerSm, 2)))
-        continue;
-      words_out[j] = want[j];
-      used += want[j];
-      ++n;
-    }
-    return n;
+  std::stable_sort(ord, ord + sh->n_joins, [&](int x, int y) { return pass[x] < pass[y]; });
+  auto usage = [&](int j, int k, int* fw, int* db) {
+    const JoinDev& d = p.joins[j];
+    if (k == kFull) *db += d.dm_words * 4;
+    if (k == kBitmap) *db += d.bm_words * 4;
+    if (k == kBloom) *fw += bloom_w[j];
   };
-  // (measured: shrinking the ring to 2 stages to fit more filters lost 6% at SF100 and gained
-  // nothing at SF10, so the ring keeps pick_stages' depth and filters take what is left)
-  int chosen[HX_MAX_JOINS];
-  p.stages = pick_stages(n_cols, p.smem_groups);
-  fit_filters(p.stages, chosen);
+  auto fits = [&](int j_new, int k_new) {
+    int fw = 0, db = 0;
+    for (int j = 0; j < sh->n_joins; ++j) usage(j, j == j_new ? k_new : kind[j], &fw, &db);
+    return k1_smem_bytes(n_cols, p.stages, p.smem_groups, fw, db) <=
+           smem_budget(std::min(kCtasPerSm, 2));
+  };
+  for (int i = 0; i < sh->n_joins; ++i) {
+    const int j = ord[i];
+    const JoinDev& d = p.joins[j];
+    if (!bloom_w[j] || 2 * pass[j] > 1.0) continue;
+    if (!d.dm) {
+      if (fits(j, kBloom)) kind[j] = kBloom;
+      continue;
+    }
+    const int full = d.dm_words * 4, bm = d.bm_words * 4, bl = bloom_w[j] * 4;
+    const int cand[3] = {full <= 2 * std::min(bm, bl) ? (int)kFull : (int)kNone,
+                         bm <= bl ? (int)kBitmap : (int)kBloom, bm <= bl ? (int)kBloom : (int)kBitmap};
+    for (int c : cand)
+      if (c != kNone && kind[j] == kNone && fits(j, c)) kind[j] = c;
+  }
+  int dms[HX_MAX_JOINS], n_dms = 0;
+  for (int j = 0; j < sh->n_joins; ++j)
+    if (p.joins[j].dm && kind[j] != kFull) dms[n_dms++] = j;
+  std::stable_sort(dms, dms + n_dms,
+                   [&](int x, int y) { return p.joins[x].dm_words < p.joins[y].dm_words; });
+  for (int i = 0; i < n_dms; ++i)
+    if (fits(dms[i], kFull)) kind[dms[i]] = kFull;
+  // offsets: Bloom filters in the filter region, maps and bitmaps in the direct-map region
   p.filter_words = 0;
+  p.dm_bytes = 0;
   for (int j = 0; j < sh->n_joins; ++j) {
-    p.joins[j].bloom_words = chosen[j];
-    p.filter_words += chosen[j];
+    JoinDev& d = p.joins[j];
+    d.bloom_words = 0;
+    d.dm_smem = -1;
+    d.bm_smem = -1;
+    if (kind[j] == kBloom) {
+      d.bloom_words = bloom_w[j];
+      p.filter_words += bloom_w[j];
+    } else if (kind[j] == kFull) {
+      d.dm_smem = p.dm_bytes;
+      p.dm_bytes += d.dm_words * 4;
+    } else if (kind[j] == kBitmap) {
+      d.bm_smem = p.dm_bytes;
+      p.dm_bytes += d.bm_words * 4;
+    }
+    d.in_s = 0;
+  }
+  // stage S (every row): the structure of the most selective direct-map join; the others run
+  // in stage C on the compacted survivors only
+  for (int i = 0; i < sh->n_joins; ++i) {
+    const int j = ord[i];
+    if (p.joins[j].dm && kind[j] != kNone && 2 * pass[j] <= 1.0) {
+      p.joins[j].in_s = 1;
+      break;
+    }
+  }
+  p.m_dm = p.m_dmsm = p.m_bm = p.m_ins = 0u;
+  for (int j = 0; j < sh->n_joins; ++j) {
+    const JoinDev& d = p.joins[j];
+    p.m_dm |= (uint32_t)(d.dm != nullptr) << j;
+    p.m_dmsm |= (uint32_t)(d.dm != nullptr && d.dm_smem >= 0) << j;
+    p.m_bm |= (uint32_t)(d.dm != nullptr && d.bm_smem >= 0) << j;
+    p.m_ins |= (uint32_t)(d.in_s != 0) << j;
   }
   if (std::getenv("HX_DEBUG")) {  // launch plan of this K1 (tuning aid)
     std::fprintf(stderr, "[hx] K1 joins=%d cols=%d stages=%d groups=%d filters:", sh->n_joins,
                  n_cols, p.stages, p.smem_groups);
     for (int j = 0; j < sh->n_joins; ++j) std::fprintf(stderr, " %d", p.joins[j].bloom_words);
-    std::fprintf(stderr, " smem=%zu\n", k1_smem_bytes(n_cols, p.stages, p.smem_groups, p.filter_words));
+    std::fprintf(stderr, " dm(words@smem/bitmap@smem):");
+    for (int j = 0; j < sh->n_joins; ++j)
+      std::fprintf(stderr, " %d@%d/%d@%d", p.joins[j].dm ? p.joins[j].dm_words : 0,
+                   p.joins[j].dm_smem, p.joins[j].bm_words, p.joins[j].bm_smem);
+    std::fprintf(stderr, " in_s:");
+    for (int j = 0; j < sh->n_joins; ++j) std::fprintf(stderr, "%d", p.joins[j].in_s);
+    std::fprintf(stderr, " smem=%zu\n",
+                 k1_smem_bytes(n_cols, p.stages, p.smem_groups, p.filter_words, p.dm_bytes));
   }
-  k.fn = pick_kernel(sh->n_joins, grouped);
-  k.smem = k1_smem_bytes(n_cols, p.stages, p.smem_groups, p.filter_words);
+  k.fn = pick_kernel(sh->n_joins, grouped, p.m_dm != 0u);
+  k.smem = k1_smem_bytes(n_cols, p.stages, p.smem_groups, p.filter_words, p.dm_bytes);
   int occ = 0;
   HX_CK(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, k.fn, kThreads, k.smem));
   occ = std::max(1, occ);

@@ -248,3 +248,75 @@ def test_device_generated_columns_match_host(ctx, sf):
         ssbgen.column_device(42, sz, col, t.data_ptr(), r0, n, torch.cuda.current_stream().cuda_stream)
         torch.cuda.synchronize()
         assert np.array_equal(t.cpu().numpy(), ssbgen.column(42, sz, col, r0, n)), col
+
+
+# ---- direct maps (plans over dense keys, R20) vs hash tables -----------------------
+def _remap_keys(db, mul, off):
+    """Apply k -> k*mul + off to every customer / supplier / part key and its foreign key
+    (a bijection: the query results are unchanged); mul=1, off=0 keeps the dense keys."""
+    out = {t: dict(cols) for t, cols in db.items()}
+    for dim, pk, fk in (("customer", "c_custkey", "lo_custkey"), ("supplier", "s_suppkey", "lo_suppkey"),
+                        ("part", "p_partkey", "lo_partkey")):
+        for t, c in ((dim, pk), ("lineorder", fk)):
+            v = out[t][c].astype(np.int64) * mul + off
+            assert v.min() >= -(1 << 31) and v.max() < (1 << 31) and not (v == -1).any()
+            out[t][c] = v.astype(np.int32)
+    return out
+
+
+@pytest.mark.parametrize("no_dm", [False, True])
+@pytest.mark.parametrize("mul,off", [(1, 0), (7919, -500000), (1 << 25, -(1 << 30))])
+def test_plans_key_encodings(ctx, monkeypatch, mul, off, no_dm):
+    """Plans choose a direct map (dense or moderately sparse keys, negative keys included) or
+    the hash table (span >= 2^27, or HX_NO_DM=1); both give the oracle's rows."""
+    if no_dm:
+        monkeypatch.setenv("HX_NO_DM", "1")
+    db = _remap_keys(tiny_db(5, n_lo=20011), mul, off)
+    dims, fact = ssb.load_db_numpy(ctx, db)
+    eng = ssb.SsbEngine(ctx, dims, fact)
+    plans = {q: eng.plan(q) for q in QUERIES}
+    order = [plans[q].hp for q in QUERIES]
+    graph = hx.capture(ctx, lambda: hx.plans_enqueue(ctx, order))
+    for _ in range(2):
+        graph.launch()
+        for q in QUERIES:
+            assert plans[q].rows() == oracle.run_query(q, db), (q, mul, no_dm)
+    graph.close()
+    for pl in plans.values():
+        pl.close()
+
+
+def test_plan_detects_changed_dimension(ctx):
+    """A direct map is sized from the passing keys a plan observed at creation: if the
+    dimension (a VIEW) later gains a passing key outside that range the execution reports
+    HX_ECAPACITY instead of writing outside the map."""
+    db = tiny_db(6, n_lo=5000)
+    keep = []
+
+    def view(cols):
+        spec = []
+        for c, v in cols.items():
+            t = torch.from_numpy(np.ascontiguousarray(v)).cuda()
+            keep.append(t)
+            spec.append((C[c], t.data_ptr(), len(v)))
+        return hx.load_columns(ctx, spec, placement=_hx.HX_PLACE_VIEW, keep=keep), keep[-len(cols):]
+
+    dims, tensors = {}, {}
+    for t in ("date", "customer", "supplier", "part"):
+        dims[t], ts = view(db[t])
+        tensors[t] = dict(zip(db[t].keys(), ts))
+    fact, _ = view(db["lineorder"])
+    torch.cuda.synchronize()
+    eng = ssb.SsbEngine(ctx, dims, fact)
+    pl = eng.plan("q3.1")  # customer c_region = ASIA, grouped by c_nation
+    pl.enqueue()
+    assert pl.rows() == oracle.run_query("q3.1", db)
+    cust = tensors["customer"]
+    asia = int(np.flatnonzero(db["customer"]["c_region"] == 2)[0])
+    cust["c_custkey"][asia] = 1 << 30  # a passing key far outside the observed range
+    torch.cuda.synchronize()
+    pl.enqueue()
+    with pytest.raises(_hx.HxError) as ei:
+        pl.rows()
+    assert ei.value.code == _hx.HX_ECAPACITY
+    pl.close()

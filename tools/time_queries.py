@@ -1,0 +1,42 @@
+"""Per-query K1 device time of prepared plans at SF (repeated), for A/B tuning.
+
+    python tools/time_queries.py [--sf 10] [--queries q2.1,q3.1] [--reps 5]
+"""
+import argparse
+import os
+import sys
+
+ROOT = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
+sys.path.insert(0, ROOT)
+sys.path.insert(0, os.path.join(ROOT, "tools"))
+
+import torch  # noqa: E402
+
+import ssbgen  # noqa: E402
+from paper_journals_pvldb_chrysogeloskaa19_b200 import hx, ssb  # noqa: E402
+from prof_query import device_db  # noqa: E402
+
+ap = argparse.ArgumentParser()
+ap.add_argument("--sf", type=float, default=10)
+ap.add_argument("--queries", default="all")
+ap.add_argument("--reps", type=int, default=5)
+a = ap.parse_args()
+ctx = hx.Context(0)
+dims, fact = device_db(ctx, ssbgen.sizes(a.sf))
+eng = ssb.SsbEngine(ctx, dims, fact)
+qs = ssb.QUERIES if a.queries == "all" else a.queries.split(",")
+plans = {q: eng.plan(q) for q in qs}
+tot = 0.0
+for q in qs:
+    ts = []
+    for _ in range(a.reps):
+        plans[q].enqueue()
+        plans[q].rows()
+        ts.append(plans[q].hp.k1_time()[0])
+    ts.sort()
+    tot += ts[len(ts) // 2]
+    print(f"{q} k1 median {ts[len(ts) // 2]:.4f} ms  min {ts[0]:.4f}  all {' '.join(f'{t:.3f}' for t in ts)}")
+print(f"sum of medians {tot:.4f} ms")
+for pl in plans.values():
+    pl.close()
+ctx.close()
