@@ -245,7 +245,8 @@ bool k1_is_host(const K1Prepared* k);
 int ring_create(hx_ctx* ctx, const K1Prepared* k, int64_t block_rows, StageRing** out);
 void ring_destroy(hx_ctx* ctx, StageRing* r);
 void k1_free(K1Prepared* k);
-int64_t k1_bytes(const K1Prepared* k);
+int64_t k1_bytes(const K1Prepared* k);          // streamed bytes (rows x 4 x staged columns)
+int k1_gathered_cols(const K1Prepared* k);      // measure columns gathered for passing rows
 const int32_t* table_col(const hx_table* t, int32_t col_id);
 bool table_has_col(const hx_table* t, int32_t col_id);
 cudaEvent_t pooled_event(hx_ctx* ctx);

@@ -28,7 +28,8 @@ struct OutHeader {
   long long n_groups;
   int32_t error;
   int32_t n_gdims;
-  int32_t pad[10];
+  long long n_pass;  // rows that passed every join (sum of the group counts)
+  int32_t pad[8];
 };
 static_assert(sizeof(OutHeader) == 64, "OutHeader is 64 bytes");
 
@@ -60,15 +61,20 @@ __global__ void k1_finalize(FinalizeArgs a) {
   using Scan = cub::BlockScan<int, 1024>;
   __shared__ typename Scan::TempStorage tmp;
   __shared__ long long running;
+  __shared__ unsigned long long n_pass;
   const long long n = a.meta->n_groups;
   int err = a.meta->error;
   for (int d = 0; d < a.n_deps && !err; ++d) err = a.deps[d]->error;
   if (!err && a.expect_groups >= 0 && n != a.expect_groups) err = HX_ECAPACITY;
-  if (threadIdx.x == 0) running = 0;
+  if (threadIdx.x == 0) {
+    running = 0;
+    n_pass = 0;
+  }
   __syncthreads();
   if (!err) {
     for (long long base = 0; base < n; base += 1024) {
       const long long g = base + threadIdx.x;
+      if (g < n && a.cnts[g]) atomicAdd(&n_pass, a.cnts[g]);
       const int flag = g < n && (a.n_gdims == 0 || a.cnts[g] > 0);
       int excl, total;
       Scan(tmp).ExclusiveSum(flag, excl, total);
@@ -97,6 +103,7 @@ __global__ void k1_finalize(FinalizeArgs a) {
     h.n_groups = n;
     h.error = err;
     h.n_gdims = a.n_gdims;
+    h.n_pass = err ? 0 : (long long)n_pass;
     *a.hdr = h;
   }
 }
@@ -412,7 +419,10 @@ int hx_plan_k1_time(hx_plan* pl, float* ms, int64_t* bytes) {
     *ms = 0.f;
     if (pl->k1_e0 && k1_bytes(pl->k1) > 0) HX_CK(cudaEventElapsedTime(ms, pl->k1_e0, pl->k1_e1));
   }
-  if (bytes) *bytes = k1_bytes(pl->k1);
+  if (bytes) {  // streamed columns + one 32-byte sector per gathered value
+    const OutHeader* h = static_cast<const OutHeader*>(pl->h_out);
+    *bytes = k1_bytes(pl->k1) + h->n_pass * 32 * k1_gathered_cols(pl->k1);
+  }
   return HX_OK;
 }
 

@@ -52,11 +52,16 @@ constexpr int kTileRows = kConsumers * kRowsPerThread;  // T = 1024
 constexpr int kCtasPerSm = HX_K1_CTAS;    // target residency (registers, smem budget)
 constexpr int kMaxStageCols = 8;
 constexpr int kSmemGroups = 1024;          // per-CTA group table capacity
-// dynamic smem: [barriers 128 | reduce 256 | head 128 | queues 8 x 256 x (1+4) B | groups | tiles]
+// dynamic smem: [barriers 128 | reduce 256 | head 128 | per-warp queues: 256 row bytes (+ 256
+// group indices, hash-table instances) | per-warp carry buffers | groups | Bloom filters |
+// direct maps | tile ring]
 constexpr int kSmemQueueOff = 512;
-constexpr int kCarryBytes = (HX_MAX_JOINS + 3) * 32 * 4;  // one CarryBuf per consumer warp
-constexpr int kSmemCarryOff = kSmemQueueOff + kConsumers * kRowsPerThread * 5;
-constexpr int kSmemFixed = kSmemCarryOff + kConsumerWarps * kCarryBytes;
+constexpr int kQueueRows = 2 * kRowsPerThread * 32;       // per warp: one tile pair's rows
+constexpr int kCarryBytes = (HX_MAX_JOINS + 4) * 32 * 4;  // one CarryBuf per consumer warp
+constexpr int smem_carry_off(bool dm) {
+  return kSmemQueueOff + kConsumerWarps * kQueueRows * (dm ? 1 : 5);
+}
+constexpr int smem_fixed(bool dm) { return smem_carry_off(dm) + kConsumerWarps * kCarryBytes; }
 
 struct JoinDev {
   int32_t c;                               // staged column of the FK
@@ -89,7 +94,12 @@ struct K1Params {
   int32_t n_preds;
   DevPred preds[HX_MAX_PREDS];
   JoinDev joins[HX_MAX_JOINS];
-  int32_t agg_op, agg_a, agg_b;
+  int32_t agg_op, agg_a, agg_b;            // measure operands: staged column (if staged)
+  // late materialisation: a measure column no predicate or join reads is not streamed; its
+  // value is gathered (one 32-byte sector) for the rows that pass every join only
+  int32_t ga, gb;                          // operand a / b gathered
+  const int32_t* gat_a;                    // fact columns indexed by fact row
+  const int32_t* gat_b;
   const AggMeta* meta;
   unsigned long long* g_sum;
   unsigned long long* g_cnt;
@@ -185,6 +195,14 @@ __device__ __forceinline__ long long measure(int op, int32_t a, int32_t b) {
   if (op == HX_AGG_SUM_MUL) return (long long)a * (long long)b;
   if (op == HX_AGG_SUM_SUB) return (long long)a - (long long)b;
   return (long long)a;
+}
+// The measure of a passing row: staged operands come with the row, gathered ones are read
+// now (the row passed every join: one sector per gathered value).
+__device__ __forceinline__ long long row_measure(const K1Params& p, int32_t a, int32_t b,
+                                                 uint32_t row) {
+  if (p.ga) a = __ldg(p.gat_a + row);
+  if (p.gb) b = __ldg(p.gat_b + row);
+  return measure(p.agg_op, a, b);
 }
 
 // Per-warp view of one join's hash table (loaded once per CTA).
@@ -298,11 +316,13 @@ __device__ __forceinline__ int32_t group_origin(const JoinState (&js)[HX_MAX_JOI
 struct CarryEntry {
   int32_t key[HX_MAX_JOINS];
   int32_t a, b, g;
+  uint32_t row;  // fact row (gathered measures)
 };
 // Per-warp buffer of the (< 32) queued rows carried to the next tile (SoA, one slot per lane).
 struct CarryBuf {
   int32_t key[HX_MAX_JOINS][32];
   int32_t a[32], b[32], g[32];
+  uint32_t row[32];
 };
 
 // Entry idx of the combined sequence [carried rows..., this tile's queue...].
@@ -311,24 +331,29 @@ __device__ __forceinline__ CarryEntry load_entry(const K1Params& p,
                                                  const JoinState (&js)[HX_MAX_JOINS],
                                                  const CarryBuf* cb, int n_carry,
                                                  const uint8_t* q_row, const int32_t* q_g,
-                                                 bool carry_g, const int32_t* wcol, int stride,
-                                                 int idx) {
+                                                 bool carry_g, const int32_t* wcol0,
+                                                 const int32_t* wcol1, uint32_t wrow0,
+                                                 uint32_t wrow1, int stride, int idx) {
   CarryEntry e;
   if (idx < n_carry) {
 #pragma unroll
     for (int jx = 0; jx < NJ; ++jx) e.key[jx] = cb->key[jx][idx];
-    e.a = cb->a[idx];
-    e.b = cb->b[idx];
+    e.a = p.ga ? 0 : cb->a[idx];
+    e.b = p.gb ? 0 : cb->b[idx];
     e.g = cb->g[idx];
+    e.row = (p.ga | p.gb) ? cb->row[idx] : 0u;
   } else {
     const int i = idx - n_carry;
-    const int r = q_row[i];
+    const int q = q_row[i];  // bit 7: which tile of the pair; bits 0-6: row in the warp's slice
+    const int32_t* wcol = (q & 128) ? wcol1 : wcol0;
+    const int r = q & 127;
 #pragma unroll
     for (int jx = 0; jx < NJ; ++jx)
       e.key[jx] = wcol[js[jx].c * stride + r];
-    e.a = wcol[p.agg_a * stride + r];
-    e.b = wcol[p.agg_b * stride + r];
+    e.a = p.ga ? 0 : wcol[p.agg_a * stride + r];
+    e.b = p.gb ? 0 : wcol[p.agg_b * stride + r];
     e.g = carry_g ? q_g[i] : 0;
+    e.row = ((q & 128) ? wrow1 : wrow0) + (uint32_t)r;
   }
   return e;
 }
@@ -422,53 +447,74 @@ __device__ __forceinline__ void stage_c_row(const K1Params& p, const JoinState (
     if (!alive) pend = 0;
   }
   if (alive)
-    accumulate<GROUPED>(p, smem_table, s_sum, s_cnt, gg, measure(p.agg_op, e.a, e.b), acc_sum,
+    accumulate<GROUPED>(p, smem_table, s_sum, s_cnt, gg, row_measure(p, e.a, e.b, e.row), acc_sum,
                         acc_cnt);
 }
 
-// Process one staged tile. Warp w owns rows [w*128, w*128+128) of the tile; lane l holds the
-// 4 consecutive rows w*128 + 4l .. +3, read with one 128-bit shared-memory load per column
-// (512 contiguous bytes per warp: conflict-free). Column c, row r of the tile is at
-// sbase[c * stride + r].
-//   stage A  predicates on lineorder columns, branch-free, for the 4 rows of each lane;
-//   stage B  (no predicates) the first join is probed in place for all 4 rows at once —
-//            4 independent 128-bit L2 loads in flight per lane;
-//   compact  survivors are appended to a per-warp queue with ballot + popc (the GPU
-//            "selection vector"), so the remaining joins and the aggregate run with every
-//            lane busy instead of mostly-masked lanes;
-//   stage C  one queued row per lane: the probes of ALL remaining joins are issued together
-//            (independent keys, so one L2 round trip instead of one per join), then the
-//            measure and the group-table atomic.
+// Process a PAIR of staged tiles (two consecutive tiles of this CTA, so the per-iteration
+// costs — compaction, the stage-C batch bookkeeping, the carry — are paid once per 256 rows
+// of a warp). Warp w owns rows [w*128, w*128+128) of each tile; lane l holds the 4
+// consecutive rows w*128 + 4l .. +3 of each, read with one 128-bit shared-memory load per
+// column and tile (512 contiguous bytes per warp: conflict-free). Row k of a lane (k = 0..7)
+// is row (k & 3) of its slice of tile k >> 2. Column c, row r of a tile is at
+// sbase[c * stride + r]; a missing second tile has rows_valid 0.
+//   stage A  predicates on lineorder columns, branch-free;
+//   stage S  (direct maps) the shared-memory structure of the most selective join: full map,
+//            membership bitmap or Bloom filter;
+//   stage F  (hash tables) the first join's Bloom filter; stage B (no predicate, no filter)
+//            the first join probed in place, 4 independent 128-bit L2 loads in flight;
+//   compact  survivors are appended to a per-warp queue (warp prefix sum of the lanes'
+//            counts), so the remaining joins run with every lane busy;
+//   stage C  in full batches of 32 queued rows, one row per lane: the remaining filters,
+//            then the lookups / probes of ALL remaining joins issued together (one L2 round
+//            trip), the measure and the group-table atomic.
 template <int NJ, bool GROUPED, bool DM>
 __device__ __forceinline__ void process_tile(const K1Params& p, const JoinState (&js)[HX_MAX_JOINS],
-                                             const unsigned char* sdm, const int32_t* sbase,
-                                             int stride, int rows_valid, int warp, int lane,
+                                             const unsigned char* sdm, const int32_t* sbase0,
+                                             const int32_t* sbase1, uint32_t frow0,
+                                             uint32_t frow1, int stride, int rows_valid0,
+                                             int rows_valid1, int warp, int lane,
                                              bool smem_table,
                                              unsigned long long* s_sum, uint32_t* s_cnt,
                                              uint8_t* q_row, int32_t* q_g, CarryBuf* cb,
                                              int& n_carry, long long& acc_sum,
                                              long long& acc_cnt) {
-  const int wbase = warp * (32 * kRowsPerThread);
-  const int r0 = wbase + lane * kRowsPerThread;
-  const int32_t* tb = sbase + r0;
+  constexpr int R = kRowsPerThread;  // rows per lane per tile
+  const int wbase = warp * (32 * R);
+  const int r0 = wbase + lane * R;
+  const int32_t* tb[2] = {sbase0 + r0, sbase1 + r0};
   uint32_t m = 0;
 #pragma unroll
-  for (int k = 0; k < kRowsPerThread; ++k) m |= (uint32_t)(r0 + k < rows_valid) << k;
+  for (int k = 0; k < R; ++k) {
+    m |= (uint32_t)(r0 + k < rows_valid0) << k;
+    m |= (uint32_t)(r0 + k < rows_valid1) << (R + k);
+  }
   if (__ballot_sync(kFull, m) == 0) return;
+  // the 8 values of staged column c for this lane
+  auto load8 = [&](int c, int32_t (&v)[2 * R]) {
+#pragma unroll
+    for (int h = 0; h < 2; ++h) {
+      const int4 x = *reinterpret_cast<const int4*>(tb[h] + c * stride);
+      v[h * R + 0] = x.x;
+      v[h * R + 1] = x.y;
+      v[h * R + 2] = x.z;
+      v[h * R + 3] = x.w;
+    }
+  };
 
   // stage A: lineorder predicates (kind is uniform: one branch per predicate, not per row)
   for (int q = 0; q < p.n_preds; ++q) {
     const DevPred& pr = p.preds[q];
-    const int4 v = *reinterpret_cast<const int4*>(tb + pr.c * stride);
-    const int32_t vv[4] = {v.x, v.y, v.z, v.w};
+    int32_t vv[2 * R];
+    load8(pr.c, vv);
     if (pr.kind == HX_PRED_RANGE) {
       const uint32_t lo = (uint32_t)pr.lo, span = (uint32_t)pr.hi - (uint32_t)pr.lo;
 #pragma unroll
-      for (int k = 0; k < kRowsPerThread; ++k)
+      for (int k = 0; k < 2 * R; ++k)
         m &= ~((uint32_t)(((uint32_t)vv[k] - lo) > span) << k);
     } else {
 #pragma unroll
-      for (int k = 0; k < kRowsPerThread; ++k) {
+      for (int k = 0; k < 2 * R; ++k) {
         bool ok = false;
 #pragma unroll
         for (int i = 0; i < 4; ++i) ok |= (i < pr.n_in) && vv[k] == pr.in[i];
@@ -477,91 +523,98 @@ __device__ __forceinline__ void process_tile(const K1Params& p, const JoinState 
     }
   }
 
-  // stage F: semi-join reduction with the shared-memory Bloom filter of the first filtered
-  // join (the most selective: joins are in ascending pass fraction) on every row; the other
-  // joins' filters are applied to the few survivors in stage C. No false negatives; the
-  // ~5% false positives are removed by the exact probe.
+  // stage F (hash tables): semi-join reduction with the shared-memory Bloom filter of the
+  // first filtered join (the most selective: joins are in ascending pass fraction) on every
+  // row; the other joins' filters are applied to the survivors in stage C. No false
+  // negatives; the ~5% false positives are removed by the exact probe.
   const int jf = first_filter<NJ, DM>(js);
 #pragma unroll
   for (int jx = 0; jx < NJ; ++jx) {
     if (jx != jf) continue;
-    const int4 kv = *reinterpret_cast<const int4*>(tb + js[jx].c * stride);
-    const int32_t key[4] = {kv.x, kv.y, kv.z, kv.w};
+    int32_t key[2 * R];
+    load8(js[jx].c, key);
 #pragma unroll
-    for (int k = 0; k < kRowsPerThread; ++k) m &= ~((uint32_t)!bloom_pass(js[jx], key[k]) << k);
+    for (int k = 0; k < 2 * R; ++k) m &= ~((uint32_t)!bloom_pass(js[jx], key[k]) << k);
   }
 
-  // stage S: the shared-memory structure of the most selective direct-map join, on every row
-  // (branch-free): a full map clears a missing row and adds (rank + 1) * stride to the group
-  // index of a hit; a bitmap or Bloom filter only clears rows
-  int32_t g[kRowsPerThread];
+  // stage S (direct maps): the shared-memory structure of the most selective join, on every
+  // row (branch-free). A full map clears a missing row (and, when it resolves the pipeline's
+  // only join, yields the group index); a bitmap or Bloom filter only clears rows.
+  const bool all_res = all_resolved_in_s<NJ, DM>(p);
+  int32_t g[2 * R];
   const int32_t g0 = group_origin<NJ, GROUPED, DM>(js);
 #pragma unroll
-  for (int k = 0; k < kRowsPerThread; ++k) g[k] = g0;
+  for (int k = 0; k < 2 * R; ++k) g[k] = g0;
 #pragma unroll
   for (int jx = 0; jx < NJ; ++jx) {
     const JoinDev& d = p.joins[jx];
     if (!DM || !jbit(p.m_ins, jx)) continue;
-    const int4 kv = *reinterpret_cast<const int4*>(tb + d.c * stride);
-    const int32_t key[4] = {kv.x, kv.y, kv.z, kv.w};
+    int32_t key[2 * R];
+    load8(d.c, key);
     if (dm_smem<DM>(p, jx)) {  // the full map: exact verdict and rank
       const uint32_t* w = reinterpret_cast<const uint32_t*>(sdm + d.dm_smem);
 #pragma unroll
-      for (int k = 0; k < kRowsPerThread; ++k) {
+      for (int k = 0; k < 2 * R; ++k) {
         const uint32_t bit = dm_bit(d, key[k]);
         const uint32_t word = dm_in(d, key[k]) ? w[bit >> 5] : 0u;
         const uint32_t v = dm_entry(d, word, bit);
         m &= ~((uint32_t)(v == 0u) << k);
-        if (GROUPED && all_resolved_in_s<NJ, DM>(p)) g[k] += (int32_t)v * js[jx].jstride;
+        if (GROUPED && all_res) g[k] += (int32_t)v * js[jx].jstride;
       }
     } else if (jbit(p.m_bm, jx)) {  // its membership bitmap: exact verdict (rank from L2)
       const uint32_t* w = reinterpret_cast<const uint32_t*>(sdm + d.bm_smem);
 #pragma unroll
-      for (int k = 0; k < kRowsPerThread; ++k) {
+      for (int k = 0; k < 2 * R; ++k) {
         const uint32_t u = (uint32_t)key[k] - (uint32_t)d.dm_kmin;
         const uint32_t word = u < d.dm_span ? w[u >> 5] : 0u;
         m &= ~((uint32_t)(((word >> (u & 31u)) & 1u) == 0u) << k);
       }
     } else {  // its Bloom filter: no false negatives
 #pragma unroll
-      for (int k = 0; k < kRowsPerThread; ++k) m &= ~((uint32_t)!bloom_pass(js[jx], key[k]) << k);
-    }
-  }
-  const int j0 = first_join_in_place<NJ, DM>(p, js);
-  if (j0) {
-    // stage B: ONE probe step of the first join for the lane's 4 rows (4 independent
-    // 128-bit loads in flight). Rows whose bucket was full without a verdict (rare at load
-    // factor 1/4) are queued with ~next_bucket in place of the group index and finish in
-    // stage C, so the warp never waits on its longest probe chain here.
-    const JoinState& j = js[0];
-    const int4 kv = *reinterpret_cast<const int4*>(tb + j.c * stride);
-    const int32_t key[4] = {kv.x, kv.y, kv.z, kv.w};
-    ulonglong2 v[kRowsPerThread];
-    uint32_t b[kRowsPerThread];
-#pragma unroll
-    for (int k = 0; k < kRowsPerThread; ++k) {
-      b[k] = bucket_of(key[k], j.shift);
-      if ((m >> k) & 1u) v[k] = __ldg(j.buckets + b[k]);
-    }
-#pragma unroll
-    for (int k = 0; k < kRowsPerThread; ++k) {
-      if (!((m >> k) & 1u)) continue;
-      bool hit, miss;
-      int32_t rank;
-      probe_step(v[k], key[k], hit, miss, rank);
-      g[k] = hit ? rank * j.jstride : (int32_t)~((b[k] + 1) & j.bmask);
-      m &= ~((uint32_t)miss << k);
+      for (int k = 0; k < 2 * R; ++k) m &= ~((uint32_t)!bloom_pass(js[jx], key[k]) << k);
     }
   }
 
-  if (NJ == 0 || all_resolved_in_s<NJ, DM>(p)) {  // every join resolved: aggregate in place
-    const int4 va = *reinterpret_cast<const int4*>(tb + p.agg_a * stride);
-    const int4 vb = *reinterpret_cast<const int4*>(tb + p.agg_b * stride);
-    const int32_t a4[4] = {va.x, va.y, va.z, va.w}, b4[4] = {vb.x, vb.y, vb.z, vb.w};
+  const int j0 = first_join_in_place<NJ, DM>(p, js);
+  if (j0) {
+    // stage B (hash tables): ONE probe step of the first join per row, 4 independent 128-bit
+    // loads in flight per tile. Rows whose bucket was full without a verdict (rare at load
+    // factor 1/4) are queued with ~next_bucket in place of the group index and finish in
+    // stage C, so the warp never waits on its longest probe chain here.
+    const JoinState& j = js[0];
+    int32_t key[2 * R];
+    load8(j.c, key);
 #pragma unroll
-    for (int k = 0; k < kRowsPerThread; ++k)
+    for (int h = 0; h < 2; ++h) {
+      ulonglong2 v[R];
+      uint32_t b[R];
+#pragma unroll
+      for (int k = 0; k < R; ++k) {
+        b[k] = bucket_of(key[h * R + k], j.shift);
+        if ((m >> (h * R + k)) & 1u) v[k] = __ldg(j.buckets + b[k]);
+      }
+#pragma unroll
+      for (int k = 0; k < R; ++k) {
+        const int kk = h * R + k;
+        if (!((m >> kk) & 1u)) continue;
+        bool hit, miss;
+        int32_t rank;
+        probe_step(v[k], key[kk], hit, miss, rank);
+        g[kk] = hit ? rank * j.jstride : (int32_t)~((b[k] + 1) & j.bmask);
+        m &= ~((uint32_t)miss << kk);
+      }
+    }
+  }
+
+  if (NJ == 0 || all_res) {  // every join resolved: aggregate in place
+    int32_t a8[2 * R] = {}, b8[2 * R] = {};
+    if (!p.ga) load8(p.agg_a, a8);
+    if (!p.gb) load8(p.agg_b, b8);
+#pragma unroll
+    for (int k = 0; k < 2 * R; ++k)
       if ((m >> k) & 1u)
-        accumulate<GROUPED>(p, smem_table, s_sum, s_cnt, g[k], measure(p.agg_op, a4[k], b4[k]),
+        accumulate<GROUPED>(p, smem_table, s_sum, s_cnt, g[k],
+                            row_measure(p, a8[k], b8[k], (k < R ? frow0 : frow1) + r0 + (k & 3)),
                             acc_sum, acc_cnt);
     return;
   }
@@ -580,32 +633,37 @@ __device__ __forceinline__ void process_tile(const K1Params& p, const JoinState 
   const bool carry_g = j0;
   for (uint32_t bits = m; bits; bits &= bits - 1u, ++pos) {
     const int k = __ffs(bits) - 1;
-    q_row[pos] = (uint8_t)(lane * kRowsPerThread + k);
+    q_row[pos] = (uint8_t)(((k >> 2) << 7) | (lane * R + (k & 3)));
     if (carry_g) {
       int32_t gv = 0;
 #pragma unroll
-      for (int kk = 0; kk < kRowsPerThread; ++kk) gv = kk == k ? g[kk] : gv;
+      for (int kk = 0; kk < 2 * R; ++kk) gv = kk == k ? g[kk] : gv;
       q_g[pos] = gv;
     }
   }
   __syncwarp();
 
-  // stage C in full batches of 32: the warp's queue of this tile is appended to the rows
-  // carried over from earlier tiles; every complete batch of 32 is processed now (one row per
-  // lane, all lanes busy), the < 32 left over are copied (as values) into the carry buffer,
-  // so the tile's shared-memory stage can be released.
-  const int32_t* wcol = sbase + wbase;
+  // stage C in full batches of 32: the warp's queue of this pair is appended to the rows
+  // carried over from earlier pairs; every complete batch of 32 is processed now (one row
+  // per lane, all lanes busy), the < 32 left over are copied (as values) into the carry
+  // buffer, so the tiles' shared-memory stages can be released.
+  const int32_t* wcol0 = sbase0 + wbase;
+  const int32_t* wcol1 = sbase1 + wbase;
+  const uint32_t wrow0 = frow0 + wbase, wrow1 = frow1 + wbase;
   const int total = n_carry + qn;
   const int full_end = total & ~31;
   for (int base = 0; base < full_end; base += 32) {
-    CarryEntry e = load_entry<NJ, DM>(p, js, cb, n_carry, q_row, q_g, carry_g, wcol, stride, base + lane);
+    CarryEntry e = load_entry<NJ, DM>(p, js, cb, n_carry, q_row, q_g, carry_g, wcol0, wcol1,
+                                      wrow0, wrow1, stride, base + lane);
     stage_c_row<NJ, GROUPED, DM>(p, js, sdm, e, j0, jf, smem_table, s_sum, s_cnt, acc_sum, acc_cnt);
   }
   {
     const int idx = full_end + lane;
     const bool has = idx < total;
     CarryEntry e{};
-    if (has) e = load_entry<NJ, DM>(p, js, cb, n_carry, q_row, q_g, carry_g, wcol, stride, idx);
+    if (has)
+      e = load_entry<NJ, DM>(p, js, cb, n_carry, q_row, q_g, carry_g, wcol0, wcol1, wrow0, wrow1,
+                             stride, idx);
     __syncwarp();
     if (has) {
 #pragma unroll
@@ -613,10 +671,11 @@ __device__ __forceinline__ void process_tile(const K1Params& p, const JoinState 
       cb->a[lane] = e.a;
       cb->b[lane] = e.b;
       cb->g[lane] = e.g;
+      cb->row[lane] = e.row;
     }
     n_carry = total - full_end;
   }
-  __syncwarp();  // the queue and the carry buffer are reused by the next tile
+  __syncwarp();  // the queue and the carry buffer are reused by the next pair
 }
 
 // The rows still carried by a warp after its last tile (fewer than 32).
@@ -633,6 +692,7 @@ __device__ __forceinline__ void drain_carry(const K1Params& p, const JoinState (
   for (int jx = 0; jx < NJ; ++jx) e.key[jx] = cb->key[jx][lane];
   e.a = cb->a[lane];
   e.b = cb->b[lane];
+  e.row = cb->row[lane];
   e.g = cb->g[lane];
   stage_c_row<NJ, GROUPED, DM>(p, js, sdm, e, j0, jf, smem_table, s_sum, s_cnt, acc_sum, acc_cnt);
 }
@@ -661,8 +721,10 @@ __global__ void __launch_bounds__(kThreads, kCtasPerSm) k1_probe_agg(const __gri
   uint64_t* empty = full + p.stages;
   long long* red = reinterpret_cast<long long*>(smem + 128);                // 2 x 8 warps
   int32_t* headbuf = reinterpret_cast<int32_t*>(smem + 128 + 256);           // 8 cols x 4
-  uint8_t* q_rows = smem + kSmemQueueOff;                                    // 8 x 256 B
-  int32_t* q_gs = reinterpret_cast<int32_t*>(smem + kSmemQueueOff + kConsumers * kRowsPerThread);
+  constexpr int kSmemFixed = smem_fixed(DM);
+  uint8_t* q_rows = smem + kSmemQueueOff;
+  int32_t* q_gs = DM ? nullptr
+                     : reinterpret_cast<int32_t*>(smem + kSmemQueueOff + kConsumerWarps * kQueueRows);
   unsigned long long* s_sum = reinterpret_cast<unsigned long long*>(smem + kSmemFixed);
   uint32_t* s_cnt = reinterpret_cast<uint32_t*>(s_sum + p.smem_groups);
   const size_t table_bytes = ((size_t)p.smem_groups * 12 + 127) & ~size_t(127);
@@ -716,9 +778,9 @@ __global__ void __launch_bounds__(kThreads, kCtasPerSm) k1_probe_agg(const __gri
 
   // ---------------- consumer warps ----------------
   const int ctid = tid;  // 0..255
-  uint8_t* q_row = q_rows + warp * (32 * kRowsPerThread);
-  int32_t* q_g = q_gs + warp * (32 * kRowsPerThread);
-  CarryBuf* cb = reinterpret_cast<CarryBuf*>(smem + kSmemCarryOff + warp * kCarryBytes);
+  uint8_t* q_row = q_rows + warp * kQueueRows;
+  int32_t* q_g = DM ? nullptr : q_gs + warp * kQueueRows;
+  CarryBuf* cb = reinterpret_cast<CarryBuf*>(smem + smem_carry_off(DM) + warp * kCarryBytes);
   int n_carry = 0;
   JoinState js[HX_MAX_JOINS];
 #pragma unroll
@@ -789,16 +851,19 @@ __global__ void __launch_bounds__(kThreads, kCtasPerSm) k1_probe_agg(const __gri
     if (ctid < p.head_rows)
       for (int c = 0; c < p.n_cols; ++c) headbuf[c * 4 + ctid] = p.head_col[c][ctid];
     consumer_sync();
-    process_tile<NJ, GROUPED, DM>(p, js, sdm, headbuf, 4, p.head_rows, warp, lane, smem_table, s_sum,
-                              s_cnt, q_row, q_g, cb, n_carry, acc_sum, acc_cnt);
+    process_tile<NJ, GROUPED, DM>(p, js, sdm, headbuf, headbuf, 0u, 0u, 4, p.head_rows, 0, warp, lane,
+                                  smem_table, s_sum, s_cnt, q_row, q_g, cb, n_carry, acc_sum,
+                                  acc_cnt);
   }
   consumer_sync();
 
+  // this CTA's tiles t = blockIdx.x + i * gridDim.x arrive in ring slots i mod stages; the
+  // consumers take them two at a time
   int s = 0;
   uint32_t ph = 0;
-  for (int64_t t = blockIdx.x; t < p.n_tiles; t += gridDim.x) {
-    mbar_wait(full + s, ph);
-    int32_t* st = stage0 + (size_t)s * stage_elems;
+  auto acquire = [&](int64_t t, int slot, uint32_t phase) -> int {
+    mbar_wait(full + slot, phase);
+    int32_t* st = stage0 + (size_t)slot * stage_elems;
     const int64_t r0 = t * kTileRows;
     const int rows = (int)std::min<int64_t>(kTileRows, p.n_rows - r0);
     const int copied = rows & ~3;
@@ -808,13 +873,45 @@ __global__ void __launch_bounds__(kThreads, kCtasPerSm) k1_probe_agg(const __gri
           st[c * kTileRows + copied + ctid] = p.col[c][r0 + copied + ctid];
       consumer_sync();
     }
-    process_tile<NJ, GROUPED, DM>(p, js, sdm, st, kTileRows, rows, warp, lane, smem_table, s_sum, s_cnt,
-                              q_row, q_g, cb, n_carry, acc_sum, acc_cnt);
+    return rows;
+  };
+  // (pairs need >= 4 ring slots so that two more tiles stream in while a pair is processed;
+  // a shallower ring takes the tiles one at a time)
+  const bool pairs = p.stages >= 4;
+  for (int64_t t = blockIdx.x; t < p.n_tiles;) {
+    const int64_t t0 = t, t1 = t + gridDim.x;
+    const bool two = pairs && t1 < p.n_tiles;
+    t = two ? t1 + gridDim.x : t1;
+    int s1 = s + 1;
+    uint32_t ph1 = ph;
+    if (s1 == p.stages) {
+      s1 = 0;
+      ph1 ^= 1u;
+    }
+    const int rows0 = acquire(t0, s, ph);
+    const int rows1 = two ? acquire(t1, s1, ph1) : 0;
+    const int32_t* st0 = stage0 + (size_t)s * stage_elems;
+    const int32_t* st1 = two ? stage0 + (size_t)s1 * stage_elems : st0;
+    const uint32_t frow0 = (uint32_t)(p.head_rows + t0 * kTileRows);
+    const uint32_t frow1 = (uint32_t)(p.head_rows + t1 * kTileRows);
+    process_tile<NJ, GROUPED, DM>(p, js, sdm, st0, st1, frow0, frow1, kTileRows, rows0, rows1, warp, lane,
+                                  smem_table, s_sum, s_cnt, q_row, q_g, cb, n_carry, acc_sum,
+                                  acc_cnt);
     __syncwarp();
-    if (lane == 0) mbar_arrive(empty + s);
-    if (++s == p.stages) {
-      s = 0;
-      ph ^= 1u;
+    if (lane == 0) {
+      mbar_arrive(empty + s);
+      if (two) mbar_arrive(empty + s1);
+    }
+    if (two) {  // advance by two slots
+      s = s1 + 1;
+      ph = ph1;
+      if (s == p.stages) {
+        s = 0;
+        ph ^= 1u;
+      }
+    } else {
+      s = s1;
+      ph = ph1;
     }
   }
 
@@ -919,21 +1016,21 @@ KernelFn pick_kernel(int nj, bool grouped, bool dm) {
   return kKernels[dm ? 1 : 0][grouped ? 1 : 0][nj];
 }
 
-size_t k1_smem_bytes(int n_cols, int stages, int smem_groups, int filter_words = 0,
+size_t k1_smem_bytes(bool dm, int n_cols, int stages, int smem_groups, int filter_words = 0,
                      int dm_bytes = 0) {
   const size_t table_bytes = ((size_t)smem_groups * 12 + 127) & ~size_t(127);
   const size_t filter_bytes = ((size_t)filter_words * 4 + 127) & ~size_t(127);
-  return kSmemFixed + table_bytes + filter_bytes + (size_t)dm_bytes +
+  return smem_fixed(dm) + table_bytes + filter_bytes + (size_t)dm_bytes +
          (size_t)stages * n_cols * kTileRows * sizeof(int32_t);
 }
 
 // Per-CTA shared memory for `ctas` resident CTAs per SM (228 KB per SM, 1 KB reserved each).
 constexpr size_t smem_budget(int ctas) { return (228 * 1024) / ctas - 1024; }
 
-int pick_stages(int n_cols, int smem_groups) {
+int pick_stages(bool dm, int n_cols, int smem_groups) {
   // as many tile stages as fit next to kCtasPerSm CTAs per SM, at least double buffering
-  // (at most ~96 KB of tiles per CTA: the rest of a large CTA is left for Bloom filters)
-  const size_t fixed = kSmemFixed + (((size_t)smem_groups * 12 + 127) & ~size_t(127));
+  // (at most HX_K1_STAGE_KB of tiles per CTA: the rest is left for filters and maps)
+  const size_t fixed = smem_fixed(dm) + (((size_t)smem_groups * 12 + 127) & ~size_t(127));
   const size_t budget = std::min<size_t>(smem_budget(kCtasPerSm), fixed + HX_K1_STAGE_KB * 1024);
   const size_t stage = (size_t)n_cols * kTileRows * 4;
   const int s = budget > fixed ? (int)((budget - fixed) / stage) : 0;
@@ -953,8 +1050,9 @@ int k1_occupancy(hx_ctx* ctx) {
     attrs = true;
   }
   int occ = 0;
-  cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, k1_probe_agg<3, true, false>, kThreads,
-                                                k1_smem_bytes(4, pick_stages(4, kSmemGroups), kSmemGroups));
+  cudaOccupancyMaxActiveBlocksPerMultiprocessor(
+      &occ, k1_probe_agg<3, true, false>, kThreads,
+      k1_smem_bytes(false, 4, pick_stages(false, 4, kSmemGroups), kSmemGroups));
   return occ;
 }
 
@@ -1031,6 +1129,7 @@ int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht*
              "hx_pipeline_probe_agg: shape differs from the agg's");
   K1Prepared k{};
   K1Params& p = k.p;
+  bool dm_mode = false;
   // distinct fact columns the shape references -> staged columns
   int32_t ids[kMaxStageCols];
   int n_cols = 0;
@@ -1081,10 +1180,39 @@ int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht*
     for (int j = 0; j < sh->n_joins; ++j) n_dm += p.joins[j].dm != nullptr;
     HX_REQUIRE(n_dm == 0 || n_dm == sh->n_joins, HX_EINVAL,
                "hx_pipeline_probe_agg: direct-map and hash-table joins in one pipeline");
+    dm_mode = n_dm > 0;
   }
   p.agg_op = sh->agg_op;
-  p.agg_a = stage_of(sh->agg_a);
-  p.agg_b = sh->agg_op == HX_AGG_SUM ? p.agg_a : stage_of(sh->agg_b);
+  // Late materialisation (R21): when every join's passing fraction is known (a
+  // plan observed it) and their product bounds the passing rows below 1/16, a measure column
+  // that no predicate or join reads is gathered for the passing rows (one 32-byte sector
+  // each) instead of streamed for every row. Device-resident fact tables only.
+  {
+    double bound = sh->n_joins > 0 ? 1.0 : 2.0;
+    for (int j = 0; j < sh->n_joins; ++j) {
+      const hx_ht* ht = hts[sh->join_ht[j]];
+      bound *= ht->known_keys < 0 ? 2.0
+                                  : (double)ht->known_keys / (double)std::max<int64_t>(1, ht->dim_rows);
+    }
+    const bool ok = bound * 16.0 <= 1.0 && fact->placement != HX_PLACE_HOST_PINNED &&
+                    fact->n_rows < (int64_t(1) << 32) && std::getenv("HX_NO_GATHER") == nullptr;
+    auto read_by_stages = [&](int32_t col) {
+      for (int q = 0; q < sh->n_preds; ++q)
+        if (sh->preds[q].col_id == col) return true;
+      for (int j = 0; j < sh->n_joins; ++j)
+        if (sh->join_fk_col[j] == col) return true;
+      return false;
+    };
+    HX_REQUIRE(table_has_col(fact, sh->agg_a) &&
+                   (sh->agg_op == HX_AGG_SUM || table_has_col(fact, sh->agg_b)),
+               HX_EINVAL, "hx_pipeline_probe_agg: measure column not in fact table");
+    p.ga = ok && !read_by_stages(sh->agg_a);
+    p.gb = sh->agg_op == HX_AGG_SUM ? p.ga : (ok && !read_by_stages(sh->agg_b));
+    p.gat_a = p.ga ? table_col(fact, sh->agg_a) : nullptr;
+    p.gat_b = p.gb ? table_col(fact, sh->agg_op == HX_AGG_SUM ? sh->agg_a : sh->agg_b) : nullptr;
+  }
+  p.agg_a = p.ga ? 0 : stage_of(sh->agg_a);
+  p.agg_b = sh->agg_op == HX_AGG_SUM ? p.agg_a : (p.gb ? 0 : stage_of(sh->agg_b));
   HX_REQUIRE(p.agg_a >= 0 && p.agg_b >= 0, HX_EINVAL,
              "hx_pipeline_probe_agg: measure column not in fact table (or > 8 columns)");
   HX_REQUIRE(k1_group_bound(sh, hts, n_hts) >= 1, HX_EINVAL, "hx_pipeline_probe_agg: bad gdim_join");
@@ -1128,7 +1256,7 @@ int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht*
   //      membership bitmap (exact) and its Bloom filter; a hash-table join its Bloom filter;
   //   2. the direct maps still read from L2 are then staged in full, smallest first (each
   //      saves one L2 lookup per surviving row), replacing their filter.
-  p.stages = pick_stages(n_cols, p.smem_groups);
+  p.stages = pick_stages(dm_mode, n_cols, p.smem_groups);
   enum { kNone = 0, kFull, kBitmap, kBloom };
   int kind[HX_MAX_JOINS] = {kNone, kNone, kNone, kNone};
   int bloom_w[HX_MAX_JOINS] = {0, 0, 0, 0};
@@ -1150,7 +1278,7 @@ int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht*
   auto fits = [&](int j_new, int k_new) {
     int fw = 0, db = 0;
     for (int j = 0; j < sh->n_joins; ++j) usage(j, j == j_new ? k_new : kind[j], &fw, &db);
-    return k1_smem_bytes(n_cols, p.stages, p.smem_groups, fw, db) <=
+    return k1_smem_bytes(dm_mode, n_cols, p.stages, p.smem_groups, fw, db) <=
            smem_budget(std::min(kCtasPerSm, 2));
   };
   for (int i = 0; i < sh->n_joins; ++i) {
@@ -1212,8 +1340,8 @@ int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht*
     p.m_ins |= (uint32_t)(d.in_s != 0) << j;
   }
   if (std::getenv("HX_DEBUG")) {  // launch plan of this K1 (tuning aid)
-    std::fprintf(stderr, "[hx] K1 joins=%d cols=%d stages=%d groups=%d filters:", sh->n_joins,
-                 n_cols, p.stages, p.smem_groups);
+    std::fprintf(stderr, "[hx] K1 joins=%d cols=%d gather=%d%d stages=%d groups=%d filters:",
+                 sh->n_joins, n_cols, p.ga, p.gb, p.stages, p.smem_groups);
     for (int j = 0; j < sh->n_joins; ++j) std::fprintf(stderr, " %d", p.joins[j].bloom_words);
     std::fprintf(stderr, " dm(words@smem/bitmap@smem):");
     for (int j = 0; j < sh->n_joins; ++j)
@@ -1222,10 +1350,10 @@ int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht*
     std::fprintf(stderr, " in_s:");
     for (int j = 0; j < sh->n_joins; ++j) std::fprintf(stderr, "%d", p.joins[j].in_s);
     std::fprintf(stderr, " smem=%zu\n",
-                 k1_smem_bytes(n_cols, p.stages, p.smem_groups, p.filter_words, p.dm_bytes));
+                 k1_smem_bytes(dm_mode, n_cols, p.stages, p.smem_groups, p.filter_words, p.dm_bytes));
   }
   k.fn = pick_kernel(sh->n_joins, grouped, p.m_dm != 0u);
-  k.smem = k1_smem_bytes(n_cols, p.stages, p.smem_groups, p.filter_words, p.dm_bytes);
+  k.smem = k1_smem_bytes(dm_mode, n_cols, p.stages, p.smem_groups, p.filter_words, p.dm_bytes);
   int occ = 0;
   HX_CK(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, k.fn, kThreads, k.smem));
   occ = std::max(1, occ);
@@ -1340,6 +1468,9 @@ int k1_enqueue(hx_ctx* ctx, const K1Prepared* k, bool fresh, cudaEvent_t e0, cud
 
 void k1_free(K1Prepared* k) { delete k; }
 int64_t k1_bytes(const K1Prepared* k) { return k->rows * 4 * k->n_cols; }
+int k1_gathered_cols(const K1Prepared* k) {
+  return k->p.ga + (k->p.agg_op != HX_AGG_SUM && k->p.gb ? 1 : 0);
+}
 
 int probe_agg(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht* const* hts,
               int n_hts, hx_agg* agg, bool fresh) {
