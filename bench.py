@@ -274,7 +274,10 @@ def main():
         gr_ = None if args.no_graph else hx.capture(ctx, lambda od_=od_: hx.plans_enqueue(ctx, od_))
         sets.append((pl_, od_, gr_))
     plans, order, graph = sets[0]
-    k1_acc = [0.0, 0, 0, 0.0]
+    # SURVEY.md §8(d) algorithmic bytes per lineorder row: the referenced columns (16 B for
+    # Q1-Q3, 24 B for Q4); the bytes K1 actually moves can be fewer (late materialisation)
+    B = {q: 4 * len(ssb.FACT_COLS[q]) for q in queries}
+    k1_acc = [0.0, 0, 0, 0.0, 0]  # ms, launches, moved bytes, span ms, algorithmic bytes
 
     def launch(st):
         if st[2] is not None:
@@ -291,6 +294,7 @@ def main():
                 k1_acc[0] += ms_
                 k1_acc[1] += 1
                 k1_acc[2] += b_
+                k1_acc[4] += n_mine * B[q]
         return out
 
     def run_steps(n, timed=False):
@@ -324,7 +328,7 @@ def main():
         dist.barrier()
     clk = clocks.stop()
     ms = e0.elapsed_time(e1)
-    k1_ms, k1_n, k1_bytes, k1_span = k1_acc
+    k1_ms, k1_n, k1_moved, k1_span, k1_bytes = k1_acc
     launches, step_h2d, step_d2h = ctx.stats(reset=True)
     if world > 1:
         t = torch.tensor([ms, float(launches)], device="cuda", dtype=torch.float64)
@@ -337,11 +341,18 @@ def main():
 
     peak, peak_src = peaks()
     achieved = (k1_bytes / (k1_ms / 1e3)) / 1e9 if k1_ms > 0 else 0.0
+    moved = (k1_moved / (k1_ms / 1e3)) / 1e9 if k1_ms > 0 else 0.0
     tr = ncu_traffic()
     roofline = {"bound": "hbm", "achieved": achieved, "peak": peak, "unit": "GB/s",
                 "frac": achieved / peak, "peak_source": peak_src,
                 "kernel": f"k1_probe_agg (fused scan->filter->probe->aggregate), {len(queries)} queries",
                 "algorithmic_bytes_per_launch": k1_bytes / max(k1_n, 1),
+                "algorithmic_bytes_definition": "SURVEY.md 8(d): 4 B x referenced lineorder columns "
+                                                "(16 B/row Q1-Q3, 24 B/row Q4) x rows",
+                "moved_bytes_per_launch": k1_moved / max(k1_n, 1),
+                "moved_bytes_definition": "streamed columns (4 B/row) + one 32-B sector per "
+                                          "gathered measure value of a row that passed every join",
+                "achieved_moved": moved, "frac_moved": moved / peak,
                 "k1_ms_per_launch": k1_ms / max(k1_n, 1),
                 "k1_busy_frac_of_step": k1_ms / ms if ms > 0 else None,
                 "k1_span_ms_per_step": k1_span / args.steps,
@@ -369,16 +380,17 @@ def main():
 
     # ---- per query (after the timed region): K1-only and whole-query time ---------------
     per_query = {}
-    B = {q: 4 * len(ssb.FACT_COLS[q]) for q in queries}
     for q in queries:
         reps = 5
         qe0, qe1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
-        kms = 0.0
+        kms, kmoved = 0.0, 0
         qe0.record(stream)
         for _ in range(reps):
             plans[q].enqueue()
             plans[q].rows()
-            kms += plans[q].hp.k1_time()[0]
+            ms_, b_ = plans[q].hp.k1_time()
+            kms += ms_
+            kmoved += b_
         qe1.record(stream)
         torch.cuda.synchronize()
         qms = qe0.elapsed_time(qe1) / reps
@@ -387,7 +399,9 @@ def main():
                         "rows_per_s": n_mine / (qms / 1e3),
                         "k1_hbm_gbps": n_mine * B[q] / (kms / 1e3) / 1e9 if kms else None,
                         "k1_frac_of_peak": (n_mine * B[q] / (kms / 1e3) / 1e9) / peak if kms else None,
-                        "bytes_per_row": B[q]}
+                        "bytes_per_row": B[q],
+                        "k1_moved_gbps": kmoved / reps / (kms / 1e3) / 1e9 if kms else None,
+                        "moved_bytes_per_row": kmoved / reps / max(n_mine, 1)}
 
     # ---- e2e through the C-ABI with HOST buffers (H2D + queries + D2H inside the clock) ---
     e2e = None

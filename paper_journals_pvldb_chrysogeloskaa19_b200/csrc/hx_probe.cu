@@ -9,17 +9,21 @@
 // and a GROUP BY (the paper does not describe its group-by; R17).
 //
 // How (B200-first, not the paper's 2019 LLVM-generated sm_61 code):
-//   * persistent CTAs (grid = SMs x resident CTAs), each with one PRODUCER warp that
-//     streams lineorder tiles (T rows x the query's columns) from HBM into a shared-memory
-//     ring with cp.async.bulk (the TMA bulk-copy engine) completing on mbarriers, L2
-//     evict-first; and 8 CONSUMER warps that process a tile while the next S-1 are in
-//     flight (mem-move's "prefetch to the consumer's local memory", done
-//     at tile granularity inside the kernel);
-//   * each consumer thread owns R rows of the tile (strided by 256 -> conflict-free LDS) and
-//     runs the pipeline stage-wise across them: predicates, then for each join the R
-//     hash probes are issued together (R independent L2 loads in flight) before any is
-//     checked; rows die as soon as a predicate or probe fails;
-//   * hash tables are read with L2 evict-last hints so the scan does not evict them;
+//   * persistent CTAs (one per SM), each with one PRODUCER warp that streams lineorder tiles
+//     (2560 rows x the query's streamed columns) from HBM into a shared-memory ring with
+//     cp.async.bulk (the TMA bulk-copy engine) completing on mbarriers, L2 evict-first, and 20
+//     CONSUMER warps that take the tiles two at a time while the next ones are in flight
+//     (mem-move's "prefetch to the consumer's local memory", done at tile
+//     granularity inside the kernel);
+//   * each consumer lane owns 4 consecutive rows of each tile (one 128-bit shared-memory load
+//     per column) and runs the pipeline stage-wise: predicates, the most selective join's
+//     shared-memory structure, compaction of the survivors into a per-warp queue, then the
+//     remaining joins for 32 queued rows at a time (one row per lane, lookups issued
+//     together);
+//   * joins are probed in direct maps (plans over dense keys: rank + 1 per key, exact, staged
+//     in shared memory when they fit) or in open-addressing hash tables with shared-memory
+//     Bloom filters (hx_build.cu); measure columns no stage reads are gathered for the rows
+//     that pass every join instead of being streamed (late materialisation);
 //   * GROUP BY: a dense per-CTA shared-memory table (int64 SUM, int32 COUNT) indexed by the
 //     mixed radix of the probed dimensions' dense ranks, flushed with one global atomic per
 //     non-empty group per CTA; ungrouped queries reduce warp -> CTA -> one global atomic.
@@ -35,7 +39,7 @@ namespace {
 
 constexpr unsigned kFull = 0xFFFFFFFFu;
 #ifndef HX_K1_WARPS
-#define HX_K1_WARPS 16  // consumer warps per CTA (tuned: tools/variants/run.sh)
+#define HX_K1_WARPS 20  // consumer warps per CTA (tuned: 16 -> 20 is -6% K1 time, 24 spills)
 #endif
 #ifndef HX_K1_STAGE_KB
 #define HX_K1_STAGE_KB 160  // max shared memory for the tile ring (the rest: Bloom filters)
@@ -48,7 +52,7 @@ constexpr int kConsumerWarps = HX_K1_WARPS;
 constexpr int kConsumers = kConsumerWarps * 32;
 constexpr int kThreads = kConsumers + 32;  // + one producer warp
 constexpr int kRowsPerThread = 4;          // R
-constexpr int kTileRows = kConsumers * kRowsPerThread;  // T = 1024
+constexpr int kTileRows = kConsumers * kRowsPerThread;  // T = 2560 rows
 constexpr int kCtasPerSm = HX_K1_CTAS;    // target residency (registers, smem budget)
 constexpr int kMaxStageCols = 8;
 constexpr int kSmemGroups = 1024;          // per-CTA group table capacity
@@ -196,15 +200,6 @@ __device__ __forceinline__ long long measure(int op, int32_t a, int32_t b) {
   if (op == HX_AGG_SUM_SUB) return (long long)a - (long long)b;
   return (long long)a;
 }
-// The measure of a passing row: staged operands come with the row, gathered ones are read
-// now (the row passed every join: one sector per gathered value).
-__device__ __forceinline__ long long row_measure(const K1Params& p, int32_t a, int32_t b,
-                                                 uint32_t row) {
-  if (p.ga) a = __ldg(p.gat_a + row);
-  if (p.gb) b = __ldg(p.gat_b + row);
-  return measure(p.agg_op, a, b);
-}
-
 // Per-warp view of one join's hash table (loaded once per CTA).
 struct JoinState {
   const ulonglong2* buckets;  // 16-byte buckets of two {key, rank} slots
@@ -318,6 +313,12 @@ struct CarryEntry {
   int32_t a, b, g;
   uint32_t row;  // fact row (gathered measures)
 };
+// A stage-C row that passed, whose accumulation is deferred by one batch so that its gathered
+// measure operands (issued loads) arrive while the next batch runs (latency hiding).
+struct Pending {
+  int32_t g, a, b;
+  bool alive;
+};
 // Per-warp buffer of the (< 32) queued rows carried to the next tile (SoA, one slot per lane).
 struct CarryBuf {
   int32_t key[HX_MAX_JOINS][32];
@@ -365,7 +366,7 @@ __device__ __forceinline__ void stage_c_row(const K1Params& p, const JoinState (
                                             const unsigned char* sdm, const CarryEntry& e,
                                             int j0, int jf, bool smem_table,
                                             unsigned long long* s_sum, uint32_t* s_cnt,
-                                            long long& acc_sum, long long& acc_cnt) {
+                                            long long& acc_sum, long long& acc_cnt, Pending& pd) {
   // (direct maps: the group index is computed here from scratch; stage S only filtered)
   int32_t gg = DM ? group_origin<NJ, GROUPED, DM>(js) : e.g;
   bool alive = true;
@@ -446,9 +447,15 @@ __device__ __forceinline__ void stage_c_row(const K1Params& p, const JoinState (
     }
     if (!alive) pend = 0;
   }
-  if (alive)
-    accumulate<GROUPED>(p, smem_table, s_sum, s_cnt, gg, row_measure(p, e.a, e.b, e.row), acc_sum,
+  Pending cur{gg, e.a, e.b, alive};
+  if (alive) {  // issue the gathers now, consume them one batch later
+    if (p.ga) cur.a = __ldg(p.gat_a + e.row);
+    if (p.gb) cur.b = __ldg(p.gat_b + e.row);
+  }
+  if (pd.alive)
+    accumulate<GROUPED>(p, smem_table, s_sum, s_cnt, pd.g, measure(p.agg_op, pd.a, pd.b), acc_sum,
                         acc_cnt);
+  pd = cur;
 }
 
 // Process a PAIR of staged tiles (two consecutive tiles of this CTA, so the per-iteration
@@ -478,7 +485,7 @@ __device__ __forceinline__ void process_tile(const K1Params& p, const JoinState 
                                              unsigned long long* s_sum, uint32_t* s_cnt,
                                              uint8_t* q_row, int32_t* q_g, CarryBuf* cb,
                                              int& n_carry, long long& acc_sum,
-                                             long long& acc_cnt) {
+                                             long long& acc_cnt, Pending& pd) {
   constexpr int R = kRowsPerThread;  // rows per lane per tile
   const int wbase = warp * (32 * R);
   const int r0 = wbase + lane * R;
@@ -610,11 +617,20 @@ __device__ __forceinline__ void process_tile(const K1Params& p, const JoinState 
     int32_t a8[2 * R] = {}, b8[2 * R] = {};
     if (!p.ga) load8(p.agg_a, a8);
     if (!p.gb) load8(p.agg_b, b8);
+    if (p.ga | p.gb) {  // gathers of every passing row first (all in flight together)
+#pragma unroll
+      for (int k = 0; k < 2 * R; ++k) {
+        const uint32_t row = (k < R ? frow0 : frow1) + r0 + (k & 3);
+        if ((m >> k) & 1u) {
+          if (p.ga) a8[k] = __ldg(p.gat_a + row);
+          if (p.gb) b8[k] = __ldg(p.gat_b + row);
+        }
+      }
+    }
 #pragma unroll
     for (int k = 0; k < 2 * R; ++k)
       if ((m >> k) & 1u)
-        accumulate<GROUPED>(p, smem_table, s_sum, s_cnt, g[k],
-                            row_measure(p, a8[k], b8[k], (k < R ? frow0 : frow1) + r0 + (k & 3)),
+        accumulate<GROUPED>(p, smem_table, s_sum, s_cnt, g[k], measure(p.agg_op, a8[k], b8[k]),
                             acc_sum, acc_cnt);
     return;
   }
@@ -655,7 +671,7 @@ __device__ __forceinline__ void process_tile(const K1Params& p, const JoinState 
   for (int base = 0; base < full_end; base += 32) {
     CarryEntry e = load_entry<NJ, DM>(p, js, cb, n_carry, q_row, q_g, carry_g, wcol0, wcol1,
                                       wrow0, wrow1, stride, base + lane);
-    stage_c_row<NJ, GROUPED, DM>(p, js, sdm, e, j0, jf, smem_table, s_sum, s_cnt, acc_sum, acc_cnt);
+    stage_c_row<NJ, GROUPED, DM>(p, js, sdm, e, j0, jf, smem_table, s_sum, s_cnt, acc_sum, acc_cnt, pd);
   }
   {
     const int idx = full_end + lane;
@@ -685,7 +701,7 @@ __device__ __forceinline__ void drain_carry(const K1Params& p, const JoinState (
                                             int n_carry, int lane, int j0,
                                             int jf, bool smem_table, unsigned long long* s_sum,
                                             uint32_t* s_cnt, long long& acc_sum,
-                                            long long& acc_cnt) {
+                                            long long& acc_cnt, Pending& pd) {
   if (lane >= n_carry) return;
   CarryEntry e;
 #pragma unroll
@@ -694,7 +710,7 @@ __device__ __forceinline__ void drain_carry(const K1Params& p, const JoinState (
   e.b = cb->b[lane];
   e.row = cb->row[lane];
   e.g = cb->g[lane];
-  stage_c_row<NJ, GROUPED, DM>(p, js, sdm, e, j0, jf, smem_table, s_sum, s_cnt, acc_sum, acc_cnt);
+  stage_c_row<NJ, GROUPED, DM>(p, js, sdm, e, j0, jf, smem_table, s_sum, s_cnt, acc_sum, acc_cnt, pd);
 }
 
 __device__ __forceinline__ void mbar_wait_sleep(uint64_t* bar, uint32_t parity) {
@@ -798,7 +814,10 @@ __global__ void __launch_bounds__(kThreads, kCtasPerSm) k1_probe_agg(const __gri
       js[j] = JoinState{nullptr, 0, 32, 0u, 0, nullptr, 0};
     }
   }
-  // stage the Bloom filters that fit their reservation into shared memory (once per CTA)
+  // stage the Bloom filters into their shared-memory reservations (once per CTA). A filter
+  // larger than its reservation (a power of two) is folded: the word index is the top bits of
+  // the hash, so OR-ing each run of F adjacent words gives the same filter with F times fewer
+  // words (more false positives, never a false negative).
   {
     uint32_t* dst = s_filters;
 #pragma unroll
@@ -806,16 +825,25 @@ __global__ void __launch_bounds__(kThreads, kCtasPerSm) k1_probe_agg(const __gri
       const int reserved = p.joins[j].bloom_words;
       if (reserved == 0) continue;
       const int lw = p.joins[j].hdr->bloom_log2w;
+      const uint32_t* src = p.joins[j].bloom;
       if ((1 << lw) <= reserved) {
-        const uint4* src = reinterpret_cast<const uint4*>(p.joins[j].bloom);
         if (lw >= 2) {
           for (int i = ctid; i < (1 << lw) / 4; i += kConsumers)
-            reinterpret_cast<uint4*>(dst)[i] = __ldg(src + i);
+            reinterpret_cast<uint4*>(dst)[i] = __ldg(reinterpret_cast<const uint4*>(src) + i);
         } else if (ctid < 2) {  // 1-2 words: replicate to two so that blw >= 1
-          dst[ctid] = __ldg(p.joins[j].bloom + (lw == 0 ? 0 : ctid));
+          dst[ctid] = __ldg(src + (lw == 0 ? 0 : ctid));
         }
         js[j].sbloom = dst;
         js[j].blw = lw == 0 ? 1 : lw;
+      } else {
+        const int fold = (1 << lw) / reserved;
+        for (int i = ctid; i < reserved; i += kConsumers) {
+          uint32_t w = 0;
+          for (int f = 0; f < fold; ++f) w |= __ldg(src + i * fold + f);
+          dst[i] = w;
+        }
+        js[j].sbloom = dst;
+        js[j].blw = 31 - __clz(reserved);
       }
       dst += reserved;
     }
@@ -846,6 +874,7 @@ __global__ void __launch_bounds__(kThreads, kCtasPerSm) k1_probe_agg(const __gri
     }
   }
   long long acc_sum = 0, acc_cnt = 0;
+  Pending pd{0, 0, 0, false};
   // misaligned head rows (views at a row offset): CTA 0 reads them directly
   if (blockIdx.x == 0 && p.head_rows > 0) {
     if (ctid < p.head_rows)
@@ -853,7 +882,7 @@ __global__ void __launch_bounds__(kThreads, kCtasPerSm) k1_probe_agg(const __gri
     consumer_sync();
     process_tile<NJ, GROUPED, DM>(p, js, sdm, headbuf, headbuf, 0u, 0u, 4, p.head_rows, 0, warp, lane,
                                   smem_table, s_sum, s_cnt, q_row, q_g, cb, n_carry, acc_sum,
-                                  acc_cnt);
+                                  acc_cnt, pd);
   }
   consumer_sync();
 
@@ -896,7 +925,7 @@ __global__ void __launch_bounds__(kThreads, kCtasPerSm) k1_probe_agg(const __gri
     const uint32_t frow1 = (uint32_t)(p.head_rows + t1 * kTileRows);
     process_tile<NJ, GROUPED, DM>(p, js, sdm, st0, st1, frow0, frow1, kTileRows, rows0, rows1, warp, lane,
                                   smem_table, s_sum, s_cnt, q_row, q_g, cb, n_carry, acc_sum,
-                                  acc_cnt);
+                                  acc_cnt, pd);
     __syncwarp();
     if (lane == 0) {
       mbar_arrive(empty + s);
@@ -918,7 +947,11 @@ __global__ void __launch_bounds__(kThreads, kCtasPerSm) k1_probe_agg(const __gri
   // the rows this warp still carries
   if (NJ > 0)
     drain_carry<NJ, GROUPED, DM>(p, js, sdm, cb, n_carry, lane, first_join_in_place<NJ, DM>(p, js),
-                             first_filter<NJ, DM>(js), smem_table, s_sum, s_cnt, acc_sum, acc_cnt);
+                             first_filter<NJ, DM>(js), smem_table, s_sum, s_cnt, acc_sum, acc_cnt,
+                             pd);
+  if (pd.alive)  // the last deferred row
+    accumulate<GROUPED>(p, smem_table, s_sum, s_cnt, pd.g, measure(p.agg_op, pd.a, pd.b), acc_sum,
+                        acc_cnt);
   __syncwarp();
 
   // ---------------- flush the CTA's partial aggregate ----------------
@@ -1285,15 +1318,25 @@ int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht*
     const int j = ord[i];
     const JoinDev& d = p.joins[j];
     if (!bloom_w[j] || 2 * pass[j] > 1.0) continue;
-    if (!d.dm) {
-      if (fits(j, kBloom)) kind[j] = kBloom;
-      continue;
+    if (d.dm) {
+      const int full = d.dm_words * 4, bm = d.bm_words * 4, bl = bloom_w[j] * 4;
+      const int cand[3] = {full <= 2 * std::min(bm, bl) ? (int)kFull : (int)kNone,
+                           bm <= bl ? (int)kBitmap : (int)kBloom,
+                           bm <= bl ? (int)kBloom : (int)kBitmap};
+      for (int c : cand)
+        if (c != kNone && kind[j] == kNone && fits(j, c)) kind[j] = c;
+    } else if (fits(j, kBloom)) {
+      kind[j] = kBloom;
     }
-    const int full = d.dm_words * 4, bm = d.bm_words * 4, bl = bloom_w[j] * 4;
-    const int cand[3] = {full <= 2 * std::min(bm, bl) ? (int)kFull : (int)kNone,
-                         bm <= bl ? (int)kBitmap : (int)kBloom, bm <= bl ? (int)kBloom : (int)kBitmap};
-    for (int c : cand)
-      if (c != kNone && kind[j] == kNone && fits(j, c)) kind[j] = c;
+    // no room at full size: a folded Bloom filter (4 or 2 bits per key) still drops most rows
+    for (int f = 2; f <= 4 && kind[j] == kNone && bloom_w[j] / f >= 4; f *= 2) {
+      const int w0 = bloom_w[j];
+      bloom_w[j] = w0 / f;
+      if (fits(j, kBloom))
+        kind[j] = kBloom;
+      else
+        bloom_w[j] = w0;
+    }
   }
   int dms[HX_MAX_JOINS], n_dms = 0;
   for (int j = 0; j < sh->n_joins; ++j)
