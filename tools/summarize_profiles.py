@@ -40,7 +40,7 @@ def main(tag, rep, launches):
                    f"{float(d[c('sm__warps_active.avg.pct_of_peak_sustained_active')]):.1f} | "
                    f"{d[c('launch__registers_per_thread')]} |")
     out += ["", f"Sum over the 13 launches: {tt:.0f} us; algorithmic {ta/1e9:.2f} GB; DRAM {tr/1e9:.2f} GB "
-                f"(traffic/algorithmic {tr/ta:.3f}: no re-reads)."]
+                f"(traffic/algorithmic {tr/ta:.3f}; below 1 where late materialisation gathers measure columns for passing rows only)."]
     with open(os.path.join(ROOT, "profiles", f"{tag}_k1_ncu_summary.md"), "w") as f:
         f.write("\n".join(out) + "\n")
     with open(os.path.join(ROOT, "profiles", "k1_traffic.json"), "w") as f:
