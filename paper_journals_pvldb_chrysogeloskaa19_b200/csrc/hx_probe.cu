@@ -28,6 +28,7 @@
 //     mixed radix of the probed dimensions' dense ranks, flushed with one global atomic per
 //     non-empty group per CTA; ungrouped queries reduce warp -> CTA -> one global atomic.
 #include <algorithm>
+#include <cmath>
 #include <cstdio>
 #include <cstdlib>
 
@@ -116,6 +117,8 @@ struct K1Params {
   uint32_t m_dmsm;                         // its full map is staged in shared memory
   uint32_t m_bm;                           // its bitmap is staged in shared memory
   uint32_t m_ins;                          // its shared-memory structure runs in stage S
+  uint32_t m_l2;                           // stage C reads its map from L2 (rank, or no
+                                           // exact shared-memory verdict)
 };
 
 // join kinds (uniform per launch: read from the kernel parameters)
@@ -129,7 +132,7 @@ __device__ __forceinline__ bool resolved_in_s(const K1Params& p, int jx) {
 }
 template <bool DM>
 __device__ __forceinline__ bool dm_l2(const K1Params& p, int jx) {
-  return DM && !jbit(p.m_dmsm, jx);
+  return DM && jbit(p.m_l2, jx);
 }
 // Direct-map entry (rank + 1, or 0) of a key from the map's 32-bit word array
 __device__ __forceinline__ uint32_t dm_bit(const JoinDev& d, int32_t key) {
@@ -1070,6 +1073,128 @@ int pick_stages(bool dm, int n_cols, int smem_groups) {
   return std::max(2, std::min(4, s));
 }
 
+enum { kStNone = 0, kStFull, kStBitmap, kStBloom };
+
+// False-positive rate of the blocked Bloom filter (one 32-bit word per key, two bits set) at
+// `bits_per_key`: the keys per word are Poisson(32 / bits_per_key); a key of a word holding
+// n keys passes when both its bits are among the word's set bits.
+double bloom_fp(double bits_per_key) {
+  if (bits_per_key <= 0.0) return 1.0;
+  const double lam = 32.0 / bits_per_key;
+  double fp = 0.0, pn = std::exp(-lam);
+  for (int n = 0; n < 256; ++n) {
+    const double q = 1.0 - std::pow(31.0 / 32.0, 2.0 * n);
+    fp += pn * q * q;
+    pn *= lam / (n + 1);
+  }
+  return std::min(1.0, fp);
+}
+
+// Relative per-row costs (issue slots) of the K1 stages, measured on SF10 SSB: a stage-S
+// filter on every row, a row entering stage C (compaction, queue, batch), a stage-C
+// shared-memory filter, an L2 lookup. HX_K1_COST="s,c,sc,l2" overrides (tuning aid).
+struct K1Cost {
+  double s = 8.0, c = 60.0, sc = 8.0, l2 = 20.0;
+};
+K1Cost k1_cost() {
+  K1Cost k;
+  if (const char* e = std::getenv("HX_K1_COST"))
+    std::sscanf(e, "%lf,%lf,%lf,%lf", &k.s, &k.c, &k.sc, &k.l2);
+  return k;
+}
+
+// Shared-memory plan of a direct-map pipeline: for every combination of per-join structures
+// that fits next to the tile ring (none; the full map: exact + rank; the membership bitmap:
+// exact; the Bloom filter at 8, 4, 2 or 1 bits per key) and every choice of the joins whose
+// structure runs on EVERY row in stage S (the rest run on the compacted survivors in stage
+// C), the expected cost per lineorder row is
+//     s * |S| + c * f_S + sc * (structures read in stage C) * f_S + l2 * (L2 maps) * f_C
+// with f_S = the fraction of rows passing stage S (pass fraction + false positives) and f_C
+// the fraction still alive when the L2 lookups are issued; a pipeline whose joins are all
+// full maps in stage S aggregates in place (no stage C). The cheapest plan is taken.
+template <class Fits>
+double plan_dm(int nj, const JoinDev* joins, const bool* known, const double* pass,
+               const int64_t* keys, const int* bloom_w0, const bool* grouped, Fits fits,
+               int* kind, int* bloom_w, int* in_s) {
+  struct Opt {
+    int kind, bw;
+    double e;
+    bool exact;
+  };
+  Opt opts[HX_MAX_JOINS][8];
+  int n_opt[HX_MAX_JOINS];
+  for (int j = 0; j < nj; ++j) {
+    const JoinDev& d = joins[j];
+    const double pj = known[j] ? pass[j] : 1.0;
+    int n = 0;
+    opts[j][n++] = {kStNone, 0, 1.0, false};
+    opts[j][n++] = {kStFull, 0, pj, true};
+    if (d.dm_lw > 0) opts[j][n++] = {kStBitmap, 0, pj, true};
+    if (known[j] && keys[j] > 0)
+      for (int f = 1; f <= 8 && bloom_w0[j] / f >= 4; f *= 2) {
+        const int bw = bloom_w0[j] / f;
+        const double e = pj + (1.0 - pj) * bloom_fp(32.0 * bw / (double)keys[j]);
+        opts[j][n++] = {kStBloom, bw, e, false};
+      }
+    n_opt[j] = n;
+  }
+  const K1Cost K = k1_cost();
+  double best = 1e300;
+  int idx[HX_MAX_JOINS] = {0, 0, 0, 0};
+  int kd[HX_MAX_JOINS], bw[HX_MAX_JOINS];
+  while (true) {
+    for (int j = 0; j < nj; ++j) {
+      kd[j] = opts[j][idx[j]].kind;
+      bw[j] = opts[j][idx[j]].bw;
+    }
+    if (fits(kd, bw)) {
+      uint32_t has = 0;
+      for (int j = 0; j < nj; ++j) has |= (uint32_t)(kd[j] != kStNone) << j;
+      // every subset of the joins that have a structure may run in stage S
+      for (uint32_t S = has;; S = (S - 1) & has) {
+        double fS = 1.0, cost = 0.0;
+        bool all_res = true;
+        for (int j = 0; j < nj; ++j) {
+          if ((S >> j) & 1u) {
+            fS *= opts[j][idx[j]].e;
+            cost += K.s;
+          }
+          all_res = all_res && ((S >> j) & 1u) && kd[j] == kStFull;
+        }
+        if (!all_res) {
+          cost += K.c * fS;
+          double fC = fS;
+          int n_l2 = 0;
+          for (int j = 0; j < nj; ++j) {
+            const bool inS = (S >> j) & 1u;
+            if (!inS && kd[j] != kStNone) {
+              cost += K.sc * fS;
+              fC *= opts[j][idx[j]].e;
+            }
+            if (inS && kd[j] == kStFull && grouped[j]) cost += K.sc * fS;  // rank re-read
+            const bool full = kd[j] == kStFull;
+            n_l2 += !full && (grouped[j] || !opts[j][idx[j]].exact);
+          }
+          cost += K.l2 * n_l2 * fC;
+        }
+        if (cost < best - 1e-12) {
+          best = cost;
+          for (int j = 0; j < nj; ++j) {
+            kind[j] = kd[j];
+            bloom_w[j] = bw[j];
+            in_s[j] = (S >> j) & 1u;
+          }
+        }
+        if (S == 0) break;
+      }
+    }
+    int j = 0;
+    while (j < nj && ++idx[j] == n_opt[j]) idx[j++] = 0;
+    if (j == nj) break;
+  }
+  return best;
+}
+
 }  // namespace
 
 int k1_occupancy(hx_ctx* ctx) {
@@ -1281,70 +1406,60 @@ int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht*
   const bool grouped = sh->n_gdims > 0;
   p.smem_groups = grouped ? (int32_t)std::min<long long>(kSmemGroups, agg->cap_groups) : 0;
   // Shared-memory plan. The tile ring keeps pick_stages' depth (measured: shrinking it to fit
-  // more filters lost 6% at SF100); the rest of the CTA's shared memory is given out in two
-  // passes over the joins whose passing key count a plan observed:
-  //   1. selective joins (at most half the dimension passes), most selective first, get a
-  //      filter that runs on every row: a direct-map join its full map (exact, also resolves
-  //      the rank) if that is at most twice its smallest filter, else the smaller of its
-  //      membership bitmap (exact) and its Bloom filter; a hash-table join its Bloom filter;
-  //   2. the direct maps still read from L2 are then staged in full, smallest first (each
-  //      saves one L2 lookup per surviving row), replacing their filter.
+  // more filters lost 6% at SF100); the rest of the CTA's shared memory holds per-join
+  // structures: hash-table pipelines get Bloom filters greedily (plan_ht below); direct-map
+  // pipelines are planned by a cost model over every combination (plan_dm).
   p.stages = pick_stages(dm_mode, n_cols, p.smem_groups);
-  enum { kNone = 0, kFull, kBitmap, kBloom };
-  int kind[HX_MAX_JOINS] = {kNone, kNone, kNone, kNone};
+  int kind[HX_MAX_JOINS] = {kStNone, kStNone, kStNone, kStNone};
   int bloom_w[HX_MAX_JOINS] = {0, 0, 0, 0};
+  int in_s[HX_MAX_JOINS] = {0, 0, 0, 0};
   double pass[HX_MAX_JOINS] = {1, 1, 1, 1};
-  int ord[HX_MAX_JOINS] = {0, 1, 2, 3};
+  bool known[HX_MAX_JOINS] = {false, false, false, false};
+  int bloom_w0[HX_MAX_JOINS] = {0, 0, 0, 0};
+  int64_t keys[HX_MAX_JOINS] = {0, 0, 0, 0};
   for (int j = 0; j < sh->n_joins; ++j) {
     const hx_ht* ht = hts[sh->join_ht[j]];
     if (ht->known_keys < 0) continue;
+    known[j] = true;
+    keys[j] = ht->known_keys;
     pass[j] = (double)ht->known_keys / (double)std::max<int64_t>(1, ht->dim_rows);
-    bloom_w[j] = std::max(4, 1 << std::min(ht->max_bloom_log2w, bloom_log2w_for(ht->known_keys)));
+    bloom_w0[j] = std::max(4, 1 << std::min(ht->max_bloom_log2w, bloom_log2w_for(ht->known_keys)));
   }
-  std::stable_sort(ord, ord + sh->n_joins, [&](int x, int y) { return pass[x] < pass[y]; });
-  auto usage = [&](int j, int k, int* fw, int* db) {
-    const JoinDev& d = p.joins[j];
-    if (k == kFull) *db += d.dm_words * 4;
-    if (k == kBitmap) *db += d.bm_words * 4;
-    if (k == kBloom) *fw += bloom_w[j];
-  };
-  auto fits = [&](int j_new, int k_new) {
+  auto fits_sizes = [&](const int* kd, const int* bw) {
     int fw = 0, db = 0;
-    for (int j = 0; j < sh->n_joins; ++j) usage(j, j == j_new ? k_new : kind[j], &fw, &db);
+    for (int j = 0; j < sh->n_joins; ++j) {
+      const JoinDev& d = p.joins[j];
+      if (kd[j] == kStFull) db += d.dm_words * 4;
+      if (kd[j] == kStBitmap) db += d.bm_words * 4;
+      if (kd[j] == kStBloom) fw += bw[j];
+    }
     return k1_smem_bytes(dm_mode, n_cols, p.stages, p.smem_groups, fw, db) <=
            smem_budget(std::min(kCtasPerSm, 2));
   };
-  for (int i = 0; i < sh->n_joins; ++i) {
-    const int j = ord[i];
-    const JoinDev& d = p.joins[j];
-    if (!bloom_w[j] || 2 * pass[j] > 1.0) continue;
-    if (d.dm) {
-      const int full = d.dm_words * 4, bm = d.bm_words * 4, bl = bloom_w[j] * 4;
-      const int cand[3] = {full <= 2 * std::min(bm, bl) ? (int)kFull : (int)kNone,
-                           bm <= bl ? (int)kBitmap : (int)kBloom,
-                           bm <= bl ? (int)kBloom : (int)kBitmap};
-      for (int c : cand)
-        if (c != kNone && kind[j] == kNone && fits(j, c)) kind[j] = c;
-    } else if (fits(j, kBloom)) {
-      kind[j] = kBloom;
-    }
-    // no room at full size: a folded Bloom filter (4 or 2 bits per key) still drops most rows
-    for (int f = 2; f <= 4 && kind[j] == kNone && bloom_w[j] / f >= 4; f *= 2) {
-      const int w0 = bloom_w[j];
-      bloom_w[j] = w0 / f;
-      if (fits(j, kBloom))
-        kind[j] = kBloom;
-      else
-        bloom_w[j] = w0;
+  double plan_cost = -1.0;
+  if (dm_mode) {
+    bool grouped_j[HX_MAX_JOINS] = {false, false, false, false};
+    for (int g = 0; g < sh->n_gdims; ++g) grouped_j[sh->gdim_join[g]] = true;
+    plan_cost = plan_dm(sh->n_joins, p.joins, known, pass, keys, bloom_w0, grouped_j, fits_sizes,
+                        kind, bloom_w, in_s);
+  } else {
+    // hash tables: selective joins (at most half the dimension passes), most selective first,
+    // get a Bloom filter (folded to 4 or 2 bits per key when the full one does not fit)
+    int ord[HX_MAX_JOINS] = {0, 1, 2, 3};
+    std::stable_sort(ord, ord + sh->n_joins, [&](int x, int y) { return pass[x] < pass[y]; });
+    for (int i = 0; i < sh->n_joins; ++i) {
+      const int j = ord[i];
+      if (!known[j] || 2 * pass[j] > 1.0) continue;
+      for (int f = 1; f <= 4 && kind[j] == kStNone && bloom_w0[j] / f >= 4; f *= 2) {
+        kind[j] = kStBloom;
+        bloom_w[j] = bloom_w0[j] / f;
+        if (!fits_sizes(kind, bloom_w)) {
+          kind[j] = kStNone;
+          bloom_w[j] = 0;
+        }
+      }
     }
   }
-  int dms[HX_MAX_JOINS], n_dms = 0;
-  for (int j = 0; j < sh->n_joins; ++j)
-    if (p.joins[j].dm && kind[j] != kFull) dms[n_dms++] = j;
-  std::stable_sort(dms, dms + n_dms,
-                   [&](int x, int y) { return p.joins[x].dm_words < p.joins[y].dm_words; });
-  for (int i = 0; i < n_dms; ++i)
-    if (fits(dms[i], kFull)) kind[dms[i]] = kFull;
   // offsets: Bloom filters in the filter region, maps and bitmaps in the direct-map region
   p.filter_words = 0;
   p.dm_bytes = 0;
@@ -1353,34 +1468,33 @@ int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht*
     d.bloom_words = 0;
     d.dm_smem = -1;
     d.bm_smem = -1;
-    if (kind[j] == kBloom) {
+    if (kind[j] == kStBloom) {
       d.bloom_words = bloom_w[j];
       p.filter_words += bloom_w[j];
-    } else if (kind[j] == kFull) {
+    } else if (kind[j] == kStFull) {
       d.dm_smem = p.dm_bytes;
       p.dm_bytes += d.dm_words * 4;
-    } else if (kind[j] == kBitmap) {
+    } else if (kind[j] == kStBitmap) {
       d.bm_smem = p.dm_bytes;
       p.dm_bytes += d.bm_words * 4;
     }
-    d.in_s = 0;
+    d.in_s = in_s[j];
   }
-  // stage S (every row): the structure of the most selective direct-map join; the others run
-  // in stage C on the compacted survivors only
-  for (int i = 0; i < sh->n_joins; ++i) {
-    const int j = ord[i];
-    if (p.joins[j].dm && kind[j] != kNone && 2 * pass[j] <= 1.0) {
-      p.joins[j].in_s = 1;
-      break;
+  p.m_dm = p.m_dmsm = p.m_bm = p.m_ins = p.m_l2 = 0u;
+  {
+    bool grouped_j[HX_MAX_JOINS] = {false, false, false, false};
+    for (int g = 0; g < sh->n_gdims; ++g) grouped_j[sh->gdim_join[g]] = true;
+    for (int j = 0; j < sh->n_joins; ++j) {
+      const JoinDev& d = p.joins[j];
+      const bool dm = d.dm != nullptr, full = dm && d.dm_smem >= 0, bm = dm && d.bm_smem >= 0;
+      p.m_dm |= (uint32_t)dm << j;
+      p.m_dmsm |= (uint32_t)full << j;
+      p.m_bm |= (uint32_t)bm << j;
+      p.m_ins |= (uint32_t)(d.in_s != 0) << j;
+      // the L2 map: for the rank of a grouping join, or for the verdict when no exact
+      // structure is staged (none, or a Bloom filter)
+      p.m_l2 |= (uint32_t)(dm && !full && (grouped_j[j] || !bm)) << j;
     }
-  }
-  p.m_dm = p.m_dmsm = p.m_bm = p.m_ins = 0u;
-  for (int j = 0; j < sh->n_joins; ++j) {
-    const JoinDev& d = p.joins[j];
-    p.m_dm |= (uint32_t)(d.dm != nullptr) << j;
-    p.m_dmsm |= (uint32_t)(d.dm != nullptr && d.dm_smem >= 0) << j;
-    p.m_bm |= (uint32_t)(d.dm != nullptr && d.bm_smem >= 0) << j;
-    p.m_ins |= (uint32_t)(d.in_s != 0) << j;
   }
   if (std::getenv("HX_DEBUG")) {  // launch plan of this K1 (tuning aid)
     std::fprintf(stderr, "[hx] K1 joins=%d cols=%d gather=%d%d stages=%d groups=%d filters:",
@@ -1392,7 +1506,7 @@ int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht*
                    p.joins[j].dm_smem, p.joins[j].bm_words, p.joins[j].bm_smem);
     std::fprintf(stderr, " in_s:");
     for (int j = 0; j < sh->n_joins; ++j) std::fprintf(stderr, "%d", p.joins[j].in_s);
-    std::fprintf(stderr, " smem=%zu\n",
+    std::fprintf(stderr, " l2:%x cost=%.2f smem=%zu\n", p.m_l2, plan_cost,
                  k1_smem_bytes(dm_mode, n_cols, p.stages, p.smem_groups, p.filter_words, p.dm_bytes));
   }
   k.fn = pick_kernel(sh->n_joins, grouped, p.m_dm != 0u);
