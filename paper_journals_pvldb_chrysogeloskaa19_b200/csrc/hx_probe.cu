@@ -91,7 +91,10 @@ struct JoinDev {
 struct K1Params {
   const int32_t* col[kMaxStageCols];       // staged fact columns (table base + head offset)
   int32_t n_cols;
-  int32_t stages;
+  int32_t stages;                          // tile ring depth (4..8)
+  int32_t prefetch;                        // L2 prefetch distance in tiles of this CTA (0: off)
+  int32_t smem_fixed;                      // bytes before the group table (no per-warp queues
+                                           // when every join resolves in stage S)
   int64_t n_rows;                          // rows after the head
   int64_t n_tiles;
   const int32_t* head_col[kMaxStageCols];  // misaligned head rows (read directly)
@@ -188,6 +191,10 @@ __device__ __forceinline__ void bulk_g2s(void* dst, const void* src, uint32_t by
       " [%0], [%1], %2, [%3], %4;" ::"r"(smem_u32(dst)),
       "l"(src), "r"(bytes), "r"(smem_u32(bar)), "l"(pol)
       : "memory");
+}
+// Prefetch `bytes` (multiple of 16) of global memory into L2 (bulk engine; no completion).
+__device__ __forceinline__ void bulk_prefetch_l2(const void* src, uint32_t bytes) {
+  asm volatile("cp.async.bulk.prefetch.L2.global [%0], %1;" ::"l"(src), "r"(bytes) : "memory");
 }
 __device__ __forceinline__ unsigned long long ld_slot(const unsigned long long* p, uint64_t pol) {
   unsigned long long v;
@@ -740,7 +747,7 @@ __global__ void __launch_bounds__(kThreads, kCtasPerSm) k1_probe_agg(const __gri
   uint64_t* empty = full + p.stages;
   long long* red = reinterpret_cast<long long*>(smem + 128);                // 2 x 8 warps
   int32_t* headbuf = reinterpret_cast<int32_t*>(smem + 128 + 256);           // 8 cols x 4
-  constexpr int kSmemFixed = smem_fixed(DM);
+  const int kSmemFixed = p.smem_fixed;
   uint8_t* q_rows = smem + kSmemQueueOff;
   int32_t* q_gs = DM ? nullptr
                      : reinterpret_cast<int32_t*>(smem + kSmemQueueOff + kConsumerWarps * kQueueRows);
@@ -780,6 +787,17 @@ __global__ void __launch_bounds__(kThreads, kCtasPerSm) k1_probe_agg(const __gri
         const int64_t rows = std::min<int64_t>(kTileRows, p.n_rows - r0);
         const uint32_t bytes = (uint32_t)(rows & ~int64_t(3)) * 4u;
         mbar_arrive_expect_tx(full + s, bytes * p.n_cols);
+        // L2 prefetch of the tile `prefetch` ring refills ahead: its bulk copy then hits L2,
+        // so the ring's bytes in flight are not bounded by its free slots alone
+        if (p.prefetch) {
+          const int64_t tp = t + (int64_t)p.prefetch * gridDim.x;
+          if (tp < p.n_tiles) {
+            const int64_t rp = tp * kTileRows;
+            const uint32_t pb = (uint32_t)(std::min<int64_t>(kTileRows, p.n_rows - rp) & ~int64_t(3)) * 4u;
+            if (pb)
+              for (int c = 0; c < p.n_cols; ++c) bulk_prefetch_l2(p.col[c] + rp, pb);
+          }
+        }
         if (bytes) {
           int32_t* dst = stage0 + (size_t)s * stage_elems;
           for (int c = 0; c < p.n_cols; ++c)
@@ -1053,10 +1071,10 @@ KernelFn pick_kernel(int nj, bool grouped, bool dm) {
 }
 
 size_t k1_smem_bytes(bool dm, int n_cols, int stages, int smem_groups, int filter_words = 0,
-                     int dm_bytes = 0) {
+                     int dm_bytes = 0, bool in_place = false) {
   const size_t table_bytes = ((size_t)smem_groups * 12 + 127) & ~size_t(127);
   const size_t filter_bytes = ((size_t)filter_words * 4 + 127) & ~size_t(127);
-  return smem_fixed(dm) + table_bytes + filter_bytes + (size_t)dm_bytes +
+  return (in_place ? kSmemQueueOff : smem_fixed(dm)) + table_bytes + filter_bytes + (size_t)dm_bytes +
          (size_t)stages * n_cols * kTileRows * sizeof(int32_t);
 }
 
@@ -1496,6 +1514,25 @@ int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht*
       p.m_l2 |= (uint32_t)(dm && !full && (grouped_j[j] || !bm)) << j;
     }
   }
+  // a pipeline whose joins all resolve in stage S aggregates in place: no per-warp queues or
+  // carry buffers. Shared memory the plan left over deepens the tile ring (up to 8 stages:
+  // more bytes in flight per SM while the consumers hold a pair of tiles).
+  const bool in_place = sh->n_joins == 0 ||
+                        (dm_mode && (p.m_dmsm & p.m_ins) == (1u << sh->n_joins) - 1u);
+  p.smem_fixed = in_place ? kSmemQueueOff : smem_fixed(dm_mode);
+  {
+    int max_stages = 8;
+    if (const char* e = std::getenv("HX_K1_MAX_STAGES")) max_stages = std::max(2, std::min(8, std::atoi(e)));
+    while (p.stages < max_stages &&
+           k1_smem_bytes(dm_mode, n_cols, p.stages + 1, p.smem_groups, p.filter_words, p.dm_bytes,
+                         in_place) <= smem_budget(std::min(kCtasPerSm, 2)))
+      ++p.stages;
+  }
+  // (measured, SF10: a distance of 2 gains 4-7% on the 4-column pipelines whose ring stays at
+  // 4 stages, and loses 3-6% on 3-column ones, whose rings are deeper or whose tiles are
+  // consumed faster)
+  p.prefetch = (n_cols >= 4 && p.stages <= 4) ? 2 : 0;
+  if (const char* e = std::getenv("HX_K1_PREFETCH")) p.prefetch = std::max(0, std::min(64, std::atoi(e)));
   if (std::getenv("HX_DEBUG")) {  // launch plan of this K1 (tuning aid)
     std::fprintf(stderr, "[hx] K1 joins=%d cols=%d gather=%d%d stages=%d groups=%d filters:",
                  sh->n_joins, n_cols, p.ga, p.gb, p.stages, p.smem_groups);
@@ -1506,11 +1543,13 @@ int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht*
                    p.joins[j].dm_smem, p.joins[j].bm_words, p.joins[j].bm_smem);
     std::fprintf(stderr, " in_s:");
     for (int j = 0; j < sh->n_joins; ++j) std::fprintf(stderr, "%d", p.joins[j].in_s);
-    std::fprintf(stderr, " l2:%x cost=%.2f smem=%zu\n", p.m_l2, plan_cost,
-                 k1_smem_bytes(dm_mode, n_cols, p.stages, p.smem_groups, p.filter_words, p.dm_bytes));
+    std::fprintf(stderr, " l2:%x cost=%.2f stages=%d smem=%zu\n", p.m_l2, plan_cost, p.stages,
+                 k1_smem_bytes(dm_mode, n_cols, p.stages, p.smem_groups, p.filter_words, p.dm_bytes,
+                               in_place));
   }
   k.fn = pick_kernel(sh->n_joins, grouped, p.m_dm != 0u);
-  k.smem = k1_smem_bytes(dm_mode, n_cols, p.stages, p.smem_groups, p.filter_words, p.dm_bytes);
+  k.smem = k1_smem_bytes(dm_mode, n_cols, p.stages, p.smem_groups, p.filter_words, p.dm_bytes,
+                         in_place);
   int occ = 0;
   HX_CK(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, k.fn, kThreads, k.smem));
   occ = std::max(1, occ);
