@@ -53,8 +53,9 @@ def parse():
     ap.add_argument("--no-graph", action="store_true", help="enqueue plans without a CUDA graph")
     ap.add_argument("--no-pipeline", action="store_true",
                     help="one plan set: the host reads a step's results before the next starts")
-    ap.add_argument("--variant", default="hbm", choices=["hbm", "host"],
-                    help="host: lineorder in pinned host memory streamed over PCIe (config 5)")
+    ap.add_argument("--variant", default="hbm", choices=["hbm", "host", "uva"],
+                    help="host: lineorder in pinned host memory streamed over PCIe (config 5, "
+                         "mem-move DMA); uva: the same memory read in place by K1 (zero-copy)")
     return ap.parse_args()
 
 
@@ -75,9 +76,11 @@ def peaks():
 
 
 def workload_name(sf, world, variant="hbm", queries=None):
-    if variant == "host":
+    if variant in ("host", "uva"):
+        how = ("streamed over PCIe (mem-move DMA into a device ring)" if variant == "host"
+               else "read in place over PCIe by K1 through UVA (zero-copy)")
         return (f"SSB {'/'.join(q.upper() for q in queries)}, SF{sf:g} per GPU (SF{sf * world:g} "
-                "total), lineorder host-resident in pinned memory, streamed over PCIe (mem-move)")
+                f"total), lineorder host-resident in pinned memory, {how}")
     return f"SSB all 13 queries, SF{sf:g} per GPU (SF{sf * world:g} total), HBM-resident"
 
 
@@ -224,7 +227,7 @@ def main():
         dist.broadcast_object_list(uid, src=0)
         ctx.comm_init(world, rank, uid[0])
     if args.queries == "all":
-        queries = ["q2.1", "q3.1", "q4.1"] if args.variant == "host" else ssb.QUERIES
+        queries = ["q2.1", "q3.1", "q4.1"] if args.variant in ("host", "uva") else ssb.QUERIES
     else:
         queries = args.queries.split(",")
     C = ssbgen.COLS
@@ -248,15 +251,17 @@ def main():
 
     dims = {t: dev_table(ssbgen.TABLE_COLS[t], 0, ssbgen.table_rows(sz, ssbgen.TABLE_COLS[t][0]))
             for t in ("date", "customer", "supplier", "part")}
-    if args.variant == "host":
+    if args.variant in ("host", "uva"):
         # §8(a) a8: lineorder stays in page-locked host memory; K1 streams it over PCIe
+        # (host: DMA into a device staging ring; uva: K1's bulk copies read it in place)
         spec = []
         for c in ssbgen.TABLE_COLS["lineorder"]:
             buf = torch.empty(max(n_mine, 1), dtype=torch.int32, pin_memory=True)
             ssbgen.column(SEED, sz, c, r0, n_mine, out=buf.numpy())
             keep.append(buf)
             spec.append((C[c], buf.data_ptr(), n_mine))
-        fact = hx.load_columns(ctx, spec, placement=hx._hx.HX_PLACE_HOST_PINNED)
+        fact = hx.load_columns(ctx, spec, placement=hx._hx.HX_PLACE_HOST_PINNED if args.variant == "host"
+                               else hx._hx.HX_PLACE_HOST_MAPPED)
     else:
         fact = dev_table(ssbgen.TABLE_COLS["lineorder"], r0, n_mine)
     torch.cuda.synchronize()
@@ -358,7 +363,7 @@ def main():
                 "k1_span_ms_per_step": k1_span / args.steps,
                 "traffic": tr["dram_bytes_per_launch"] if tr else None,
                 "traffic_source": tr["source"] if tr else None}
-    if args.variant == "host":
+    if args.variant in ("host", "uva"):
         # the streamed pipeline (H2D copies overlapped with K1) is bound by the host link:
         # peak = this run's own pinned H2D copy bandwidth (1 GiB, best of 3)
         hb = torch.empty(1 << 28, dtype=torch.int32, pin_memory=True)
@@ -374,8 +379,11 @@ def main():
         del hb, db_
         roofline.update({"bound": "pcie", "peak": best, "frac": achieved / best,
                          "peak_source": "measured in this run: pinned H2D cudaMemcpyAsync, 1 GiB, best of 3",
-                         "kernel": "mem-move H2D ring + k1_probe_agg per block (achieved = streamed "
-                                   "referenced-column bytes / span of the query's K1 launches)",
+                         "kernel": ("mem-move H2D ring + k1_probe_agg per block (achieved = streamed "
+                                    "referenced-column bytes / span of the query's K1 launches)")
+                         if args.variant == "host" else
+                         "k1_probe_agg reading mapped host memory through UVA (achieved = "
+                         "referenced-column bytes / K1 time)",
                          "traffic": None, "traffic_source": None})
 
     # ---- per query (after the timed region): K1-only and whole-query time ---------------
@@ -405,13 +413,16 @@ def main():
 
     # ---- e2e through the C-ABI with HOST buffers (H2D + queries + D2H inside the clock) ---
     e2e = None
-    if args.variant == "host":
+    if args.variant in ("host", "uva"):
         # the timed step already moves every input from pinned host memory (H2D ring) and
         # reads the results back: it IS the end-to-end measurement
         e2e = {"value": value, "unit": UNIT, "h2d_bytes_per_step": step_h2d // args.steps,
                "d2h_bytes_per_step": step_d2h // args.steps, "ms_per_step": ms_step,
-               "path": "plans over a HX_PLACE_HOST_PINNED fact table: H2D staging ring + K1 "
-                       "per block + merge + finalize + D2H, one CUDA graph per step"}
+               "path": ("plans over a HX_PLACE_HOST_PINNED fact table: H2D staging ring + K1 "
+                        "per block + merge + finalize + D2H, one CUDA graph per step")
+                       if args.variant == "host" else
+                       ("plans over a HX_PLACE_HOST_MAPPED fact table: K1 reads pinned host "
+                        "memory in place over PCIe + merge + finalize + D2H, one CUDA graph per step")}
     elif not args.no_e2e:
         host = {}
         for t in ("lineorder", "date", "customer", "supplier", "part"):

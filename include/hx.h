@@ -92,8 +92,13 @@ int hx_partition_free(hx_partition* p);
  *                    contiguous range (always true for part == NULL).
  *   HX_PLACE_HOST_PINNED : no copy; `data` must be page-locked host memory; K1 then streams
  *                    blocks over PCIe through a device staging ring (mem-move, §8(a) a8).
+ *   HX_PLACE_HOST_MAPPED : no copy; `data` must be page-locked, device-mapped host memory
+ *                    (cudaHostAlloc / cudaHostRegister; UVA); K1's bulk copies read it
+ *                    directly over PCIe (zero-copy, the UVA access of the paper's GPU
+ *                    baselines, §6.4).
+ *                    Fact tables only (dimension builds return HX_EUNSUPPORTED).
  * All columns of one table must have the same number of rows. At most HX_MAX_COLS. */
-enum { HX_PLACE_COPY = 0, HX_PLACE_VIEW = 1, HX_PLACE_HOST_PINNED = 2 };
+enum { HX_PLACE_COPY = 0, HX_PLACE_VIEW = 1, HX_PLACE_HOST_PINNED = 2, HX_PLACE_HOST_MAPPED = 3 };
 #define HX_MAX_COLS 16
 typedef struct { int32_t col_id; int32_t reserved; const int32_t* data; int64_t n_rows; } hx_col;
 typedef struct hx_table hx_table;

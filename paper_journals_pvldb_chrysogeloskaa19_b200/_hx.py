@@ -16,7 +16,7 @@ LIB_PATH = os.environ.get("HX_LIB", os.path.join(_HERE, "libhx.so"))  # HX_LIB: 
 HX_OK, HX_EINVAL, HX_ECUDA, HX_ENCCL, HX_ENOMEM, HX_ECAPACITY, HX_EDUPKEY, HX_EUNSUPPORTED = (
     0, -1, -2, -3, -4, -5, -6, -7)
 HX_POLICY_RANGE, HX_POLICY_ROUND_ROBIN = 0, 1
-HX_PLACE_COPY, HX_PLACE_VIEW, HX_PLACE_HOST_PINNED = 0, 1, 2
+HX_PLACE_COPY, HX_PLACE_VIEW, HX_PLACE_HOST_PINNED, HX_PLACE_HOST_MAPPED = 0, 1, 2, 3
 HX_PRED_RANGE, HX_PRED_IN = 0, 1
 HX_AGG_SUM, HX_AGG_SUM_MUL, HX_AGG_SUM_SUB = 0, 1, 2
 HX_MAX_COLS, HX_MAX_PREDS, HX_MAX_JOINS, HX_MAX_GDIMS = 16, 3, 4, 3

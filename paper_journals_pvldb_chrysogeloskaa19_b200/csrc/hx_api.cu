@@ -241,7 +241,7 @@ int hx_load_columns(hx_ctx* ctx, const hx_col* cols, int n_cols, const hx_partit
                     int part_index, int placement, hx_table** out) {
   HX_REQUIRE(ctx && out && n_cols >= 1 && cols, HX_EINVAL, "hx_load_columns: bad argument");
   HX_REQUIRE(n_cols <= HX_MAX_COLS, HX_ECAPACITY, "hx_load_columns: too many columns");
-  HX_REQUIRE(placement >= HX_PLACE_COPY && placement <= HX_PLACE_HOST_PINNED, HX_EINVAL,
+  HX_REQUIRE(placement >= HX_PLACE_COPY && placement <= HX_PLACE_HOST_MAPPED, HX_EINVAL,
              "hx_load_columns: bad placement");
   const int64_t n_src = cols[0].n_rows;
   for (int c = 0; c < n_cols; ++c) {
@@ -306,20 +306,32 @@ int hx_load_columns(hx_ctx* ctx, const hx_col* cols, int n_cols, const hx_partit
     const int64_t first = ranges.empty() ? 0 : ranges[0].first;
     for (int c = 0; c < n_cols; ++c) {
       cudaPointerAttributes a{};
+      const int32_t* base = cols[c].data;
       if (n_src > 0 && cudaPointerGetAttributes(&a, cols[c].data) == cudaSuccess) {
         const bool ok = placement == HX_PLACE_VIEW ? a.type == cudaMemoryTypeDevice ||
                                                          a.type == cudaMemoryTypeManaged
-                                                   : a.type == cudaMemoryTypeHost;
+                        : placement == HX_PLACE_HOST_MAPPED
+                            ? a.type == cudaMemoryTypeHost && a.devicePointer != nullptr
+                            : a.type == cudaMemoryTypeHost;
         if (!ok) {
           delete t;
           return fail(HX_EINVAL, placement == HX_PLACE_VIEW
                                      ? "hx_load_columns: HX_PLACE_VIEW needs device memory"
+                                 : placement == HX_PLACE_HOST_MAPPED
+                                     ? "hx_load_columns: HX_PLACE_HOST_MAPPED needs mapped pinned memory"
                                      : "hx_load_columns: HX_PLACE_HOST_PINNED needs pinned memory");
         }
+        // zero-copy: the device's address of the mapped pages (equal to the host address
+        // under UVA)
+        if (placement == HX_PLACE_HOST_MAPPED) base = static_cast<const int32_t*>(a.devicePointer);
       } else {
         cudaGetLastError();
+        if (placement == HX_PLACE_HOST_MAPPED && n_src > 0) {
+          delete t;
+          return fail(HX_EINVAL, "hx_load_columns: HX_PLACE_HOST_MAPPED needs mapped pinned memory");
+        }
       }
-      t->dev[c] = const_cast<int32_t*>(cols[c].data) + first;
+      t->dev[c] = const_cast<int32_t*>(base) + first;
     }
   }
   *out = t;

@@ -264,7 +264,8 @@ int ht_create(hx_ctx* ctx, const hx_table* dim, int32_t key_col, const hx_pred* 
   HX_REQUIRE(ctx && dim && out, HX_EINVAL, "hx_build_dim_ht: null argument");
   HX_REQUIRE(n_preds >= 0 && n_preds <= HX_MAX_PREDS && (n_preds == 0 || preds), HX_EINVAL,
              "hx_build_dim_ht: bad predicate list");
-  HX_REQUIRE(dim->placement != HX_PLACE_HOST_PINNED, HX_EUNSUPPORTED,
+  HX_REQUIRE(dim->placement != HX_PLACE_HOST_PINNED && dim->placement != HX_PLACE_HOST_MAPPED,
+             HX_EUNSUPPORTED,
              "hx_build_dim_ht: dimension tables must be device resident");
   HX_REQUIRE(dim->n_rows < (1ll << 30), HX_ECAPACITY, "hx_build_dim_ht: dimension too large");
   BuildParams p{};

@@ -1249,6 +1249,7 @@ struct K1Prepared {
   // host-resident fact table (§8(a) a8): the staged columns live in pinned host memory and
   // are streamed block by block through a device staging ring (mem-move)
   bool host = false;
+  bool mapped = false;  // HX_PLACE_HOST_MAPPED: K1 reads host memory in place (zero-copy)
   const int32_t* host_col[kMaxStageCols] = {};
   int occ = 1;
 };
@@ -1371,6 +1372,7 @@ int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht*
                                   : (double)ht->known_keys / (double)std::max<int64_t>(1, ht->dim_rows);
     }
     const bool ok = bound * 16.0 <= 1.0 && fact->placement != HX_PLACE_HOST_PINNED &&
+                    fact->placement != HX_PLACE_HOST_MAPPED &&
                     fact->n_rows < (int64_t(1) << 32) && std::getenv("HX_NO_GATHER") == nullptr;
     auto read_by_stages = [&](int32_t col) {
       for (int q = 0; q < sh->n_preds; ++q)
@@ -1403,6 +1405,7 @@ int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht*
   // tiles: the head rows up to 16-byte alignment are handled separately (device tables; a
   // host-resident table is staged block by block into aligned device buffers instead)
   k.host = fact->placement == HX_PLACE_HOST_PINNED;
+  k.mapped = fact->placement == HX_PLACE_HOST_MAPPED;
   const uintptr_t mis = k.host ? 0 : reinterpret_cast<uintptr_t>(table_col(fact, ids[0])) & 15u;
   for (int c = 0; c < n_cols && !k.host; ++c)
     HX_REQUIRE((reinterpret_cast<uintptr_t>(table_col(fact, ids[c])) & 15u) == mis &&
@@ -1531,7 +1534,7 @@ int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht*
   // (measured, SF10: a distance of 2 gains 4-7% on the 4-column pipelines whose ring stays at
   // 4 stages, and loses 3-6% on 3-column ones, whose rings are deeper or whose tiles are
   // consumed faster)
-  p.prefetch = (n_cols >= 4 && p.stages <= 4) ? 2 : 0;
+  p.prefetch = (n_cols >= 4 && p.stages <= 4 && fact->placement != HX_PLACE_HOST_MAPPED) ? 2 : 0;
   if (const char* e = std::getenv("HX_K1_PREFETCH")) p.prefetch = std::max(0, std::min(64, std::atoi(e)));
   if (std::getenv("HX_DEBUG")) {  // launch plan of this K1 (tuning aid)
     std::fprintf(stderr, "[hx] K1 joins=%d cols=%d gather=%d%d stages=%d groups=%d filters:",
@@ -1658,6 +1661,7 @@ int k1_enqueue(hx_ctx* ctx, const K1Prepared* k, bool fresh, cudaEvent_t e0, cud
   k->fn<<<(unsigned)k->grid, kThreads, k->smem, ctx->stream>>>(p);
   HX_CK_LAUNCH("k1_probe_agg");
   ctx->launches += 1;
+  if (k->mapped) ctx->h2d_bytes += k1_bytes(k);  // read over PCIe by the kernel itself
   if (e1) HX_CK(record_event(e1, ctx->stream));
   return HX_OK;
 }

@@ -240,11 +240,14 @@ def load_db_numpy(ctx: hx.Context, db: Dict[str, Dict[str, np.ndarray]],
     return dims, fact
 
 
-def load_db_host_resident(ctx: hx.Context, db: Dict[str, Dict[str, np.ndarray]], pin):
-    """Dimensions to the device; lineorder stays in page-locked host memory
-    (HX_PLACE_HOST_PINNED): K1 streams it block by block over PCIe (mem-move, §8(a) a8).
-    `pin(n)` returns a page-locked int32 buffer of n values with .ctypes / data_ptr access
-    (e.g. lambda n: torch.empty(n, dtype=torch.int32, pin_memory=True))."""
+def load_db_host_resident(ctx: hx.Context, db: Dict[str, Dict[str, np.ndarray]], pin,
+                          placement: int = _hx.HX_PLACE_HOST_PINNED):
+    """Dimensions to the device; lineorder stays in page-locked host memory.
+    HX_PLACE_HOST_PINNED: K1 streams it block by block over PCIe (mem-move, §8(a) a8);
+    HX_PLACE_HOST_MAPPED: K1 reads it in place through UVA (zero-copy, §8(f) NEXT-3).
+    `pin(n)` returns a page-locked (and, for MAPPED, device-mapped) int32 buffer of n values
+    with .ctypes / data_ptr access (e.g. lambda n: torch.empty(n, dtype=torch.int32,
+    pin_memory=True): the CUDA caching host allocator maps its pages)."""
     dims = {t: hx.load_numpy(ctx, {C[c]: v for c, v in db[t].items()})
             for t in ("date", "customer", "supplier", "part")}
     keep, spec = [], []
@@ -254,5 +257,5 @@ def load_db_host_resident(ctx: hx.Context, db: Dict[str, Dict[str, np.ndarray]],
         arr[: len(v)] = v
         keep.append(buf)
         spec.append((C[c], arr.ctypes.data, len(v)))
-    fact = hx.load_columns(ctx, spec, placement=_hx.HX_PLACE_HOST_PINNED, keep=keep)
+    fact = hx.load_columns(ctx, spec, placement=placement, keep=keep)
     return dims, fact

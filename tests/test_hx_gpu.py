@@ -197,6 +197,30 @@ def test_host_resident_streaming(ctx, sf):
         pl.close()
 
 
+@pytest.mark.parametrize("sf", [0.002, 0.4])
+def test_host_mapped_zero_copy(ctx, sf):
+    """§8(f) NEXT-3: lineorder in mapped pinned host memory read in place by K1's bulk copies
+    through UVA (HX_PLACE_HOST_MAPPED), plain and planned paths, every query."""
+    db = ssbgen.database(17, ssbgen.sizes(sf))
+    pin = lambda n: torch.empty(n, dtype=torch.int32, pin_memory=True)
+    dims, fact = ssb.load_db_host_resident(ctx, db, pin, _hx.HX_PLACE_HOST_MAPPED)
+    eng = ssb.SsbEngine(ctx, dims, fact)
+    for q in QUERIES:
+        want = oracle.run_query(q, db)
+        assert eng.run(q) == want, q
+        pl = eng.plan(q)
+        pl.enqueue()
+        assert pl.rows() == want, q
+        pl.close()
+
+
+def test_host_mapped_rejects_device_memory(ctx):
+    t = torch.zeros(16, dtype=torch.int32, device="cuda")
+    with pytest.raises(_hx.HxError):
+        hx.load_columns(ctx, [(C["lo_orderdate"], t.data_ptr(), 16)],
+                        placement=_hx.HX_PLACE_HOST_MAPPED)
+
+
 @pytest.mark.parametrize("sf", [10, 100])
 def test_parity_full_size_bench_configuration(ctx, sf):
     """BASELINE.json configs[1] (SF10, 60 M lineorder rows) and configs[2]'s 1-GPU leg (SF100,
