@@ -56,6 +56,11 @@ def parse():
     ap.add_argument("--variant", default="hbm", choices=["hbm", "host", "uva"],
                     help="host: lineorder in pinned host memory streamed over PCIe (config 5, "
                          "mem-move DMA); uva: the same memory read in place by K1 (zero-copy)")
+    ap.add_argument("--workload", default="ssb", choices=["ssb", "sum", "join"],
+                    help="sum / join: the paper's §6.4 micro-benchmarks (SUM over one 23 GB "
+                         "column; COUNT of a 1:N join with a 7.7 MB build side)")
+    ap.add_argument("--micro-rows", type=int, default=0,
+                    help="fact rows per GPU of the micro-benchmarks (default: the paper's 23 GB)")
     return ap.parse_args()
 
 
@@ -202,6 +207,117 @@ def cpu_baseline(args, world):
                       f"(full dims), single-threaded, {dt:.1f} s"}
 
 
+def run_micro(args, world, rank, local, ctx, stream, torch, dist, hx):
+    """--workload sum|join: §6.4 micro-benchmarks, one step = one
+    execution of the prepared plan (join: K2 build of the 7.7 MB side + K1 probe; sum: K1
+    scan) + merge + finalize + result to the host, in a CUDA graph."""
+    from paper_journals_pvldb_chrysogeloskaa19_b200 import micro
+    n_gpu = args.micro_rows or ssbgen.MICRO_PAPER_ROWS
+    sz = ssbgen.micro_sizes(n_gpu * world, ssbgen.MICRO_PAPER_BUILD)
+    r0 = rank * n_gpu
+    keep = []
+    C = ssbgen.COLS
+
+    def dev_table(cols, row_begin, n):
+        spec = []
+        for c in cols:
+            t = torch.empty(max(n, 1), dtype=torch.int32, device="cuda")
+            ssbgen.column_device(SEED, sz, c, t.data_ptr(), row_begin, n, stream.cuda_stream)
+            keep.append(t)
+            spec.append((C[c], t.data_ptr(), n))
+        return hx.load_columns(ctx, spec, placement=hx._hx.HX_PLACE_VIEW)
+
+    cols = ["mb_value"] if args.workload == "sum" else ["mb_value", "mb_probekey"]
+    fact = dev_table(cols, r0, n_gpu)
+    build = dev_table(["mb_buildkey"], 0, sz["n_part"])
+    torch.cuda.synchronize()
+    eng = micro.MicroEngine(ctx, fact, build)
+    plans = [eng.plan_sum() if args.workload == "sum" else eng.plan_join() for _ in range(2)]
+    graphs = [hx.capture(ctx, lambda p=p: hx.plans_enqueue(ctx, [p])) for p in plans]
+    k1 = [0.0, 0]
+
+    def run(n, timed=False):
+        for i in range(n):
+            graphs[i % 2].launch()
+            if i:
+                eng.plan_value(plans[(i - 1) % 2], args.workload)
+                if timed:
+                    k1[0] += plans[(i - 1) % 2].k1_time()[0]
+                    k1[1] += 1
+        if n:
+            eng.plan_value(plans[(n - 1) % 2], args.workload)
+            if timed:
+                k1[0] += plans[(n - 1) % 2].k1_time()[0]
+                k1[1] += 1
+
+    run(args.warmup)
+    clocks = Clocks(local)
+    if world > 1:
+        dist.barrier()
+    torch.cuda.synchronize()
+    clocks.start()
+    e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+    e0.record(stream)
+    run(args.steps, timed=True)
+    e1.record(stream)
+    torch.cuda.synchronize()
+    if world > 1:
+        dist.barrier()
+    clk = clocks.stop()
+    ms = e0.elapsed_time(e1)
+    launches, _, _ = ctx.stats(reset=True)
+    if world > 1:
+        t = torch.tensor([ms], device="cuda", dtype=torch.float64)
+        dist.all_reduce(t, op=dist.ReduceOp.MAX)
+        ms = float(t[0])
+    ms_step = ms / args.steps
+    bpr = 4 * len(cols)
+    peak, peak_src = peaks()
+    k1_ms = k1[0] / max(k1[1], 1)
+    achieved = n_gpu * bpr / (k1_ms / 1e3) / 1e9 if k1_ms > 0 else 0.0
+    cpu = None
+    if rank == 0 and world == 1 and not args.no_cpu_baseline:
+        from oracle import micro as omicro
+        sample = min(n_gpu, 200_000_000)
+        v = ssbgen.column(SEED, sz, "mb_value", 0, sample)
+        t0 = time.perf_counter()
+        if args.workload == "sum":
+            omicro.sum_column([v])
+        else:
+            pk = ssbgen.column(SEED, sz, "mb_probekey", 0, sample)
+            bk = ssbgen.column(SEED, sz, "mb_buildkey")
+            t0 = time.perf_counter()
+            omicro.join_count(bk, [(pk, v)])
+        dt = time.perf_counter() - t0
+        cpu = {"value": sample / dt, "unit": "fact rows/s", "cores": 1, "kind": "oracle",
+               "sample": f"oracle/micro.py (numpy) over fact rows [0, {sample}), {dt:.1f} s"}
+    if rank == 0:
+        name = ("§6.4 SUM over one int32 column" if args.workload == "sum" else
+                "§6.4 COUNT (and SUM) of a non-partitioned 1:N join")
+        line = {"metric": f"micro-benchmark fact rows/sec & HBM GB/s ({args.workload})",
+                "value": n_gpu * world / (ms_step / 1e3), "unit": "fact rows/s",
+                "n_gpus": world, "steps": args.steps, "warmup": args.warmup,
+                "ms_per_step": ms_step, "higher_is_better": True, "scaling": "weak",
+                "vs_baseline": None, "dtype": "int32 columns, int64 accumulate",
+                "data": f"synthetic (ssbgen mb_* columns, seed {SEED}), generated in HBM",
+                "config": {"workload": f"{name}: {n_gpu * 4 / 1e9:.1f} GB per column per GPU, "
+                                       f"build side {sz['n_part'] * 4 / 1e6:.1f} MB (PAPER.md:1364-1366)",
+                           "fact_rows_per_gpu": n_gpu, "build_rows": sz["n_part"],
+                           "l2": "inputs larger than L2; no flush"},
+                "roofline": {"bound": "hbm", "achieved": achieved, "peak": peak, "unit": "GB/s",
+                             "frac": achieved / peak, "peak_source": peak_src,
+                             "kernel": "k1_probe_agg", "algorithmic_bytes_per_launch": n_gpu * bpr,
+                             "k1_ms_per_launch": k1_ms, "traffic": None},
+                "cpu_baseline": cpu, "e2e": None, "clocks": clk, "gpu_launches": launches}
+        print(json.dumps(line), flush=True)
+    for g in graphs:
+        g.close()
+    for p in plans:
+        p.close()
+    fact.close()
+    build.close()
+
+
 def main():
     args = parse()
     world, rank, local = dist_env()
@@ -226,6 +342,12 @@ def main():
         uid = [hx.comm_unique_id() if rank == 0 else None]
         dist.broadcast_object_list(uid, src=0)
         ctx.comm_init(world, rank, uid[0])
+    if args.workload != "ssb":
+        run_micro(args, world, rank, local, ctx, stream, torch, dist, hx)
+        ctx.close()
+        if world > 1:
+            dist.destroy_process_group()
+        return
     if args.queries == "all":
         queries = ["q2.1", "q3.1", "q4.1"] if args.variant in ("host", "uva") else ssb.QUERIES
     else:

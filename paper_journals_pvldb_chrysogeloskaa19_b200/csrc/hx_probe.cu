@@ -121,7 +121,10 @@ struct K1Params {
   uint32_t m_bm;                           // its bitmap is staged in shared memory
   uint32_t m_ins;                          // its shared-memory structure runs in stage S
   uint32_t m_l2;                           // stage C reads its map from L2 (rank, or no
-                                           // exact shared-memory verdict)
+                                           // exact verdict yet)
+  uint32_t m_l2s;                          // stage S reads its map from L2 on every row (no
+                                           // shared-memory structure: exact verdict + rank)
+  uint32_t m_res;                          // resolved in stage S (full map staged, or m_l2s)
 };
 
 // join kinds (uniform per launch: read from the kernel parameters)
@@ -296,7 +299,7 @@ __device__ __forceinline__ int first_filter(const JoinState (&js)[HX_MAX_JOINS])
 }
 template <int NJ, bool DM>
 __device__ __forceinline__ bool all_resolved_in_s(const K1Params& p) {
-  return DM && (p.m_dmsm & p.m_ins & ((1u << NJ) - 1u)) == ((1u << NJ) - 1u);
+  return DM && (p.m_res & ((1u << NJ) - 1u)) == ((1u << NJ) - 1u);
 }
 // 1 when stage B probes the first join in place (hash-table joins, no lineorder predicate,
 // no filter on the first join).
@@ -585,6 +588,17 @@ __device__ __forceinline__ void process_tile(const K1Params& p, const JoinState 
         const uint32_t u = (uint32_t)key[k] - (uint32_t)d.dm_kmin;
         const uint32_t word = u < d.dm_span ? w[u >> 5] : 0u;
         m &= ~((uint32_t)(((word >> (u & 31u)) & 1u) == 0u) << k);
+      }
+    } else if (jbit(p.m_l2s, jx)) {  // its map from L2, every live row (8 loads in flight)
+      uint32_t w[2 * R];
+#pragma unroll
+      for (int k = 0; k < 2 * R; ++k)
+        w[k] = ((m >> k) & 1u) && dm_in(d, key[k]) ? __ldg(d.dm + (dm_bit(d, key[k]) >> 5)) : 0u;
+#pragma unroll
+      for (int k = 0; k < 2 * R; ++k) {
+        const uint32_t v = dm_entry(d, w[k], dm_bit(d, key[k]));
+        m &= ~((uint32_t)(v == 0u) << k);
+        if (GROUPED && all_res) g[k] += (int32_t)v * js[jx].jstride;
       }
     } else {  // its Bloom filter: no false negatives
 #pragma unroll
@@ -1015,6 +1029,171 @@ __global__ void __launch_bounds__(kThreads, kCtasPerSm) k1_probe_agg(const __gri
   }
 }
 
+// K1 for join-less pipelines (the §6.4 SUM micro-benchmark; any shape
+// with no join): Listing 1 pipeline 9 in its plain form — unpack,
+// predicate, register accumulator, then warp shuffle -> CTA -> one leader atomic. There is no
+// structure to stage and no survivor to compact, so the consumers only read their rows:
+// one producer warp streams 32 KB stages of the columns (kScanRows(NC) rows) HBM -> shared
+// memory with cp.async.bulk into a kScanStages-deep mbarrier ring (evict-first), and each of
+// the kScanThreads consumer threads reads 4 consecutive rows per column with one 128-bit
+// shared-memory load. (Plain 128-bit global loads measured 5.5 TB/s on one column; the
+// bulk-copy ring reaches the read-stream ceiling, tools/stream_roofline.cu.)
+constexpr int kScanThreads = 512;  // consumer threads (+ one producer warp)
+constexpr int kScanStages = 6;
+constexpr int scan_rows(int nc) { return nc == 1 ? 8192 : nc == 2 ? 4096 : 2048; }
+constexpr size_t scan_smem(int nc) { return 128 + (size_t)kScanStages * nc * scan_rows(nc) * 4; }
+template <int NC>
+__global__ void __launch_bounds__(kScanThreads + 32, 1) k1_scan_agg(const __grid_constant__ K1Params p) {
+  constexpr int kRows = scan_rows(NC);
+  extern __shared__ __align__(128) unsigned char smem[];
+  uint64_t* full = reinterpret_cast<uint64_t*>(smem);
+  uint64_t* empty = full + kScanStages;
+  int32_t* ring = reinterpret_cast<int32_t*>(smem + 128);
+  __shared__ long long red[2][kScanThreads / 32];
+  const int tid = threadIdx.x, warp = tid >> 5, lane = tid & 31;
+  const int64_t n_tiles = (p.n_rows + kRows - 1) / kRows;
+  if (tid == kScanThreads) {
+    for (int st = 0; st < kScanStages; ++st) {
+      mbar_init(full + st, 1);
+      mbar_init(empty + st, kScanThreads / 32);
+    }
+    asm volatile("fence.mbarrier_init.release.cluster;" ::: "memory");
+  }
+  __syncthreads();
+  if (warp == kScanThreads / 32) {  // producer
+    if (lane == 0) {
+      const uint64_t pol = policy_evict_first();
+      int st = 0;
+      uint32_t ph = 0;
+      int64_t k = 0;
+      for (int64_t t = blockIdx.x; t < n_tiles; t += gridDim.x, ++k) {
+        if (k >= kScanStages) mbar_wait_sleep(empty + st, ph ^ 1u);
+        const int64_t r0 = t * kRows;
+        const uint32_t bytes = (uint32_t)(std::min<int64_t>(kRows, p.n_rows - r0) & ~int64_t(3)) * 4u;
+        mbar_arrive_expect_tx(full + st, bytes * NC);
+        if (bytes)
+          for (int c = 0; c < NC; ++c)
+            bulk_g2s(ring + ((size_t)st * NC + c) * kRows, p.col[c] + r0, bytes, full + st, pol);
+        if (++st == kScanStages) {
+          st = 0;
+          ph ^= 1u;
+        }
+      }
+    }
+    return;
+  }
+  long long acc_sum = 0, acc_cnt = 0;
+  auto row = [&](const int32_t (&v)[NC]) {
+    bool ok = true;
+    for (int q = 0; q < p.n_preds; ++q) {
+      const DevPred& pr = p.preds[q];
+      int32_t x = v[0];
+#pragma unroll
+      for (int c = 1; c < NC; ++c) x = pr.c == c ? v[c] : x;
+      ok = ok && pred_pass(pr, x);
+    }
+    int32_t a = v[0], b = v[0];
+#pragma unroll
+    for (int c = 1; c < NC; ++c) {
+      a = p.agg_a == c ? v[c] : a;
+      b = p.agg_b == c ? v[c] : b;
+    }
+    if (ok) {
+      acc_sum += measure(p.agg_op, a, b);
+      acc_cnt += 1;
+    }
+  };
+  const bool plain_sum = p.n_preds == 0 && p.agg_op == HX_AGG_SUM;
+  // misaligned head rows (views at a row offset; before the first 16-byte boundary)
+  if (blockIdx.x == 0 && tid < p.head_rows) {
+    int32_t v[NC];
+#pragma unroll
+    for (int c = 0; c < NC; ++c) v[c] = p.head_col[c][tid];
+    row(v);
+  }
+  int st = 0;
+  uint32_t ph = 0;
+  for (int64_t t = blockIdx.x; t < n_tiles; t += gridDim.x) {
+    mbar_wait(full + st, ph);
+    const int64_t r0 = t * kRows;
+    const int rows = (int)std::min<int64_t>(kRows, p.n_rows - r0);
+    const int32_t* sb = ring + (size_t)st * NC * kRows;
+    if (rows == kRows && plain_sum) {  // SUM(a), no predicate: 4 rows per 128-bit load
+#pragma unroll 4
+      for (int i = tid; i < kRows / 4; i += kScanThreads) {
+        const int4 x = reinterpret_cast<const int4*>(sb + p.agg_a * kRows)[i];
+        acc_sum += ((long long)x.x + (long long)x.y) + ((long long)x.z + (long long)x.w);
+      }
+      acc_cnt += kRows / kScanThreads;
+    } else if (rows == kRows) {
+#pragma unroll 2
+      for (int i = tid; i < kRows / 4; i += kScanThreads) {
+        int4 x[NC];
+#pragma unroll
+        for (int c = 0; c < NC; ++c) x[c] = reinterpret_cast<const int4*>(sb + c * kRows)[i];
+        // predicates column-wise on the 4 rows (kind uniform per predicate), then the measure
+        uint32_t m = 0xFu;
+        for (int q = 0; q < p.n_preds; ++q) {
+          const DevPred& pr = p.preds[q];
+          int4 y = x[0];
+#pragma unroll
+          for (int c = 1; c < NC; ++c) y = pr.c == c ? x[c] : y;
+          const int32_t yv[4] = {y.x, y.y, y.z, y.w};
+#pragma unroll
+          for (int k = 0; k < 4; ++k) m &= ~((uint32_t)!pred_pass(pr, yv[k]) << k);
+        }
+        int4 a4 = x[0], b4 = x[0];
+#pragma unroll
+        for (int c = 1; c < NC; ++c) {
+          a4 = p.agg_a == c ? x[c] : a4;
+          b4 = p.agg_b == c ? x[c] : b4;
+        }
+        const int32_t av[4] = {a4.x, a4.y, a4.z, a4.w}, bv[4] = {b4.x, b4.y, b4.z, b4.w};
+#pragma unroll
+        for (int k = 0; k < 4; ++k)
+          if ((m >> k) & 1u) acc_sum += measure(p.agg_op, av[k], bv[k]);
+        acc_cnt += __popc(m);
+      }
+    } else {  // the last, partial tile: its < 4 ragged rows were not copied
+      const int copied = rows & ~3;
+      for (int r = tid; r < rows; r += kScanThreads) {
+        int32_t v[NC];
+#pragma unroll
+        for (int c = 0; c < NC; ++c) v[c] = r < copied ? sb[c * kRows + r] : p.col[c][r0 + r];
+        row(v);
+      }
+    }
+    __syncwarp();
+    if (lane == 0) mbar_arrive(empty + st);
+    if (++st == kScanStages) {
+      st = 0;
+      ph ^= 1u;
+    }
+  }
+  // neighbourhood reduce + leader atomic (Listing 1 L27-29)
+#pragma unroll
+  for (int o = 16; o > 0; o >>= 1) {
+    acc_sum += __shfl_xor_sync(kFull, acc_sum, o);
+    acc_cnt += __shfl_xor_sync(kFull, acc_cnt, o);
+  }
+  if (lane == 0) {
+    red[0][warp] = acc_sum;
+    red[1][warp] = acc_cnt;
+  }
+  asm volatile("bar.sync 1, %0;" ::"n"(kScanThreads) : "memory");
+  if (tid == 0) {
+    long long s = 0, c = 0;
+    for (int w = 0; w < kScanThreads / 32; ++w) {
+      s += red[0][w];
+      c += red[1][w];
+    }
+    if (c) {
+      atomicAdd(p.g_sum, (unsigned long long)s);
+      atomicAdd(p.g_cnt, (unsigned long long)c);
+    }
+  }
+}
+
 // Group layout from the dimension ranks (device-side; no host round trip) and zeroing of
 // the group arrays. Every CTA computes n_groups; CTA 0 publishes the meta.
 __global__ void k1_prepare(AggMeta* meta, const HtHeader* g0, const HtHeader* g1,
@@ -1112,12 +1291,12 @@ double bloom_fp(double bits_per_key) {
 // filter on every row, a row entering stage C (compaction, queue, batch), a stage-C
 // shared-memory filter, an L2 lookup. HX_K1_COST="s,c,sc,l2" overrides (tuning aid).
 struct K1Cost {
-  double s = 8.0, c = 60.0, sc = 8.0, l2 = 20.0;
+  double s = 8.0, c = 60.0, sc = 8.0, l2 = 20.0, s2 = 16.0;  // s2: an L2 map read in stage S
 };
 K1Cost k1_cost() {
   K1Cost k;
   if (const char* e = std::getenv("HX_K1_COST"))
-    std::sscanf(e, "%lf,%lf,%lf,%lf", &k.s, &k.c, &k.sc, &k.l2);
+    std::sscanf(e, "%lf,%lf,%lf,%lf,%lf", &k.s, &k.c, &k.sc, &k.l2, &k.s2);
   return k;
 }
 
@@ -1166,18 +1345,18 @@ double plan_dm(int nj, const JoinDev* joins, const bool* known, const double* pa
       bw[j] = opts[j][idx[j]].bw;
     }
     if (fits(kd, bw)) {
-      uint32_t has = 0;
-      for (int j = 0; j < nj; ++j) has |= (uint32_t)(kd[j] != kStNone) << j;
-      // every subset of the joins that have a structure may run in stage S
+      // every subset of the joins may run in stage S: a join with a shared-memory structure
+      // applies it there; one without reads its map from L2 there (exact, like a full map)
+      const uint32_t has = (1u << nj) - 1u;
       for (uint32_t S = has;; S = (S - 1) & has) {
         double fS = 1.0, cost = 0.0;
         bool all_res = true;
         for (int j = 0; j < nj; ++j) {
           if ((S >> j) & 1u) {
-            fS *= opts[j][idx[j]].e;
-            cost += K.s;
+            fS *= kd[j] == kStNone ? (known[j] ? pass[j] : 1.0) : opts[j][idx[j]].e;
+            cost += kd[j] == kStNone ? K.s2 : K.s;
           }
-          all_res = all_res && ((S >> j) & 1u) && kd[j] == kStFull;
+          all_res = all_res && ((S >> j) & 1u) && (kd[j] == kStFull || kd[j] == kStNone);
         }
         if (!all_res) {
           cost += K.c * fS;
@@ -1191,7 +1370,8 @@ double plan_dm(int nj, const JoinDev* joins, const bool* known, const double* pa
             }
             if (inS && kd[j] == kStFull && grouped[j]) cost += K.sc * fS;  // rank re-read
             const bool full = kd[j] == kStFull;
-            n_l2 += !full && (grouped[j] || !opts[j][idx[j]].exact);
+            const bool exact = opts[j][idx[j]].exact || (inS && kd[j] == kStNone);
+            n_l2 += !full && (grouped[j] || !exact);
           }
           cost += K.l2 * n_l2 * fC;
         }
@@ -1223,6 +1403,10 @@ int k1_occupancy(hx_ctx* ctx) {
         for (int j = 0; j <= HX_MAX_JOINS; ++j)
           cudaFuncSetAttribute(kKernels[d][g][j], cudaFuncAttributeMaxDynamicSharedMemorySize,
                                227 * 1024);
+    cudaFuncSetAttribute(k1_scan_agg<1>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)scan_smem(1));
+    cudaFuncSetAttribute(k1_scan_agg<2>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)scan_smem(2));
+    cudaFuncSetAttribute(k1_scan_agg<3>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)scan_smem(3));
+    cudaFuncSetAttribute(k1_scan_agg<4>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)scan_smem(4));
     attrs = true;
   }
   int occ = 0;
@@ -1250,6 +1434,9 @@ struct K1Prepared {
   // are streamed block by block through a device staging ring (mem-move)
   bool host = false;
   bool mapped = false;  // HX_PLACE_HOST_MAPPED: K1 reads host memory in place (zero-copy)
+  KernelFn scan = nullptr;  // join-less pipeline: k1_scan_agg<NC> instead of k1_probe_agg
+  int scan_grid = 0;
+  size_t scan_smem = 0;
   const int32_t* host_col[kMaxStageCols] = {};
   int occ = 1;
 };
@@ -1501,7 +1688,7 @@ int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht*
     }
     d.in_s = in_s[j];
   }
-  p.m_dm = p.m_dmsm = p.m_bm = p.m_ins = p.m_l2 = 0u;
+  p.m_dm = p.m_dmsm = p.m_bm = p.m_ins = p.m_l2 = p.m_l2s = p.m_res = 0u;
   {
     bool grouped_j[HX_MAX_JOINS] = {false, false, false, false};
     for (int g = 0; g < sh->n_gdims; ++g) grouped_j[sh->gdim_join[g]] = true;
@@ -1512,16 +1699,19 @@ int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht*
       p.m_dmsm |= (uint32_t)full << j;
       p.m_bm |= (uint32_t)bm << j;
       p.m_ins |= (uint32_t)(d.in_s != 0) << j;
-      // the L2 map: for the rank of a grouping join, or for the verdict when no exact
-      // structure is staged (none, or a Bloom filter)
-      p.m_l2 |= (uint32_t)(dm && !full && (grouped_j[j] || !bm)) << j;
+      const bool l2s = dm && d.in_s && !full && !bm && d.bloom_words == 0;
+      p.m_l2s |= (uint32_t)l2s << j;
+      p.m_res |= (uint32_t)(d.in_s && (full || l2s)) << j;
+      // the L2 map in stage C: for the rank of a grouping join, or for the verdict when no
+      // exact one is known (no structure, or a Bloom filter)
+      p.m_l2 |= (uint32_t)(dm && !full && (grouped_j[j] || !(bm || l2s))) << j;
     }
   }
   // a pipeline whose joins all resolve in stage S aggregates in place: no per-warp queues or
   // carry buffers. Shared memory the plan left over deepens the tile ring (up to 8 stages:
   // more bytes in flight per SM while the consumers hold a pair of tiles).
   const bool in_place = sh->n_joins == 0 ||
-                        (dm_mode && (p.m_dmsm & p.m_ins) == (1u << sh->n_joins) - 1u);
+                        (dm_mode && p.m_res == (1u << sh->n_joins) - 1u);
   p.smem_fixed = in_place ? kSmemQueueOff : smem_fixed(dm_mode);
   {
     int max_stages = 8;
@@ -1546,7 +1736,7 @@ int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht*
                    p.joins[j].dm_smem, p.joins[j].bm_words, p.joins[j].bm_smem);
     std::fprintf(stderr, " in_s:");
     for (int j = 0; j < sh->n_joins; ++j) std::fprintf(stderr, "%d", p.joins[j].in_s);
-    std::fprintf(stderr, " l2:%x cost=%.2f stages=%d smem=%zu\n", p.m_l2, plan_cost, p.stages,
+    std::fprintf(stderr, " l2:%x l2s:%x cost=%.2f stages=%d smem=%zu\n", p.m_l2, p.m_l2s, plan_cost, p.stages,
                  k1_smem_bytes(dm_mode, n_cols, p.stages, p.smem_groups, p.filter_words, p.dm_bytes,
                                in_place));
   }
@@ -1560,6 +1750,14 @@ int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht*
   k.grid = (int)std::max<int64_t>(1, std::min<int64_t>(p.n_tiles, (int64_t)ctx->n_sms * occ));
   k.rows = fact->n_rows;
   k.n_cols = n_cols;
+  if (sh->n_joins == 0 && n_cols >= 1 && n_cols <= 4 && !k.host &&
+      std::getenv("HX_NO_SCAN") == nullptr) {
+    const KernelFn scans[4] = {k1_scan_agg<1>, k1_scan_agg<2>, k1_scan_agg<3>, k1_scan_agg<4>};
+    k.scan = scans[n_cols - 1];
+    k.scan_smem = scan_smem(n_cols);
+    const int64_t tiles = (p.n_rows + scan_rows(n_cols) - 1) / scan_rows(n_cols);
+    k.scan_grid = (int)std::max<int64_t>(1, std::min<int64_t>(tiles, (int64_t)ctx->n_sms));
+  }
   *out = new K1Prepared(k);
   return HX_OK;
 }
@@ -1658,8 +1856,13 @@ int k1_enqueue(hx_ctx* ctx, const K1Prepared* k, bool fresh, cudaEvent_t e0, cud
   if (k->rows == 0) return HX_OK;
   if (k->host) return k1_enqueue_host(ctx, k, ring, e0, e1);
   if (e0) HX_CK(record_event(e0, ctx->stream));
-  k->fn<<<(unsigned)k->grid, kThreads, k->smem, ctx->stream>>>(p);
-  HX_CK_LAUNCH("k1_probe_agg");
+  if (k->scan) {
+    k->scan<<<(unsigned)k->scan_grid, kScanThreads + 32, k->scan_smem, ctx->stream>>>(p);
+    HX_CK_LAUNCH("k1_scan_agg");
+  } else {
+    k->fn<<<(unsigned)k->grid, kThreads, k->smem, ctx->stream>>>(p);
+    HX_CK_LAUNCH("k1_probe_agg");
+  }
   ctx->launches += 1;
   if (k->mapped) ctx->h2d_bytes += k1_bytes(k);  // read over PCIe by the kernel itself
   if (e1) HX_CK(record_event(e1, ctx->stream));

@@ -26,6 +26,8 @@ COLS: Dict[str, int] = {
     "c_custkey": 32, "c_city": 33, "c_nation": 34, "c_region": 35,
     "s_suppkey": 48, "s_city": 49, "s_nation": 50, "s_region": 51,
     "p_partkey": 64, "p_mfgr": 65, "p_category": 66, "p_brand1": 67,
+    # §6.4 micro-benchmarks (ssbgen.h MB_*): fact value / probe-key columns, build keys
+    "mb_value": 9, "mb_probekey": 10, "mb_buildkey": 68,
 }
 TABLE_COLS = {
     "lineorder": [c for c in COLS if c.startswith("lo_")],
@@ -100,6 +102,19 @@ def sizes(sf: float) -> Dict[str, int]:
         "n_part": n_part,
         "n_date": N_DATE,
     }
+
+
+# PAPER.md:1364-1366 §6.4: "a single column of 23GB" (sum; the join's probe side) and "a
+# 7.7MB column" (the join's build side), as int32 values.
+MICRO_PAPER_ROWS = 23_000_000_000 // 4
+MICRO_PAPER_BUILD = 7_700_000 // 4
+
+
+def micro_sizes(n_rows: int, n_build: int = MICRO_PAPER_BUILD) -> Dict[str, int]:
+    """Sizes of the §6.4 micro-benchmark tables: n_rows fact rows (mb_value, mb_probekey),
+    n_build build keys (mb_buildkey)."""
+    return {"n_lineorder": int(n_rows), "n_customer": 1, "n_supplier": 1,
+            "n_part": max(1, int(n_build)), "n_date": N_DATE}
 
 
 class _Sizes(ctypes.Structure):

@@ -19,6 +19,7 @@
  *   customer/supplier nation U[0,24]; region = TPC-H map; city = nation*10 + U[0,9]
  *   part              mfgr U[0,4]; category = mfgr*5 + U[0,4]; brand1 = category*40 + U[0,39]
  *   date              the full calendar 1992-01-01 .. 1998-12-31 (2,557 rows)
+ *   micro-benchmarks  mb_value U[0,2^20); mb_probekey U[1, 2*n_part]; mb_buildkey 2*row+1
  * Dictionary codes are order-preserving (alphabetical regions/nations, see ssbgen/__init__.py).
  */
 #ifndef SSBGEN_H
@@ -40,6 +41,11 @@ enum {
   SSB_LO_ORDERDATE = 0, SSB_LO_CUSTKEY = 1, SSB_LO_PARTKEY = 2, SSB_LO_SUPPKEY = 3,
   SSB_LO_QUANTITY = 4, SSB_LO_EXTENDEDPRICE = 5, SSB_LO_DISCOUNT = 6, SSB_LO_REVENUE = 7,
   SSB_LO_SUPPLYCOST = 8,
+  /* §6.4 micro-benchmark inputs: a fact table
+     of n_lineorder rows with a value column (SUM query) and a probe-key column (1:N join),
+     and a build table of n_part rows whose keys are the odd numbers 1, 3, .., 2*n_part-1.
+     Probe keys are uniform over [1, 2*n_part], so about half of them match one build key. */
+  MB_VALUE = 9, MB_PROBEKEY = 10, MB_BUILDKEY = 68,
   SSB_D_DATEKEY = 16, SSB_D_YEAR = 17, SSB_D_YEARMONTHNUM = 18, SSB_D_WEEKNUMINYEAR = 19,
   SSB_D_DAYNUMINYEAR = 20, SSB_D_MONTHNUMINYEAR = 21,
   SSB_C_CUSTKEY = 32, SSB_C_CITY = 33, SSB_C_NATION = 34, SSB_C_REGION = 35,
@@ -60,7 +66,8 @@ enum {
   SSBGEN_ST_ORDERDAY = 1, SSBGEN_ST_CUSTKEY = 2, SSBGEN_ST_PARTKEY = 3, SSBGEN_ST_SUPPKEY = 4,
   SSBGEN_ST_QUANTITY = 5, SSBGEN_ST_DISCOUNT = 6,
   SSBGEN_ST_C_NATION = 17, SSBGEN_ST_C_CITY = 18, SSBGEN_ST_S_NATION = 19, SSBGEN_ST_S_CITY = 20,
-  SSBGEN_ST_P_MFGR = 21, SSBGEN_ST_P_CAT = 22, SSBGEN_ST_P_BRAND = 23
+  SSBGEN_ST_P_MFGR = 21, SSBGEN_ST_P_CAT = 22, SSBGEN_ST_P_BRAND = 23,
+  SSBGEN_ST_MB_VALUE = 24, SSBGEN_ST_MB_PROBE = 25
 };
 
 SSBGEN_FN uint64_t ssbgen_splitmix64(uint64_t x) {
@@ -200,6 +207,10 @@ SSBGEN_FN int32_t ssbgen_value(uint64_t seed, const ssbgen_sizes* sz, int col, i
     case SSB_P_BRAND1:
       return ssbgen_p_category(seed, row) * 40 +
              (int32_t)ssbgen_uniform(seed, SSBGEN_ST_P_BRAND, row, 40);
+    case MB_VALUE: return (int32_t)ssbgen_uniform(seed, SSBGEN_ST_MB_VALUE, row, 1u << 20);
+    case MB_PROBEKEY:
+      return 1 + (int32_t)ssbgen_uniform(seed, SSBGEN_ST_MB_PROBE, row, (uint32_t)(2 * sz->n_part));
+    case MB_BUILDKEY: return (int32_t)(2 * row + 1);
     default: return 0;
   }
 }
