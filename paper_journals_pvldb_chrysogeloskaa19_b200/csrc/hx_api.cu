@@ -2,6 +2,7 @@
 // router, mem-move (column placement), hash-table objects, pipeline launch, union-router
 // merge and measurement. The kernels live in hx_build.cu (K2) and hx_probe.cu (K1).
 #include <algorithm>
+#include <cstdlib>
 #include <cstring>
 #include <string>
 
@@ -96,6 +97,13 @@ int hx_init(int device, void* stream, hx_ctx** out) {
     cudaMemPoolSetAttribute(pool, cudaMemPoolAttrReleaseThreshold, &thr);
   }
   ctx->k1_ctas_per_sm = std::max(1, k1_occupancy(ctx));
+  {
+    int least = 0, greatest = 0;
+    if (cudaDeviceGetStreamPriorityRange(&least, &greatest) == cudaSuccess &&
+        std::getenv("HX_NO_K1_PRIORITY") == nullptr)
+      ctx->k1_priority = greatest;
+    cudaGetLastError();
+  }
   for (int a = 0; a < hx_ctx::kAux; ++a) {
     HX_CK(cudaStreamCreateWithFlags(&ctx->aux[a], cudaStreamNonBlocking));
     HX_CK(cudaEventCreateWithFlags(&ctx->join_ev[a], cudaEventDisableTiming));

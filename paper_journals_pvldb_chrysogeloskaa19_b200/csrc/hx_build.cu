@@ -55,52 +55,23 @@ __device__ __forceinline__ bool row_pass(const BuildParams& p, int64_t i) {
   return ok;
 }
 
-// Count passing rows and their key range; flag the group codes present among them.
-__global__ void k2_filter_mark(BuildParams p) {
-  int local = 0;
-  uint32_t emin = 0xFFFFFFFFu, emax = 0u;
-  const int64_t stride = (int64_t)gridDim.x * blockDim.x;
-  for (int64_t i = (int64_t)blockIdx.x * blockDim.x + threadIdx.x; i < p.n_rows; i += stride) {
-    if (!row_pass(p, i)) continue;
-    ++local;
-    const int32_t key = __ldg(p.key + i);
-    if (key == kEmptyKey) atomicExch(&p.hdr->error, HX_EINVAL);  // reserved key
-    emin = min(emin, key_enc(key));
-    emax = max(emax, key_enc(key));
-    if (p.group) {
-      int32_t code = __ldg(p.group + i) - p.group_lo;
-      if (code < 0 || code >= p.domain)
-        atomicExch(&p.hdr->error, HX_EINVAL);
-      else
-        p.c2r[code] = 1;  // benign race: every writer stores 1
-    }
-  }
-#pragma unroll
-  for (int o = 16; o > 0; o >>= 1) local += __shfl_xor_sync(kFull, local, o);
-  emin = __reduce_min_sync(kFull, emin);
-  emax = __reduce_max_sync(kFull, emax);
-  if ((threadIdx.x & 31) == 0 && local) {
-    atomicAdd(&p.hdr->n_keys, local);
-    atomicMax(&p.hdr->kmin_inv, ~emin);
-    atomicMax(&p.hdr->kmax_enc, emax);
-  }
-}
-
-// One CTA: dense ranks of the present group codes (exclusive scan of the flags), rank->code
-// map, and the table capacity from the passing count.
-__global__ void k2_rank(BuildParams p) {
-  using Scan = cub::BlockScan<int, 1024>;
+// The dense ranks of the present group codes (exclusive scan of the flags), the rank->code
+// map, and the table capacity / Bloom size from the passing count: run by ONE CTA of NT
+// threads once every flag and counter is final.
+template <int NT>
+__device__ void rank_codes(const BuildParams& p) {
+  using Scan = cub::BlockScan<int, NT>;
   __shared__ typename Scan::TempStorage tmp;
   __shared__ int running;
   if (threadIdx.x == 0) running = 0;
   __syncthreads();
   if (p.group) {
-    for (int base = 0; base < p.domain; base += 1024) {
-      int code = base + threadIdx.x;
-      int flag = code < p.domain ? p.c2r[code] : 0;
+    for (int base = 0; base < p.domain; base += NT) {
+      const int code = base + threadIdx.x;
+      const int flag = code < p.domain ? __ldcg(p.c2r + code) : 0;
       int excl, total;
       Scan(tmp).ExclusiveSum(flag, excl, total);
-      int rank = running + excl;
+      const int rank = running + excl;
       if (flag) {
         p.c2r[code] = rank;
         p.r2c[rank] = code + p.group_lo;
@@ -111,7 +82,7 @@ __global__ void k2_rank(BuildParams p) {
     }
   }
   if (threadIdx.x == 0) {
-    int n = p.hdr->n_keys;
+    const int n = __ldcg(&p.hdr->n_keys);
     int lg = kMinLog2Cap;
     while (lg < p.max_log2cap && (1ll << lg) < (long long)kLoadInv * n) ++lg;
     p.hdr->log2cap = lg;
@@ -123,15 +94,91 @@ __global__ void k2_rank(BuildParams p) {
   }
 }
 
-// Empty the slots and Bloom words in use (their sizes are only known on the device).
+// Count passing rows and their key range; flag the group codes present among them; zero the
+// Bloom filter (all of its words) and, for a direct-map build, the map and bitmap (the
+// insert kernel runs after this one). The LAST CTA to finish (threadfence + counter) then
+// ranks the codes and sizes the table, so the build needs no separate rank launch.
+// The passing count, key range and code flags are reduced in shared memory first: one set of
+// global atomics per CTA (same-address atomics from every warp serialise at one L2 slice).
+constexpr int kFilterThreads = 256;
+constexpr int kSmemCodeWords = 1024;  // code-presence bitmap in shared memory (32 K codes)
+__global__ void __launch_bounds__(kFilterThreads) k2_filter_mark(BuildParams p) {
+  __shared__ uint32_t s_codes[kSmemCodeWords];
+  __shared__ int s_n;
+  __shared__ uint32_t s_min, s_max;
+  const bool smem_codes = p.group && p.domain <= kSmemCodeWords * 32;
+  const int code_words = smem_codes ? (p.domain + 31) / 32 : 0;
+  for (int w = threadIdx.x; w < code_words; w += blockDim.x) s_codes[w] = 0u;
+  if (threadIdx.x == 0) {
+    s_n = 0;
+    s_min = 0xFFFFFFFFu;
+    s_max = 0u;
+  }
+  __syncthreads();
+  int local = 0;
+  uint32_t emin = 0xFFFFFFFFu, emax = 0u;
+  const int64_t stride = (int64_t)gridDim.x * blockDim.x;
+  const int64_t gtid = (int64_t)blockIdx.x * blockDim.x + threadIdx.x;
+  const int64_t bloom_words = int64_t(1) << p.max_bloom_log2w;
+  for (int64_t i = gtid; i < bloom_words; i += stride) p.bloom[i] = 0u;
+  if (p.dm) {
+    for (int64_t i = gtid; i < p.dm_words; i += stride) p.dm[i] = 0u;
+    if (p.dm_bm)
+      for (int64_t i = gtid; i < p.bm_words; i += stride) p.dm_bm[i] = 0u;
+  }
+  for (int64_t i = gtid; i < p.n_rows; i += stride) {
+    if (!row_pass(p, i)) continue;
+    ++local;
+    const int32_t key = __ldg(p.key + i);
+    if (key == kEmptyKey) atomicExch(&p.hdr->error, HX_EINVAL);  // reserved key
+    emin = min(emin, key_enc(key));
+    emax = max(emax, key_enc(key));
+    if (p.group) {
+      int32_t code = __ldg(p.group + i) - p.group_lo;
+      if (code < 0 || code >= p.domain)
+        atomicExch(&p.hdr->error, HX_EINVAL);
+      else if (smem_codes)
+        atomicOr(s_codes + (code >> 5), 1u << (code & 31));
+      else
+        p.c2r[code] = 1;  // benign race: every writer stores 1
+    }
+  }
+#pragma unroll
+  for (int o = 16; o > 0; o >>= 1) local += __shfl_xor_sync(kFull, local, o);
+  emin = __reduce_min_sync(kFull, emin);
+  emax = __reduce_max_sync(kFull, emax);
+  if ((threadIdx.x & 31) == 0 && local) {
+    atomicAdd(&s_n, local);
+    atomicMin(&s_min, emin);
+    atomicMax(&s_max, emax);
+  }
+  __syncthreads();
+  if (threadIdx.x == 0 && s_n) {
+    atomicAdd(&p.hdr->n_keys, s_n);
+    atomicMax(&p.hdr->kmin_inv, ~s_min);
+    atomicMax(&p.hdr->kmax_enc, s_max);
+  }
+  for (int w = threadIdx.x; w < code_words; w += blockDim.x)
+    for (uint32_t bits = s_codes[w]; bits; bits &= bits - 1u)
+      p.c2r[w * 32 + __ffs(bits) - 1] = 1;
+  // last-CTA-done: publish this CTA's flags and counters, then count it in
+  __shared__ bool last;
+  __threadfence();
+  __syncthreads();
+  if (threadIdx.x == 0) last = atomicAdd(&p.hdr->done, 1u) == gridDim.x - 1;
+  __syncthreads();
+  if (!last) return;
+  __threadfence();
+  rank_codes<kFilterThreads>(p);
+}
+
+// Empty the slots in use (their count is only known on the device; the Bloom filter was
+// zeroed by the filter kernel).
 __global__ void k2_clear(BuildParams p) {
   const int64_t cap = 1ll << p.hdr->log2cap;
-  const int64_t words = 1ll << p.hdr->bloom_log2w;
   const int64_t stride = (int64_t)gridDim.x * blockDim.x;
-  for (int64_t i = (int64_t)blockIdx.x * blockDim.x + threadIdx.x; i < cap; i += stride) {
+  for (int64_t i = (int64_t)blockIdx.x * blockDim.x + threadIdx.x; i < cap; i += stride)
     p.slots[i] = kEmptySlot;
-    if (i < words) p.bloom[i] = 0u;
-  }
 }
 
 // Warp-cooperative linear-probing insert of every passing row.
@@ -208,14 +255,6 @@ __global__ void k2_insert(BuildParams p) {
       }
     }
   }
-}
-
-// Empty the Bloom words in use (direct-map builds have no slots to clear).
-__global__ void k2_clear_bloom(BuildParams p) {
-  const int64_t words = 1ll << p.hdr->bloom_log2w;
-  for (int64_t i = (int64_t)blockIdx.x * blockDim.x + threadIdx.x; i < words;
-       i += (int64_t)gridDim.x * blockDim.x)
-    p.bloom[i] = 0u;
 }
 
 // Direct-map build: entry (key - kmin) |= rank + 1 for every passing row, plus the key's
@@ -326,7 +365,8 @@ int ht_create(hx_ctx* ctx, const hx_table* dim, int32_t key_col, const hx_pred* 
   return HX_OK;
 }
 
-// Enqueue the four build kernels (asynchronous; CUDA-graph capturable). Re-running a build
+// Enqueue the build (a header memset + 2 kernels for a direct map, + 3 for a hash table;
+// asynchronous; CUDA-graph capturable). Re-running a build
 // on the same table rebuilds it from scratch.
 int ht_enqueue_build(hx_ctx* ctx, hx_ht* ht, cudaStream_t stream) {
   const BuildParams& p = *static_cast<const BuildParams*>(ht->build);
@@ -334,19 +374,14 @@ int ht_enqueue_build(hx_ctx* ctx, hx_ht* ht, cudaStream_t stream) {
   HX_CK(cudaMemsetAsync(ht->base, 0, sizeof(HtHeader) + p.domain * sizeof(int32_t), s));
   const int64_t want = (p.n_rows + 255) / 256;
   const int grid = (int)std::max<int64_t>(1, std::min<int64_t>(want, (int64_t)ctx->n_sms * 8));
-  k2_filter_mark<<<grid, 256, 0, s>>>(p);
+  // (at most 2 CTAs per SM for the filter: its per-CTA flush is the serial part)
+  const int fgrid = (int)std::max<int64_t>(1, std::min<int64_t>(want, (int64_t)ctx->n_sms * 2));
+  k2_filter_mark<<<fgrid, kFilterThreads, 0, s>>>(p);  // + zeroing, + rank (last CTA)
   HX_CK_LAUNCH("k2_filter_mark");
-  k2_rank<<<1, 1024, 0, s>>>(p);
-  HX_CK_LAUNCH("k2_rank");
   if (p.dm) {  // direct map (+ bitmap, Bloom filter) instead of slots
-    HX_CK(cudaMemsetAsync(p.dm, 0, (size_t)(p.dm_words + p.bm_words) * sizeof(uint32_t), s));
-    const int bgrid = (int)std::min<int64_t>(((int64_t(1) << p.max_bloom_log2w) + 255) / 256,
-                                             (int64_t)ctx->n_sms * 4);
-    k2_clear_bloom<<<bgrid, 256, 0, s>>>(p);
-    HX_CK_LAUNCH("k2_clear_bloom");
     k2_dm_insert<<<grid, 256, 0, s>>>(p);
     HX_CK_LAUNCH("k2_dm_insert");
-    ctx->launches += 4;
+    ctx->launches += 2;
     return HX_OK;
   }
   const int64_t slots_max = int64_t(1) << p.max_log2cap;
@@ -355,7 +390,7 @@ int ht_enqueue_build(hx_ctx* ctx, hx_ht* ht, cudaStream_t stream) {
   HX_CK_LAUNCH("k2_clear");
   k2_insert<<<grid, 256, 0, s>>>(p);
   HX_CK_LAUNCH("k2_insert");
-  ctx->launches += 4;
+  ctx->launches += 3;
   return HX_OK;
 }
 

@@ -45,6 +45,7 @@ struct HtHeader {
   // keeps ~min and max with atomicMax so that a zeroed header is the neutral element
   uint32_t kmin_inv;
   uint32_t kmax_enc;
+  uint32_t done;     // CTAs of the filter kernel finished (the last one ranks)
 };
 __host__ __device__ __forceinline__ uint32_t key_enc(int32_t k) { return (uint32_t)k ^ 0x80000000u; }
 __host__ __device__ __forceinline__ int32_t key_dec(uint32_t e) { return (int32_t)(e ^ 0x80000000u); }
@@ -126,6 +127,7 @@ struct hx_ctx {
   bool own_stream = false;
   int n_sms = 0;
   int k1_ctas_per_sm = 0;
+  int k1_priority = 0;  // launch priority of K1 (the device's greatest; builds keep the default)
   ncclComm_t comm = nullptr;
   int rank = 0, nranks = 1;
   // K1 profiling: event pairs around each launch

@@ -316,6 +316,9 @@ int hx_plans_enqueue(hx_ctx* ctx, hx_plan* const* plans, int n) {
     int rc = plan_enqueue_builds(ctx, plans[i]);
     if (rc != HX_OK) return rc;
   }
+  if (std::getenv("HX_SERIAL_BUILDS")) {  // A/B: every build done before the first pipeline
+    for (int i = 0; i < n; ++i) HX_CK(cudaStreamWaitEvent(ctx->stream, plans[i]->built_ev[0], 0));
+  }
   for (int i = 0; i < n; ++i) {
     int rc = plan_enqueue_probe(ctx, plans[i]);
     if (rc != HX_OK) return rc;
@@ -466,7 +469,9 @@ int hx_graph_end(hx_ctx* ctx, hx_graph** out) {
   hx_graph* g = new hx_graph();
   g->ctx = ctx;
   cudaError_t e = cudaStreamEndCapture(ctx->stream, &g->graph);
-  if (e == cudaSuccess) e = cudaGraphInstantiate(&g->exec, g->graph, 0);
+  // node priorities (K1's launch priority) are honoured only with this flag
+  if (e == cudaSuccess)
+    e = cudaGraphInstantiateWithFlags(&g->exec, g->graph, cudaGraphInstantiateFlagUseNodePriority);
   g->launches = ctx->launches - ctx->capture_launches;
   ctx->launches = ctx->capture_launches;  // captured, not executed
   g->d2h = ctx->d2h_bytes - ctx->capture_d2h;

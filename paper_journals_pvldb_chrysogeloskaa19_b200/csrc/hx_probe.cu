@@ -1234,6 +1234,24 @@ __global__ void k1_prepare(AggMeta* meta, const HtHeader* g0, const HtHeader* g1
 
 using KernelFn = void (*)(K1Params);
 
+// K1 launches carry the device's greatest priority: the builds of later queries (forked on
+// auxiliary streams so they overlap) then only take SMs that K1 leaves idle (its tail), and
+// the next K1's CTAs are dispatched ahead of queued build CTAs.
+cudaError_t launch_k1(KernelFn fn, int grid, int block, size_t smem, cudaStream_t s,
+                      const K1Params& p, int priority) {
+  cudaLaunchConfig_t cfg{};
+  cfg.gridDim = dim3((unsigned)grid);
+  cfg.blockDim = dim3((unsigned)block);
+  cfg.dynamicSmemBytes = smem;
+  cfg.stream = s;
+  cudaLaunchAttribute attr[1];
+  attr[0].id = cudaLaunchAttributePriority;
+  attr[0].val.priority = priority;
+  cfg.attrs = attr;
+  cfg.numAttrs = 1;
+  return cudaLaunchKernelEx(&cfg, fn, p);
+}
+
 // [direct maps][grouped][joins]; join-less pipelines use the hash-table instances
 const KernelFn kKernels[2][2][HX_MAX_JOINS + 1] = {
     {{k1_probe_agg<0, false, false>, k1_probe_agg<1, false, false>, k1_probe_agg<2, false, false>,
@@ -1823,8 +1841,7 @@ static int k1_enqueue_host(hx_ctx* ctx, const K1Prepared* k, StageRing* ring, cu
     p.n_rows = rows;
     p.n_tiles = (rows + kTileRows - 1) / kTileRows;
     const int grid = (int)std::max<int64_t>(1, std::min<int64_t>(p.n_tiles, (int64_t)ctx->n_sms * k->occ));
-    k->fn<<<(unsigned)grid, kThreads, k->smem, ctx->stream>>>(p);
-    HX_CK_LAUNCH("k1_probe_agg");
+    HX_CK(launch_k1(k->fn, grid, kThreads, k->smem, ctx->stream, p, ctx->k1_priority));
     ctx->launches += 1;
     HX_CK(cudaEventRecord(ring->freed[s], ctx->stream));
   }
@@ -1856,13 +1873,11 @@ int k1_enqueue(hx_ctx* ctx, const K1Prepared* k, bool fresh, cudaEvent_t e0, cud
   if (k->rows == 0) return HX_OK;
   if (k->host) return k1_enqueue_host(ctx, k, ring, e0, e1);
   if (e0) HX_CK(record_event(e0, ctx->stream));
-  if (k->scan) {
-    k->scan<<<(unsigned)k->scan_grid, kScanThreads + 32, k->scan_smem, ctx->stream>>>(p);
-    HX_CK_LAUNCH("k1_scan_agg");
-  } else {
-    k->fn<<<(unsigned)k->grid, kThreads, k->smem, ctx->stream>>>(p);
-    HX_CK_LAUNCH("k1_probe_agg");
-  }
+  if (k->scan)
+    HX_CK(launch_k1(k->scan, k->scan_grid, kScanThreads + 32, k->scan_smem, ctx->stream, p,
+                    ctx->k1_priority));
+  else
+    HX_CK(launch_k1(k->fn, k->grid, kThreads, k->smem, ctx->stream, p, ctx->k1_priority));
   ctx->launches += 1;
   if (k->mapped) ctx->h2d_bytes += k1_bytes(k);  // read over PCIe by the kernel itself
   if (e1) HX_CK(record_event(e1, ctx->stream));
