@@ -27,11 +27,16 @@ def main(tag, rep, launches):
            "planned execution of each query). ncu times are cold-cache and serialised: compare shares.", "",
            "| query | kernel | ncu us | algorithmic GB | DRAM r+w GB | traffic/alg | L2 hit % | issue active % | warps active % | regs |",
            "|---|---|---|---|---|---|---|---|---|---|"]
+    def scaled(d, name):  # ncu raw values carry their unit in the second header row
+        unit = rows[1][c(name)]
+        mult = {"byte": 1, "Kbyte": 1e3, "Mbyte": 1e6, "Gbyte": 1e9, "KB": 1e3, "MB": 1e6, "GB": 1e9}
+        return float(d[c(name)] or 0) * mult.get(unit, 1)
+
     tt = ta = tr = 0.0
     for q, d in zip(QS, data):
         t = float(d[c("gpu__time_duration.sum")])
-        rd = float(d[c("dram__bytes_read.sum")]) * 1e9
-        wr = float(d[c("dram__bytes_write.sum")]) * 1e6
+        rd = scaled(d, "dram__bytes_read.sum")
+        wr = scaled(d, "dram__bytes_write.sum")
         alg = N * BROW[q[1]]
         tt, ta, tr = tt + t, ta + alg, tr + rd + wr
         out.append(f"| {q} | {d[c('Kernel Name')].split('(')[0].split('::')[-1]} | {t:.1f} | {alg/1e9:.3f} | "
