@@ -139,7 +139,8 @@ struct hx_graph {
 };
 
 static int plan_enqueue_builds(hx_ctx* ctx, hx_plan* pl);
-static int plan_enqueue_probe(hx_ctx* ctx, hx_plan* pl);
+static int plan_enqueue_probe(hx_ctx* ctx, hx_plan* pl, bool merge = true);
+static int plan_enqueue_finish(hx_ctx* ctx, hx_plan* pl);
 static int join_fin(hx_ctx* ctx);
 
 static void plan_destroy(hx_plan* pl) {
@@ -319,9 +320,31 @@ int hx_plans_enqueue(hx_ctx* ctx, hx_plan* const* plans, int n) {
   if (std::getenv("HX_SERIAL_BUILDS")) {  // A/B: every build done before the first pipeline
     for (int i = 0; i < n; ++i) HX_CK(cudaStreamWaitEvent(ctx->stream, plans[i]->built_ev[0], 0));
   }
+  // > 1 rank: the pipelines run back to back and the union-router merges of all plans go
+  // out as ONE grouped NCCL launch after the last of them (a per-plan allreduce would put
+  // 13 collective latencies between the pipelines)
+  const bool grouped = ctx->comm && ctx->nranks > 1 && n > 1;
   for (int i = 0; i < n; ++i) {
-    int rc = plan_enqueue_probe(ctx, plans[i]);
+    int rc = plan_enqueue_probe(ctx, plans[i], /*merge=*/!grouped);
     if (rc != HX_OK) return rc;
+  }
+  if (grouped) {
+    HX_REQUIRE(ncclGroupStart() == ncclSuccess, HX_ENCCL, "ncclGroupStart");
+    for (int i = 0; i < n; ++i) {
+      ncclResult_t r = ncclAllReduce(plans[i]->agg.sums, plans[i]->agg.sums,
+                                     2 * (size_t)plans[i]->n_groups, ncclUint64, ncclSum,
+                                     ctx->comm, ctx->stream);
+      if (r != ncclSuccess) {
+        ncclGroupEnd();
+        return fail(HX_ENCCL, std::string("ncclAllReduce: ") + ncclGetErrorString(r));
+      }
+    }
+    ncclResult_t r = ncclGroupEnd();
+    HX_REQUIRE(r == ncclSuccess, HX_ENCCL, std::string("ncclGroupEnd: ") + ncclGetErrorString(r));
+    for (int i = 0; i < n; ++i) {
+      int rc = plan_enqueue_finish(ctx, plans[i]);
+      if (rc != HX_OK) return rc;
+    }
   }
   return n > 0 ? join_fin(ctx) : HX_OK;
 }
@@ -349,16 +372,23 @@ static int plan_enqueue_builds(hx_ctx* ctx, hx_plan* pl) {
 
 // K1 (after the plan's builds) -> merge on the main stream; finalize -> D2H on the finalize
 // stream, so the next plan's K1 starts as soon as this one's merge is done
-static int plan_enqueue_probe(hx_ctx* ctx, hx_plan* pl) {
+static int plan_enqueue_probe(hx_ctx* ctx, hx_plan* pl, bool merge) {
   HX_CK(cudaStreamWaitEvent(ctx->stream, pl->built_ev[0], 0));
   int rc = k1_enqueue(ctx, pl->k1, true, pl->k1_e0, pl->k1_e1, pl->ring, /*prepare=*/false);
   if (rc != HX_OK) return rc;
+  if (!merge) return HX_OK;  // the caller merges (grouped) and finishes
   if (ctx->comm && ctx->nranks > 1) {
     // union router: partial {sum,cnt} arrays are adjacent, one allreduce over NVLink
     ncclResult_t r = ncclAllReduce(pl->agg.sums, pl->agg.sums, 2 * (size_t)pl->n_groups,
                                    ncclUint64, ncclSum, ctx->comm, ctx->stream);
     HX_REQUIRE(r == ncclSuccess, HX_ENCCL, std::string("ncclAllReduce: ") + ncclGetErrorString(r));
   }
+  return plan_enqueue_finish(ctx, pl);
+}
+
+// after the (merged) group arrays are final on the main stream: finalize -> D2H on the
+// finalize stream
+static int plan_enqueue_finish(hx_ctx* ctx, hx_plan* pl) {
   HX_CK(cudaEventRecord(pl->probed, ctx->stream));
   HX_CK(cudaStreamWaitEvent(ctx->fin_stream, pl->probed, 0));
   k1_finalize<<<1, 1024, 0, ctx->fin_stream>>>(pl->fin);
