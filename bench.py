@@ -86,7 +86,9 @@ def workload_name(sf, world, variant="hbm", queries=None):
                else "read in place over PCIe by K1 through UVA (zero-copy)")
         return (f"SSB {'/'.join(q.upper() for q in queries)}, SF{sf:g} per GPU (SF{sf * world:g} "
                 f"total), lineorder host-resident in pinned memory, {how}")
-    return f"SSB all 13 queries, SF{sf:g} per GPU (SF{sf * world:g} total), HBM-resident"
+    which = ("all 13 queries" if queries is None or len(queries) == 13
+             else "/".join(q.upper() for q in queries))
+    return f"SSB {which}, SF{sf:g} per GPU (SF{sf * world:g} total), HBM-resident"
 
 
 def config(args, world, n_rows_gpu, queries):
@@ -353,6 +355,10 @@ def main():
     else:
         queries = args.queries.split(",")
     C = ssbgen.COLS
+    # only the lineorder columns the selected queries reference are placed (SF1000 on one
+    # GPU: the 6 columns of Q2-Q4 = 144 GB or the 4 of Q1 = 96 GB fit HBM; all 9 do not)
+    need = set().union(*(ssb.FACT_COLS[q] for q in queries))
+    lo_cols = [c for c in ssbgen.TABLE_COLS["lineorder"] if C[c] in need]
 
     # ---- data in HBM: this rank's router blocks of lineorder, full replicated dims -------
     sz = ssbgen.sizes(args.sf * world)
@@ -377,7 +383,7 @@ def main():
         # §8(a) a8: lineorder stays in page-locked host memory; K1 streams it over PCIe
         # (host: DMA into a device staging ring; uva: K1's bulk copies read it in place)
         spec = []
-        for c in ssbgen.TABLE_COLS["lineorder"]:
+        for c in lo_cols:
             buf = torch.empty(max(n_mine, 1), dtype=torch.int32, pin_memory=True)
             ssbgen.column(SEED, sz, c, r0, n_mine, out=buf.numpy())
             keep.append(buf)
@@ -385,7 +391,7 @@ def main():
         fact = hx.load_columns(ctx, spec, placement=hx._hx.HX_PLACE_HOST_PINNED if args.variant == "host"
                                else hx._hx.HX_PLACE_HOST_MAPPED)
     else:
-        fact = dev_table(ssbgen.TABLE_COLS["lineorder"], r0, n_mine)
+        fact = dev_table(lo_cols, r0, n_mine)
     torch.cuda.synchronize()
     eng = ssb.SsbEngine(ctx, dims, fact)
     # one prepared plan per query (HT + group buffers allocated once, builds sized once);
@@ -393,7 +399,8 @@ def main():
     # the 13 host reads of the finalized results. Two such plan sets alternate (steps i and
     # i+1 use different buffers), so the host reads step i's results while the device
     # already runs step i+1 — every step still builds, probes, merges and reads everything.
-    n_sets = 1 if (args.no_graph or args.no_pipeline) else 2
+    big = n_mine * 4 * len(lo_cols) > (64 << 30)  # SF >= ~300 per GPU: one plan set fits
+    n_sets = 1 if (args.no_graph or args.no_pipeline or big) else 2
     sets = []
     for _ in range(n_sets):
         pl_ = {q: eng.plan(q) for q in queries}
@@ -545,11 +552,14 @@ def main():
                        if args.variant == "host" else
                        ("plans over a HX_PLACE_HOST_MAPPED fact table: K1 reads pinned host "
                         "memory in place over PCIe + merge + finalize + D2H, one CUDA graph per step")}
+    elif not args.no_e2e and n_mine * 4 * len(lo_cols) > (32 << 30):
+        e2e = {"value": None, "unit": UNIT, "skipped": "lineorder partition larger than the "
+               "32 GB of pinned host memory this run allocates for the e2e leg"}
     elif not args.no_e2e:
         host = {}
         for t in ("lineorder", "date", "customer", "supplier", "part"):
             host[t] = {}
-            for c in ssbgen.TABLE_COLS[t]:
+            for c in (lo_cols if t == "lineorder" else ssbgen.TABLE_COLS[t]):
                 n = n_mine if t == "lineorder" else ssbgen.table_rows(sz, c)
                 buf = torch.empty(max(n, 1), dtype=torch.int32, pin_memory=True)
                 ssbgen.column(SEED, sz, c, r0 if t == "lineorder" else 0, n, out=buf.numpy())

@@ -104,13 +104,13 @@ const std::vector<R>& lookup(const Index<R>& idx, int32_t key) {
   return it == idx.end() ? none : it->second;
 }
 
-struct Db {
-  const oracle_db& t;
+// The dimension indexes (built once per database) and the lineorder columns a query scans.
+struct Indexes {
   Index<DateRow> date;
   Index<CustRow> cust;
   Index<SuppRow> supp;
   Index<PartRow> part;
-  explicit Db(const oracle_db& db) : t(db) {
+  explicit Indexes(const oracle_db& db) {
     for (int64_t i = 0; i < db.n_date; ++i)
       date[db.d_datekey[i]].push_back({db.d_year[i], db.d_yearmonthnum[i], db.d_weeknuminyear[i]});
     for (int64_t i = 0; i < db.n_cust; ++i)
@@ -120,6 +120,10 @@ struct Db {
     for (int64_t i = 0; i < db.n_part; ++i)
       part[db.p_partkey[i]].push_back({db.p_mfgr[i], db.p_category[i], db.p_brand1[i]});
   }
+};
+struct Db {
+  const oracle_db& t;   // lineorder columns
+  const Indexes* ix;    // dimension rows by primary key
 };
 
 using Key = std::array<int32_t, 3>;
@@ -138,14 +142,14 @@ inline void add(Groups& g, Key k, int64_t v) {
 void q1_1(const Db& db, int64_t b, int64_t e, Groups& g) {
   const oracle_db& t = db.t;
   for (int64_t i = b; i < e; ++i)
-    for (const DateRow& d : lookup(db.date, t.lo_orderdate[i]))
+    for (const DateRow& d : lookup(db.ix->date, t.lo_orderdate[i]))
       if (d.year == 1993 && t.lo_discount[i] >= 1 && t.lo_discount[i] <= 3 && t.lo_quantity[i] < 25)
         add(g, {0, 0, 0}, (int64_t)t.lo_extendedprice[i] * t.lo_discount[i]);
 }
 void q1_2(const Db& db, int64_t b, int64_t e, Groups& g) {
   const oracle_db& t = db.t;
   for (int64_t i = b; i < e; ++i)
-    for (const DateRow& d : lookup(db.date, t.lo_orderdate[i]))
+    for (const DateRow& d : lookup(db.ix->date, t.lo_orderdate[i]))
       if (d.yearmonthnum == 199401 && t.lo_discount[i] >= 4 && t.lo_discount[i] <= 6 &&
           t.lo_quantity[i] >= 26 && t.lo_quantity[i] <= 35)
         add(g, {0, 0, 0}, (int64_t)t.lo_extendedprice[i] * t.lo_discount[i]);
@@ -153,7 +157,7 @@ void q1_2(const Db& db, int64_t b, int64_t e, Groups& g) {
 void q1_3(const Db& db, int64_t b, int64_t e, Groups& g) {
   const oracle_db& t = db.t;
   for (int64_t i = b; i < e; ++i)
-    for (const DateRow& d : lookup(db.date, t.lo_orderdate[i]))
+    for (const DateRow& d : lookup(db.ix->date, t.lo_orderdate[i]))
       if (d.weeknuminyear == 6 && d.year == 1994 && t.lo_discount[i] >= 5 &&
           t.lo_discount[i] <= 7 && t.lo_quantity[i] >= 26 && t.lo_quantity[i] <= 35)
         add(g, {0, 0, 0}, (int64_t)t.lo_extendedprice[i] * t.lo_discount[i]);
@@ -166,9 +170,9 @@ template <class PartPred, class SuppPred>
 void q2(const Db& db, int64_t b, int64_t e, Groups& g, PartPred pp, SuppPred sp) {
   const oracle_db& t = db.t;
   for (int64_t i = b; i < e; ++i)
-    for (const DateRow& d : lookup(db.date, t.lo_orderdate[i]))
-      for (const PartRow& p : lookup(db.part, t.lo_partkey[i]))
-        for (const SuppRow& s : lookup(db.supp, t.lo_suppkey[i]))
+    for (const DateRow& d : lookup(db.ix->date, t.lo_orderdate[i]))
+      for (const PartRow& p : lookup(db.ix->part, t.lo_partkey[i]))
+        for (const SuppRow& s : lookup(db.ix->supp, t.lo_suppkey[i]))
           if (pp(p) && sp(s)) add(g, {d.year, p.brand1, 0}, t.lo_revenue[i]);
 }
 void q2_1(const Db& db, int64_t b, int64_t e, Groups& g) {
@@ -195,9 +199,9 @@ template <class CP, class SP, class DP, class CK, class SK>
 void q3(const Db& db, int64_t b, int64_t e, Groups& g, CP cp, SP sp, DP dp, CK ck, SK sk) {
   const oracle_db& t = db.t;
   for (int64_t i = b; i < e; ++i)
-    for (const CustRow& c : lookup(db.cust, t.lo_custkey[i]))
-      for (const SuppRow& s : lookup(db.supp, t.lo_suppkey[i]))
-        for (const DateRow& d : lookup(db.date, t.lo_orderdate[i]))
+    for (const CustRow& c : lookup(db.ix->cust, t.lo_custkey[i]))
+      for (const SuppRow& s : lookup(db.ix->supp, t.lo_suppkey[i]))
+        for (const DateRow& d : lookup(db.ix->date, t.lo_orderdate[i]))
           if (cp(c) && sp(s) && dp(d)) add(g, {ck(c), sk(s), d.year}, t.lo_revenue[i]);
 }
 void q3_1(const Db& db, int64_t b, int64_t e, Groups& g) {
@@ -238,10 +242,10 @@ template <class Pred, class KeyF>
 void q4(const Db& db, int64_t b, int64_t e, Groups& g, Pred pred, KeyF key) {
   const oracle_db& t = db.t;
   for (int64_t i = b; i < e; ++i)
-    for (const DateRow& d : lookup(db.date, t.lo_orderdate[i]))
-      for (const CustRow& c : lookup(db.cust, t.lo_custkey[i]))
-        for (const SuppRow& s : lookup(db.supp, t.lo_suppkey[i]))
-          for (const PartRow& p : lookup(db.part, t.lo_partkey[i]))
+    for (const DateRow& d : lookup(db.ix->date, t.lo_orderdate[i]))
+      for (const CustRow& c : lookup(db.ix->cust, t.lo_custkey[i]))
+        for (const SuppRow& s : lookup(db.ix->supp, t.lo_suppkey[i]))
+          for (const PartRow& p : lookup(db.ix->part, t.lo_partkey[i]))
             if (pred(d, c, s, p))
               add(g, key(d, c, s, p), (int64_t)t.lo_revenue[i] - (int64_t)t.lo_supplycost[i]);
 }
@@ -292,6 +296,8 @@ const QueryDef kQueries[] = {
     {"q4.1", q4_1, 2, 1}, {"q4.2", q4_2, 3, 1}, {"q4.3", q4_3, 3, 1},
 };
 
+int64_t run_query(const char* qname, const Indexes& ix, const oracle_db* db, int64_t row_begin,
+                  int64_t row_end, oracle_row* out, int64_t cap);
 }  // namespace
 
 extern "C" {
@@ -303,12 +309,36 @@ extern "C" {
    row count, -1 for an unknown query or bad range, -2 if cap is too small. */
 int64_t oracle_ssb_query(const char* qname, const oracle_db* db, int64_t row_begin,
                          int64_t row_end, oracle_row* out, int64_t cap) {
+  if (!db) return -1;
+  const Indexes ix(*db);
+  return run_query(qname, ix, db, row_begin, row_end, out, cap);
+}
+
+/* The same over a prebuilt index of the dimension tables (oracle_index_new), so that many
+   lineorder chunks (e.g. SF1000 regenerated 100 M rows at a time, on several threads) are
+   evaluated without rebuilding the dimension maps: `lo` supplies only the lineorder columns
+   (its dimension fields are ignored). The index is read-only here and may be shared. */
+int64_t oracle_ssb_query_idx(const char* qname, const void* index, const oracle_db* lo,
+                             int64_t row_begin, int64_t row_end, oracle_row* out, int64_t cap) {
+  if (!index) return -1;
+  return run_query(qname, *static_cast<const Indexes*>(index), lo, row_begin, row_end, out, cap);
+}
+
+/* Builds the dimension indexes of `db` (its lineorder fields are ignored); caller frees. */
+void* oracle_index_new(const oracle_db* db) { return db ? new Indexes(*db) : nullptr; }
+void oracle_index_free(void* index) { delete static_cast<Indexes*>(index); }
+
+}  // extern "C"
+
+namespace {
+int64_t run_query(const char* qname, const Indexes& ix, const oracle_db* db, int64_t row_begin,
+                  int64_t row_end, oracle_row* out, int64_t cap) {
   if (!qname || !db || row_begin < 0 || row_end < row_begin || row_end > db->n_lo) return -1;
   const QueryDef* q = nullptr;
   for (const QueryDef& d : kQueries)
     if (std::strcmp(d.name, qname) == 0) q = &d;
   if (!q) return -1;
-  Db index(*db);
+  const Db index{*db, &ix};
   Groups g;
   q->run(index, row_begin, row_end, g);
   std::vector<std::pair<Key, Acc>> rows(g.begin(), g.end());  // std::map: keys ascending
@@ -327,6 +357,9 @@ int64_t oracle_ssb_query(const char* qname, const oracle_db* db, int64_t row_beg
   }
   return (int64_t)rows.size();
 }
+}  // namespace
+
+extern "C" {
 
 /* Encodes an SSB string literal with the oracle's own dictionary (kind: 0 region,
    1 nation, 2 city, 3 mfgr, 4 category, 5 brand1). Exposed so tests can check it agrees with

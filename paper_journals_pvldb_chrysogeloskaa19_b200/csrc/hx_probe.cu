@@ -54,6 +54,8 @@ constexpr int kConsumers = kConsumerWarps * 32;
 constexpr int kThreads = kConsumers + 32;  // + one producer warp
 constexpr int kRowsPerThread = 4;          // R
 constexpr int kTileRows = kConsumers * kRowsPerThread;  // T = 2560 rows
+// rows per K1 launch: whole tiles, < 2^32 - kTileRows (32-bit row offsets inside a launch)
+constexpr int64_t kSegRows = int64_t(kTileRows) * (int64_t(1) << 20);  // 2.68e9 rows
 constexpr int kCtasPerSm = HX_K1_CTAS;    // target residency (registers, smem budget)
 constexpr int kMaxStageCols = 8;
 constexpr int kSmemGroups = 1024;          // per-CTA group table capacity
@@ -1457,6 +1459,7 @@ struct K1Prepared {
   size_t scan_smem = 0;
   const int32_t* host_col[kMaxStageCols] = {};
   int occ = 1;
+  int64_t seg_rows = kSegRows;  // rows per launch (HX_K1_SEG_TILES overrides, for tests)
 };
 
 // Device staging ring of the mem-move for a host-resident fact table: kRingStages buffers of
@@ -1768,6 +1771,10 @@ int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht*
   k.grid = (int)std::max<int64_t>(1, std::min<int64_t>(p.n_tiles, (int64_t)ctx->n_sms * occ));
   k.rows = fact->n_rows;
   k.n_cols = n_cols;
+  if (const char* e = std::getenv("HX_K1_SEG_TILES")) {
+    const long long t = std::atoll(e);
+    if (t > 0 && t <= (1LL << 20)) k.seg_rows = t * kTileRows;
+  }
   if (sh->n_joins == 0 && n_cols >= 1 && n_cols <= 4 && !k.host &&
       std::getenv("HX_NO_SCAN") == nullptr) {
     const KernelFn scans[4] = {k1_scan_agg<1>, k1_scan_agg<2>, k1_scan_agg<3>, k1_scan_agg<4>};
@@ -1873,12 +1880,29 @@ int k1_enqueue(hx_ctx* ctx, const K1Prepared* k, bool fresh, cudaEvent_t e0, cud
   if (k->rows == 0) return HX_OK;
   if (k->host) return k1_enqueue_host(ctx, k, ring, e0, e1);
   if (e0) HX_CK(record_event(e0, ctx->stream));
-  if (k->scan)
+  if (k->scan) {
     HX_CK(launch_k1(k->scan, k->scan_grid, kScanThreads + 32, k->scan_smem, ctx->stream, p,
                     ctx->k1_priority));
-  else
-    HX_CK(launch_k1(k->fn, k->grid, kThreads, k->smem, ctx->stream, p, ctx->k1_priority));
-  ctx->launches += 1;
+    ctx->launches += 1;
+  } else {
+    // K1 addresses gathered measures and carried rows by a 32-bit row offset: a table of
+    // more rows (one GPU's SF1000 partition: 6e9) runs as consecutive launches over segments
+    // of kSegRows rows (whole tiles, 16-byte aligned), accumulating into the same groups.
+    for (int64_t s0 = 0; s0 < p.n_rows; s0 += k->seg_rows) {
+      K1Params q = p;
+      if (s0 > 0) {
+        for (int c = 0; c < p.n_cols; ++c) q.col[c] = q.head_col[c] = p.col[c] + s0;
+        q.head_rows = 0;
+        if (p.ga) q.gat_a = p.gat_a + p.head_rows + s0;
+        if (p.gb) q.gat_b = p.gat_b + p.head_rows + s0;
+      }
+      q.n_rows = std::min<int64_t>(k->seg_rows, p.n_rows - s0);
+      q.n_tiles = (q.n_rows + kTileRows - 1) / kTileRows;
+      const int grid = (int)std::max<int64_t>(1, std::min<int64_t>(q.n_tiles, (int64_t)k->grid));
+      HX_CK(launch_k1(k->fn, grid, kThreads, k->smem, ctx->stream, q, ctx->k1_priority));
+      ctx->launches += 1;
+    }
+  }
   if (k->mapped) ctx->h2d_bytes += k1_bytes(k);  // read over PCIe by the kernel itself
   if (e1) HX_CK(record_event(e1, ctx->stream));
   return HX_OK;

@@ -141,6 +141,27 @@ def test_misaligned_views(ctx, offset):
         assert eng.run(q) == oracle.run_query(q, db, offset, n - 7), q
 
 
+@pytest.mark.parametrize("seg_tiles,offset", [(1, 0), (3, 3), (7, 1)])
+def test_k1_launch_segments(ctx, monkeypatch, seg_tiles, offset):
+    """A fact table beyond 32-bit row offsets (one GPU's SF1000 partition, 6e9 rows) runs as
+    consecutive K1 launches over whole-tile segments accumulating into the same groups.
+    HX_K1_SEG_TILES shrinks the segment to 1-7 tiles so that SF0.05 (117 tiles, a ragged
+    tail, misaligned head rows) crosses dozens of boundaries; gathered measures included."""
+    monkeypatch.setenv("HX_K1_SEG_TILES", str(seg_tiles))
+    db = ssbgen.database(9, ssbgen.sizes(0.05))
+    dims, fact = ssb.load_db_numpy(ctx, db)
+    n = fact.n_rows
+    sl = fact.slice(offset, n) if offset else fact
+    eng = ssb.SsbEngine(ctx, dims, sl)
+    for q in QUERIES:
+        want = oracle.run_query(q, db, offset, n)
+        assert eng.run(q) == want, q
+        pl = eng.plan(q)
+        pl.enqueue()
+        assert pl.rows() == want, q
+        pl.close()
+
+
 @pytest.mark.parametrize("seed", [3, 8])
 def test_plans_and_graph_replay(ctx, seed):
     """Prepared plans (device finalize) and a CUDA graph of all 13 executions, replayed

@@ -185,3 +185,16 @@ def test_selectivity_sf1(sf1, q):
     pf = _expected_fraction(q, sf1)
     mu, sigma = n * pf, np.sqrt(n * pf * (1 - pf))
     assert abs(survivors - mu) < 5 * sigma + 1, (q, survivors, mu, sigma)
+
+
+def test_dim_index_chunks_equal_run_query():
+    """oracle.DimIndex (dimension maps built once, lineorder evaluated chunk by chunk on
+    threads, partials summed) gives run_query's result: the SF1000 parity helper."""
+    sz = ssbgen.sizes(0.2)
+    db = ssbgen.database(5, sz)
+    lo = db["lineorder"]
+    n = sz["n_lineorder"]
+    got = oracle.run_queries_generated(oracle.QUERIES, db, lambda b, k: {c: v[b:b + k] for c, v in lo.items()},
+                                       [(0, 400_000), (400_000, n)], 3, chunk_rows=300_001)
+    for q in oracle.QUERIES:
+        assert got[q] == oracle.as_dict(oracle.run_query(q, db)), q

@@ -15,7 +15,7 @@ import ssbgen  # noqa: E402
 from paper_journals_pvldb_chrysogeloskaa19_b200 import _hx, hx, ssb  # noqa: E402
 
 
-def device_db(ctx, sz, seed=42):
+def device_db(ctx, sz, seed=42, lo_rows=None, lo_cols=None):
     keep, stream = [], torch.cuda.current_stream().cuda_stream
 
     def table(cols, n):
@@ -29,7 +29,8 @@ def device_db(ctx, sz, seed=42):
 
     dims = {t: table(ssbgen.TABLE_COLS[t], ssbgen.table_rows(sz, ssbgen.TABLE_COLS[t][0]))
             for t in ("date", "customer", "supplier", "part")}
-    fact = table(ssbgen.TABLE_COLS["lineorder"], sz["n_lineorder"])
+    n = sz["n_lineorder"] if lo_rows is None else min(lo_rows, sz["n_lineorder"])
+    fact = table(lo_cols or ssbgen.TABLE_COLS["lineorder"], n)
     torch.cuda.synchronize()
     return dims, fact
 

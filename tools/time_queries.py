@@ -20,11 +20,14 @@ ap = argparse.ArgumentParser()
 ap.add_argument("--sf", type=float, default=10)
 ap.add_argument("--queries", default="all")
 ap.add_argument("--reps", type=int, default=5)
+ap.add_argument("--lo-rows", type=int, default=0, help="first rows of lineorder only (SF1000 dims)")
 a = ap.parse_args()
 ctx = hx.Context(0)
-dims, fact = device_db(ctx, ssbgen.sizes(a.sf))
-eng = ssb.SsbEngine(ctx, dims, fact)
 qs = ssb.QUERIES if a.queries == "all" else a.queries.split(",")
+need = set().union(*(ssb.FACT_COLS[q] for q in qs))
+dims, fact = device_db(ctx, ssbgen.sizes(a.sf), lo_rows=a.lo_rows or None,
+                       lo_cols=[c for c in ssbgen.TABLE_COLS["lineorder"] if ssbgen.COLS[c] in need])
+eng = ssb.SsbEngine(ctx, dims, fact)
 plans = {q: eng.plan(q) for q in qs}
 tot = 0.0
 for q in qs:
@@ -35,7 +38,8 @@ for q in qs:
         ts.append(plans[q].hp.k1_time()[0])
     ts.sort()
     tot += ts[len(ts) // 2]
-    print(f"{q} k1 median {ts[len(ts) // 2]:.4f} ms  min {ts[0]:.4f}  all {' '.join(f'{t:.3f}' for t in ts)}")
+    n = fact.n_rows
+    print(f"{q} {n * 4 * len(ssb.FACT_COLS[q]) / (ts[len(ts) // 2] / 1e3) / 1e9:7.0f} GB/s  k1 median {ts[len(ts) // 2]:.4f} ms  min {ts[0]:.4f}  all {' '.join(f'{t:.3f}' for t in ts)}")
 print(f"sum of medians {tot:.4f} ms")
 for pl in plans.values():
     pl.close()
