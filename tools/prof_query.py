@@ -40,11 +40,14 @@ def main():
     ap.add_argument("--sf", type=float, default=10)
     ap.add_argument("--queries", default="q1.1,q2.1,q3.1,q4.1")
     ap.add_argument("--reps", type=int, default=2)
+    ap.add_argument("--lo-rows", type=int, default=0, help="first rows of lineorder only")
     a = ap.parse_args()
     ctx = hx.Context(0, torch.cuda.current_stream().cuda_stream)
-    dims, fact = device_db(ctx, ssbgen.sizes(a.sf))
-    eng = ssb.SsbEngine(ctx, dims, fact)
     qs = ssb.QUERIES if a.queries == "all" else a.queries.split(",")
+    need = set().union(*(ssb.FACT_COLS[q] for q in qs))
+    dims, fact = device_db(ctx, ssbgen.sizes(a.sf), lo_rows=a.lo_rows or None,
+                           lo_cols=[c for c in ssbgen.TABLE_COLS["lineorder"] if ssbgen.COLS[c] in need])
+    eng = ssb.SsbEngine(ctx, dims, fact)
     plans = {q: eng.plan(q) for q in qs}  # the bench's execution path (prepared plans)
     for _ in range(a.reps):
         for q in qs:
