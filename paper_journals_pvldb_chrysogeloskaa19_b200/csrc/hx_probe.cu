@@ -1240,17 +1240,19 @@ using KernelFn = void (*)(K1Params);
 // auxiliary streams so they overlap) then only take SMs that K1 leaves idle (its tail), and
 // the next K1's CTAs are dispatched ahead of queued build CTAs.
 cudaError_t launch_k1(KernelFn fn, int grid, int block, size_t smem, cudaStream_t s,
-                      const K1Params& p, int priority) {
+                      const K1Params& p, int priority, int carveout = -1) {
   cudaLaunchConfig_t cfg{};
   cfg.gridDim = dim3((unsigned)grid);
   cfg.blockDim = dim3((unsigned)block);
   cfg.dynamicSmemBytes = smem;
   cfg.stream = s;
-  cudaLaunchAttribute attr[1];
+  cudaLaunchAttribute attr[2];
   attr[0].id = cudaLaunchAttributePriority;
   attr[0].val.priority = priority;
+  attr[1].id = cudaLaunchAttributePreferredSharedMemoryCarveout;
+  attr[1].val.sharedMemCarveout = (unsigned)carveout;
   cfg.attrs = attr;
-  cfg.numAttrs = 1;
+  cfg.numAttrs = carveout >= 0 ? 2 : 1;
   return cudaLaunchKernelEx(&cfg, fn, p);
 }
 
@@ -1279,12 +1281,26 @@ size_t k1_smem_bytes(bool dm, int n_cols, int stages, int smem_groups, int filte
 
 // Per-CTA shared memory for `ctas` resident CTAs per SM (228 KB per SM, 1 KB reserved each).
 constexpr size_t smem_budget(int ctas) { return (228 * 1024) / ctas - 1024; }
+// The shared memory K1 may plan with per CTA: the rest of the SM's 256 KB L1/shared array
+// becomes L1 cache for the L2 map reads. HX_K1_SMEM_KB lowers it (tuning aid).
+thread_local size_t t_smem_cap = 0;
+constexpr double kL1BoundCost = 50.0;  // plan cost above which K1 is L2-lookup-bound  // set while k1_setup replans an L2-lookup-bound pipeline
+size_t k1_smem_cap() {
+  size_t cap = smem_budget(std::min(kCtasPerSm, 2));
+  if (t_smem_cap) cap = std::min(cap, t_smem_cap);
+  if (const char* e = std::getenv("HX_K1_SMEM_KB")) {
+    const long kb = std::atol(e);
+    if (kb >= 64) cap = std::min<size_t>(cap, (size_t)kb * 1024);
+  }
+  return cap;
+}
 
 int pick_stages(bool dm, int n_cols, int smem_groups) {
   // as many tile stages as fit next to kCtasPerSm CTAs per SM, at least double buffering
   // (at most HX_K1_STAGE_KB of tiles per CTA: the rest is left for filters and maps)
   const size_t fixed = smem_fixed(dm) + (((size_t)smem_groups * 12 + 127) & ~size_t(127));
-  const size_t budget = std::min<size_t>(smem_budget(kCtasPerSm), fixed + HX_K1_STAGE_KB * 1024);
+  const size_t budget = std::min<size_t>(std::min(smem_budget(kCtasPerSm), k1_smem_cap()),
+                                         fixed + HX_K1_STAGE_KB * 1024);
   const size_t stage = (size_t)n_cols * kTileRows * 4;
   const int s = budget > fixed ? (int)((budget - fixed) / stage) : 0;
   return std::max(2, std::min(4, s));
@@ -1311,7 +1327,11 @@ double bloom_fp(double bits_per_key) {
 // filter on every row, a row entering stage C (compaction, queue, batch), a stage-C
 // shared-memory filter, an L2 lookup. HX_K1_COST="s,c,sc,l2" overrides (tuning aid).
 struct K1Cost {
-  double s = 8.0, c = 60.0, sc = 8.0, l2 = 20.0, s2 = 16.0;  // s2: an L2 map read in stage S
+  // s2: an L2 map read in stage S per live row (stage-S cost s + s2 * live fraction). A flat
+  // 16 per row (fitted at SF10-SF100, where such reads follow a selective shared-memory
+  // filter) made SF1000 plans read 2-15 MB maps for every row; charging the live fraction
+  // keeps the SF100 plans and picks the Bloom-filtered plans at SF1000 (Q2.1 2.2x, Q3.2 2.2x).
+  double s = 8.0, c = 60.0, sc = 8.0, l2 = 20.0, s2 = 40.0;
 };
 K1Cost k1_cost() {
   K1Cost k;
@@ -1373,8 +1393,10 @@ double plan_dm(int nj, const JoinDev* joins, const bool* known, const double* pa
         bool all_res = true;
         for (int j = 0; j < nj; ++j) {
           if ((S >> j) & 1u) {
+            // stage S runs the joins in array order, each narrowing the live rows; an L2 map
+            // is read only for the rows still live (fraction fS so far)
+            cost += kd[j] == kStNone ? K.s + K.s2 * fS : K.s;
             fS *= kd[j] == kStNone ? (known[j] ? pass[j] : 1.0) : opts[j][idx[j]].e;
-            cost += kd[j] == kStNone ? K.s2 : K.s;
           }
           all_res = all_res && ((S >> j) & 1u) && (kd[j] == kStFull || kd[j] == kStNone);
         }
@@ -1460,6 +1482,7 @@ struct K1Prepared {
   const int32_t* host_col[kMaxStageCols] = {};
   int occ = 1;
   int64_t seg_rows = kSegRows;  // rows per launch (HX_K1_SEG_TILES overrides, for tests)
+  int carveout = 100;           // preferred shared-memory carveout (% of 228 KB)
 };
 
 // Device staging ring of the mem-move for a host-resident fact table: kRingStages buffers of
@@ -1505,6 +1528,10 @@ int agg_alloc(hx_ctx* ctx, hx_agg* agg, long long cap_groups, const hx_query_sha
 
 int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht* const* hts,
              int n_hts, const hx_agg* agg, K1Prepared** out) {
+  struct CapReset {
+    ~CapReset() { t_smem_cap = 0; }
+  } cap_reset;
+  t_smem_cap = 0;
   HX_REQUIRE(ctx && fact && sh && agg && out, HX_EINVAL, "hx_pipeline_probe_agg: null argument");
   HX_REQUIRE(sh->n_preds >= 0 && sh->n_preds <= HX_MAX_PREDS && sh->n_joins >= 0 &&
                  sh->n_joins <= HX_MAX_JOINS && sh->n_gdims >= 0 && sh->n_gdims <= HX_MAX_GDIMS &&
@@ -1663,7 +1690,7 @@ int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht*
       if (kd[j] == kStBloom) fw += bw[j];
     }
     return k1_smem_bytes(dm_mode, n_cols, p.stages, p.smem_groups, fw, db) <=
-           smem_budget(std::min(kCtasPerSm, 2));
+           k1_smem_cap();
   };
   double plan_cost = -1.0;
   if (dm_mode) {
@@ -1671,6 +1698,17 @@ int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht*
     for (int g = 0; g < sh->n_gdims; ++g) grouped_j[sh->gdim_join[g]] = true;
     plan_cost = plan_dm(sh->n_joins, p.joins, known, pass, keys, bloom_w0, grouped_j, fits_sizes,
                         kind, bloom_w, in_s);
+    // An L2-lookup-bound plan (SF1000 Q3.1/Q4.1: 2-15 MB maps read for most rows) runs faster
+    // with less shared memory and the freed part of the SM's array as L1 for the map reads:
+    // replan within 164 KB (measured at SF1000: Q3.1 4.68 -> 3.59 ms, Q4.1 6.55 -> 5.04 ms per
+    // 600 M rows; plans below the threshold — every SF10/SF100 plan — lose with the cap).
+    if (plan_cost > kL1BoundCost && !std::getenv("HX_K1_SMEM_KB")) {
+      t_smem_cap = 164 * 1024;
+      p.stages = pick_stages(dm_mode, n_cols, p.smem_groups);
+      for (int j = 0; j < HX_MAX_JOINS; ++j) kind[j] = kStNone, bloom_w[j] = 0, in_s[j] = 0;
+      plan_cost = plan_dm(sh->n_joins, p.joins, known, pass, keys, bloom_w0, grouped_j,
+                          fits_sizes, kind, bloom_w, in_s);
+    }
   } else {
     // hash tables: selective joins (at most half the dimension passes), most selective first,
     // get a Bloom filter (folded to 4 or 2 bits per key when the full one does not fit)
@@ -1739,7 +1777,7 @@ int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht*
     if (const char* e = std::getenv("HX_K1_MAX_STAGES")) max_stages = std::max(2, std::min(8, std::atoi(e)));
     while (p.stages < max_stages &&
            k1_smem_bytes(dm_mode, n_cols, p.stages + 1, p.smem_groups, p.filter_words, p.dm_bytes,
-                         in_place) <= smem_budget(std::min(kCtasPerSm, 2)))
+                         in_place) <= k1_smem_cap())
       ++p.stages;
   }
   // (measured, SF10: a distance of 2 gains 4-7% on the 4-column pipelines whose ring stays at
@@ -1764,6 +1802,9 @@ int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht*
   k.fn = pick_kernel(sh->n_joins, grouped, p.m_dm != 0u);
   k.smem = k1_smem_bytes(dm_mode, n_cols, p.stages, p.smem_groups, p.filter_words, p.dm_bytes,
                          in_place);
+  // the smallest shared-memory carveout that holds the plan: the rest of the SM's L1/shared
+  // array caches the maps read from L2
+  k.carveout = (int)std::min<size_t>(100, ((k.smem + 1024) * 100 + 228 * 1024 - 1) / (228 * 1024));
   int occ = 0;
   HX_CK(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, k.fn, kThreads, k.smem));
   occ = std::max(1, occ);
@@ -1899,7 +1940,7 @@ int k1_enqueue(hx_ctx* ctx, const K1Prepared* k, bool fresh, cudaEvent_t e0, cud
       q.n_rows = std::min<int64_t>(k->seg_rows, p.n_rows - s0);
       q.n_tiles = (q.n_rows + kTileRows - 1) / kTileRows;
       const int grid = (int)std::max<int64_t>(1, std::min<int64_t>(q.n_tiles, (int64_t)k->grid));
-      HX_CK(launch_k1(k->fn, grid, kThreads, k->smem, ctx->stream, q, ctx->k1_priority));
+      HX_CK(launch_k1(k->fn, grid, kThreads, k->smem, ctx->stream, q, ctx->k1_priority, k->carveout));
       ctx->launches += 1;
     }
   }
