@@ -506,10 +506,15 @@ __device__ __forceinline__ void process_tile(const K1Params& p, const JoinState 
   const int r0 = wbase + lane * R;
   const int32_t* tb[2] = {sbase0 + r0, sbase1 + r0};
   uint32_t m = 0;
+  if (rows_valid0 == kTileRows) {  // full tiles (all but the last): no per-row bound checks
+    m = rows_valid1 == kTileRows ? (1u << (2 * R)) - 1u : rows_valid1 == 0 ? (1u << R) - 1u : 0u;
+  }
+  if (m == 0u) {
 #pragma unroll
-  for (int k = 0; k < R; ++k) {
-    m |= (uint32_t)(r0 + k < rows_valid0) << k;
-    m |= (uint32_t)(r0 + k < rows_valid1) << (R + k);
+    for (int k = 0; k < R; ++k) {
+      m |= (uint32_t)(r0 + k < rows_valid0) << k;
+      m |= (uint32_t)(r0 + k < rows_valid1) << (R + k);
+    }
   }
   if (__ballot_sync(kFull, m) == 0) return;
   // the 8 values of staged column c for this lane
@@ -533,14 +538,14 @@ __device__ __forceinline__ void process_tile(const K1Params& p, const JoinState 
       const uint32_t lo = (uint32_t)pr.lo, span = (uint32_t)pr.hi - (uint32_t)pr.lo;
 #pragma unroll
       for (int k = 0; k < 2 * R; ++k)
-        m &= ~((uint32_t)(((uint32_t)vv[k] - lo) > span) << k);
+        if (((uint32_t)vv[k] - lo) > span) m &= ~(1u << k);
     } else {
 #pragma unroll
       for (int k = 0; k < 2 * R; ++k) {
         bool ok = false;
 #pragma unroll
         for (int i = 0; i < 4; ++i) ok |= (i < pr.n_in) && vv[k] == pr.in[i];
-        m &= ~((uint32_t)(!ok) << k);
+        if (!ok) m &= ~(1u << k);
       }
     }
   }
@@ -556,7 +561,7 @@ __device__ __forceinline__ void process_tile(const K1Params& p, const JoinState 
     int32_t key[2 * R];
     load8(js[jx].c, key);
 #pragma unroll
-    for (int k = 0; k < 2 * R; ++k) m &= ~((uint32_t)!bloom_pass(js[jx], key[k]) << k);
+    for (int k = 0; k < 2 * R; ++k) if (!bloom_pass(js[jx], key[k])) m &= ~(1u << k);
   }
 
   // stage S (direct maps): the shared-memory structure of the most selective join, on every
@@ -580,7 +585,7 @@ __device__ __forceinline__ void process_tile(const K1Params& p, const JoinState 
         const uint32_t bit = dm_bit(d, key[k]);
         const uint32_t word = dm_in(d, key[k]) ? w[bit >> 5] : 0u;
         const uint32_t v = dm_entry(d, word, bit);
-        m &= ~((uint32_t)(v == 0u) << k);
+        if (v == 0u) m &= ~(1u << k);
         if (GROUPED && all_res) g[k] += (int32_t)v * js[jx].jstride;
       }
     } else if (jbit(p.m_bm, jx)) {  // its membership bitmap: exact verdict (rank from L2)
@@ -589,7 +594,7 @@ __device__ __forceinline__ void process_tile(const K1Params& p, const JoinState 
       for (int k = 0; k < 2 * R; ++k) {
         const uint32_t u = (uint32_t)key[k] - (uint32_t)d.dm_kmin;
         const uint32_t word = u < d.dm_span ? w[u >> 5] : 0u;
-        m &= ~((uint32_t)(((word >> (u & 31u)) & 1u) == 0u) << k);
+        if (((word >> (u & 31u)) & 1u) == 0u) m &= ~(1u << k);
       }
     } else if (jbit(p.m_l2s, jx)) {  // its map from L2, every live row (8 loads in flight)
       uint32_t w[2 * R];
@@ -599,12 +604,12 @@ __device__ __forceinline__ void process_tile(const K1Params& p, const JoinState 
 #pragma unroll
       for (int k = 0; k < 2 * R; ++k) {
         const uint32_t v = dm_entry(d, w[k], dm_bit(d, key[k]));
-        m &= ~((uint32_t)(v == 0u) << k);
+        if (v == 0u) m &= ~(1u << k);
         if (GROUPED && all_res) g[k] += (int32_t)v * js[jx].jstride;
       }
     } else {  // its Bloom filter: no false negatives
 #pragma unroll
-      for (int k = 0; k < 2 * R; ++k) m &= ~((uint32_t)!bloom_pass(js[jx], key[k]) << k);
+      for (int k = 0; k < 2 * R; ++k) if (!bloom_pass(js[jx], key[k])) m &= ~(1u << k);
     }
   }
 
@@ -634,7 +639,7 @@ __device__ __forceinline__ void process_tile(const K1Params& p, const JoinState 
         int32_t rank;
         probe_step(v[k], key[kk], hit, miss, rank);
         g[kk] = hit ? rank * j.jstride : (int32_t)~((b[k] + 1) & j.bmask);
-        m &= ~((uint32_t)miss << kk);
+        if (miss) m &= ~(1u << kk);
       }
     }
   }
@@ -652,6 +657,15 @@ __device__ __forceinline__ void process_tile(const K1Params& p, const JoinState 
           if (p.gb) b8[k] = __ldg(p.gat_b + row);
         }
       }
+    }
+    if (!GROUPED) {  // branch-free: predicated adds, one population count
+      long long sum = 0;
+#pragma unroll
+      for (int k = 0; k < 2 * R; ++k)
+        sum += ((m >> k) & 1u) ? measure(p.agg_op, a8[k], b8[k]) : 0ll;
+      acc_sum += sum;
+      acc_cnt += __popc(m);
+      return;
     }
 #pragma unroll
     for (int k = 0; k < 2 * R; ++k)
@@ -1142,7 +1156,7 @@ __global__ void __launch_bounds__(kScanThreads + 32, 1) k1_scan_agg(const __grid
           for (int c = 1; c < NC; ++c) y = pr.c == c ? x[c] : y;
           const int32_t yv[4] = {y.x, y.y, y.z, y.w};
 #pragma unroll
-          for (int k = 0; k < 4; ++k) m &= ~((uint32_t)!pred_pass(pr, yv[k]) << k);
+          for (int k = 0; k < 4; ++k) if (!pred_pass(pr, yv[k])) m &= ~(1u << k);
         }
         int4 a4 = x[0], b4 = x[0];
 #pragma unroll
