@@ -1714,10 +1714,12 @@ int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht*
                         kind, bloom_w, in_s);
     // An L2-lookup-bound plan (SF1000 Q3.1/Q4.1: 2-15 MB maps read for most rows) runs faster
     // with less shared memory and the freed part of the SM's array as L1 for the map reads:
-    // replan within 164 KB (measured at SF1000: Q3.1 4.68 -> 3.59 ms, Q4.1 6.55 -> 5.04 ms per
-    // 600 M rows; plans below the threshold — every SF10/SF100 plan — lose with the cap).
+    // replan within 164 KB, or within a 4-stage ring (tile pairs) for wide pipelines
+    // (measured at SF1000 per 600 M rows: Q3.1 4.68 -> 3.59 ms, Q4.1 6.55 -> 4.02 ms; a
+    // 3-stage ring (no pairs) gave Q4.1 5.03; plans below the threshold — every SF10/SF100
+    // plan — lose with the cap).
     if (plan_cost > kL1BoundCost && !std::getenv("HX_K1_SMEM_KB")) {
-      t_smem_cap = 164 * 1024;
+      t_smem_cap = std::max<size_t>(164 * 1024, k1_smem_bytes(dm_mode, n_cols, 4, p.smem_groups));
       p.stages = pick_stages(dm_mode, n_cols, p.smem_groups);
       for (int j = 0; j < HX_MAX_JOINS; ++j) kind[j] = kStNone, bloom_w[j] = 0, in_s[j] = 0;
       plan_cost = plan_dm(sh->n_joins, p.joins, known, pass, keys, bloom_w0, grouped_j,
