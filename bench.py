@@ -487,6 +487,10 @@ def main():
                 "moved_bytes_definition": "streamed columns (4 B/row) + one 32-B sector per "
                                           "gathered measure value of a row that passed every join",
                 "achieved_moved": moved, "frac_moved": moved / peak,
+                "peak_nominal": 8000.0, "frac_nominal": achieved / 8000.0,
+                "peak_read_stream": 7100.0,
+                "peak_read_stream_source": "tools/stream_roofline.cu: the same bulk-copy ring with "
+                                           "trivial consumers, 7.0-7.2 TB/s on this B200 (DESIGN.md 7)",
                 "k1_ms_per_launch": k1_ms / max(k1_n, 1),
                 "k1_busy_frac_of_step": k1_ms / ms if ms > 0 else None,
                 "k1_span_ms_per_step": k1_span / args.steps,
