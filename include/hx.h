@@ -108,6 +108,9 @@ int hx_table_info(const hx_table* t, int64_t* n_rows, int* n_cols);
 /* A view of rows [row_begin, row_end) of `t` (no copy; lifetime bounded by `t`). */
 int hx_table_slice(const hx_table* t, int64_t row_begin, int64_t row_end, hx_table** out);
 int hx_table_free(hx_table* t);
+/* Copies rows [row_begin, row_begin + n) of column `col_id` of `t` (device or host resident)
+   into caller host memory `dst` (n int32). Synchronises the ctx stream. */
+int hx_table_read(const hx_table* t, int32_t col_id, int64_t row_begin, int64_t n, int32_t* dst);
 
 /* ---- dimension filter + hash-table build (§8(a) a3, kernel K2) ----------------------
  * PAPER.md:1160-1163 §6.1 (broadcast-hash-join plans: the build side is the filtered
@@ -147,6 +150,40 @@ int hx_ht_info(hx_ht* ht, int64_t* n_keys, int64_t* n_slots, int32_t* n_ranks,
    (any preds — its contents are replaced). Requires hx_comm_init. */
 int hx_ht_broadcast(hx_ctx* ctx, hx_ht* ht, int root);
 int hx_ht_free(hx_ht* ht);
+/* hx_build_dim_ht with build flags. HX_BUILD_IDENTITY_RANKS: the rank of group code c is
+   c - group_lo for every code of [group_lo, group_hi] (n_ranks = the domain size), not its
+   position among the codes present — so tables built over DIFFERENT row subsets of one
+   dimension (the partitions of a hash-partitioned join, §8(f) NEXT-1) give every group the
+   same index, and their partial aggregates add element-wise (union router). */
+enum { HX_BUILD_IDENTITY_RANKS = 1 };
+int hx_build_dim_ht_ex(hx_ctx* ctx, const hx_table* dim, int32_t key_col, const hx_pred* preds,
+                       int n_preds, int32_t group_col, int32_t group_lo, int32_t group_hi,
+                       int flags, hx_ht** out);
+
+/* ---- hash-partitioned join: hash-pack + hash-routing exchange (§8(f) NEXT-1) ---------
+ * PAPER.md:405-428 §3.1 (hash-based routing policies: the router sends each block's rows to
+ * the consumer chosen by a hash of a key, after a hash-pack operator groups the rows by
+ * destination), PAPER.md:557-561, 582-587 (Fig. 1d/e: hash-partitioned joins exchange both
+ * inputs so that matching keys meet on one device). The alternative to broadcasting a
+ * dimension too large to replicate.
+ * hx_hash_partition (hash-pack, kernel K3): the rows of the device table `t` are permuted so
+ * that the rows of part p = hx_part_of(key, n_parts) are contiguous and in part order (order
+ * within a part unspecified). *out: a new library-owned device table with t's columns;
+ * part_offsets (caller array of n_parts + 1 int64, host memory): part p is rows
+ * [part_offsets[p], part_offsets[p+1]). 1 <= n_parts <= HX_MAX_PARTS. Synchronises (the
+ * offsets are read back to size the exchange).
+ * Part function: p = ((uint64)(uint32)(key * 0x9E3779B1) * n_parts) >> 32 (Fibonacci hash,
+ * multiply-shift range reduction; keys of one value always meet in one part). */
+#define HX_MAX_PARTS 64
+int hx_hash_partition(hx_ctx* ctx, const hx_table* t, int32_t key_col, int n_parts,
+                      hx_table** out, int64_t* part_offsets);
+/* The hash-routing exchange: part p of `parted` (from hx_hash_partition with n_parts ==
+   nranks) goes to rank p; *out receives, in rank order, the rows every rank routed here — one
+   grouped set of ncclSend/ncclRecv per column over NVLink after an ncclAllGather of the part
+   sizes. Collective over the communicator. Without a communicator of > 1 ranks it returns a
+   copy of part 0 (n_parts must be 1 then). Synchronises. */
+int hx_exchange_partitions(hx_ctx* ctx, const hx_table* parted, const int64_t* part_offsets,
+                           int n_parts, hx_table** out);
 
 /* ---- fused scan → filter → probe×k → aggregate (§8(a) a5, kernel K1) ----------------
  * PAPER.md:859-869 Listing 1 pipeline 9 (grid-stride unpack, predicate, thread-local

@@ -20,6 +20,8 @@ HX_PLACE_COPY, HX_PLACE_VIEW, HX_PLACE_HOST_PINNED, HX_PLACE_HOST_MAPPED = 0, 1,
 HX_PRED_RANGE, HX_PRED_IN = 0, 1
 HX_AGG_SUM, HX_AGG_SUM_MUL, HX_AGG_SUM_SUB = 0, 1, 2
 HX_MAX_COLS, HX_MAX_PREDS, HX_MAX_JOINS, HX_MAX_GDIMS = 16, 3, 4, 3
+HX_BUILD_IDENTITY_RANKS = 1
+HX_MAX_PARTS = 64
 
 _NAMES = {0: "HX_OK", -1: "HX_EINVAL", -2: "HX_ECUDA", -3: "HX_ENCCL", -4: "HX_ENOMEM",
           -5: "HX_ECAPACITY", -6: "HX_EDUPKEY", -7: "HX_EUNSUPPORTED"}
@@ -85,7 +87,11 @@ _SIGS = {
     "hx_table_info": ([_P, _PI64, ctypes.POINTER(_I)], _I),
     "hx_table_slice": ([_P, _I64, _I64, _PP], _I),
     "hx_table_free": ([_P], _I),
+    "hx_table_read": ([_P, _I32, _I64, _I64, _PI32], _I),
     "hx_build_dim_ht": ([_P, _P, _I32, ctypes.POINTER(hx_pred), _I, _I32, _I32, _I32, _PP], _I),
+    "hx_build_dim_ht_ex": ([_P, _P, _I32, ctypes.POINTER(hx_pred), _I, _I32, _I32, _I32, _I, _PP], _I),
+    "hx_hash_partition": ([_P, _P, _I32, _I, _PP, _PI64], _I),
+    "hx_exchange_partitions": ([_P, _P, _PI64, _I, _PP], _I),
     "hx_ht_info": ([_P, _PI64, _PI64, _PI32, _PI32], _I),
     "hx_ht_broadcast": ([_P, _P, _I], _I),
     "hx_ht_free": ([_P], _I),

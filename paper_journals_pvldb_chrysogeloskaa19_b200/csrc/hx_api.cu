@@ -365,6 +365,19 @@ int hx_table_slice(const hx_table* t, int64_t row_begin, int64_t row_end, hx_tab
   return HX_OK;
 }
 
+int hx_table_read(const hx_table* t, int32_t col_id, int64_t row_begin, int64_t n, int32_t* dst) {
+  HX_REQUIRE(t && (dst || n == 0) && row_begin >= 0 && n >= 0 && row_begin + n <= t->n_rows,
+             HX_EINVAL, "hx_table_read: bad argument");
+  HX_REQUIRE(table_has_col(t, col_id), HX_EINVAL, "hx_table_read: column not in table");
+  if (n == 0) return HX_OK;
+  HX_CK(cudaSetDevice(t->ctx->device));
+  HX_CK(cudaMemcpyAsync(dst, table_col(t, col_id) + row_begin, (size_t)n * 4, cudaMemcpyDefault,
+                        t->ctx->stream));
+  HX_CK(cudaStreamSynchronize(t->ctx->stream));
+  t->ctx->d2h_bytes += n * 4;
+  return HX_OK;
+}
+
 int hx_table_free(hx_table* t) {
   HX_REQUIRE(t, HX_EINVAL, "hx_table_free: null table");
   if (t->owned) {
@@ -382,6 +395,14 @@ int hx_build_dim_ht(hx_ctx* ctx, const hx_table* dim, int32_t key_col, const hx_
                     hx_ht** out) {
   if (ctx) HX_CK(cudaSetDevice(ctx->device));
   return build_dim_ht(ctx, dim, key_col, preds, n_preds, group_col, group_lo, group_hi, out);
+}
+
+int hx_build_dim_ht_ex(hx_ctx* ctx, const hx_table* dim, int32_t key_col, const hx_pred* preds,
+                       int n_preds, int32_t group_col, int32_t group_lo, int32_t group_hi,
+                       int flags, hx_ht** out) {
+  if (ctx) HX_CK(cudaSetDevice(ctx->device));
+  return build_dim_ht(ctx, dim, key_col, preds, n_preds, group_col, group_lo, group_hi, out,
+                      flags);
 }
 
 int hx_ht_info(hx_ht* ht, int64_t* n_keys, int64_t* n_slots, int32_t* n_ranks,

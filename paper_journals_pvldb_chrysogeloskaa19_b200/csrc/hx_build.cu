@@ -45,6 +45,7 @@ struct BuildParams {
   int32_t dm_kmin;
   uint32_t dm_span;
   int32_t dm_lw;
+  int32_t identity_ranks;  // HX_BUILD_IDENTITY_RANKS: rank = code - group_lo for every code
 };
 
 __device__ __forceinline__ bool row_pass(const BuildParams& p, int64_t i) {
@@ -68,7 +69,7 @@ __device__ void rank_codes(const BuildParams& p) {
   if (p.group) {
     for (int base = 0; base < p.domain; base += NT) {
       const int code = base + threadIdx.x;
-      const int flag = code < p.domain ? __ldcg(p.c2r + code) : 0;
+      const int flag = code < p.domain ? (p.identity_ranks ? 1 : __ldcg(p.c2r + code)) : 0;
       int excl, total;
       Scan(tmp).ExclusiveSum(flag, excl, total);
       const int rank = running + excl;
@@ -299,7 +300,8 @@ int ceil_log2(int64_t x) {
 
 // Validate a build and allocate its table (no kernels launched).
 int ht_create(hx_ctx* ctx, const hx_table* dim, int32_t key_col, const hx_pred* preds,
-              int n_preds, int32_t group_col, int32_t group_lo, int32_t group_hi, hx_ht** out) {
+              int n_preds, int32_t group_col, int32_t group_lo, int32_t group_hi, hx_ht** out,
+              int flags) {
   HX_REQUIRE(ctx && dim && out, HX_EINVAL, "hx_build_dim_ht: null argument");
   HX_REQUIRE(n_preds >= 0 && n_preds <= HX_MAX_PREDS && (n_preds == 0 || preds), HX_EINVAL,
              "hx_build_dim_ht: bad predicate list");
@@ -328,6 +330,8 @@ int ht_create(hx_ctx* ctx, const hx_table* dim, int32_t key_col, const hx_pred* 
                "hx_build_dim_ht: bad group code range");
     domain = (int64_t)group_hi - group_lo + 1;
   }
+  HX_REQUIRE((flags & ~HX_BUILD_IDENTITY_RANKS) == 0, HX_EINVAL, "hx_build_dim_ht: bad flags");
+  p.identity_ranks = (flags & HX_BUILD_IDENTITY_RANKS) && group_col >= 0 ? 1 : 0;
   p.n_rows = dim->n_rows;
   p.group_lo = group_lo;
   p.domain = (int32_t)domain;
@@ -338,6 +342,7 @@ int ht_create(hx_ctx* ctx, const hx_table* dim, int32_t key_col, const hx_pred* 
   ht->domain = (int32_t)domain;
   ht->group_lo = group_lo;
   ht->has_group = group_col >= 0;
+  ht->identity_ranks = p.identity_ranks != 0;
   ht->max_log2cap = p.max_log2cap;
   ht->dim_rows = dim->n_rows;
   p.max_bloom_log2w = bloom_log2w_for(std::max<int64_t>(dim->n_rows, 1));
@@ -428,9 +433,9 @@ void ht_destroy(hx_ht* ht) {
 
 int build_dim_ht(hx_ctx* ctx, const hx_table* dim, int32_t key_col, const hx_pred* preds,
                  int n_preds, int32_t group_col, int32_t group_lo, int32_t group_hi,
-                 hx_ht** out) {
+                 hx_ht** out, int flags) {
   hx_ht* ht = nullptr;
-  int rc = ht_create(ctx, dim, key_col, preds, n_preds, group_col, group_lo, group_hi, &ht);
+  int rc = ht_create(ctx, dim, key_col, preds, n_preds, group_col, group_lo, group_hi, &ht, flags);
   if (rc != HX_OK) return rc;
   rc = ht_enqueue_build(ctx, ht);
   if (rc != HX_OK) {

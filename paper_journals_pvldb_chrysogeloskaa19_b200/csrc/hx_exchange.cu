@@ -1,0 +1,261 @@
+// hx_exchange.cu — the hash-partitioned join's data movement:
+// hash-pack (kernel K3: group a table's rows by the part of their key) and the hash-routing
+// exchange (part p -> rank p over NCCL). PAPER.md:405-428 §3.1 (hash-based routing; the
+// hash-pack operator), PAPER.md:557-561, 582-587 (Fig. 1d/e hash-partitioned joins).
+//
+// K3 is a three-pass radix scatter over whole rows, bound by HBM (each row is read twice and
+// written once: 12 B per 4-byte column):
+//   k3_count    each CTA counts the rows of its contiguous chunk per part (shared-memory
+//               counters), writes counts[part][cta];
+//   k3_scan     one CTA: exclusive scan over (part, cta) -> each CTA's write cursor per part,
+//               and the part offsets;
+//   k3_scatter  each CTA re-reads its chunk and writes every column of a row to its part's
+//               next slot (warp-aggregated shared-memory cursors: one atomic per part per
+//               warp instruction).
+#include <cub/block/block_scan.cuh>
+
+#include <algorithm>
+#include <vector>
+
+#include "hx_internal.cuh"
+
+namespace hx {
+namespace {
+
+constexpr int kK3Threads = 512;
+
+__host__ __device__ __forceinline__ int part_of(int32_t key, int n_parts) {
+  return (int)(((unsigned long long)((uint32_t)key * 0x9E3779B1u) * (unsigned)n_parts) >> 32);
+}
+
+struct K3Params {
+  const int32_t* key;
+  const int32_t* src[HX_MAX_COLS];
+  int32_t* dst[HX_MAX_COLS];
+  int32_t n_cols;
+  int32_t n_parts;
+  int64_t n_rows;
+  int64_t chunk;            // rows per CTA
+  int64_t* counts;          // [n_parts][grid]: counts, then (after the scan) write cursors
+  int64_t* part_offsets;    // [n_parts + 1]
+};
+
+__global__ void __launch_bounds__(kK3Threads) k3_count(K3Params p) {
+  __shared__ unsigned int cnt[HX_MAX_PARTS];
+  for (int i = threadIdx.x; i < p.n_parts; i += blockDim.x) cnt[i] = 0;
+  __syncthreads();
+  const int64_t r0 = (int64_t)blockIdx.x * p.chunk;
+  const int64_t r1 = min(p.n_rows, r0 + p.chunk);
+  for (int64_t r = r0 + threadIdx.x; r < r1; r += blockDim.x)
+    atomicAdd(&cnt[part_of(__ldg(p.key + r), p.n_parts)], 1u);
+  __syncthreads();
+  for (int i = threadIdx.x; i < p.n_parts; i += blockDim.x)
+    p.counts[(int64_t)i * gridDim.x + blockIdx.x] = cnt[i];
+}
+
+// exclusive scan of counts in (part, cta) order: the rows of part 0 from every CTA, then
+// part 1, ... — each CTA's rows of a part land contiguously at its cursor
+__global__ void __launch_bounds__(1024) k3_scan(K3Params p, int grid) {
+  using Scan = cub::BlockScan<long long, 1024>;
+  __shared__ typename Scan::TempStorage tmp;
+  __shared__ long long running;
+  if (threadIdx.x == 0) running = 0;
+  __syncthreads();
+  const int64_t n = (int64_t)p.n_parts * grid;
+  for (int64_t base = 0; base < n; base += 1024) {
+    const int64_t i = base + threadIdx.x;
+    const long long v = i < n ? p.counts[i] : 0;
+    long long excl, total;
+    Scan(tmp).ExclusiveSum(v, excl, total);
+    if (i < n) {
+      p.counts[i] = running + excl;
+      if (i % grid == 0) p.part_offsets[i / grid] = running + excl;
+    }
+    __syncthreads();
+    if (threadIdx.x == 0) running += total;
+    __syncthreads();
+  }
+  if (threadIdx.x == 0) p.part_offsets[p.n_parts] = running;
+}
+
+__global__ void __launch_bounds__(kK3Threads) k3_scatter(K3Params p) {
+  __shared__ unsigned long long cur[HX_MAX_PARTS];
+  for (int i = threadIdx.x; i < p.n_parts; i += blockDim.x)
+    cur[i] = (unsigned long long)p.counts[(int64_t)i * gridDim.x + blockIdx.x];
+  __syncthreads();
+  const int64_t r0 = (int64_t)blockIdx.x * p.chunk;
+  const int64_t r1 = min(p.n_rows, r0 + p.chunk);
+  const int lane = threadIdx.x & 31;
+  for (int64_t base = r0; base < r1; base += blockDim.x) {
+    const int64_t r = base + threadIdx.x;
+    const bool live = r < r1;
+    const int part = live ? part_of(__ldg(p.key + r), p.n_parts) : -1;
+    // warp-aggregated cursor: the lanes of one part take consecutive slots
+    const unsigned act = __ballot_sync(0xFFFFFFFFu, live);
+    unsigned long long pos = 0;
+    if (live) {
+      const unsigned same = __match_any_sync(act, part);
+      const int leader = __ffs(same) - 1;
+      unsigned long long b = 0;
+      if (lane == leader) b = atomicAdd(&cur[part], (unsigned long long)__popc(same));
+      b = __shfl_sync(same, b, leader);
+      pos = b + __popc(same & ((1u << lane) - 1u));
+      for (int c = 0; c < p.n_cols; ++c) p.dst[c][pos] = __ldg(p.src[c] + r);
+    }
+  }
+}
+
+int table_alloc_like(hx_ctx* ctx, const hx_table* t, int64_t n_rows, hx_table** out) {
+  hx_table* o = new hx_table();
+  o->ctx = ctx;
+  o->n_cols = t->n_cols;
+  o->n_rows = n_rows;
+  o->placement = HX_PLACE_COPY;
+  o->owned = true;
+  for (int c = 0; c < t->n_cols; ++c) {
+    o->col_id[c] = t->col_id[c];
+    o->dev[c] = nullptr;
+    if (n_rows == 0) continue;
+    cudaError_t e = cudaMallocAsync(&o->dev[c], ((size_t)n_rows * 4 + 255) & ~size_t(255), ctx->stream);
+    if (e != cudaSuccess) {
+      for (int d = 0; d < c; ++d) cudaFreeAsync(o->dev[d], ctx->stream);
+      delete o;
+      return cuda_fail(e, "cudaMallocAsync(partitioned column)", __FILE__, __LINE__);
+    }
+  }
+  *out = o;
+  return HX_OK;
+}
+
+}  // namespace
+}  // namespace hx
+
+using namespace hx;
+
+extern "C" {
+
+int hx_hash_partition(hx_ctx* ctx, const hx_table* t, int32_t key_col, int n_parts,
+                      hx_table** out, int64_t* part_offsets) {
+  HX_REQUIRE(ctx && t && out && part_offsets, HX_EINVAL, "hx_hash_partition: null argument");
+  HX_REQUIRE(n_parts >= 1 && n_parts <= HX_MAX_PARTS, HX_EINVAL, "hx_hash_partition: bad n_parts");
+  HX_REQUIRE(t->placement == HX_PLACE_COPY || t->placement == HX_PLACE_VIEW, HX_EUNSUPPORTED,
+             "hx_hash_partition: the table must be device resident");
+  HX_REQUIRE(table_has_col(t, key_col), HX_EINVAL, "hx_hash_partition: key column not in table");
+  HX_CK(cudaSetDevice(ctx->device));
+  hx_table* o = nullptr;
+  int rc = table_alloc_like(ctx, t, t->n_rows, &o);
+  if (rc != HX_OK) return rc;
+  if (t->n_rows == 0) {
+    for (int i = 0; i <= n_parts; ++i) part_offsets[i] = 0;
+    *out = o;
+    return HX_OK;
+  }
+  const int64_t grid = std::max<int64_t>(1, std::min<int64_t>((int64_t)ctx->n_sms * 4,
+                                                             (t->n_rows + 4095) / 4096));
+  K3Params p{};
+  p.key = table_col(t, key_col);
+  p.n_cols = t->n_cols;
+  for (int c = 0; c < t->n_cols; ++c) {
+    p.src[c] = t->dev[c];
+    p.dst[c] = o->dev[c];
+  }
+  p.n_parts = n_parts;
+  p.n_rows = t->n_rows;
+  p.chunk = (t->n_rows + grid - 1) / grid;
+  void* scratch = nullptr;
+  const size_t sbytes = sizeof(int64_t) * ((size_t)n_parts * grid + n_parts + 1);
+  cudaError_t e = cudaMallocAsync(&scratch, sbytes, ctx->stream);
+  if (e != cudaSuccess) {
+    hx_table_free(o);
+    return cuda_fail(e, "cudaMallocAsync(partition counters)", __FILE__, __LINE__);
+  }
+  p.counts = static_cast<int64_t*>(scratch);
+  p.part_offsets = p.counts + (size_t)n_parts * grid;
+  k3_count<<<(unsigned)grid, kK3Threads, 0, ctx->stream>>>(p);
+  k3_scan<<<1, 1024, 0, ctx->stream>>>(p, (int)grid);
+  k3_scatter<<<(unsigned)grid, kK3Threads, 0, ctx->stream>>>(p);
+  ctx->launches += 3;
+  e = cudaGetLastError();
+  if (e == cudaSuccess)
+    e = cudaMemcpyAsync(part_offsets, p.part_offsets, sizeof(int64_t) * (n_parts + 1),
+                        cudaMemcpyDeviceToHost, ctx->stream);
+  cudaFreeAsync(scratch, ctx->stream);
+  if (e == cudaSuccess) e = cudaStreamSynchronize(ctx->stream);
+  if (e != cudaSuccess) {
+    hx_table_free(o);
+    return cuda_fail(e, "hx_hash_partition", __FILE__, __LINE__);
+  }
+  ctx->d2h_bytes += sizeof(int64_t) * (n_parts + 1);
+  *out = o;
+  return HX_OK;
+}
+
+int hx_exchange_partitions(hx_ctx* ctx, const hx_table* parted, const int64_t* part_offsets,
+                           int n_parts, hx_table** out) {
+  HX_REQUIRE(ctx && parted && part_offsets && out, HX_EINVAL, "hx_exchange_partitions: null argument");
+  HX_REQUIRE(part_offsets[0] == 0 && part_offsets[n_parts] == parted->n_rows, HX_EINVAL,
+             "hx_exchange_partitions: offsets do not match the table");
+  HX_CK(cudaSetDevice(ctx->device));
+  const int nr = ctx->comm ? ctx->nranks : 1;
+  HX_REQUIRE(n_parts == nr, HX_EINVAL, "hx_exchange_partitions: n_parts must equal the rank count");
+  if (nr == 1) {  // no exchange: this rank keeps its one part (a library-owned copy)
+    hx_table* o = nullptr;
+    int rc = table_alloc_like(ctx, parted, parted->n_rows, &o);
+    if (rc != HX_OK) return rc;
+    for (int c = 0; c < parted->n_cols; ++c)
+      if (parted->n_rows)
+        HX_CK(cudaMemcpyAsync(o->dev[c], parted->dev[c], (size_t)parted->n_rows * 4,
+                              cudaMemcpyDeviceToDevice, ctx->stream));
+    HX_CK(cudaStreamSynchronize(ctx->stream));
+    *out = o;
+    return HX_OK;
+  }
+  // part sizes of every rank: sizes[src * nr + dst]
+  int64_t* dsz = nullptr;
+  HX_CK(cudaMallocAsync(&dsz, sizeof(int64_t) * nr * (nr + 1), ctx->stream));
+  std::vector<int64_t> mine(nr), sizes((size_t)nr * nr);
+  for (int p = 0; p < nr; ++p) mine[p] = part_offsets[p + 1] - part_offsets[p];
+  HX_CK(cudaMemcpyAsync(dsz, mine.data(), sizeof(int64_t) * nr, cudaMemcpyHostToDevice, ctx->stream));
+  ncclResult_t r = ncclAllGather(dsz, dsz + nr, nr, ncclInt64, ctx->comm, ctx->stream);
+  if (r != ncclSuccess) {
+    cudaFreeAsync(dsz, ctx->stream);
+    return fail(HX_ENCCL, std::string("ncclAllGather: ") + ncclGetErrorString(r));
+  }
+  HX_CK(cudaMemcpyAsync(sizes.data(), dsz + nr, sizeof(int64_t) * nr * nr, cudaMemcpyDeviceToHost,
+                        ctx->stream));
+  HX_CK(cudaStreamSynchronize(ctx->stream));
+  cudaFreeAsync(dsz, ctx->stream);
+  int64_t n_in = 0;
+  std::vector<int64_t> recv_off(nr);
+  for (int s = 0; s < nr; ++s) {
+    recv_off[s] = n_in;
+    n_in += sizes[(size_t)s * nr + ctx->rank];
+  }
+  hx_table* o = nullptr;
+  int rc = table_alloc_like(ctx, parted, n_in, &o);
+  if (rc != HX_OK) return rc;
+  r = ncclGroupStart();
+  for (int c = 0; c < parted->n_cols && r == ncclSuccess; ++c) {
+    for (int peer = 0; peer < nr && r == ncclSuccess; ++peer) {
+      const int64_t ns = part_offsets[peer + 1] - part_offsets[peer];
+      const int64_t nrv = sizes[(size_t)peer * nr + ctx->rank];
+      if (ns > 0)
+        r = ncclSend(parted->dev[c] + part_offsets[peer], (size_t)ns, ncclInt32, peer, ctx->comm,
+                     ctx->stream);
+      if (r == ncclSuccess && nrv > 0)
+        r = ncclRecv(o->dev[c] + recv_off[peer], (size_t)nrv, ncclInt32, peer, ctx->comm,
+                     ctx->stream);
+    }
+  }
+  const ncclResult_t r2 = ncclGroupEnd();
+  if (r == ncclSuccess) r = r2;
+  if (r != ncclSuccess) {
+    hx_table_free(o);
+    return fail(HX_ENCCL, std::string("hash-routing exchange: ") + ncclGetErrorString(r));
+  }
+  HX_CK(cudaStreamSynchronize(ctx->stream));
+  *out = o;
+  return HX_OK;
+}
+
+}  // extern "C"

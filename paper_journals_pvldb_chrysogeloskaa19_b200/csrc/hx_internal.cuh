@@ -180,6 +180,7 @@ struct hx_ht {
   int32_t domain = 1;              // group code range size (1 when no group column)
   int32_t group_lo = 0;
   bool has_group = false;
+  bool identity_ranks = false;     // HX_BUILD_IDENTITY_RANKS: n_ranks == domain
   int64_t dim_rows = 0;
   void* build = nullptr;           // hx::BuildParams (hx_build.cu): re-enqueueable build
   uint32_t* bloom = nullptr;       // Bloom filter words (after the slots)
@@ -220,9 +221,10 @@ namespace hx {
 // launchers implemented in hx_build.cu / hx_probe.cu
 int build_dim_ht(hx_ctx* ctx, const hx_table* dim, int32_t key_col, const hx_pred* preds,
                  int n_preds, int32_t group_col, int32_t group_lo, int32_t group_hi,
-                 hx_ht** out);
+                 hx_ht** out, int flags = 0);
 int ht_create(hx_ctx* ctx, const hx_table* dim, int32_t key_col, const hx_pred* preds,
-              int n_preds, int32_t group_col, int32_t group_lo, int32_t group_hi, hx_ht** out);
+              int n_preds, int32_t group_col, int32_t group_lo, int32_t group_hi, hx_ht** out,
+              int flags = 0);
 int ht_enqueue_build(hx_ctx* ctx, hx_ht* ht, cudaStream_t stream = nullptr);
 void ht_destroy(hx_ht* ht);
 // switch a table's builds to a direct map over keys [kmin, kmin + span) with 2^lw-bit entries

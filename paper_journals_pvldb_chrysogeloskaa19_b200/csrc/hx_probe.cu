@@ -1519,7 +1519,9 @@ long long k1_group_bound(const hx_query_shape* sh, hx_ht* const* hts, int n_hts)
     for (int g2 = 0; g2 < g; ++g2)
       if (sh->gdim_join[g2] == j) return -1;
     const hx_ht* ht = hts[sh->join_ht[j]];
-    bound *= std::max<long long>(1, std::min<long long>(ht->domain, std::max<int64_t>(ht->dim_rows, 1)));
+    // (dense ranks: at most one per passing row; identity ranks: the whole domain)
+    bound *= std::max<long long>(1, ht->identity_ranks ? ht->domain
+                                     : std::min<long long>(ht->domain, std::max<int64_t>(ht->dim_rows, 1)));
     bound = std::min<long long>(bound, (long long)HX_MAX_GROUPS + 1);
   }
   return bound;

@@ -40,6 +40,12 @@ class Context:
         buf = ctypes.create_string_buffer(uid, 128)
         call("hx_comm_init", self.h, nranks, rank, buf)
 
+    def comm_info(self) -> Tuple[int, int]:
+        """(rank, nranks); (0, 1) without a communicator."""
+        a, b = ctypes.c_int(), ctypes.c_int()
+        call("hx_comm_info", self.h, ctypes.byref(a), ctypes.byref(b))
+        return a.value, b.value
+
     def profile_enable(self, on: bool = True) -> None:
         call("hx_profile_enable", self.h, int(on))
 
@@ -139,6 +145,15 @@ class Table:
         call("hx_table_slice", self.h, row_begin, row_end, ctypes.byref(h))
         return Table(self.ctx, h, parent=self)
 
+    def read(self, col_id: int, row_begin: int = 0, n: Optional[int] = None) -> np.ndarray:
+        """Rows of one column, copied to the host (synchronous)."""
+        if n is None:
+            n = self.n_rows - row_begin
+        out = np.empty(n, dtype=np.int32)
+        call("hx_table_read", self.h, col_id, row_begin, n,
+             out.ctypes.data_as(ctypes.POINTER(ctypes.c_int32)))
+        return out
+
     def close(self):
         if getattr(self, "h", None):
             call("hx_table_free", self.h)
@@ -205,12 +220,34 @@ class HashTable:
 
 
 def build_dim_ht(ctx: Context, dim: Table, key_col: int, preds: Sequence[_hx.hx_pred] = (),
-                 group_col: int = -1, group_lo: int = 0, group_hi: int = 0) -> HashTable:
+                 group_col: int = -1, group_lo: int = 0, group_hi: int = 0,
+                 flags: int = 0) -> HashTable:
     arr = (_hx.hx_pred * max(1, len(preds)))(*preds)
     h = ctypes.c_void_p()
-    call("hx_build_dim_ht", ctx.h, dim.h, key_col, arr, len(preds), group_col, group_lo,
-         group_hi, ctypes.byref(h))
+    if flags:
+        call("hx_build_dim_ht_ex", ctx.h, dim.h, key_col, arr, len(preds), group_col, group_lo,
+             group_hi, flags, ctypes.byref(h))
+    else:
+        call("hx_build_dim_ht", ctx.h, dim.h, key_col, arr, len(preds), group_col, group_lo,
+             group_hi, ctypes.byref(h))
     return HashTable(ctx, h, dim)
+
+
+def hash_partition(ctx: Context, t: Table, key_col: int, n_parts: int) -> Tuple[Table, List[int]]:
+    """Hash-pack (K3): a new device table with t's rows grouped by part of `key_col`, and the
+    part offsets (n_parts + 1)."""
+    offs = (ctypes.c_int64 * (n_parts + 1))()
+    h = ctypes.c_void_p()
+    call("hx_hash_partition", ctx.h, t.h, key_col, n_parts, ctypes.byref(h), offs)
+    return Table(ctx, h), list(offs)
+
+
+def exchange_partitions(ctx: Context, parted: Table, offsets: Sequence[int]) -> Table:
+    """Hash-routing exchange: part p to rank p (NCCL); the rows routed to this rank."""
+    offs = (ctypes.c_int64 * len(offsets))(*offsets)
+    h = ctypes.c_void_p()
+    call("hx_exchange_partitions", ctx.h, parted.h, offs, len(offsets) - 1, ctypes.byref(h))
+    return Table(ctx, h)
 
 
 def query_shape(preds=(), joins=(), agg_op=_hx.HX_AGG_SUM, agg_a=0, agg_b=0,

@@ -181,6 +181,78 @@ class SsbEngine:
     def run(self, q: str) -> List[Tuple]:
         return self.finish(self.start(q))
 
+    # ---- hash-partitioned join of one dimension -------------------
+    def _partitioned_build(self, b: DimBuild, dim_rows: hx.Table) -> hx.HashTable:
+        g = b.group
+        return hx.build_dim_ht(self.ctx, dim_rows, C[b.key], [_hx_pred(t) for t in b.preds],
+                               C[g[0]] if g else -1, g[1] if g else 0, g[2] if g else 0,
+                               flags=_hx.HX_BUILD_IDENTITY_RANKS)
+
+    def _join_of(self, plan: Plan, dim: str) -> int:
+        js = [i for i, (_, b) in enumerate(plan.joins) if b.table == dim]
+        if len(js) != 1:
+            raise ValueError(f"{plan.name} does not join {dim} once")
+        return js[0]
+
+    def run_hash_partitioned(self, q: str, dim: str, n_parts: int) -> List[Tuple]:
+        """Hash-partitioned join on ONE GPU: lineorder and dimension `dim` are hash-packed on
+        the join key into n_parts parts (K3, hx_hash_partition); part p of lineorder meets only
+        part p of the dimension — the rows rank p would hold after the hash-routing exchange
+         — while the other dimensions stay broadcast. The
+        partitioned dimension's table of each part is built with identity ranks, so every
+        part's partial aggregate has one group layout; the parts accumulate into one
+        aggregate (the union router) and merge."""
+        plan = PLANS[q]
+        j = self._join_of(plan, dim)
+        fk, b = plan.joins[j]
+        fparts, foffs = hx.hash_partition(self.ctx, self.fact, C[fk], n_parts)
+        dparts, doffs = hx.hash_partition(self.ctx, self.dims[dim], C[b.key], n_parts)
+        hts = [self.build(bb) if i != j else None for i, (_, bb) in enumerate(plan.joins)]
+        shape = self.shape(plan)
+        agg, keep = None, []
+        for p in range(n_parts):
+            fp = fparts.slice(foffs[p], foffs[p + 1])
+            dp = dparts.slice(doffs[p], doffs[p + 1])
+            htp = self._partitioned_build(b, dp)
+            hts_p = list(hts)
+            hts_p[j] = htp
+            if agg is None:
+                agg = hx.pipeline_probe_agg(self.ctx, fp, shape, hts_p)
+            else:
+                hx.pipeline_probe_agg_into(self.ctx, fp, shape, hts_p, agg)
+            keep += [fp, dp, htp]
+        hts[j] = keep[2]
+        rows = self.finish(Pending(plan, [t for t in hts if t is not None], agg))
+        for o in keep:
+            o.close()
+        fparts.close()
+        dparts.close()
+        return rows
+
+    def run_hash_routed(self, q: str, dim: str, root: int = -1) -> List[Tuple]:
+        """The multi-GPU form: every rank hash-packs its lineorder rows and its rows of `dim`
+        into nranks parts, the hash-routing exchange (hx_exchange_partitions, NCCL send/recv
+        over NVLink) gives rank r part r of everyone, each rank joins what it received
+        (identity ranks for the partitioned dimension, broadcast tables for the others), and
+        the union router merges the partials (allreduce). With one rank: a copy of itself."""
+        plan = PLANS[q]
+        j = self._join_of(plan, dim)
+        fk, b = plan.joins[j]
+        nr = self.ctx.comm_info()[1]
+        fparts, foffs = hx.hash_partition(self.ctx, self.fact, C[fk], nr)
+        dparts, doffs = hx.hash_partition(self.ctx, self.dims[dim], C[b.key], nr)
+        f_in = hx.exchange_partitions(self.ctx, fparts, foffs)
+        d_in = hx.exchange_partitions(self.ctx, dparts, doffs)
+        fparts.close()
+        dparts.close()
+        hts = [self.build(bb) if i != j else self._partitioned_build(bb, d_in)
+               for i, (_, bb) in enumerate(plan.joins)]
+        agg = hx.pipeline_probe_agg(self.ctx, f_in, self.shape(plan), hts)
+        rows = self.finish(Pending(plan, hts, agg), root)
+        f_in.close()
+        d_in.close()
+        return rows
+
     # ---- prepared plans (allocation- and sync-free executions, graph capturable) ----------
     DIM_ORDER = ("date", "customer", "supplier", "part")
 

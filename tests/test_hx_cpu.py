@@ -140,3 +140,88 @@ def test_two_rank_partition_merge_gloo():
         for qq, merged in res.items():
             want = oracle.as_dict(oracle.run_query(qq, db))
             assert {k: v for k, v in merged.items() if v[1] > 0} == want, (rank, qq)
+
+
+# ---- world_size 2 over gloo: the hash-partitioned join's exchange (§8(f) NEXT-1) ----------
+def _part_of(keys, n_parts):
+    """include/hx.h part function: ((uint64)(uint32)(key * 0x9E3779B1) * n_parts) >> 32."""
+    h = (keys.astype(np.int64).astype(np.uint64) * np.uint64(0x9E3779B1)) & np.uint64(0xFFFFFFFF)
+    return ((h * np.uint64(n_parts)) >> np.uint64(32)).astype(np.int64)
+
+
+def _hash_rank_main(rank, world, port, out):
+    """Each rank owns round-robin router blocks of lineorder and a disjoint half of the
+    customer rows; both are hash-packed on the customer key and exchanged (all_to_all over
+    gloo, the host stand-in for hx_exchange_partitions' NCCL send/recv); each rank evaluates
+    the query on what it received, with the other dimensions replicated; the partials merge
+    by group codes (union router). The routing host logic is what libhx runs per rank."""
+    import torch
+    import torch.distributed as dist
+
+    import oracle
+    from ssb_tiny import tiny_db
+
+    os.environ.update(MASTER_ADDR="127.0.0.1", MASTER_PORT=str(port))
+    dist.init_process_group("gloo", rank=rank, world_size=world)
+    db = tiny_db(23, n_lo=15013)
+    lo, cu = db["lineorder"], db["customer"]
+    n = len(lo["lo_orderdate"])
+    part = hx.router_partition(n, world, 997, _hx.HX_POLICY_ROUND_ROBIN)
+    mine = np.concatenate([np.arange(b, e) for b, e, p in part.blocks() if p == rank])
+    cmine = np.arange(rank, len(cu["c_custkey"]), world)  # this rank's customer rows
+
+    def exchange(cols, key):
+        dest = _part_of(key, world)
+        order = np.argsort(dest, kind="stable")
+        send_counts = np.bincount(dest, minlength=world)
+        recv_counts = torch.zeros(world, dtype=torch.int64)
+        dist.all_to_all_single(recv_counts, torch.from_numpy(send_counts.astype(np.int64)))
+        got = {}
+        for name, v in cols.items():
+            buf = torch.empty(int(recv_counts.sum()), dtype=torch.int32)
+            dist.all_to_all_single(buf, torch.from_numpy(np.ascontiguousarray(v[order])),
+                                   recv_counts.tolist(), send_counts.tolist())
+            got[name] = buf.numpy()
+        return got
+
+    lo_in = exchange({k: v[mine] for k, v in lo.items()}, lo["lo_custkey"][mine])
+    cu_in = exchange({k: v[cmine] for k, v in cu.items()}, cu["c_custkey"][cmine])
+    assert (_part_of(lo_in["lo_custkey"], world) == rank).all()
+    assert (_part_of(cu_in["c_custkey"], world) == rank).all()
+    local = dict(db, lineorder=lo_in, customer=cu_in)
+    results = {}
+    for q in ("q3.1", "q3.2", "q4.1", "q4.2"):
+        parts = [None] * world
+        dist.all_gather_object(parts, oracle.as_dict(oracle.run_query(q, local)))
+        m = oracle.merge(parts)
+        results[q] = {k: v for k, v in m.items() if v[1] > 0} if oracle.N_KEYS[q] else m
+    out.put((rank, results))
+    dist.destroy_process_group()
+
+
+def test_two_rank_hash_partitioned_join_gloo():
+    import multiprocessing as mp
+    import socket
+    import sys
+
+    sys.path.insert(0, os.path.join(ROOT, "tests"))
+    import oracle
+    from ssb_tiny import tiny_db
+
+    s = socket.socket()
+    s.bind(("127.0.0.1", 0))
+    port = s.getsockname()[1]
+    s.close()
+    ctx = mp.get_context("spawn")
+    q = ctx.Queue()
+    procs = [ctx.Process(target=_hash_rank_main, args=(r, 2, port, q)) for r in range(2)]
+    for p in procs:
+        p.start()
+    got = [q.get(timeout=240) for _ in procs]
+    for p in procs:
+        p.join(timeout=60)
+        assert p.exitcode == 0
+    db = tiny_db(23, n_lo=15013)
+    for rank, res in got:
+        for qq, merged in res.items():
+            assert merged == oracle.as_dict(oracle.run_query(qq, db)), (rank, qq)
