@@ -172,8 +172,10 @@ int hx_build_dim_ht_ex(hx_ctx* ctx, const hx_table* dim, int32_t key_col, const 
  * part_offsets (caller array of n_parts + 1 int64, host memory): part p is rows
  * [part_offsets[p], part_offsets[p+1]). 1 <= n_parts <= HX_MAX_PARTS. Synchronises (the
  * offsets are read back to size the exchange).
- * Part function: p = ((uint64)(uint32)(key * 0x9E3779B1) * n_parts) >> 32 (Fibonacci hash,
- * multiply-shift range reduction; keys of one value always meet in one part). */
+ * Part function: h = fmix32((uint32)key) (murmur3 finaliser: h ^= h >> 16; h *= 0x85EBCA6B;
+ * h ^= h >> 13; h *= 0xC2B2AE35; h ^= h >> 16), p = ((uint64)h * n_parts) >> 32 — keys of
+ * one value always meet in one part, and the parts are independent of the hash tables'
+ * bucket function. */
 #define HX_MAX_PARTS 64
 int hx_hash_partition(hx_ctx* ctx, const hx_table* t, int32_t key_col, int n_parts,
                       hx_table** out, int64_t* part_offsets);

@@ -9,9 +9,8 @@
 //               counters), writes counts[part][cta];
 //   k3_scan     one CTA: exclusive scan over (part, cta) -> each CTA's write cursor per part,
 //               and the part offsets;
-//   k3_scatter  each CTA re-reads its chunk and writes every column of a row to its part's
-//               next slot (warp-aggregated shared-memory cursors: one atomic per part per
-//               warp instruction).
+//   k3_scatter  each CTA re-reads its chunk tile by tile, regroups each tile by part in
+//               shared memory and writes one contiguous run per part (coalesced).
 #include <cub/block/block_scan.cuh>
 
 #include <algorithm>
@@ -24,8 +23,18 @@ namespace {
 
 constexpr int kK3Threads = 512;
 
+// (murmur3's fmix32 finaliser, then multiply-shift range reduction. NOT the hash tables'
+// Fibonacci hash: a part function correlated with the bucket function would crowd each part's
+// keys into 1/n_parts of its table's buckets — measured 15 s instead of 10 ms for Q3.1 with
+// 8 parts when both were Fibonacci hashes.)
 __host__ __device__ __forceinline__ int part_of(int32_t key, int n_parts) {
-  return (int)(((unsigned long long)((uint32_t)key * 0x9E3779B1u) * (unsigned)n_parts) >> 32);
+  uint32_t h = (uint32_t)key;
+  h ^= h >> 16;
+  h *= 0x85EBCA6Bu;
+  h ^= h >> 13;
+  h *= 0xC2B2AE35u;
+  h ^= h >> 16;
+  return (int)(((unsigned long long)h * (unsigned)n_parts) >> 32);
 }
 
 struct K3Params {
@@ -78,30 +87,83 @@ __global__ void __launch_bounds__(1024) k3_scan(K3Params p, int grid) {
   if (threadIdx.x == 0) p.part_offsets[p.n_parts] = running;
 }
 
+// Scatter through shared memory: each 2,048-row tile is first regrouped by part in shared
+// memory (one column at a time), then written out as one contiguous run per part (~T/P rows),
+// so the writes coalesce like a copy instead of landing row by row in P places.
+constexpr int kK3Tile = 2048;
+constexpr int kK3PerThread = kK3Tile / kK3Threads;
 __global__ void __launch_bounds__(kK3Threads) k3_scatter(K3Params p) {
-  __shared__ unsigned long long cur[HX_MAX_PARTS];
-  for (int i = threadIdx.x; i < p.n_parts; i += blockDim.x)
+  __shared__ unsigned long long cur[HX_MAX_PARTS];  // next output row of each part
+  __shared__ unsigned tcnt[HX_MAX_PARTS], tstart[HX_MAX_PARTS];
+  __shared__ int32_t buf[kK3Tile];
+  __shared__ uint8_t psorted[kK3Tile];
+  const int tid = threadIdx.x, lane = tid & 31;
+  for (int i = tid; i < p.n_parts; i += blockDim.x)
     cur[i] = (unsigned long long)p.counts[(int64_t)i * gridDim.x + blockIdx.x];
-  __syncthreads();
   const int64_t r0 = (int64_t)blockIdx.x * p.chunk;
   const int64_t r1 = min(p.n_rows, r0 + p.chunk);
-  const int lane = threadIdx.x & 31;
-  for (int64_t base = r0; base < r1; base += blockDim.x) {
-    const int64_t r = base + threadIdx.x;
-    const bool live = r < r1;
-    const int part = live ? part_of(__ldg(p.key + r), p.n_parts) : -1;
-    // warp-aggregated cursor: the lanes of one part take consecutive slots
-    const unsigned act = __ballot_sync(0xFFFFFFFFu, live);
-    unsigned long long pos = 0;
-    if (live) {
-      const unsigned same = __match_any_sync(act, part);
-      const int leader = __ffs(same) - 1;
-      unsigned long long b = 0;
-      if (lane == leader) b = atomicAdd(&cur[part], (unsigned long long)__popc(same));
-      b = __shfl_sync(same, b, leader);
-      pos = b + __popc(same & ((1u << lane) - 1u));
-      for (int c = 0; c < p.n_cols; ++c) p.dst[c][pos] = __ldg(p.src[c] + r);
+  for (int64_t t0 = r0; t0 < r1; t0 += kK3Tile) {
+    const int rows = (int)(r1 - t0 < kK3Tile ? r1 - t0 : (int64_t)kK3Tile);
+    for (int i = tid; i < p.n_parts; i += blockDim.x) tcnt[i] = 0;
+    __syncthreads();
+    int mypart[kK3PerThread], myslot[kK3PerThread];
+#pragma unroll
+    for (int k = 0; k < kK3PerThread; ++k) {
+      const int j = tid + k * kK3Threads;
+      const bool live = j < rows;
+      const int part = live ? part_of(__ldg(p.key + t0 + j), p.n_parts) : 0;
+      const unsigned act = __ballot_sync(0xFFFFFFFFu, live);
+      int slot = 0;
+      if (live) {  // warp-aggregated slot within the tile's part
+        const unsigned same = __match_any_sync(act, part);
+        const int leader = __ffs(same) - 1;
+        unsigned base = 0;
+        if (lane == leader) base = atomicAdd(&tcnt[part], (unsigned)__popc(same));
+        base = __shfl_sync(same, base, leader);
+        slot = (int)(base + __popc(same & ((1u << lane) - 1u)));
+      }
+      mypart[k] = part;
+      myslot[k] = live ? slot : -1;
     }
+    __syncthreads();
+    if (tid < 32) {  // exclusive scan of the (<= 64) tile counts
+      const unsigned a = lane < p.n_parts ? tcnt[lane] : 0u;
+      const unsigned b = lane + 32 < p.n_parts ? tcnt[lane + 32] : 0u;
+      unsigned ia = a;
+#pragma unroll
+      for (int o = 1; o < 32; o <<= 1) {
+        const unsigned v = __shfl_up_sync(0xFFFFFFFFu, ia, o);
+        if (lane >= o) ia += v;
+      }
+      const unsigned tot_a = __shfl_sync(0xFFFFFFFFu, ia, 31);
+      unsigned ib = b;
+#pragma unroll
+      for (int o = 1; o < 32; o <<= 1) {
+        const unsigned v = __shfl_up_sync(0xFFFFFFFFu, ib, o);
+        if (lane >= o) ib += v;
+      }
+      if (lane < p.n_parts) tstart[lane] = ia - a;
+      if (lane + 32 < p.n_parts) tstart[lane + 32] = tot_a + ib - b;
+    }
+    __syncthreads();
+#pragma unroll
+    for (int k = 0; k < kK3PerThread; ++k)
+      if (myslot[k] >= 0) psorted[tstart[mypart[k]] + myslot[k]] = (uint8_t)mypart[k];
+    for (int c = 0; c < p.n_cols; ++c) {
+      const int32_t* src = p.src[c] + t0;
+#pragma unroll
+      for (int k = 0; k < kK3PerThread; ++k)
+        if (myslot[k] >= 0) buf[tstart[mypart[k]] + myslot[k]] = __ldg(src + tid + k * kK3Threads);
+      __syncthreads();
+      int32_t* dst = p.dst[c];
+      for (int i = tid; i < rows; i += kK3Threads) {
+        const int part = psorted[i];
+        dst[cur[part] + (unsigned)(i - (int)tstart[part])] = buf[i];
+      }
+      __syncthreads();
+    }
+    for (int i = tid; i < p.n_parts; i += blockDim.x) cur[i] += tcnt[i];
+    __syncthreads();
   }
 }
 

@@ -35,8 +35,14 @@ def ctx():
 
 
 def part_of(keys: np.ndarray, n_parts: int) -> np.ndarray:
-    """include/hx.h: p = ((uint64)(uint32)(key * 0x9E3779B1) * n_parts) >> 32."""
-    h = (keys.astype(np.int64).astype(np.uint64) * np.uint64(0x9E3779B1)) & np.uint64(0xFFFFFFFF)
+    """include/hx.h part function: fmix32 (murmur3 finaliser), then ((uint64)h * n_parts) >> 32."""
+    m = np.uint64(0xFFFFFFFF)
+    h = keys.astype(np.int64).astype(np.uint64) & m
+    h ^= h >> np.uint64(16)
+    h = (h * np.uint64(0x85EBCA6B)) & m
+    h ^= h >> np.uint64(13)
+    h = (h * np.uint64(0xC2B2AE35)) & m
+    h ^= h >> np.uint64(16)
     return ((h * np.uint64(n_parts)) >> np.uint64(32)).astype(np.int64)
 
 

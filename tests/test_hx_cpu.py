@@ -144,8 +144,14 @@ def test_two_rank_partition_merge_gloo():
 
 # ---- world_size 2 over gloo: the hash-partitioned join's exchange (§8(f) NEXT-1) ----------
 def _part_of(keys, n_parts):
-    """include/hx.h part function: ((uint64)(uint32)(key * 0x9E3779B1) * n_parts) >> 32."""
-    h = (keys.astype(np.int64).astype(np.uint64) * np.uint64(0x9E3779B1)) & np.uint64(0xFFFFFFFF)
+    """include/hx.h part function: fmix32 (murmur3 finaliser), then ((uint64)h * n_parts) >> 32."""
+    m = np.uint64(0xFFFFFFFF)
+    h = keys.astype(np.int64).astype(np.uint64) & m
+    h ^= h >> np.uint64(16)
+    h = (h * np.uint64(0x85EBCA6B)) & m
+    h ^= h >> np.uint64(13)
+    h = (h * np.uint64(0xC2B2AE35)) & m
+    h ^= h >> np.uint64(16)
     return ((h * np.uint64(n_parts)) >> np.uint64(32)).astype(np.int64)
 
 
