@@ -179,6 +179,7 @@ int hx_comm_init(hx_ctx* ctx, int nranks, int rank, const void* id128) {
   std::memcpy(&id, id128, sizeof(id));
   HX_CK(cudaSetDevice(ctx->device));
   HX_NCCL(ncclCommInitRank(&ctx->comm, nranks, id, rank));
+  ctx->force_coll = std::getenv("HX_FORCE_COLLECTIVES") != nullptr;
   ctx->rank = rank;
   ctx->nranks = nranks;
   return HX_OK;
@@ -501,7 +502,7 @@ int hx_merge_aggregates(hx_ctx* ctx, hx_agg* agg, int root, int64_t* sums, int64
   }
   if (m.error) return fail(m.error, "hx_pipeline_probe_agg: group capacity exceeded");
   const int64_t ng = m.n_groups;
-  if (ctx->comm && ctx->nranks > 1 && ng > 0) {
+  if (use_collectives(ctx) && ng > 0) {
     HX_REQUIRE(root < ctx->nranks, HX_EINVAL, "hx_merge_aggregates: bad root");
     // sums and cnts are adjacent regions of cap_groups each: reduce both with one call each
     if (root < 0) {

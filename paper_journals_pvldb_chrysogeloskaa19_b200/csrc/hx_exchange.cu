@@ -260,7 +260,7 @@ int hx_exchange_partitions(hx_ctx* ctx, const hx_table* parted, const int64_t* p
   HX_CK(cudaSetDevice(ctx->device));
   const int nr = ctx->comm ? ctx->nranks : 1;
   HX_REQUIRE(n_parts == nr, HX_EINVAL, "hx_exchange_partitions: n_parts must equal the rank count");
-  if (nr == 1) {  // no exchange: this rank keeps its one part (a library-owned copy)
+  if (!use_collectives(ctx)) {  // no exchange: this rank keeps its one part (a library-owned copy)
     hx_table* o = nullptr;
     int rc = table_alloc_like(ctx, parted, parted->n_rows, &o);
     if (rc != HX_OK) return rc;

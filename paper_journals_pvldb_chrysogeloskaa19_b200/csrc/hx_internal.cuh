@@ -130,6 +130,9 @@ struct hx_ctx {
   int k1_priority = 0;  // launch priority of K1 (the device's greatest; builds keep the default)
   ncclComm_t comm = nullptr;
   int rank = 0, nranks = 1;
+  // run the collectives even on a 1-rank communicator (HX_FORCE_COLLECTIVES=1 at
+  // hx_comm_init): the multi-GPU call sequence, exercised on one GPU by the tests
+  bool force_coll = false;
   // K1 profiling: event pairs around each launch
   bool prof_on = false;
   std::vector<std::pair<cudaEvent_t, cudaEvent_t>> prof_events;
@@ -218,6 +221,10 @@ struct AggMeta {
 };
 
 namespace hx {
+// the union-router merge / exchange go through NCCL (a communicator of > 1 ranks, or forced)
+inline bool use_collectives(const hx_ctx* ctx) {
+  return ctx->comm && (ctx->nranks > 1 || ctx->force_coll);
+}
 // launchers implemented in hx_build.cu / hx_probe.cu
 int build_dim_ht(hx_ctx* ctx, const hx_table* dim, int32_t key_col, const hx_pred* preds,
                  int n_preds, int32_t group_col, int32_t group_lo, int32_t group_hi,

@@ -323,7 +323,7 @@ int hx_plans_enqueue(hx_ctx* ctx, hx_plan* const* plans, int n) {
   // > 1 rank: the pipelines run back to back and the union-router merges of all plans go
   // out as ONE grouped NCCL launch after the last of them (a per-plan allreduce would put
   // 13 collective latencies between the pipelines)
-  const bool grouped = ctx->comm && ctx->nranks > 1 && n > 1;
+  const bool grouped = use_collectives(ctx) && n > 1;
   for (int i = 0; i < n; ++i) {
     int rc = plan_enqueue_probe(ctx, plans[i], /*merge=*/!grouped);
     if (rc != HX_OK) return rc;
@@ -377,7 +377,7 @@ static int plan_enqueue_probe(hx_ctx* ctx, hx_plan* pl, bool merge) {
   int rc = k1_enqueue(ctx, pl->k1, true, pl->k1_e0, pl->k1_e1, pl->ring, /*prepare=*/false);
   if (rc != HX_OK) return rc;
   if (!merge) return HX_OK;  // the caller merges (grouped) and finishes
-  if (ctx->comm && ctx->nranks > 1) {
+  if (use_collectives(ctx)) {
     // union router: partial {sum,cnt} arrays are adjacent, one allreduce over NVLink
     ncclResult_t r = ncclAllReduce(pl->agg.sums, pl->agg.sums, 2 * (size_t)pl->n_groups,
                                    ncclUint64, ncclSum, ctx->comm, ctx->stream);
