@@ -59,6 +59,9 @@ def parse():
     ap.add_argument("--workload", default="ssb", choices=["ssb", "sum", "join"],
                     help="sum / join: the paper's §6.4 micro-benchmarks (SUM over one 23 GB "
                          "column; COUNT of a 1:N join with a 7.7 MB build side)")
+    ap.add_argument("--force-collectives", action="store_true",
+                    help="N=1: a 1-rank NCCL communicator with HX_FORCE_COLLECTIVES=1, so the "
+                         "step includes the union-router allreduce a multi-GPU step issues")
     ap.add_argument("--micro-rows", type=int, default=0,
                     help="fact rows per GPU of the micro-benchmarks (default: the paper's 23 GB)")
     return ap.parse_args()
@@ -97,7 +100,9 @@ def config(args, world, n_rows_gpu, queries):
             "sf_total": args.sf * world, "queries": queries,
             "lineorder_rows_per_gpu": n_rows_gpu, "router_block_rows": BLOCK_ROWS,
             "parallelism": f"lineorder block-partitioned over {world} GPU(s); dims replicated; "
-                           "partials merged by NCCL allreduce" if world > 1 else "1 GPU",
+                           "partials merged by NCCL allreduce" if world > 1 else
+                           ("1 GPU, 1-rank NCCL communicator issuing the merge allreduce"
+                            if getattr(args, "force_collectives", False) else "1 GPU"),
             "l2": "inputs larger than L2 (each query scans >= 0.96 GB/GPU vs 126 MB L2); no flush"}
 
 
@@ -344,6 +349,9 @@ def main():
         uid = [hx.comm_unique_id() if rank == 0 else None]
         dist.broadcast_object_list(uid, src=0)
         ctx.comm_init(world, rank, uid[0])
+    elif args.force_collectives:
+        os.environ["HX_FORCE_COLLECTIVES"] = "1"
+        ctx.comm_init(1, 0, hx.comm_unique_id())
     if args.workload != "ssb":
         run_micro(args, world, rank, local, ctx, stream, torch, dist, hx)
         ctx.close()

@@ -140,7 +140,7 @@ struct hx_graph {
 
 static int plan_enqueue_builds(hx_ctx* ctx, hx_plan* pl);
 static int plan_enqueue_probe(hx_ctx* ctx, hx_plan* pl, bool merge = true);
-static int plan_enqueue_finish(hx_ctx* ctx, hx_plan* pl);
+static int plan_enqueue_finish(hx_ctx* ctx, hx_plan* pl, bool on_fin = false);
 static int join_fin(hx_ctx* ctx);
 
 static void plan_destroy(hx_plan* pl) {
@@ -320,10 +320,12 @@ int hx_plans_enqueue(hx_ctx* ctx, hx_plan* const* plans, int n) {
   if (std::getenv("HX_SERIAL_BUILDS")) {  // A/B: every build done before the first pipeline
     for (int i = 0; i < n; ++i) HX_CK(cudaStreamWaitEvent(ctx->stream, plans[i]->built_ev[0], 0));
   }
-  // > 1 rank: the pipelines run back to back and the union-router merges of all plans go
-  // out as ONE grouped NCCL launch after the last of them (a per-plan allreduce would put
-  // 13 collective latencies between the pipelines)
-  const bool grouped = use_collectives(ctx) && n > 1;
+  // > 1 rank: each plan's union-router allreduce runs on the finalize stream, overlapping
+  // the next pipelines (HX_GROUPED_MERGE: one grouped NCCL launch after the last pipeline
+  // instead — measured 2.87 vs 2.64 ms per SF10 step with a 1-rank communicator: the
+  // finalizes then no longer overlap the pipelines)
+  static const bool grouped_env = std::getenv("HX_GROUPED_MERGE") != nullptr;  // A/B
+  const bool grouped = grouped_env && use_collectives(ctx) && n > 1;
   for (int i = 0; i < n; ++i) {
     int rc = plan_enqueue_probe(ctx, plans[i], /*merge=*/!grouped);
     if (rc != HX_OK) return rc;
@@ -378,19 +380,25 @@ static int plan_enqueue_probe(hx_ctx* ctx, hx_plan* pl, bool merge) {
   if (rc != HX_OK) return rc;
   if (!merge) return HX_OK;  // the caller merges (grouped) and finishes
   if (use_collectives(ctx)) {
-    // union router: partial {sum,cnt} arrays are adjacent, one allreduce over NVLink
+    // union router: partial {sum,cnt} arrays are adjacent, one allreduce over NVLink — on the
+    // finalize stream, so the next plan's K1 does not wait for the collective
+    HX_CK(cudaEventRecord(pl->probed, ctx->stream));
+    HX_CK(cudaStreamWaitEvent(ctx->fin_stream, pl->probed, 0));
     ncclResult_t r = ncclAllReduce(pl->agg.sums, pl->agg.sums, 2 * (size_t)pl->n_groups,
-                                   ncclUint64, ncclSum, ctx->comm, ctx->stream);
+                                   ncclUint64, ncclSum, ctx->comm, ctx->fin_stream);
     HX_REQUIRE(r == ncclSuccess, HX_ENCCL, std::string("ncclAllReduce: ") + ncclGetErrorString(r));
+    return plan_enqueue_finish(ctx, pl, /*on_fin=*/true);
   }
   return plan_enqueue_finish(ctx, pl);
 }
 
 // after the (merged) group arrays are final on the main stream: finalize -> D2H on the
 // finalize stream
-static int plan_enqueue_finish(hx_ctx* ctx, hx_plan* pl) {
-  HX_CK(cudaEventRecord(pl->probed, ctx->stream));
-  HX_CK(cudaStreamWaitEvent(ctx->fin_stream, pl->probed, 0));
+static int plan_enqueue_finish(hx_ctx* ctx, hx_plan* pl, bool on_fin) {
+  if (!on_fin) {  // the group arrays are final on the main stream
+    HX_CK(cudaEventRecord(pl->probed, ctx->stream));
+    HX_CK(cudaStreamWaitEvent(ctx->fin_stream, pl->probed, 0));
+  }
   k1_finalize<<<1, 1024, 0, ctx->fin_stream>>>(pl->fin);
   HX_CK_LAUNCH("k1_finalize");
   ctx->launches += 1;
