@@ -63,8 +63,8 @@ __host__ __device__ __forceinline__ int64_t dm_words_for(int64_t span, int lw) {
 
 // Blocked Bloom filter over the passing keys (one 32-bit word per key, two bits set), built
 // with the table. K1 stages it in shared memory to drop most non-matching rows before any
-// L2 probe (semi-join reduction). kBloomBitsPerKey bits per key: false positives ~5%.
-constexpr int kBloomBitsPerKey = 8;
+// L2 probe (semi-join reduction). kBloomBitsPerKey bits per key: false positives ~1.5% (K1 folds it to 8..1).
+constexpr int kBloomBitsPerKey = 16;
 __host__ __device__ __forceinline__ int bloom_log2w_for(long long n_keys) {
   long long bits = n_keys * kBloomBitsPerKey;
   int l = 5;

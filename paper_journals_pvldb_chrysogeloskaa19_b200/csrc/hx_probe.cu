@@ -1382,7 +1382,7 @@ double plan_dm(int nj, const JoinDev* joins, const bool* known, const double* pa
     opts[j][n++] = {kStFull, 0, pj, true};
     if (d.dm_lw > 0) opts[j][n++] = {kStBitmap, 0, pj, true};
     if (known[j] && keys[j] > 0)
-      for (int f = 1; f <= 8 && bloom_w0[j] / f >= 4; f *= 2) {
+      for (int f = 1; f <= 16 && bloom_w0[j] / f >= 4; f *= 2) {
         const int bw = bloom_w0[j] / f;
         const double e = pj + (1.0 - pj) * bloom_fp(32.0 * bw / (double)keys[j]);
         opts[j][n++] = {kStBloom, bw, e, false};
@@ -1740,7 +1740,7 @@ int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht*
     for (int i = 0; i < sh->n_joins; ++i) {
       const int j = ord[i];
       if (!known[j] || 2 * pass[j] > 1.0) continue;
-      for (int f = 1; f <= 4 && kind[j] == kStNone && bloom_w0[j] / f >= 4; f *= 2) {
+      for (int f = 1; f <= 8 && kind[j] == kStNone && bloom_w0[j] / f >= 4; f *= 2) {
         kind[j] = kStBloom;
         bloom_w[j] = bloom_w0[j] / f;
         if (!fits_sizes(kind, bloom_w)) {
