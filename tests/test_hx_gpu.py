@@ -372,3 +372,35 @@ def test_plan_detects_changed_dimension(ctx):
         pl.rows()
     assert ei.value.code == _hx.HX_ECAPACITY
     pl.close()
+
+
+# ---- probe-order invariance (the join order cannot change the result) --------
+@pytest.mark.parametrize("seed", [0, 1])
+def test_probe_order_permutations(ctx, seed):
+    """Every permutation of a query's joins (probe order = array order; the group key keeps
+    the SELECT order through gdim_join) gives the oracle's rows."""
+    import itertools
+    db = ssbgen.database(21 + seed, ssbgen.sizes(0.01))
+    dims, fact = ssb.load_db_numpy(ctx, db)
+    eng = ssb.SsbEngine(ctx, dims, fact)
+    rng = np.random.default_rng(seed)
+    for q in ("q2.1", "q3.1", "q3.3", "q4.1", "q4.2", "q4.3"):
+        plan = ssb.PLANS[q]
+        want = oracle.run_query(q, db)
+        hts = [eng.build(b) for _, b in plan.joins]
+        perms = list(itertools.permutations(range(len(plan.joins))))
+        for perm in [perms[i] for i in rng.choice(len(perms), size=min(6, len(perms)), replace=False)]:
+            pos = {j: i for i, j in enumerate(perm)}  # original join j probed at position pos[j]
+            shape = hx.query_shape(
+                preds=[ssb._hx_pred(t) for t in plan.fact_preds],
+                joins=[(C[plan.joins[j][0]], j) for j in perm],
+                agg_op=plan.agg[0], agg_a=C[plan.agg[1]], agg_b=C[plan.agg[2]],
+                gdims=[pos[g] for g in plan.gdims])
+            agg = hx.pipeline_probe_agg(ctx, fact, shape, hts)
+            keys, sums, cnts = hx.merge_aggregates(ctx, agg)
+            rows = ssb.order_by(plan, [tuple(int(x) for x in keys[i]) + (int(sums[i]), int(cnts[i]))
+                                       for i in range(len(sums))])
+            agg.close()
+            assert rows == want, (q, perm)
+        for t in hts:
+            t.close()
