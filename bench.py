@@ -577,38 +577,74 @@ def main():
                 ssbgen.column(SEED, sz, c, r0 if t == "lineorder" else 0, n, out=buf.numpy())
                 host[t][c] = (buf, n)
 
+        def timed(step, n):
+            step()
+            ctx.stats(reset=True)
+            if world > 1:
+                dist.barrier()
+            torch.cuda.synchronize()
+            t0 = time.perf_counter()
+            for _ in range(n):
+                step()
+            torch.cuda.synchronize()
+            dt_ = (time.perf_counter() - t0) / n
+            _, h2d_, d2h_ = ctx.stats(reset=True)
+            if world > 1:
+                t = torch.tensor([dt_], device="cuda", dtype=torch.float64)
+                dist.all_reduce(t, op=dist.ReduceOp.MAX)
+                dt_ = float(t[0])
+            return dt_, h2d_ // n, d2h_ // n
+
+        # (1) the serving pattern: device tables and prepared plans created once (outside the
+        # clock); every step copies ALL inputs host -> HBM into them (hx_table_write), runs
+        # the 13 plans (one graph launch) and reads the 13 results back
+        etabs = {t: hx.load_columns(ctx, [(C[c], b_.data_ptr(), n_) for c, (b_, n_) in host[t].items()])
+                 for t in host}
+        eeng = ssb.SsbEngine(ctx, {t: etabs[t] for t in ("date", "customer", "supplier", "part")},
+                             etabs["lineorder"])
+        eplans = {q: eeng.plan(q) for q in queries}
+        eorder = [eplans[q].hp for q in queries]
+        egraph = hx.capture(ctx, lambda: hx.plans_enqueue(ctx, eorder))
+
         def e2e_step():
+            for t, cols_ in host.items():
+                for c, (b_, n_) in cols_.items():
+                    etabs[t].write(C[c], b_.data_ptr(), n_)
+            egraph.launch()
+            return [eplans[q].rows() for q in queries]
+
+        # (2) one-shot: fresh device tables every step and the unprepared calls
+        def e2e_fresh_step():
             def load(t):
-                return hx.load_columns(ctx, [(C[c], b.data_ptr(), n) for c, (b, n) in host[t].items()])
+                return hx.load_columns(ctx, [(C[c], b_.data_ptr(), n_) for c, (b_, n_) in host[t].items()])
             d = {t: load(t) for t in ("date", "customer", "supplier", "part")}
             f = load("lineorder")
             e = ssb.SsbEngine(ctx, d, f)
             pend = [e.start(q) for q in queries]
-            out = [e.finish(p) for p in pend]
+            out = [e.finish(p_) for p_ in pend]
             for tb in list(d.values()) + [f]:
                 tb.close()
             return out
 
-        e2e_step()
-        ctx.stats(reset=True)
-        if world > 1:
-            dist.barrier()
-        torch.cuda.synchronize()
-        t0 = time.perf_counter()
-        for _ in range(args.steps):
-            e2e_step()
-        torch.cuda.synchronize()
-        dt = (time.perf_counter() - t0) / args.steps
-        _, h2d, d2h = ctx.stats(reset=True)
-        if world > 1:
-            t = torch.tensor([dt], device="cuda", dtype=torch.float64)
-            dist.all_reduce(t, op=dist.ReduceOp.MAX)
-            dt = float(t[0])
+        assert e2e_step() == e2e_fresh_step()  # both paths give the same 13 results
+        dt, h2d, d2h = timed(e2e_step, args.steps)
+        dtf, h2df, d2hf = timed(e2e_fresh_step, max(3, args.steps // 5))
         e2e = {"value": len(queries) * total_rows / dt, "unit": UNIT,
-               "h2d_bytes_per_step": h2d // args.steps, "d2h_bytes_per_step": d2h // args.steps,
-               "ms_per_step": dt * 1e3,
-               "path": "hx_load_columns(pinned host -> HBM) + 13 x (hx_build_dim_ht.. + "
-                       "hx_pipeline_probe_agg + hx_merge_aggregates -> host)"}
+               "h2d_bytes_per_step": h2d, "d2h_bytes_per_step": d2h, "ms_per_step": dt * 1e3,
+               "path": "hx_table_write of every lineorder and dimension column (pinned host -> "
+                       "HBM, into the tables the prepared plans were created on) + one graph "
+                       "launch of the 13 plans (builds, K1, merge, finalize, D2H) + 13 host "
+                       "result reads",
+               "fresh": {"value": len(queries) * total_rows / dtf, "ms_per_step": dtf * 1e3,
+                         "h2d_bytes_per_step": h2df, "d2h_bytes_per_step": d2hf,
+                         "path": "hx_load_columns(pinned host -> new HBM tables) + 13 x "
+                                 "(hx_build_dim_ht.. + hx_pipeline_probe_agg + "
+                                 "hx_merge_aggregates -> host)"}}
+        egraph.close()
+        for pl in eplans.values():
+            pl.close()
+        for tb in etabs.values():
+            tb.close()
 
     cpu = None
     if rank == 0 and world == 1 and not args.no_cpu_baseline:

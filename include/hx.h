@@ -111,6 +111,13 @@ int hx_table_free(hx_table* t);
 /* Copies rows [row_begin, row_begin + n) of column `col_id` of `t` (device or host resident)
    into caller host memory `dst` (n int32). Synchronises the ctx stream. */
 int hx_table_read(const hx_table* t, int32_t col_id, int64_t row_begin, int64_t n, int32_t* dst);
+/* Copies n int32 values from caller memory `src` (host — pinned for an asynchronous copy — or
+   device) into rows [row_begin, row_begin + n) of column `col_id` of the device table `t`
+   (HX_PLACE_COPY or HX_PLACE_VIEW), on the ctx stream; asynchronous, `src` must stay valid
+   until the stream reaches the copy. Refreshes the data under prepared plans (mem-move into
+   existing HBM buffers); a plan must be re-created if a dimension's keys or group codes
+   change beyond what it was sized for (hx_plan_enqueue reports it). */
+int hx_table_write(hx_table* t, int32_t col_id, int64_t row_begin, int64_t n, const int32_t* src);
 
 /* ---- dimension filter + hash-table build (§8(a) a3, kernel K2) ----------------------
  * PAPER.md:1160-1163 §6.1 (broadcast-hash-join plans: the build side is the filtered

@@ -379,6 +379,25 @@ int hx_table_read(const hx_table* t, int32_t col_id, int64_t row_begin, int64_t 
   return HX_OK;
 }
 
+int hx_table_write(hx_table* t, int32_t col_id, int64_t row_begin, int64_t n, const int32_t* src) {
+  HX_REQUIRE(t && (src || n == 0) && row_begin >= 0 && n >= 0 && row_begin + n <= t->n_rows,
+             HX_EINVAL, "hx_table_write: bad argument");
+  HX_REQUIRE(t->placement == HX_PLACE_COPY || t->placement == HX_PLACE_VIEW, HX_EUNSUPPORTED,
+             "hx_table_write: the table must be device resident");
+  HX_REQUIRE(table_has_col(t, col_id), HX_EINVAL, "hx_table_write: column not in table");
+  if (n == 0) return HX_OK;
+  HX_CK(cudaSetDevice(t->ctx->device));
+  cudaPointerAttributes pa{};
+  bool src_host = true;
+  if (cudaPointerGetAttributes(&pa, src) == cudaSuccess)
+    src_host = pa.type != cudaMemoryTypeDevice && pa.type != cudaMemoryTypeManaged;
+  cudaGetLastError();
+  HX_CK(cudaMemcpyAsync(const_cast<int32_t*>(table_col(t, col_id)) + row_begin, src, (size_t)n * 4,
+                        cudaMemcpyDefault, t->ctx->stream));
+  if (src_host) t->ctx->h2d_bytes += n * 4;
+  return HX_OK;
+}
+
 int hx_table_free(hx_table* t) {
   HX_REQUIRE(t, HX_EINVAL, "hx_table_free: null table");
   if (t->owned) {

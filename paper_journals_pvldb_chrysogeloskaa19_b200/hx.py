@@ -154,6 +154,11 @@ class Table:
              out.ctypes.data_as(ctypes.POINTER(ctypes.c_int32)))
         return out
 
+    def write(self, col_id: int, src_ptr: int, n: int, row_begin: int = 0) -> None:
+        """Copy n int32 values from `src_ptr` (pinned host or device memory) into a column
+        (asynchronous, on the ctx stream)."""
+        call("hx_table_write", self.h, col_id, row_begin, n, src_ptr)
+
     def close(self):
         if getattr(self, "h", None):
             call("hx_table_free", self.h)

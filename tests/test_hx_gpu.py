@@ -404,3 +404,30 @@ def test_probe_order_permutations(ctx, seed):
             assert rows == want, (q, perm)
         for t in hts:
             t.close()
+
+
+def test_table_write_read_and_plans_on_refreshed_data(ctx):
+    """hx_table_write refreshes the HBM columns under prepared plans (the serving pattern of
+    bench.py's e2e leg): rewrite every lineorder column from host memory (first with another
+    seed's lineorder rows, then the original ones) and the same plan returns each database's
+    oracle rows; hx_table_read returns what was written."""
+    db1 = ssbgen.database(31, ssbgen.sizes(0.01))
+    db2 = ssbgen.database(32, ssbgen.sizes(0.01))
+    dims, fact = ssb.load_db_numpy(ctx, db1)
+    eng = ssb.SsbEngine(ctx, dims, fact)
+    plans = {q: eng.plan(q) for q in ("q1.1", "q2.1", "q4.3")}
+    # (the dimension tables stay db1's: the second database contributes its lineorder rows)
+    for db in (dict(db1, lineorder=db2["lineorder"]), db1):
+        keep = []
+        for c, v in db["lineorder"].items():
+            v = np.ascontiguousarray(v, dtype=np.int32)
+            keep.append(v)
+            fact.write(C[c], v.ctypes.data, len(v))
+        torch.cuda.synchronize()
+        for c, v in db["lineorder"].items():
+            assert np.array_equal(fact.read(C[c]), v), c
+        for q, pl in plans.items():
+            pl.enqueue()
+            assert pl.rows() == oracle.run_query(q, db), q
+    for pl in plans.values():
+        pl.close()
