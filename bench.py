@@ -439,11 +439,17 @@ def main():
                 k1_acc[4] += n_mine * B[q]
         return out
 
+    step_ev = []  # an event after each timed step's launch: per-step device times
+
     def run_steps(n, timed=False):
         prev = None
         for i in range(n):
             cur = sets[i % n_sets]
             launch(cur)
+            if timed:
+                ev = torch.cuda.Event(enable_timing=True)
+                ev.record(stream)
+                step_ev.append(ev)
             if n_sets == 1:
                 collect(cur, timed)
                 continue
@@ -478,6 +484,7 @@ def main():
         dist.all_reduce(t[1:], op=dist.ReduceOp.SUM)
         ms, launches = float(t[0]), int(t[1])
     ms_step = ms / args.steps
+    per_step = [e0.elapsed_time(step_ev[0])] + [a.elapsed_time(b) for a, b in zip(step_ev, step_ev[1:])]
     total_rows = sz["n_lineorder"]
     value = len(queries) * total_rows / (ms_step / 1e3)
 
@@ -654,6 +661,7 @@ def main():
         n_sms, ctas = ctx.info()
         line = {"metric": METRIC, "value": value, "unit": UNIT, "n_gpus": world,
                 "steps": args.steps, "warmup": args.warmup, "ms_per_step": ms_step,
+                "ms_per_step_median": statistics.median(per_step), "ms_per_step_min": min(per_step),
                 "higher_is_better": True, "scaling": "weak", "vs_baseline": None,
                 "dtype": "int32 columns, int64 accumulate",
                 "data": f"synthetic (ssbgen dbgen-shaped SSB distributions, seed {SEED}), "
