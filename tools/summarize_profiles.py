@@ -25,8 +25,8 @@ def main(tag, rep, launches):
            "Captured with `ncu --set full --clock-control none --import-source on -k regex:k1_probe_agg "
            "-s 13 -c 13 python tools/prof_query.py --sf 10 --queries all --reps 2` (the second, "
            "planned execution of each query). ncu times are cold-cache and serialised: compare shares.", "",
-           "| query | kernel | ncu us | algorithmic GB | DRAM r+w GB | traffic/alg | L2 hit % | issue active % | warps active % | regs |",
-           "|---|---|---|---|---|---|---|---|---|---|"]
+           "| query | kernel | ncu us | algorithmic GB | DRAM r+w GB | traffic/alg | DRAM GB/s (% of 8 TB/s) | L2 hit % | issue active % | warps active % | regs |",
+           "|---|---|---|---|---|---|---|---|---|---|---|"]
     def scaled(d, name):  # ncu raw values carry their unit in the second header row
         unit = rows[1][c(name)]
         mult = {"byte": 1, "Kbyte": 1e3, "Mbyte": 1e6, "Gbyte": 1e9, "KB": 1e3, "MB": 1e6, "GB": 1e9}
@@ -40,7 +40,8 @@ def main(tag, rep, launches):
         alg = N * BROW[q[1]]
         tt, ta, tr = tt + t, ta + alg, tr + rd + wr
         out.append(f"| {q} | {d[c('Kernel Name')].split('(')[0].split('::')[-1]} | {t:.1f} | {alg/1e9:.3f} | "
-                   f"{(rd+wr)/1e9:.3f} | {(rd+wr)/alg:.3f} | {float(d[c('lts__t_sector_hit_rate.pct')]):.1f} | "
+                   f"{(rd+wr)/1e9:.3f} | {(rd+wr)/alg:.3f} | {(rd+wr)/(t*1e3):.0f} ({(rd+wr)/(t*1e3)/80:.0f}%) | "
+                   f"{float(d[c('lts__t_sector_hit_rate.pct')]):.1f} | "
                    f"{float(d[c('smsp__issue_active.avg.pct_of_peak_sustained_active')]):.1f} | "
                    f"{float(d[c('sm__warps_active.avg.pct_of_peak_sustained_active')]):.1f} | "
                    f"{d[c('launch__registers_per_thread')]} |")
