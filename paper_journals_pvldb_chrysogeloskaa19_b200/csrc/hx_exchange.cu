@@ -9,8 +9,9 @@
 //               counters), writes counts[part][cta];
 //   k3_scan     one CTA: exclusive scan over (part, cta) -> each CTA's write cursor per part,
 //               and the part offsets;
-//   k3_scatter  each CTA re-reads its chunk tile by tile, regroups each tile by part in
-//               shared memory and writes one contiguous run per part (coalesced).
+//   k3_scatter  each CTA re-reads its chunk tile by tile, regroups each tile (every column at
+//               once: more bytes in flight) by part in shared memory and writes one
+//               contiguous run per part (coalesced).
 #include <cub/block/block_scan.cuh>
 
 #include <algorithm>
@@ -95,7 +96,7 @@ constexpr int kK3PerThread = kK3Tile / kK3Threads;
 __global__ void __launch_bounds__(kK3Threads) k3_scatter(K3Params p) {
   __shared__ unsigned long long cur[HX_MAX_PARTS];  // next output row of each part
   __shared__ unsigned tcnt[HX_MAX_PARTS], tstart[HX_MAX_PARTS];
-  __shared__ int32_t buf[kK3Tile];
+  extern __shared__ int32_t buf[];  // [n_cols][kK3Tile]: every column of the tile in flight at once
   __shared__ uint8_t psorted[kK3Tile];
   const int tid = threadIdx.x, lane = tid & 31;
   for (int i = tid; i < p.n_parts; i += blockDim.x)
@@ -151,17 +152,21 @@ __global__ void __launch_bounds__(kK3Threads) k3_scatter(K3Params p) {
       if (myslot[k] >= 0) psorted[tstart[mypart[k]] + myslot[k]] = (uint8_t)mypart[k];
     for (int c = 0; c < p.n_cols; ++c) {
       const int32_t* src = p.src[c] + t0;
+      int32_t* b = buf + c * kK3Tile;
 #pragma unroll
       for (int k = 0; k < kK3PerThread; ++k)
-        if (myslot[k] >= 0) buf[tstart[mypart[k]] + myslot[k]] = __ldg(src + tid + k * kK3Threads);
-      __syncthreads();
+        if (myslot[k] >= 0) b[tstart[mypart[k]] + myslot[k]] = __ldg(src + tid + k * kK3Threads);
+    }
+    __syncthreads();
+    for (int c = 0; c < p.n_cols; ++c) {
       int32_t* dst = p.dst[c];
+      const int32_t* b = buf + c * kK3Tile;
       for (int i = tid; i < rows; i += kK3Threads) {
         const int part = psorted[i];
-        dst[cur[part] + (unsigned)(i - (int)tstart[part])] = buf[i];
+        dst[cur[part] + (unsigned)(i - (int)tstart[part])] = b[i];
       }
-      __syncthreads();
     }
+    __syncthreads();
     for (int i = tid; i < p.n_parts; i += blockDim.x) cur[i] += tcnt[i];
     __syncthreads();
   }
@@ -212,7 +217,12 @@ int hx_hash_partition(hx_ctx* ctx, const hx_table* t, int32_t key_col, int n_par
     *out = o;
     return HX_OK;
   }
-  const int64_t grid = std::max<int64_t>(1, std::min<int64_t>((int64_t)ctx->n_sms * 4,
+  // one wave of the scatter kernel (its shared memory grows with the column count)
+  const size_t scatter_smem = (size_t)t->n_cols * kK3Tile * sizeof(int32_t);
+  cudaFuncSetAttribute(k3_scatter, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)scatter_smem);
+  int occ = 1;
+  cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, k3_scatter, kK3Threads, scatter_smem);
+  const int64_t grid = std::max<int64_t>(1, std::min<int64_t>((int64_t)ctx->n_sms * std::max(1, occ),
                                                              (t->n_rows + 4095) / 4096));
   K3Params p{};
   p.key = table_col(t, key_col);
@@ -235,7 +245,7 @@ int hx_hash_partition(hx_ctx* ctx, const hx_table* t, int32_t key_col, int n_par
   p.part_offsets = p.counts + (size_t)n_parts * grid;
   k3_count<<<(unsigned)grid, kK3Threads, 0, ctx->stream>>>(p);
   k3_scan<<<1, 1024, 0, ctx->stream>>>(p, (int)grid);
-  k3_scatter<<<(unsigned)grid, kK3Threads, 0, ctx->stream>>>(p);
+  k3_scatter<<<(unsigned)grid, kK3Threads, scatter_smem, ctx->stream>>>(p);
   ctx->launches += 3;
   e = cudaGetLastError();
   if (e == cudaSuccess)
