@@ -230,27 +230,30 @@ class SsbEngine:
         return rows
 
     def run_hash_routed(self, q: str, dim: str, root: int = -1) -> List[Tuple]:
-        """The multi-GPU form: every rank hash-packs its lineorder rows and its rows of `dim`
-        into nranks parts, the hash-routing exchange (hx_exchange_partitions, NCCL send/recv
-        over NVLink) gives rank r part r of everyone, each rank joins what it received
-        (identity ranks for the partitioned dimension, broadcast tables for the others), and
-        the union router merges the partials (allreduce). With one rank: a copy of itself."""
+        """The multi-GPU form: every rank hash-packs its lineorder rows into nranks parts and
+        the hash-routing exchange (hx_exchange_partitions, NCCL send/recv over NVLink) gives
+        rank r part r of everyone's rows; rank r joins them with part r of the (replicated)
+        dimension (identity ranks; the other dimensions broadcast), and the union router
+        merges the partials (allreduce). With one rank: a copy of itself."""
         plan = PLANS[q]
         j = self._join_of(plan, dim)
         fk, b = plan.joins[j]
-        nr = self.ctx.comm_info()[1]
+        rank, nr = self.ctx.comm_info()
         fparts, foffs = hx.hash_partition(self.ctx, self.fact, C[fk], nr)
-        dparts, doffs = hx.hash_partition(self.ctx, self.dims[dim], C[b.key], nr)
         f_in = hx.exchange_partitions(self.ctx, fparts, foffs)
-        d_in = hx.exchange_partitions(self.ctx, dparts, doffs)
         fparts.close()
-        dparts.close()
+        # the dimension tables are replicated on every GPU (§8(a) a1), so rank r's part of the
+        # dimension is already local: hash-pack it and keep part r (exchanging it too would
+        # deliver nranks copies of every key)
+        dparts, doffs = hx.hash_partition(self.ctx, self.dims[dim], C[b.key], nr)
+        d_in = dparts.slice(doffs[rank], doffs[rank + 1])
         hts = [self.build(bb) if i != j else self._partitioned_build(bb, d_in)
                for i, (_, bb) in enumerate(plan.joins)]
         agg = hx.pipeline_probe_agg(self.ctx, f_in, self.shape(plan), hts)
         rows = self.finish(Pending(plan, hts, agg), root)
         f_in.close()
         d_in.close()
+        dparts.close()
         return rows
 
     # ---- prepared plans (allocation- and sync-free executions, graph capturable) ----------
