@@ -1,7 +1,7 @@
 """The multi-GPU (NCCL) call sequences on ONE GPU: a 1-rank communicator with
 HX_FORCE_COLLECTIVES=1 makes libhx issue every collective it would issue with N ranks — the
-union-router allreduce / reduce of hx_merge_aggregates, the grouped allreduce of a multi-plan
-step (inside a captured CUDA graph), the mem-move broadcast of a built hash table, and the
+union-router allreduce / reduce of hx_merge_aggregates, the per-plan allreduces of a
+multi-plan step (on the finalize stream, inside a captured CUDA graph), the mem-move broadcast of a built hash table, and the
 hash-routing exchange's allgather + send/recv — so their buffers, sizes and ordering are
 checked bit-exactly against the oracle. (NCCL refuses two ranks on one device; the N-rank
 data flow is covered by the gloo tests in test_hx_cpu.py.)
@@ -49,7 +49,8 @@ def test_merge_allreduce_and_reduce(nctx, db, root):
         assert eng.finish(eng.start(q), root) == oracle.run_query(q, db), (q, root)
 
 
-def test_plans_grouped_allreduce_in_graph(nctx, db):
+def test_plans_allreduce_in_graph(nctx, db):
+    """Each plan's union-router allreduce on the finalize stream, inside a captured graph."""
     dims, fact = ssb.load_db_numpy(nctx, db)
     eng = ssb.SsbEngine(nctx, dims, fact)
     plans = {q: eng.plan(q) for q in QUERIES}
