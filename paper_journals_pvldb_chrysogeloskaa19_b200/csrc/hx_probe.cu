@@ -1624,7 +1624,8 @@ int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht*
     }
     const bool ok = bound * 16.0 <= 1.0 && fact->placement != HX_PLACE_HOST_PINNED &&
                     fact->placement != HX_PLACE_HOST_MAPPED &&
-                    fact->n_rows < (int64_t(1) << 32) && std::getenv("HX_NO_GATHER") == nullptr;
+                    std::getenv("HX_NO_GATHER") == nullptr;  // (any size: launch segments keep
+                                                             // row offsets 32-bit)
     auto read_by_stages = [&](int32_t col) {
       for (int q = 0; q < sh->n_preds; ++q)
         if (sh->preds[q].col_id == col) return true;
