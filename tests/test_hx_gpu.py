@@ -431,3 +431,27 @@ def test_table_write_read_and_plans_on_refreshed_data(ctx):
             assert pl.rows() == oracle.run_query(q, db), q
     for pl in plans.values():
         pl.close()
+
+
+@pytest.mark.parametrize("case", ["no_passing_part", "empty_supplier", "empty_date"])
+def test_degenerate_dimensions(ctx, case):
+    """A dimension filter that passes nothing, and empty dimension tables: every dependent
+    query yields the oracle's (empty, or count-0) result — plain calls and prepared plans."""
+    db = tiny_db(29, n_lo=9001)
+    db = {t: dict(cols) for t, cols in db.items()}
+    if case == "no_passing_part":
+        db["part"]["p_category"] = np.full_like(db["part"]["p_category"], 24)
+        db["part"]["p_brand1"] = np.full_like(db["part"]["p_brand1"], 24 * 40)
+        db["part"]["p_mfgr"] = np.full_like(db["part"]["p_mfgr"], 4)
+    else:
+        t = case.split("_")[1]
+        db[t] = {k: v[:0] for k, v in db[t].items()}
+    dims, fact = ssb.load_db_numpy(ctx, db)
+    eng = ssb.SsbEngine(ctx, dims, fact)
+    for q in QUERIES:
+        want = oracle.run_query(q, db)
+        assert eng.run(q) == want, (case, q)
+        pl = eng.plan(q)
+        pl.enqueue()
+        assert pl.rows() == want, (case, q)
+        pl.close()
