@@ -182,7 +182,9 @@ int hx_build_dim_ht_ex(hx_ctx* ctx, const hx_table* dim, int32_t key_col, const 
  * Part function: h = fmix32((uint32)key) (murmur3 finaliser: h ^= h >> 16; h *= 0x85EBCA6B;
  * h ^= h >> 13; h *= 0xC2B2AE35; h ^= h >> 16), p = ((uint64)h * n_parts) >> 32 — keys of
  * one value always meet in one part, and the parts are independent of the hash tables'
- * bucket function. */
+ * bucket function.
+ * Errors: HX_EINVAL (null argument, n_parts outside 1..HX_MAX_PARTS, key column not in t),
+ * HX_EUNSUPPORTED (t not device resident), HX_ENOMEM / HX_ECUDA (allocation, launch). */
 #define HX_MAX_PARTS 64
 int hx_hash_partition(hx_ctx* ctx, const hx_table* t, int32_t key_col, int n_parts,
                       hx_table** out, int64_t* part_offsets);
@@ -190,7 +192,9 @@ int hx_hash_partition(hx_ctx* ctx, const hx_table* t, int32_t key_col, int n_par
    nranks) goes to rank p; *out receives, in rank order, the rows every rank routed here — one
    grouped set of ncclSend/ncclRecv per column over NVLink after an ncclAllGather of the part
    sizes. Collective over the communicator. Without a communicator of > 1 ranks it returns a
-   copy of part 0 (n_parts must be 1 then). Synchronises. */
+   copy of part 0 (n_parts must be 1 then). Synchronises. Errors: HX_EINVAL (offsets that do
+   not match the table, n_parts != the rank count), HX_ENCCL (a collective failed; message in
+   hx_last_error), HX_ENOMEM / HX_ECUDA. *out is library-owned (hx_table_free). */
 int hx_exchange_partitions(hx_ctx* ctx, const hx_table* parted, const int64_t* part_offsets,
                            int n_parts, hx_table** out);
 
