@@ -6,14 +6,19 @@ lineorder partition: filter + hash-table build of every joined dimension (K2), t
 scan -> filter -> probe x k -> aggregate pipeline (K1), and the union-router merge of the
 partial aggregates (NCCL allreduce when N > 1) with the result copied to the host.
 
-Workload (config.workload): SSB SF10 per GPU, HBM-resident (BASELINE.json configs[1] at
-N=1; weak scaling: N GPUs run SF 10*N with lineorder range-partitioned in 2^22-row router
-blocks and the dimensions replicated). Synthetic dbgen-shaped data from ssbgen (seed 42),
-generated directly in HBM outside the timed region. Each query scans 0.96-1.44 GB per GPU,
-larger than the 126 MB L2, so no L2 flush is needed between queries.
+Workload (config.workload): SSB SF100 per GPU, HBM-resident — BASELINE.json configs[2], the
+largest configuration that fits one GPU (N=1); weak scaling: N GPUs run SF 100*N with
+lineorder range-partitioned in 2^22-row router blocks and the dimensions replicated.
+Synthetic dbgen-shaped data from ssbgen (seed 42), generated directly in HBM outside the
+timed region. Each query scans 9.6-14.4 GB per GPU, far larger than the 126 MB L2, so no L2
+flush is needed between queries (--l2-flush flushes between steps for the SF1 C1 case).
 
     python bench.py [--gpus N] [--steps K] [--warmup W] [--sf SF_PER_GPU] [--impl reference]
     python -m torch.distributed.run --nproc-per-node N ... bench.py --gpus N ...
+
+`--gpus N > 1` without a torch.distributed launcher re-executes itself under
+`python -m torch.distributed.run --nproc-per-node N` (one process per GPU); under a launcher,
+WORLD_SIZE must equal N (a mismatch is an error, never a silent 1-GPU run).
 """
 from __future__ import annotations
 
@@ -40,12 +45,12 @@ SEED = 42
 BLOCK_ROWS = 1 << 22
 
 
-def parse():
+def parse(argv=None):
     ap = argparse.ArgumentParser()
     ap.add_argument("--gpus", type=int, default=1)
     ap.add_argument("--steps", type=int, default=50)
     ap.add_argument("--warmup", type=int, default=3)
-    ap.add_argument("--sf", type=float, default=10.0, help="SSB scale factor per GPU")
+    ap.add_argument("--sf", type=float, default=100.0, help="SSB scale factor per GPU")
     ap.add_argument("--impl", default="hx", choices=["hx", "reference"])
     ap.add_argument("--no-cpu-baseline", action="store_true")
     ap.add_argument("--no-e2e", action="store_true")
@@ -64,7 +69,15 @@ def parse():
                          "step includes the union-router allreduce a multi-GPU step issues")
     ap.add_argument("--micro-rows", type=int, default=0,
                     help="fact rows per GPU of the micro-benchmarks (default: the paper's 23 GB)")
-    return ap.parse_args()
+    ap.add_argument("--sizeup", action="store_true",
+                    help="with --workload sum|join: the §6.4 size-up sweep (0.125-16 GB per "
+                         "column), one JSON line per size")
+    ap.add_argument("--no-ht-path", action="store_true",
+                    help="skip the ht_path block (the same plans on open-addressing hash tables)")
+    ap.add_argument("--l2-flush", action="store_true",
+                    help="flush L2 (write 2x its size) between timed steps, outside the per-step "
+                         "events (small inputs, e.g. C1 = --sf 1 --queries q1.1)")
+    return ap.parse_args(argv)
 
 
 def dist_env():
@@ -72,6 +85,35 @@ def dist_env():
     rank = int(os.environ.get("RANK", "0"))
     local = int(os.environ.get("LOCAL_RANK", "0"))
     return world, rank, local
+
+
+def free_port():
+    import socket
+    s = socket.socket()
+    s.bind(("127.0.0.1", 0))
+    port = s.getsockname()[1]
+    s.close()
+    return port
+
+
+def launch_plan(gpus, env, argv):
+    """How this invocation runs: ("run", None) in this process, ("relaunch", cmd) under
+    torch.distributed.run with one process per GPU, or ("error", message).
+    `--gpus N > 1` without WORLD_SIZE re-executes under the launcher; with WORLD_SIZE set it
+    must equal N (the driver's torchrun launch), never a silent 1-GPU run."""
+    if gpus < 1:
+        return "error", f"bench.py: --gpus {gpus} < 1"
+    ws = env.get("WORLD_SIZE")
+    if ws is None:
+        if gpus == 1:
+            return "run", None
+        cmd = [sys.executable, "-m", "torch.distributed.run", "--nnodes=1",
+               f"--nproc-per-node={gpus}", "--master-addr=127.0.0.1",
+               f"--master-port={free_port()}", os.path.abspath(__file__)] + list(argv)
+        return "relaunch", cmd
+    if int(ws) != gpus:
+        return "error", f"bench.py: --gpus {gpus} but WORLD_SIZE={ws} (launch one process per GPU)"
+    return "run", None
 
 
 def peaks():
@@ -103,7 +145,10 @@ def config(args, world, n_rows_gpu, queries):
                            "partials merged by NCCL allreduce" if world > 1 else
                            ("1 GPU, 1-rank NCCL communicator issuing the merge allreduce"
                             if getattr(args, "force_collectives", False) else "1 GPU"),
-            "l2": "inputs larger than L2 (each query scans >= 0.96 GB/GPU vs 126 MB L2); no flush"}
+            "l2": ("L2 flushed between steps (a 256 MB buffer written outside the per-step "
+                   "events)" if getattr(args, "l2_flush", False) else
+                   f"inputs larger than L2 (each query scans >= {0.096 * args.sf:.2f} GB/GPU vs "
+                   f"126 MB L2); no flush")}
 
 
 class Clocks:
@@ -210,7 +255,10 @@ def run_reference(args, world, rank):
             "steps": args.steps, "warmup": args.warmup, "ms_per_step": dt * 1e3,
             "higher_is_better": True, "scaling": "weak", "vs_baseline": None, "dtype": "int64",
             "data": f"synthetic (ssbgen dbgen-shaped SSB, seed {SEED})",
-            "config": config(args, world, sz["n_lineorder"] // world, queries),
+            "config": dict(config(args, world, sz["n_lineorder"] // world, queries),
+                           executed_as=f"reference arm: the CPU oracle (oracle/ssb_oracle.cpp) "
+                                       f"over lineorder rows [0, {sample}) in host memory, not "
+                                       f"the HBM-resident GPU path", sample_rows=sample),
             "cpu_baseline": {"value": value, "unit": UNIT, "cores": threads, "kind": "oracle",
                              "sample": samp},
             "e2e": {"value": value, "unit": UNIT, "h2d_bytes_per_step": 0, "d2h_bytes_per_step": 0}}
@@ -221,7 +269,7 @@ def cpu_baseline(args, world):
     """The oracle, single-threaded as it stands, on a bounded sample (rank 0, N=1)."""
     import oracle
     sz = ssbgen.sizes(args.sf * world)
-    sample = min(sz["n_lineorder"], 2_000_000)
+    sample = min(sz["n_lineorder"], 12_000_000)  # ~10 s of single-threaded oracle work
     db = ssbgen.database(SEED, sz, 0, sample)
     idx = oracle.DimIndex(db)  # the dimension maps, built once (not timed: SURVEY.md 8(d))
     t0 = time.perf_counter()
@@ -348,7 +396,19 @@ def run_micro(args, world, rank, local, ctx, stream, torch, dist, hx):
 
 def main():
     args = parse()
+    how, what = launch_plan(args.gpus, os.environ, sys.argv[1:])
+    if how == "error":
+        print(what, file=sys.stderr, flush=True)
+        sys.exit(2)
+    if how == "relaunch":
+        env = dict(os.environ)
+        env.setdefault("NCCL_DEBUG", "INFO")  # the communicator log shows nranks = N
+        env.setdefault("NCCL_DEBUG_SUBSYS", "INIT")
+        sys.exit(subprocess.run(what, env=env).returncode)
     world, rank, local = dist_env()
+    if world > 1:
+        os.environ.setdefault("NCCL_DEBUG", "INFO")
+        os.environ.setdefault("NCCL_DEBUG_SUBSYS", "INIT")
     if args.impl == "reference":
         run_reference(args, world, rank)
         return
@@ -357,6 +417,10 @@ def main():
     import torch.distributed as dist
     from paper_journals_pvldb_chrysogeloskaa19_b200 import hx, ssb
 
+    if torch.cuda.device_count() <= local:
+        print(f"bench.py: rank {rank} needs GPU {local} but {torch.cuda.device_count()} are visible",
+              file=sys.stderr, flush=True)
+        sys.exit(2)
     torch.cuda.set_device(local)
     if world > 1:
         dist.init_process_group("nccl", device_id=torch.device("cuda", local))
@@ -429,7 +493,7 @@ def main():
     # i+1 use different buffers), so the host reads step i's results while the device
     # already runs step i+1 — every step still builds, probes, merges and reads everything.
     big = n_mine * 4 * len(lo_cols) > (64 << 30)  # SF >= ~300 per GPU: one plan set fits
-    n_sets = 1 if (args.no_graph or args.no_pipeline or big) else 2
+    n_sets = 1 if (args.no_graph or args.no_pipeline or big or args.l2_flush) else 2
     sets = []
     for _ in range(n_sets):
         pl_ = {q: eng.plan(q) for q in queries}
@@ -462,10 +526,21 @@ def main():
 
     step_ev = []  # an event after each timed step's launch: per-step device times
 
+    # --l2-flush: a 2 x L2 buffer is written between steps (outside the per-step events), so
+    # every step starts with a cold L2 (inputs smaller than L2, e.g. C1 = SF1 Q1.1, 96 MB)
+    flush_buf = torch.empty(64 << 20, dtype=torch.int32, device="cuda") if args.l2_flush else None
+    flush_ev = []
+
     def run_steps(n, timed=False):
         prev = None
         for i in range(n):
             cur = sets[i % n_sets]
+            if flush_buf is not None:
+                flush_buf.fill_(i)
+                if timed:
+                    ev = torch.cuda.Event(enable_timing=True)
+                    ev.record(stream)
+                    flush_ev.append(ev)
             launch(cur)
             if timed:
                 ev = torch.cuda.Event(enable_timing=True)
@@ -497,6 +572,8 @@ def main():
         dist.barrier()
     clk = clocks.stop()
     ms = e0.elapsed_time(e1)
+    if flush_buf is not None:  # the steps only: each from its flush's end to its own end
+        ms = sum(a.elapsed_time(b) for a, b in zip(flush_ev, step_ev))
     k1_ms, k1_n, k1_moved, k1_span, k1_bytes = k1_acc
     launches, step_h2d, step_d2h = ctx.stats(reset=True)
     if world > 1:
@@ -505,7 +582,8 @@ def main():
         dist.all_reduce(t[1:], op=dist.ReduceOp.SUM)
         ms, launches = float(t[0]), int(t[1])
     ms_step = ms / args.steps
-    per_step = [e0.elapsed_time(step_ev[0])] + [a.elapsed_time(b) for a, b in zip(step_ev, step_ev[1:])]
+    per_step = ([a.elapsed_time(b) for a, b in zip(flush_ev, step_ev)] if flush_buf is not None else
+                [e0.elapsed_time(step_ev[0])] + [a.elapsed_time(b) for a, b in zip(step_ev, step_ev[1:])])
     total_rows = sz["n_lineorder"]
     value = len(queries) * total_rows / (ms_step / 1e3)
 
@@ -578,7 +656,61 @@ def main():
                         "k1_frac_of_peak": (n_mine * B[q] / (kms / 1e3) / 1e9) / peak if kms else None,
                         "bytes_per_row": B[q],
                         "k1_moved_gbps": kmoved / reps / (kms / 1e3) / 1e9 if kms else None,
+                        "k1_frac_moved": kmoved / reps / (kms / 1e3) / 1e9 / peak if kms else None,
                         "moved_bytes_per_row": kmoved / reps / max(n_mine, 1)}
+
+    # ---- ht_path: the same step on open-addressing hash tables (north_star's layout) -------
+    # Plans created under HX_OPT_JOIN_LAYOUT = HX_JOIN_HASH probe the hash tables of the
+    # dimension builds instead of direct maps (R20); same
+    # results, timed the same way (one graph per step, K steps), per query K1 as above.
+    ht_path = None
+    if args.variant == "hbm" and not args.no_ht_path and not big:
+        ctx.set_option(hx._hx.HX_OPT_JOIN_LAYOUT, hx._hx.HX_JOIN_HASH)
+        hpl = {q: eng.plan(q) for q in queries}
+        ctx.set_option(hx._hx.HX_OPT_JOIN_LAYOUT, hx._hx.HX_JOIN_AUTO)
+        hod = [hpl[q].hp for q in queries]
+        hgr = hx.capture(ctx, lambda: hx.plans_enqueue(ctx, hod))
+        same = True
+        for _ in range(max(1, args.warmup)):
+            hgr.launch()
+            same = same and all(hpl[q].rows() == plans[q].rows() for q in queries)
+        if world > 1:
+            dist.barrier()
+        torch.cuda.synchronize()
+        he0, he1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+        hk = {q: [0.0, 0] for q in queries}
+        he0.record(stream)
+        for _ in range(args.steps):
+            hgr.launch()
+            for q in queries:
+                hpl[q].rows()
+                ms_, b_ = hpl[q].hp.k1_time()
+                hk[q][0] += ms_
+                hk[q][1] += b_
+        he1.record(stream)
+        torch.cuda.synchronize()
+        hms = he0.elapsed_time(he1)
+        if world > 1:
+            t = torch.tensor([hms], device="cuda", dtype=torch.float64)
+            dist.all_reduce(t, op=dist.ReduceOp.MAX)
+            hms = float(t[0])
+        hms_step = hms / args.steps
+        hq = {}
+        for q in queries:
+            kms = hk[q][0] / args.steps
+            hq[q] = {"k1_ms": round(kms, 4),
+                     "k1_frac_of_peak": n_mine * B[q] / (kms / 1e3) / 1e9 / peak if kms else None,
+                     "k1_frac_moved": hk[q][1] / args.steps / (kms / 1e3) / 1e9 / peak if kms else None,
+                     "k1_vs_direct_map": kms / per_query[q]["k1_ms"] if per_query[q]["k1_ms"] else None}
+        hvalue = len(queries) * total_rows / (hms_step / 1e3)
+        ht_path = {"value": hvalue, "unit": UNIT, "ms_per_step": hms_step,
+                   "vs_direct_map": hvalue / value, "results_identical": same,
+                   "layout": "open addressing, 16-byte buckets of two {key, rank} slots, load "
+                             "<= 1/4, Bloom filters in shared memory (hx_build_dim_ht)",
+                   "per_query": hq}
+        hgr.close()
+        for pl in hpl.values():
+            pl.close()
 
     # ---- e2e through the C-ABI with HOST buffers (H2D + queries + D2H inside the clock) ---
     e2e = None
@@ -592,18 +724,26 @@ def main():
                        if args.variant == "host" else
                        ("plans over a HX_PLACE_HOST_MAPPED fact table: K1 reads pinned host "
                         "memory in place over PCIe + merge + finalize + D2H, one CUDA graph per step")}
-    elif not args.no_e2e and n_mine * 4 * len(lo_cols) > (32 << 30):
-        e2e = {"value": None, "unit": UNIT, "skipped": "lineorder partition larger than the "
-               "32 GB of pinned host memory this run allocates for the e2e leg"}
+    elif not args.no_e2e and (n_mine * 4 * len(lo_cols) > (32 << 30)
+                              or world * n_mine * 4 * len(lo_cols) > (256 << 30)):
+        e2e = {"value": None, "unit": UNIT, "skipped": "lineorder partitions larger than the "
+               "pinned host memory the e2e leg allocates (32 GB per rank, 256 GB per node)"}
     elif not args.no_e2e:
+        # the host copies of this rank's inputs, in page-locked memory (filled from the same
+        # seeded generator: generated in HBM and copied down, outside the clock)
         host = {}
         for t in ("lineorder", "date", "customer", "supplier", "part"):
             host[t] = {}
             for c in (lo_cols if t == "lineorder" else ssbgen.TABLE_COLS[t]):
                 n = n_mine if t == "lineorder" else ssbgen.table_rows(sz, c)
                 buf = torch.empty(max(n, 1), dtype=torch.int32, pin_memory=True)
-                ssbgen.column(SEED, sz, c, r0 if t == "lineorder" else 0, n, out=buf.numpy())
+                tmp = torch.empty(max(n, 1), dtype=torch.int32, device="cuda")
+                ssbgen.column_device(SEED, sz, c, tmp.data_ptr(), r0 if t == "lineorder" else 0, n,
+                                     stream.cuda_stream)
+                buf.copy_(tmp)
+                del tmp
                 host[t][c] = (buf, n)
+        torch.cuda.synchronize()
 
         def timed(step, n, flush=None, ctxs=(ctx,)):
             step()
@@ -729,7 +869,7 @@ def main():
                                             "step i+1" if n_sets == 2 else "none"),
                 "hbm_gbps_per_gpu": sum(n_mine * B[q] for q in queries) / (ms_step / 1e3) / 1e9,
                 "roofline": roofline, "cpu_baseline": cpu, "e2e": e2e, "clocks": clk,
-                "gpu_launches": launches, "per_query": per_query,
+                "gpu_launches": launches, "per_query": per_query, "ht_path": ht_path,
                 "k1_ctas_per_sm": ctas, "n_sms": n_sms}
         print(json.dumps(line), flush=True)
     # release library objects before their context

@@ -48,6 +48,16 @@ int hx_finalize(hx_ctx* ctx);
 int hx_ctx_stream(hx_ctx* ctx, void** stream);
 /* Number of SMs and resident K1 CTAs per SM chosen for this device (for reporting). */
 int hx_ctx_info(hx_ctx* ctx, int* n_sms, int* k1_ctas_per_sm);
+/* Context options (read when a plan is created, hx_plan_create):
+   HX_OPT_JOIN_LAYOUT: HX_JOIN_AUTO (default) lets a plan whose dimension keys are dense
+   (span < 2^27, map no larger than the rule in DESIGN.md R20) probe a direct map — the hash
+   table under the identity hash; HX_JOIN_HASH keeps the open-addressing hash tables
+    for every plan. Same results either way (keys are unique).
+   HX_OPT_L2_PERSIST: 1 (default) gives each K1 launch an L2 access-policy window
+   (persisting) over its largest probe structure read from L2; 0 disables it. */
+enum { HX_OPT_JOIN_LAYOUT = 1, HX_OPT_L2_PERSIST = 2 };
+enum { HX_JOIN_AUTO = 0, HX_JOIN_HASH = 1 };
+int hx_ctx_set_option(hx_ctx* ctx, int option, int value);
 
 /* ---- communicator (NCCL over NVLink/NVSwitch; one rank per GPU) ------------------- */
 /* The 128-byte ncclUniqueId, created on rank 0 and shipped to the others by the caller
@@ -55,6 +65,19 @@ int hx_ctx_info(hx_ctx* ctx, int* n_sms, int* k1_ctas_per_sm);
 int hx_comm_unique_id(void* id128);
 int hx_comm_init(hx_ctx* ctx, int nranks, int rank, const void* id128);
 int hx_comm_info(hx_ctx* ctx, int* rank, int* nranks);
+/* Collective trace: every NCCL data call libhx issues on this ctx (at issue time on the host;
+   a call captured into a CUDA graph is recorded once, at capture) is appended as one record:
+   the operation, the element count and element size it was issued with, the root (reduce,
+   broadcast) or peer (send, recv; -1 otherwise) and the device buffer. A 1-rank communicator
+   turns allreduce / broadcast into identities, so this is how the tests check the sizes the
+   multi-rank path would move (2 x n_groups per plan merge, the HT's bytes per broadcast).
+   hx_comm_trace copies up to `cap` of the oldest retained records (the last 4096 are kept) into
+   `out`, stores the number retained in *n, and clears them if `reset`. Host only; no sync. */
+enum { HX_COLL_ALLREDUCE = 1, HX_COLL_REDUCE = 2, HX_COLL_BROADCAST = 3, HX_COLL_ALLGATHER = 4,
+       HX_COLL_SEND = 5, HX_COLL_RECV = 6 };
+typedef struct { int32_t op; int32_t root_or_peer; int64_t count; int32_t elem_bytes;
+                 int32_t reserved; uint64_t buf; } hx_coll_rec;
+int hx_comm_trace(hx_ctx* ctx, hx_coll_rec* out, int cap, int* n, int reset);
 
 /* ---- router: segmenter + range / round-robin policy (§8(a) a2) ---------------------
  * PAPER.md:469-473 §3.1 (the segmenter splits the input into block-shaped partitions; the

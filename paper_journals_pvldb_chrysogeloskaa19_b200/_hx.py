@@ -22,6 +22,10 @@ HX_AGG_SUM, HX_AGG_SUM_MUL, HX_AGG_SUM_SUB = 0, 1, 2
 HX_MAX_COLS, HX_MAX_PREDS, HX_MAX_JOINS, HX_MAX_GDIMS = 16, 3, 4, 3
 HX_BUILD_IDENTITY_RANKS = 1
 HX_MAX_PARTS = 64
+HX_OPT_JOIN_LAYOUT, HX_OPT_L2_PERSIST = 1, 2
+HX_JOIN_AUTO, HX_JOIN_HASH = 0, 1
+(HX_COLL_ALLREDUCE, HX_COLL_REDUCE, HX_COLL_BROADCAST, HX_COLL_ALLGATHER, HX_COLL_SEND,
+ HX_COLL_RECV) = 1, 2, 3, 4, 5, 6
 
 _NAMES = {0: "HX_OK", -1: "HX_EINVAL", -2: "HX_ECUDA", -3: "HX_ENCCL", -4: "HX_ENOMEM",
           -5: "HX_ECAPACITY", -6: "HX_EDUPKEY", -7: "HX_EUNSUPPORTED"}
@@ -62,6 +66,11 @@ class hx_build_spec(ctypes.Structure):
                 ("group_lo", ctypes.c_int32), ("group_hi", ctypes.c_int32)]
 
 
+class hx_coll_rec(ctypes.Structure):
+    _fields_ = [("op", ctypes.c_int32), ("root_or_peer", ctypes.c_int32), ("count", ctypes.c_int64),
+                ("elem_bytes", ctypes.c_int32), ("reserved", ctypes.c_int32), ("buf", ctypes.c_uint64)]
+
+
 _P = ctypes.c_void_p
 _PP = ctypes.POINTER(ctypes.c_void_p)
 _I = ctypes.c_int
@@ -76,9 +85,11 @@ _SIGS = {
     "hx_finalize": ([_P], _I),
     "hx_ctx_stream": ([_P, _PP], _I),
     "hx_ctx_info": ([_P, ctypes.POINTER(_I), ctypes.POINTER(_I)], _I),
+    "hx_ctx_set_option": ([_P, _I, _I], _I),
     "hx_comm_unique_id": ([_P], _I),
     "hx_comm_init": ([_P, _I, _I, _P], _I),
     "hx_comm_info": ([_P, ctypes.POINTER(_I), ctypes.POINTER(_I)], _I),
+    "hx_comm_trace": ([_P, ctypes.POINTER(hx_coll_rec), _I, ctypes.POINTER(_I), _I], _I),
     "hx_router_partition": ([_I64, _I, _I64, _I, _PP], _I),
     "hx_partition_info": ([_P, _PI64, ctypes.POINTER(ctypes.POINTER(hx_block))], _I),
     "hx_partition_rows": ([_P, _I, _PI64], _I),

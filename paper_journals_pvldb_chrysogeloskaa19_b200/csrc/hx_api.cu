@@ -98,6 +98,22 @@ int hx_init(int device, void* stream, hx_ctx** out) {
   }
   ctx->k1_ctas_per_sm = std::max(1, k1_occupancy(ctx));
   {
+    // L2 set-aside for persisting accesses (the probe structures' access-policy windows):
+    // the device maximum (HX_L2_PERSIST_MB lowers it; 0 disables)
+    int pmax = 0, wmax = 0;
+    cudaDeviceGetAttribute(&pmax, cudaDevAttrMaxPersistingL2CacheSize, device);
+    cudaDeviceGetAttribute(&wmax, cudaDevAttrMaxAccessPolicyWindowSize, device);
+    int64_t want = pmax;
+    if (const char* e = std::getenv("HX_L2_PERSIST_MB")) want = std::min<int64_t>(want, std::atoll(e) << 20);
+    if (want > 0 && wmax > 0 && cudaDeviceSetLimit(cudaLimitPersistingL2CacheSize, (size_t)want) == cudaSuccess) {
+      size_t got = 0;
+      cudaDeviceGetLimit(&got, cudaLimitPersistingL2CacheSize);
+      ctx->l2_persist_max = (int64_t)got;
+      ctx->l2_window_max = wmax;
+    }
+    cudaGetLastError();
+  }
+  {
     int least = 0, greatest = 0;
     if (cudaDeviceGetStreamPriorityRange(&least, &greatest) == cudaSuccess &&
         std::getenv("HX_NO_K1_PRIORITY") == nullptr)
@@ -446,6 +462,28 @@ int hx_ht_info(hx_ht* ht, int64_t* n_keys, int64_t* n_slots, int32_t* n_ranks,
   return HX_OK;
 }
 
+int hx_ctx_set_option(hx_ctx* ctx, int option, int value) {
+  HX_REQUIRE(ctx, HX_EINVAL, "hx_ctx_set_option: null ctx");
+  if (option == HX_OPT_JOIN_LAYOUT) {
+    HX_REQUIRE(value == HX_JOIN_AUTO || value == HX_JOIN_HASH, HX_EINVAL,
+               "hx_ctx_set_option: bad join layout");
+    ctx->join_layout = value;
+  } else if (option == HX_OPT_L2_PERSIST) {
+    ctx->l2_persist = value != 0;
+  } else {
+    return fail(HX_EINVAL, "hx_ctx_set_option: unknown option");
+  }
+  return HX_OK;
+}
+
+int hx_comm_trace(hx_ctx* ctx, hx_coll_rec* out, int cap, int* n, int reset) {
+  HX_REQUIRE(ctx && n && cap >= 0 && (cap == 0 || out), HX_EINVAL, "hx_comm_trace: bad argument");
+  *n = (int)ctx->coll_trace.size();
+  for (int i = 0; i < std::min(cap, *n); ++i) out[i] = ctx->coll_trace[i];
+  if (reset) ctx->coll_trace.clear();
+  return HX_OK;
+}
+
 int hx_ht_broadcast(hx_ctx* ctx, hx_ht* ht, int root) {
   HX_REQUIRE(ctx && ht, HX_EINVAL, "hx_ht_broadcast: null argument");
   HX_REQUIRE(ctx->comm, HX_ENCCL, "hx_ht_broadcast: no communicator (hx_comm_init)");
@@ -453,6 +491,7 @@ int hx_ht_broadcast(hx_ctx* ctx, hx_ht* ht, int root) {
   HX_CK(cudaSetDevice(ctx->device));
   // 1) header + rank maps (same layout on every rank: same dimension and group range)
   const size_t maps = (sizeof(HtHeader) + 2 * (size_t)ht->domain * sizeof(int32_t) + 255) & ~size_t(255);
+  coll_log(ctx, HX_COLL_BROADCAST, ht->base, (int64_t)maps, 1, root);
   HX_NCCL(ncclBroadcast(ht->base, ht->base, maps, ncclUint8, root, ctx->comm, ctx->stream));
   // 2) the slots in use: every rank learns the capacity from the broadcast header
   HtHeader h{};
@@ -460,10 +499,12 @@ int hx_ht_broadcast(hx_ctx* ctx, hx_ht* ht, int root) {
   HX_CK(cudaStreamSynchronize(ctx->stream));
   HX_REQUIRE(h.log2cap <= ht->max_log2cap, HX_EINVAL,
              "hx_ht_broadcast: tables differ in size across ranks");
+  coll_log(ctx, HX_COLL_BROADCAST, ht->slots, (int64_t(1) << h.log2cap) * 8, 1, root);
   HX_NCCL(ncclBroadcast(ht->slots, ht->slots, (size_t(1) << h.log2cap) * 8, ncclUint8, root,
                         ctx->comm, ctx->stream));
   HX_REQUIRE(h.bloom_log2w <= ht->max_bloom_log2w, HX_EINVAL,
              "hx_ht_broadcast: tables differ in size across ranks");
+  coll_log(ctx, HX_COLL_BROADCAST, ht->bloom, (int64_t(1) << h.bloom_log2w) * 4, 1, root);
   HX_NCCL(ncclBroadcast(ht->bloom, ht->bloom, (size_t(1) << h.bloom_log2w) * 4, ncclUint8, root,
                         ctx->comm, ctx->stream));
   return HX_OK;
@@ -513,22 +554,48 @@ int hx_merge_aggregates(hx_ctx* ctx, hx_agg* agg, int root, int64_t* sums, int64
   HX_CK(cudaMemcpyAsync(&m, agg->meta, sizeof(m), cudaMemcpyDeviceToHost, ctx->stream));
   HX_CK(cudaStreamSynchronize(ctx->stream));
   // builds this pipeline depended on
+  int err = 0;
+  const char* msg = nullptr;
   for (const hx_ht* ht : agg->deps) {
     HtHeader h{};
     HX_CK(cudaMemcpy(&h, ht->hdr, sizeof(h), cudaMemcpyDeviceToHost));
-    if (h.error == HX_EDUPKEY) return fail(HX_EDUPKEY, "dimension build: duplicate primary key");
-    if (h.error) return fail(HX_EINVAL, "dimension build: group code outside its range");
+    if (!err && h.error == HX_EDUPKEY) err = HX_EDUPKEY, msg = "dimension build: duplicate primary key";
+    if (!err && h.error) err = HX_EINVAL, msg = "dimension build: group code outside its range";
   }
-  if (m.error) return fail(m.error, "hx_pipeline_probe_agg: group capacity exceeded");
+  if (!err && m.error) err = m.error, msg = "hx_pipeline_probe_agg: group capacity exceeded";
+  if (!err && root >= ctx->nranks) err = HX_EINVAL, msg = "hx_merge_aggregates: bad root";
   const int64_t ng = m.n_groups;
+  if (use_collectives(ctx)) {
+    // every rank reaches this collective, also one that failed locally: agree on {any error,
+    // max n_groups} first, so that an error is reported on every rank instead of leaving the
+    // others blocked in the data collective below
+    int64_t st[2] = {err ? 1 : 0, ng};
+    int64_t* dst = nullptr;
+    HX_CK(cudaMallocAsync(reinterpret_cast<void**>(&dst), sizeof(st), ctx->stream));
+    HX_CK(cudaMemcpyAsync(dst, st, sizeof(st), cudaMemcpyHostToDevice, ctx->stream));
+    coll_log(ctx, HX_COLL_ALLREDUCE, dst, 2, 8);
+    const ncclResult_t nr = ncclAllReduce(dst, dst, 2, ncclInt64, ncclMax, ctx->comm, ctx->stream);
+    cudaMemcpyAsync(st, dst, sizeof(st), cudaMemcpyDeviceToHost, ctx->stream);
+    cudaFreeAsync(dst, ctx->stream);
+    HX_CK(cudaStreamSynchronize(ctx->stream));
+    if (nr != ncclSuccess) return fail(HX_ENCCL, ncclGetErrorString(nr));
+    if (err) return fail(err, msg);
+    if (st[0]) return fail(HX_EINVAL, "hx_merge_aggregates: the merge failed on another rank");
+    if (st[1] != ng) return fail(HX_EINVAL, "hx_merge_aggregates: ranks disagree on n_groups");
+  } else if (err) {
+    return fail(err, msg);
+  }
   if (use_collectives(ctx) && ng > 0) {
-    HX_REQUIRE(root < ctx->nranks, HX_EINVAL, "hx_merge_aggregates: bad root");
     // sums and cnts are adjacent regions of cap_groups each: reduce both with one call each
     if (root < 0) {
+      coll_log(ctx, HX_COLL_ALLREDUCE, agg->sums, ng, 8);
       HX_NCCL(ncclAllReduce(agg->sums, agg->sums, ng, ncclUint64, ncclSum, ctx->comm, ctx->stream));
+      coll_log(ctx, HX_COLL_ALLREDUCE, agg->cnts, ng, 8);
       HX_NCCL(ncclAllReduce(agg->cnts, agg->cnts, ng, ncclUint64, ncclSum, ctx->comm, ctx->stream));
     } else {
+      coll_log(ctx, HX_COLL_REDUCE, agg->sums, ng, 8, root);
       HX_NCCL(ncclReduce(agg->sums, agg->sums, ng, ncclUint64, ncclSum, root, ctx->comm, ctx->stream));
+      coll_log(ctx, HX_COLL_REDUCE, agg->cnts, ng, 8, root);
       HX_NCCL(ncclReduce(agg->cnts, agg->cnts, ng, ncclUint64, ncclSum, root, ctx->comm, ctx->stream));
       if (ctx->rank != root) {
         HX_CK(cudaStreamSynchronize(ctx->stream));

@@ -288,6 +288,7 @@ int hx_exchange_partitions(hx_ctx* ctx, const hx_table* parted, const int64_t* p
   std::vector<int64_t> mine(nr), sizes((size_t)nr * nr);
   for (int p = 0; p < nr; ++p) mine[p] = part_offsets[p + 1] - part_offsets[p];
   HX_CK(cudaMemcpyAsync(dsz, mine.data(), sizeof(int64_t) * nr, cudaMemcpyHostToDevice, ctx->stream));
+  coll_log(ctx, HX_COLL_ALLGATHER, dsz, nr, 8);
   ncclResult_t r = ncclAllGather(dsz, dsz + nr, nr, ncclInt64, ctx->comm, ctx->stream);
   if (r != ncclSuccess) {
     cudaFreeAsync(dsz, ctx->stream);
@@ -311,9 +312,11 @@ int hx_exchange_partitions(hx_ctx* ctx, const hx_table* parted, const int64_t* p
     for (int peer = 0; peer < nr && r == ncclSuccess; ++peer) {
       const int64_t ns = part_offsets[peer + 1] - part_offsets[peer];
       const int64_t nrv = sizes[(size_t)peer * nr + ctx->rank];
+      if (ns > 0) coll_log(ctx, HX_COLL_SEND, parted->dev[c] + part_offsets[peer], ns, 4, peer);
       if (ns > 0)
         r = ncclSend(parted->dev[c] + part_offsets[peer], (size_t)ns, ncclInt32, peer, ctx->comm,
                      ctx->stream);
+      if (r == ncclSuccess && nrv > 0) coll_log(ctx, HX_COLL_RECV, o->dev[c] + recv_off[peer], nrv, 4, peer);
       if (r == ncclSuccess && nrv > 0)
         r = ncclRecv(o->dev[c] + recv_off[peer], (size_t)nrv, ncclInt32, peer, ctx->comm,
                      ctx->stream);

@@ -152,7 +152,25 @@ struct hx_ctx {
   // wait for them; joined back into the main stream at the end of every enqueue call
   cudaStream_t fin_stream = nullptr;
   cudaEvent_t fin_join_ev = nullptr;
+  // hx_ctx_set_option
+  int join_layout = HX_JOIN_AUTO;
+  int l2_persist = 1;
+  int64_t l2_persist_max = 0;   // persisting L2 set-aside (bytes) set at hx_init
+  int64_t l2_window_max = 0;    // cudaDevAttrMaxAccessPolicyWindowSize
+  // hx_comm_trace: the NCCL data calls issued on this ctx (last kTraceCap kept)
+  static constexpr size_t kTraceCap = 4096;
+  std::vector<hx_coll_rec> coll_trace;
 };
+namespace hx {
+// Record one NCCL data call (hx_comm_trace); call it right before issuing the collective.
+inline void coll_log(hx_ctx* ctx, int op, const void* buf, int64_t count, int elem_bytes,
+                     int root_or_peer = -1) {
+  if (ctx->coll_trace.size() >= hx_ctx::kTraceCap)
+    ctx->coll_trace.erase(ctx->coll_trace.begin(), ctx->coll_trace.begin() + hx_ctx::kTraceCap / 2);
+  ctx->coll_trace.push_back(hx_coll_rec{op, root_or_peer, count, elem_bytes, 0,
+                                        (uint64_t)reinterpret_cast<uintptr_t>(buf)});
+}
+}  // namespace hx
 
 struct hx_partition {
   int64_t n_rows = 0, block_rows = 0;

@@ -212,7 +212,7 @@ int hx_plan_create(hx_ctx* ctx, const hx_table* fact, hx_table* const* dims, int
   // range instead of hash tables when the map is no larger than kDirectMaxBytes (or than
   // twice the hash table); HX_NO_DM=1 keeps hash tables (A/B measurements, tests)
   // (all builds or none: one K1 instance probes either kind)
-  bool use_dm = std::getenv("HX_NO_DM") == nullptr;
+  bool use_dm = std::getenv("HX_NO_DM") == nullptr && ctx->join_layout == HX_JOIN_AUTO;
   int32_t dm_kmin[HX_MAX_JOINS] = {0, 0, 0, 0};
   int64_t dm_span[HX_MAX_JOINS] = {0, 0, 0, 0};
   int dm_lw[HX_MAX_JOINS] = {0, 0, 0, 0};
@@ -333,6 +333,7 @@ int hx_plans_enqueue(hx_ctx* ctx, hx_plan* const* plans, int n) {
   if (grouped) {
     HX_REQUIRE(ncclGroupStart() == ncclSuccess, HX_ENCCL, "ncclGroupStart");
     for (int i = 0; i < n; ++i) {
+      coll_log(ctx, HX_COLL_ALLREDUCE, plans[i]->agg.sums, 2 * (int64_t)plans[i]->n_groups, 8);
       ncclResult_t r = ncclAllReduce(plans[i]->agg.sums, plans[i]->agg.sums,
                                      2 * (size_t)plans[i]->n_groups, ncclUint64, ncclSum,
                                      ctx->comm, ctx->stream);
@@ -384,6 +385,7 @@ static int plan_enqueue_probe(hx_ctx* ctx, hx_plan* pl, bool merge) {
     // finalize stream, so the next plan's K1 does not wait for the collective
     HX_CK(cudaEventRecord(pl->probed, ctx->stream));
     HX_CK(cudaStreamWaitEvent(ctx->fin_stream, pl->probed, 0));
+    coll_log(ctx, HX_COLL_ALLREDUCE, pl->agg.sums, 2 * (int64_t)pl->n_groups, 8);
     ncclResult_t r = ncclAllReduce(pl->agg.sums, pl->agg.sums, 2 * (size_t)pl->n_groups,
                                    ncclUint64, ncclSum, ctx->comm, ctx->fin_stream);
     HX_REQUIRE(r == ncclSuccess, HX_ENCCL, std::string("ncclAllReduce: ") + ncclGetErrorString(r));

@@ -31,6 +31,7 @@
 #include <cmath>
 #include <cstdio>
 #include <cstdlib>
+#include <mutex>
 
 #include "hx_internal.cuh"
 
@@ -127,6 +128,7 @@ struct K1Params {
   uint32_t m_l2s;                          // stage S reads its map from L2 on every row (no
                                            // shared-memory structure: exact verdict + rank)
   uint32_t m_res;                          // resolved in stage S (full map staged, or m_l2s)
+  int32_t l2_hint;                         // 1: probe loads evict_last (0: evict_normal; A/B)
 };
 
 // join kinds (uniform per launch: read from the kernel parameters)
@@ -201,11 +203,37 @@ __device__ __forceinline__ void bulk_g2s(void* dst, const void* src, uint32_t by
 __device__ __forceinline__ void bulk_prefetch_l2(const void* src, uint32_t bytes) {
   asm volatile("cp.async.bulk.prefetch.L2.global [%0], %1;" ::"l"(src), "r"(bytes) : "memory");
 }
-__device__ __forceinline__ unsigned long long ld_slot(const unsigned long long* p, uint64_t pol) {
-  unsigned long long v;
-  asm volatile("ld.global.nc.L2::cache_hint.u64 %0, [%1], %2;" : "=l"(v) : "l"(p), "l"(pol));
+__device__ __forceinline__ uint64_t policy_evict_normal() {
+  uint64_t pol;
+  asm volatile("createpolicy.fractional.L2::evict_normal.b64 %0, 1.0;" : "=l"(pol));
+  return pol;
+}
+// Loads of the probe structures (direct-map words, hash-table buckets) and of gathered
+// measures, with an L2 eviction-priority hint: probes evict_last (the maps and tables stay
+// L2-resident against the evict-first lineorder stream; ncu then counts their sectors as
+// evict_last, which isolates the probe tables' L2 hit rate), gathers evict_first (read once).
+// Not volatile: pure loads of read-only data that the compiler may schedule freely.
+__device__ __forceinline__ uint32_t ld_hint(const uint32_t* p, uint64_t pol) {
+  uint32_t v;
+  asm("ld.global.nc.L2::cache_hint.u32 %0, [%1], %2;" : "=r"(v) : "l"(p), "l"(pol));
   return v;
 }
+__device__ __forceinline__ int32_t ld_hint(const int32_t* p, uint64_t pol) {
+  int32_t v;
+  asm("ld.global.nc.L2::cache_hint.s32 %0, [%1], %2;" : "=r"(v) : "l"(p), "l"(pol));
+  return v;
+}
+__device__ __forceinline__ ulonglong2 ld_hint(const ulonglong2* p, uint64_t pol) {
+  ulonglong2 v;
+  asm("ld.global.nc.L2::cache_hint.v2.u64 {%0, %1}, [%2], %3;"
+      : "=l"(v.x), "=l"(v.y)
+      : "l"(p), "l"(pol));
+  return v;
+}
+// The two policies of a K1 launch (created once per thread).
+struct Pols {
+  uint64_t probe, gather;
+};
 __device__ __forceinline__ void consumer_sync() {
   asm volatile("bar.sync 1, %0;" ::"n"(kConsumers) : "memory");
 }
@@ -247,18 +275,6 @@ __device__ __forceinline__ void probe_step(const ulonglong2 v, int32_t key, bool
   hit = h0 || h1;
   miss = !hit && (int32_t)(uint32_t)v.y == kEmptyKey;
   rank = (int32_t)((h0 ? v.x : v.y) >> 32);
-}
-
-// Full probe of one row (loops over buckets until hit or miss).
-__device__ __forceinline__ bool probe_row(const JoinState& j, int32_t key, int32_t& rank) {
-  uint32_t b = bucket_of(key, j.shift);
-  while (true) {
-    bool hit, miss;
-    probe_step(__ldg(j.buckets + b), key, hit, miss, rank);
-    if (hit) return true;
-    if (miss) return false;
-    b = (b + 1) & j.bmask;
-  }
 }
 
 template <bool GROUPED>
@@ -381,7 +397,8 @@ __device__ __forceinline__ void stage_c_row(const K1Params& p, const JoinState (
                                             const unsigned char* sdm, const CarryEntry& e,
                                             int j0, int jf, bool smem_table,
                                             unsigned long long* s_sum, uint32_t* s_cnt,
-                                            long long& acc_sum, long long& acc_cnt, Pending& pd) {
+                                            long long& acc_sum, long long& acc_cnt, Pending& pd,
+                                            const Pols& pol) {
   // (direct maps: the group index is computed here from scratch; stage S only filtered)
   int32_t gg = DM ? group_origin<NJ, GROUPED, DM>(js) : e.g;
   bool alive = true;
@@ -418,7 +435,7 @@ __device__ __forceinline__ void stage_c_row(const K1Params& p, const JoinState (
     const JoinDev& d = p.joins[jx];
     wdm[jx] = 0u;
     if (dm_l2<DM>(p, jx) && alive && dm_in(d, e.key[jx]))
-      wdm[jx] = __ldg(d.dm + (dm_bit(d, e.key[jx]) >> 5));
+      wdm[jx] = ld_hint(d.dm + (dm_bit(d, e.key[jx]) >> 5), pol.probe);
   }
 #pragma unroll
   for (int jx = 0; jx < NJ; ++jx) {
@@ -448,7 +465,7 @@ __device__ __forceinline__ void stage_c_row(const K1Params& p, const JoinState (
     ulonglong2 v[NJ > 0 ? NJ : 1];
 #pragma unroll
     for (int jx = 0; jx < NJ; ++jx)
-      if ((pend >> jx) & 1u) v[jx] = __ldg(js[jx].buckets + b[jx]);
+      if ((pend >> jx) & 1u) v[jx] = ld_hint(js[jx].buckets + b[jx], pol.probe);
 #pragma unroll
     for (int jx = 0; jx < NJ; ++jx) {
       if (!((pend >> jx) & 1u)) continue;
@@ -464,8 +481,8 @@ __device__ __forceinline__ void stage_c_row(const K1Params& p, const JoinState (
   }
   Pending cur{gg, e.a, e.b, alive};
   if (alive) {  // issue the gathers now, consume them one batch later
-    if (p.ga) cur.a = __ldg(p.gat_a + e.row);
-    if (p.gb) cur.b = __ldg(p.gat_b + e.row);
+    if (p.ga) cur.a = ld_hint(p.gat_a + e.row, pol.gather);
+    if (p.gb) cur.b = ld_hint(p.gat_b + e.row, pol.gather);
   }
   if (pd.alive)
     accumulate<GROUPED>(p, smem_table, s_sum, s_cnt, pd.g, measure(p.agg_op, pd.a, pd.b), acc_sum,
@@ -500,7 +517,7 @@ __device__ __forceinline__ void process_tile(const K1Params& p, const JoinState 
                                              unsigned long long* s_sum, uint32_t* s_cnt,
                                              uint8_t* q_row, int32_t* q_g, CarryBuf* cb,
                                              int& n_carry, long long& acc_sum,
-                                             long long& acc_cnt, Pending& pd) {
+                                             long long& acc_cnt, Pending& pd, const Pols& pol) {
   constexpr int R = kRowsPerThread;  // rows per lane per tile
   const int wbase = warp * (32 * R);
   const int r0 = wbase + lane * R;
@@ -600,7 +617,7 @@ __device__ __forceinline__ void process_tile(const K1Params& p, const JoinState 
       uint32_t w[2 * R];
 #pragma unroll
       for (int k = 0; k < 2 * R; ++k)
-        w[k] = ((m >> k) & 1u) && dm_in(d, key[k]) ? __ldg(d.dm + (dm_bit(d, key[k]) >> 5)) : 0u;
+        w[k] = ((m >> k) & 1u) && dm_in(d, key[k]) ? ld_hint(d.dm + (dm_bit(d, key[k]) >> 5), pol.probe) : 0u;
 #pragma unroll
       for (int k = 0; k < 2 * R; ++k) {
         const uint32_t v = dm_entry(d, w[k], dm_bit(d, key[k]));
@@ -629,7 +646,7 @@ __device__ __forceinline__ void process_tile(const K1Params& p, const JoinState 
 #pragma unroll
       for (int k = 0; k < R; ++k) {
         b[k] = bucket_of(key[h * R + k], j.shift);
-        if ((m >> (h * R + k)) & 1u) v[k] = __ldg(j.buckets + b[k]);
+        if ((m >> (h * R + k)) & 1u) v[k] = ld_hint(j.buckets + b[k], pol.probe);
       }
 #pragma unroll
       for (int k = 0; k < R; ++k) {
@@ -653,8 +670,8 @@ __device__ __forceinline__ void process_tile(const K1Params& p, const JoinState 
       for (int k = 0; k < 2 * R; ++k) {
         const uint32_t row = (k < R ? frow0 : frow1) + r0 + (k & 3);
         if ((m >> k) & 1u) {
-          if (p.ga) a8[k] = __ldg(p.gat_a + row);
-          if (p.gb) b8[k] = __ldg(p.gat_b + row);
+          if (p.ga) a8[k] = ld_hint(p.gat_a + row, pol.gather);
+          if (p.gb) b8[k] = ld_hint(p.gat_b + row, pol.gather);
         }
       }
     }
@@ -711,7 +728,8 @@ __device__ __forceinline__ void process_tile(const K1Params& p, const JoinState 
   for (int base = 0; base < full_end; base += 32) {
     CarryEntry e = load_entry<NJ, DM>(p, js, cb, n_carry, q_row, q_g, carry_g, wcol0, wcol1,
                                       wrow0, wrow1, stride, base + lane);
-    stage_c_row<NJ, GROUPED, DM>(p, js, sdm, e, j0, jf, smem_table, s_sum, s_cnt, acc_sum, acc_cnt, pd);
+    stage_c_row<NJ, GROUPED, DM>(p, js, sdm, e, j0, jf, smem_table, s_sum, s_cnt, acc_sum, acc_cnt, pd,
+                                 pol);
   }
   {
     const int idx = full_end + lane;
@@ -741,7 +759,7 @@ __device__ __forceinline__ void drain_carry(const K1Params& p, const JoinState (
                                             int n_carry, int lane, int j0,
                                             int jf, bool smem_table, unsigned long long* s_sum,
                                             uint32_t* s_cnt, long long& acc_sum,
-                                            long long& acc_cnt, Pending& pd) {
+                                            long long& acc_cnt, Pending& pd, const Pols& pol) {
   if (lane >= n_carry) return;
   CarryEntry e;
 #pragma unroll
@@ -750,7 +768,8 @@ __device__ __forceinline__ void drain_carry(const K1Params& p, const JoinState (
   e.b = cb->b[lane];
   e.row = cb->row[lane];
   e.g = cb->g[lane];
-  stage_c_row<NJ, GROUPED, DM>(p, js, sdm, e, j0, jf, smem_table, s_sum, s_cnt, acc_sum, acc_cnt, pd);
+  stage_c_row<NJ, GROUPED, DM>(p, js, sdm, e, j0, jf, smem_table, s_sum, s_cnt, acc_sum, acc_cnt, pd,
+                                 pol);
 }
 
 __device__ __forceinline__ void mbar_wait_sleep(uint64_t* bar, uint32_t parity) {
@@ -844,7 +863,8 @@ __global__ void __launch_bounds__(kThreads, kCtasPerSm) k1_probe_agg(const __gri
   }
 
   // ---------------- consumer warps ----------------
-  const int ctid = tid;  // 0..255
+  const int ctid = tid;  // 0..kConsumers-1
+  const Pols pol{p.l2_hint ? policy_evict_last() : policy_evict_normal(), policy_evict_first()};
   uint8_t* q_row = q_rows + warp * kQueueRows;
   int32_t* q_g = DM ? nullptr : q_gs + warp * kQueueRows;
   CarryBuf* cb = reinterpret_cast<CarryBuf*>(smem + smem_carry_off(DM) + warp * kCarryBytes);
@@ -933,7 +953,7 @@ __global__ void __launch_bounds__(kThreads, kCtasPerSm) k1_probe_agg(const __gri
     consumer_sync();
     process_tile<NJ, GROUPED, DM>(p, js, sdm, headbuf, headbuf, 0u, 0u, 4, p.head_rows, 0, warp, lane,
                                   smem_table, s_sum, s_cnt, q_row, q_g, cb, n_carry, acc_sum,
-                                  acc_cnt, pd);
+                                  acc_cnt, pd, pol);
   }
   consumer_sync();
 
@@ -976,7 +996,7 @@ __global__ void __launch_bounds__(kThreads, kCtasPerSm) k1_probe_agg(const __gri
     const uint32_t frow1 = (uint32_t)(p.head_rows + t1 * kTileRows);
     process_tile<NJ, GROUPED, DM>(p, js, sdm, st0, st1, frow0, frow1, kTileRows, rows0, rows1, warp, lane,
                                   smem_table, s_sum, s_cnt, q_row, q_g, cb, n_carry, acc_sum,
-                                  acc_cnt, pd);
+                                  acc_cnt, pd, pol);
     __syncwarp();
     if (lane == 0) {
       mbar_arrive(empty + s);
@@ -999,7 +1019,7 @@ __global__ void __launch_bounds__(kThreads, kCtasPerSm) k1_probe_agg(const __gri
   if (NJ > 0)
     drain_carry<NJ, GROUPED, DM>(p, js, sdm, cb, n_carry, lane, first_join_in_place<NJ, DM>(p, js),
                              first_filter<NJ, DM>(js), smem_table, s_sum, s_cnt, acc_sum, acc_cnt,
-                             pd);
+                             pd, pol);
   if (pd.alive)  // the last deferred row
     accumulate<GROUPED>(p, smem_table, s_sum, s_cnt, pd.g, measure(p.agg_op, pd.a, pd.b), acc_sum,
                         acc_cnt);
@@ -1253,20 +1273,40 @@ using KernelFn = void (*)(K1Params);
 // K1 launches carry the device's greatest priority: the builds of later queries (forked on
 // auxiliary streams so they overlap) then only take SMs that K1 leaves idle (its tail), and
 // the next K1's CTAs are dispatched ahead of queued build CTAs.
+// An L2 access-policy window (persisting) over the launch's main probe structure, when set:
+// the lines of [base, base + bytes) get persisting priority in the L2 set-aside region
+// (cudaLimitPersistingL2CacheSize, set at hx_init), hit ratio = set-aside / window bytes.
+struct L2Window {
+  void* base = nullptr;
+  size_t bytes = 0;
+  float hit_ratio = 0.f;
+};
 cudaError_t launch_k1(KernelFn fn, int grid, int block, size_t smem, cudaStream_t s,
-                      const K1Params& p, int priority, int carveout = -1) {
+                      const K1Params& p, int priority, int carveout = -1,
+                      const L2Window* win = nullptr) {
   cudaLaunchConfig_t cfg{};
   cfg.gridDim = dim3((unsigned)grid);
   cfg.blockDim = dim3((unsigned)block);
   cfg.dynamicSmemBytes = smem;
   cfg.stream = s;
-  cudaLaunchAttribute attr[2];
-  attr[0].id = cudaLaunchAttributePriority;
-  attr[0].val.priority = priority;
-  attr[1].id = cudaLaunchAttributePreferredSharedMemoryCarveout;
-  attr[1].val.sharedMemCarveout = (unsigned)carveout;
+  cudaLaunchAttribute attr[3];
+  int n = 0;
+  attr[n].id = cudaLaunchAttributePriority;
+  attr[n++].val.priority = priority;
+  if (carveout >= 0) {
+    attr[n].id = cudaLaunchAttributePreferredSharedMemoryCarveout;
+    attr[n++].val.sharedMemCarveout = (unsigned)carveout;
+  }
+  if (win && win->bytes) {
+    attr[n].id = cudaLaunchAttributeAccessPolicyWindow;
+    attr[n].val.accessPolicyWindow.base_ptr = win->base;
+    attr[n].val.accessPolicyWindow.num_bytes = win->bytes;
+    attr[n].val.accessPolicyWindow.hitRatio = win->hit_ratio;
+    attr[n].val.accessPolicyWindow.hitProp = cudaAccessPropertyPersisting;
+    attr[n++].val.accessPolicyWindow.missProp = cudaAccessPropertyStreaming;
+  }
   cfg.attrs = attr;
-  cfg.numAttrs = carveout >= 0 ? 2 : 1;
+  cfg.numAttrs = n;
   return cudaLaunchKernelEx(&cfg, fn, p);
 }
 
@@ -1452,8 +1492,13 @@ double plan_dm(int nj, const JoinDev* joins, const bool* known, const double* pa
 }  // namespace
 
 int k1_occupancy(hx_ctx* ctx) {
-  static bool attrs = false;
-  if (!attrs) {
+  // cudaFuncSetAttribute applies to the CURRENT device only: set it once per device (a
+  // process may hold contexts on several GPUs, created from several threads)
+  static std::mutex mu;
+  static uint64_t done = 0;  // bit d: device d configured
+  std::lock_guard<std::mutex> lock(mu);
+  const uint64_t bit = ctx->device < 64 ? (uint64_t(1) << ctx->device) : 0;
+  if (!bit || !(done & bit)) {
     for (int d = 0; d < 2; ++d)
       for (int g = 0; g < 2; ++g)
         for (int j = 0; j <= HX_MAX_JOINS; ++j)
@@ -1463,7 +1508,7 @@ int k1_occupancy(hx_ctx* ctx) {
     cudaFuncSetAttribute(k1_scan_agg<2>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)scan_smem(2));
     cudaFuncSetAttribute(k1_scan_agg<3>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)scan_smem(3));
     cudaFuncSetAttribute(k1_scan_agg<4>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)scan_smem(4));
-    attrs = true;
+    done |= bit;
   }
   int occ = 0;
   cudaOccupancyMaxActiveBlocksPerMultiprocessor(
@@ -1497,6 +1542,7 @@ struct K1Prepared {
   int occ = 1;
   int64_t seg_rows = kSegRows;  // rows per launch (HX_K1_SEG_TILES overrides, for tests)
   int carveout = 100;           // preferred shared-memory carveout (% of 228 KB)
+  L2Window win;                 // persisting window over the largest L2-read probe structure
 };
 
 // Device staging ring of the mem-move for a host-resident fact table: kRingStages buffers of
@@ -1576,6 +1622,10 @@ int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht*
     HX_REQUIRE(pr.kind == HX_PRED_RANGE || (pr.kind == HX_PRED_IN && pr.n_in >= 1 && pr.n_in <= 4),
                HX_EINVAL, "hx_pipeline_probe_agg: bad predicate");
     p.preds[q] = DevPred{c, pr.kind, pr.lo, pr.hi, pr.n_in, {pr.in[0], pr.in[1], pr.in[2], pr.in[3]}};
+    // an empty BETWEEN (lo > hi) selects nothing; stage A tests ranges as one unsigned
+    // compare (v - lo) > (hi - lo), which would wrap: compile it to an IN over no values
+    if (pr.kind == HX_PRED_RANGE && pr.lo > pr.hi)
+      p.preds[q] = DevPred{c, HX_PRED_IN, 0, -1, 0, {0, 0, 0, 0}};
   }
   p.n_preds = sh->n_preds;
   for (int j = 0; j < sh->n_joins; ++j) {
@@ -1808,6 +1858,41 @@ int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht*
   // 4 stages, and loses 3-6% on 3-column ones, whose rings are deeper or whose tiles are
   // consumed faster)
   p.prefetch = (n_cols >= 4 && p.stages <= 4 && fact->placement != HX_PLACE_HOST_MAPPED) ? 2 : 0;
+  // L2 residency of the probe structures (north_star; PAPER.md:1016-1022 operator state in
+  // device memory): probe loads carry an evict_last hint, and the largest structure K1 reads
+  // from L2 (a direct map not staged in shared memory, or a hash table's slots) gets a
+  // persisting access-policy window. HX_L2_HINT=0 / hx_ctx_set_option(HX_OPT_L2_PERSIST, 0):
+  // A/B switches.
+  p.l2_hint = 1;
+  if (const char* e = std::getenv("HX_L2_HINT")) p.l2_hint = std::atoi(e) != 0;
+  if (ctx->l2_persist && ctx->l2_persist_max > 0) {
+    for (int j = 0; j < sh->n_joins; ++j) {
+      const JoinDev& d = p.joins[j];
+      const hx_ht* ht = hts[sh->join_ht[j]];
+      void* base = nullptr;
+      size_t bytes = 0;
+      if (d.dm) {
+        if (d.dm_smem < 0 && (((p.m_l2 | p.m_l2s) >> j) & 1u)) {
+          base = const_cast<uint32_t*>(d.dm);
+          bytes = (size_t)d.dm_words * 4;
+        }
+      } else {
+        int lg = ht->max_log2cap;
+        if (ht->known_keys >= 0) {
+          lg = kMinLog2Cap;
+          while (lg < ht->max_log2cap && (int64_t(1) << lg) < 4 * ht->known_keys) ++lg;
+        }
+        base = ht->slots;
+        bytes = (size_t(1) << lg) * 8;
+      }
+      if (bytes > k.win.bytes) {
+        k.win.base = base;
+        k.win.bytes = std::min<size_t>(bytes, (size_t)ctx->l2_window_max);
+      }
+    }
+    if (k.win.bytes)
+      k.win.hit_ratio = (float)std::min(1.0, (double)ctx->l2_persist_max / (double)k.win.bytes);
+  }
   if (const char* e = std::getenv("HX_K1_PREFETCH")) p.prefetch = std::max(0, std::min(64, std::atoi(e)));
   if (std::getenv("HX_DEBUG")) {  // launch plan of this K1 (tuning aid)
     std::fprintf(stderr, "[hx] K1 joins=%d cols=%d gather=%d%d stages=%d groups=%d filters:",
@@ -1964,7 +2049,8 @@ int k1_enqueue(hx_ctx* ctx, const K1Prepared* k, bool fresh, cudaEvent_t e0, cud
       q.n_rows = std::min<int64_t>(k->seg_rows, p.n_rows - s0);
       q.n_tiles = (q.n_rows + kTileRows - 1) / kTileRows;
       const int grid = (int)std::max<int64_t>(1, std::min<int64_t>(q.n_tiles, (int64_t)k->grid));
-      HX_CK(launch_k1(k->fn, grid, kThreads, k->smem, ctx->stream, q, ctx->k1_priority, k->carveout));
+      HX_CK(launch_k1(k->fn, grid, kThreads, k->smem, ctx->stream, q, ctx->k1_priority, k->carveout,
+                      &k->win));
       ctx->launches += 1;
     }
   }

@@ -36,6 +36,10 @@ class Context:
         call("hx_ctx_info", self.h, ctypes.byref(a), ctypes.byref(b))
         return a.value, b.value
 
+    def set_option(self, option: int, value: int) -> None:
+        """hx_ctx_set_option (HX_OPT_JOIN_LAYOUT: HX_JOIN_AUTO | HX_JOIN_HASH; HX_OPT_L2_PERSIST)."""
+        call("hx_ctx_set_option", self.h, option, value)
+
     def comm_init(self, nranks: int, rank: int, uid: bytes) -> None:
         buf = ctypes.create_string_buffer(uid, 128)
         call("hx_comm_init", self.h, nranks, rank, buf)
@@ -45,6 +49,18 @@ class Context:
         a, b = ctypes.c_int(), ctypes.c_int()
         call("hx_comm_info", self.h, ctypes.byref(a), ctypes.byref(b))
         return a.value, b.value
+
+    def comm_trace(self, reset: bool = True) -> List[dict]:
+        """The NCCL data calls libhx issued on this context (hx_comm_trace), oldest first."""
+        n = ctypes.c_int()
+        call("hx_comm_trace", self.h, None, 0, ctypes.byref(n), 0)
+        recs = (_hx.hx_coll_rec * max(1, n.value))()
+        call("hx_comm_trace", self.h, recs, n.value, ctypes.byref(n), 1 if reset else 0)
+        names = {_hx.HX_COLL_ALLREDUCE: "allreduce", _hx.HX_COLL_REDUCE: "reduce",
+                 _hx.HX_COLL_BROADCAST: "broadcast", _hx.HX_COLL_ALLGATHER: "allgather",
+                 _hx.HX_COLL_SEND: "send", _hx.HX_COLL_RECV: "recv"}
+        return [{"op": names[r.op], "root_or_peer": r.root_or_peer, "count": r.count,
+                 "elem_bytes": r.elem_bytes, "buf": r.buf} for r in recs[:n.value]]
 
     def profile_enable(self, on: bool = True) -> None:
         call("hx_profile_enable", self.h, int(on))

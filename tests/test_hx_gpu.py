@@ -455,3 +455,43 @@ def test_degenerate_dimensions(ctx, case):
         pl.enqueue()
         assert pl.rows() == want, (case, q)
         pl.close()
+
+
+# ---- an empty BETWEEN on lineorder (lo > hi) selects nothing, with and without joins ------
+@pytest.mark.parametrize("q", ["q1.1", "q2.1", "q4.3"])
+def test_empty_fact_range_selects_nothing(ctx, q):
+    """SQL `x BETWEEN 30 AND 20` is empty. K1 tests ranges with one unsigned compare, so
+    k1_setup must compile lo > hi to always-false (it used to wrap and pass
+    nearly every row of a pipeline with joins)."""
+    import dataclasses
+    db = tiny_db(5, n_lo=20011)
+    dims, fact = ssb.load_db_numpy(ctx, db)
+    eng = ssb.SsbEngine(ctx, dims, fact)
+    base = ssb.PLANS[q]
+    plan = dataclasses.replace(base, fact_preds=list(base.fact_preds) + [("lo_quantity", 30, 20)])
+    hts = [eng.build(b) for _, b in plan.joins]
+    agg = hx.pipeline_probe_agg(ctx, fact, eng.shape(plan), hts)
+    rows = eng.finish(ssb.Pending(plan, hts, agg))
+    # ungrouped: one row, count 0 (SQL NULL sum, DESIGN.md R7); grouped: no group at all
+    assert rows == ([(0, 0)] if not plan.gdims else []), (q, rows[:3])
+
+
+@pytest.mark.parametrize("table,col", [("customer", "c_custkey"), ("date", "d_datekey")])
+def test_reserved_key_minus_one_rejected(ctx, table, col):
+    """Key -1 is the empty-slot marker (R18): a dimension holding it is refused
+    with HX_EINVAL by the plain calls and by plan creation, never silently mis-joined."""
+    db = tiny_db(4, n_lo=4097)
+    db[table][col] = db[table][col].copy()
+    db[table][col][3] = -1
+    if table == "customer":  # the row must pass Q3.1's customer filter (c_region = ASIA)
+        db[table]["c_region"] = db[table]["c_region"].copy()
+        db[table]["c_region"][3] = 2
+    dims, fact = ssb.load_db_numpy(ctx, db)
+    eng = ssb.SsbEngine(ctx, dims, fact)
+    q = "q3.1"
+    with pytest.raises(_hx.HxError) as ei:
+        eng.run(q)
+    assert ei.value.code == _hx.HX_EINVAL
+    with pytest.raises(_hx.HxError) as ei:
+        eng.plan(q)
+    assert ei.value.code == _hx.HX_EINVAL

@@ -2,10 +2,13 @@
 HX_FORCE_COLLECTIVES=1 makes libhx issue every collective it would issue with N ranks — the
 union-router allreduce / reduce of hx_merge_aggregates, the per-plan allreduces of a
 multi-plan step (on the finalize stream, inside a captured CUDA graph), the mem-move broadcast of a built hash table, and the
-hash-routing exchange's allgather + send/recv — so their buffers, sizes and ordering are
-checked bit-exactly against the oracle. (NCCL refuses two ranks on one device; the N-rank
-data flow is covered by the gloo tests in test_hx_cpu.py.)
+hash-routing exchange's allgather + send/recv — and the results are checked bit-exactly
+against the oracle. A 1-rank allreduce or broadcast is an identity whatever its count, so the
+element counts and byte sizes libhx issues are checked separately, from its collective trace
+(hx_comm_trace), against values computed independently with numpy. (NCCL refuses two ranks on
+one device: the 2-rank NCCL run is tests/test_multigpu_gpu.py, skipped with fewer than 2 GPUs.)
 """
+import numpy as np
 import pytest
 
 import oracle
@@ -87,3 +90,104 @@ def test_hash_routing_exchange(nctx, db):
     eng = ssb.SsbEngine(nctx, dims, fact)
     for q, dim in (("q2.1", "part"), ("q3.1", "customer"), ("q4.3", "supplier")):
         assert eng.run_hash_routed(q, dim) == oracle.run_query(q, db), (q, dim)
+
+
+# ---- the sizes of the collectives, from the collective trace (hx_comm_trace) ----------------
+# A 1-rank allreduce / broadcast is an identity whatever its count, so the counts libhx
+# issues are checked here against values computed independently from the generated tables
+# with numpy, following the query texts: a grouping dimension contributes the
+# number of distinct group codes among its rows that pass the dimension's filter (the dense
+# ranks, R17), and the group array is their product.
+AMERICA, ASIA, US, KI = 1, 2, 23, (221, 225)
+
+
+def _groups(db, q):
+    d, c, s, p = db["date"], db["customer"], db["supplier"], db["part"]
+    year = d["d_year"]
+    y9297 = (year >= 1992) & (year <= 1997)
+    y9798 = (year == 1997) | (year == 1998)
+    brand, cat = p["p_brand1"], p["p_category"]
+    spec = {
+        "q1.1": [], "q1.2": [], "q1.3": [],
+        "q2.1": [(year, year == year), (brand, cat == 1)],
+        "q2.2": [(year, year == year), (brand, (brand >= 260) & (brand <= 267))],
+        "q2.3": [(year, year == year), (brand, brand == 278)],
+        "q3.1": [(c["c_nation"], c["c_region"] == ASIA), (s["s_nation"], s["s_region"] == ASIA),
+                 (year, y9297)],
+        "q3.2": [(c["c_city"], c["c_nation"] == US), (s["s_city"], s["s_nation"] == US),
+                 (year, y9297)],
+        "q3.3": [(c["c_city"], np.isin(c["c_city"], KI)), (s["s_city"], np.isin(s["s_city"], KI)),
+                 (year, y9297)],
+        "q3.4": [(c["c_city"], np.isin(c["c_city"], KI)), (s["s_city"], np.isin(s["s_city"], KI)),
+                 (year, d["d_yearmonthnum"] == 199712)],
+        "q4.1": [(year, year == year), (c["c_nation"], c["c_region"] == AMERICA)],
+        "q4.2": [(year, y9798), (s["s_nation"], s["s_region"] == AMERICA),
+                 (cat, np.isin(p["p_mfgr"], (0, 1)))],
+        "q4.3": [(year, y9798), (s["s_city"], s["s_nation"] == US), (brand, cat == 3)],
+    }[q]
+    n = 1
+    for col, mask in spec:
+        n *= max(1, len(np.unique(col[mask])))
+    return n
+
+
+def test_trace_merge_counts(nctx, db):
+    """hx_merge_aggregates: an error-status allreduce (2 int64) on every rank, then the sums
+    and the counts, n_groups elements each (allreduce, or reduce to the root)."""
+    dims, fact = ssb.load_db_numpy(nctx, db)
+    eng = ssb.SsbEngine(nctx, dims, fact)
+    for root in (-1, 0):
+        for q in QUERIES:
+            nctx.comm_trace(reset=True)
+            eng.finish(eng.start(q), root)
+            tr = nctx.comm_trace(reset=True)
+            ng = _groups(db, q)
+            op = "allreduce" if root < 0 else "reduce"
+            assert [(r["op"], r["count"], r["elem_bytes"]) for r in tr] == [
+                ("allreduce", 2, 8), (op, ng, 8), (op, ng, 8)], (q, root, tr)
+
+
+def test_trace_plan_allreduce_counts(nctx, db):
+    """A multi-plan step: one union-router allreduce per plan over its adjacent {sums, counts}
+    arrays, 2 x n_groups uint64 elements, issued in plan order."""
+    dims, fact = ssb.load_db_numpy(nctx, db)
+    eng = ssb.SsbEngine(nctx, dims, fact)
+    plans = {q: eng.plan(q) for q in QUERIES}
+    nctx.comm_trace(reset=True)
+    hx.plans_enqueue(nctx, [plans[q].hp for q in QUERIES])
+    for q in QUERIES:
+        plans[q].rows()
+    tr = nctx.comm_trace(reset=True)
+    assert [(r["op"], r["count"], r["elem_bytes"]) for r in tr] == [
+        ("allreduce", 2 * _groups(db, q), 8) for q in QUERIES]
+    for pl in plans.values():
+        pl.close()
+
+
+def _next_pow2(x):
+    return 1 << max(0, int(x - 1).bit_length())
+
+
+def test_trace_ht_broadcast_sizes(nctx, db):
+    """hx_ht_broadcast moves the header + rank maps, then the slots in use (8 B each, a power
+    of two >= 4 per passing key, at least 16) and the Bloom filter (a power of two of 32-bit
+    words >= 16 bits per passing key), from the root."""
+    dims, fact = ssb.load_db_numpy(nctx, db)
+    eng = ssb.SsbEngine(nctx, dims, fact)
+    c, s = db["customer"], db["supplier"]
+    cases = [("q3.1", "customer", int(np.sum(c["c_region"] == ASIA))),
+             ("q3.2", "supplier", int(np.sum(s["s_nation"] == US))),
+             ("q4.1", "customer", int(np.sum(c["c_region"] == AMERICA)))]
+    for q, dim, n_pass in cases:
+        plan = ssb.PLANS[q]
+        (b,) = [b for _, b in plan.joins if b.table == dim]
+        t = eng.build(b)
+        nctx.comm_trace(reset=True)
+        t.broadcast(0)
+        tr = nctx.comm_trace(reset=True)
+        assert [r["op"] for r in tr] == ["broadcast"] * 3 and all(r["root_or_peer"] == 0 for r in tr)
+        assert tr[0]["count"] % 256 == 0
+        assert tr[1]["count"] == 8 * max(16, _next_pow2(4 * n_pass)), (q, dim, tr)
+        assert tr[2]["count"] == 4 * max(1, _next_pow2(16 * n_pass) // 32), (q, dim, tr)
+        assert t.info()["n_keys"] == n_pass
+        t.close()
