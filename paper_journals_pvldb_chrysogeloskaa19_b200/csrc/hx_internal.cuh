@@ -154,7 +154,7 @@ struct hx_ctx {
   cudaEvent_t fin_join_ev = nullptr;
   // hx_ctx_set_option
   int join_layout = HX_JOIN_AUTO;
-  int l2_persist = 1;
+  int l2_persist = 0;           // measured: the persisting window costs ~2%
   int64_t l2_persist_max = 0;   // persisting L2 set-aside (bytes) set at hx_init
   int64_t l2_window_max = 0;    // cudaDevAttrMaxAccessPolicyWindowSize
   // hx_comm_trace: the NCCL data calls issued on this ctx (last kTraceCap kept)

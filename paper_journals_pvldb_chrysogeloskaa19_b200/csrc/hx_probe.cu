@@ -46,6 +46,20 @@ constexpr unsigned kFull = 0xFFFFFFFFu;
 #ifndef HX_K1_STAGE_KB
 #define HX_K1_STAGE_KB 160  // max shared memory for the tile ring (the rest: Bloom filters)
 #endif
+#ifndef HX_PROBE_HINT
+#define HX_PROBE_HINT 0   // probe loads with an L2 evict_last hint (0: plain ld.global.nc;
+                          // measured: the hint costs 2-9% on Q4.x)
+#endif
+#ifndef HX_GATHER_HINT
+#define HX_GATHER_HINT 0  // gathered measures with an L2 evict_first hint (0: plain)
+#endif
+#ifndef HX_CLAIM_AHEAD
+#define HX_CLAIM_AHEAD 0  // claim the next chunk before processing the current one (measured:
+                          // a reserved chunk waits for its warp and delays its stage, -5%)
+#endif
+#ifndef HX_TAG_SLEEP
+#define HX_TAG_SLEEP 20   // ns slept between polls of a ring slot's tile tag (0: spin)
+#endif
 #ifndef HX_K1_CTAS
 #define HX_K1_CTAS 1    // resident CTAs per SM the launch bounds / smem budget target
                         // (one CTA per SM shares one copy of the Bloom filters)
@@ -55,15 +69,35 @@ constexpr int kConsumers = kConsumerWarps * 32;
 constexpr int kThreads = kConsumers + 32;  // + one producer warp
 constexpr int kRowsPerThread = 4;          // R
 constexpr int kTileRows = kConsumers * kRowsPerThread;  // T = 2560 rows
+// A CHUNK is one consumer warp's unit of work: 256 consecutive rows of a tile, two halves of
+// 128 (lane l holds rows 4l..4l+3 of each half: one conflict-free 128-bit shared-memory load
+// per column and half). Warps claim chunks dynamically (a shared counter), so a warp that
+// drew a chunk with many survivors does not hold the others back.
+constexpr int kHalfRows = 32 * kRowsPerThread;             // 128
+constexpr int kChunkRows = 2 * kHalfRows;                  // 256
+constexpr int kChunksPerTile = kTileRows / kChunkRows;     // 10
+static_assert(kTileRows % kChunkRows == 0, "a tile is a whole number of chunks");
 // rows per K1 launch: whole tiles, < 2^32 - kTileRows (32-bit row offsets inside a launch)
 constexpr int64_t kSegRows = int64_t(kTileRows) * (int64_t(1) << 20);  // 2.68e9 rows
 constexpr int kCtasPerSm = HX_K1_CTAS;    // target residency (registers, smem budget)
 constexpr int kMaxStageCols = 8;
 constexpr int kSmemGroups = 1024;          // per-CTA group table capacity
-// dynamic smem: [barriers 128 | reduce 256 | head 128 | per-warp queues: 256 row bytes (+ 256
-// group indices, hash-table instances) | per-warp carry buffers | groups | Bloom filters |
-// direct maps | tile ring]
-constexpr int kSmemQueueOff = 512;
+// dynamic smem: [barriers 128 | head 8 cols x 4 rows | chunk scheduling | per-warp queues: 256
+// row bytes (+ 256 group indices, hash-table instances) | per-warp carry buffers | groups |
+// Bloom filters | direct maps | tile ring]. (The ungrouped final reduce writes the warps' partials
+// at kSmemQueueOff once every consumer is done — all of those regions are dead by then — so it
+// needs no region of its own.)
+constexpr int kSmemBarOff = 0;                                    // 2 x 8 stages x 8 B
+constexpr int kSmemHeadOff = 128;
+constexpr int kSmemHeadBytes = 128;                               // kMaxStageCols x 4 x 4 B
+// chunk scheduling: [next chunk counter | ring slot tags (the tile each slot was last filled
+// with) x 8]
+constexpr int kSmemCtlOff = kSmemHeadOff + kSmemHeadBytes;
+constexpr int kSmemCtlBytes = 64;
+constexpr int kSmemQueueOff = kSmemCtlOff + kSmemCtlBytes;       // 320
+static_assert(kSmemHeadOff - kSmemBarOff >= 2 * 8 * 8, "barriers overlap the head rows");
+static_assert(kSmemCtlBytes >= 4 * (1 + 8), "counter + 8 slot tags");
+static_assert(kSmemQueueOff % 64 == 0, "queues / carry buffers / group table alignment");
 constexpr int kQueueRows = 2 * kRowsPerThread * 32;       // per warp: one tile pair's rows
 constexpr int kCarryBytes = (HX_MAX_JOINS + 4) * 32 * 4;  // one CarryBuf per consumer warp
 constexpr int smem_carry_off(bool dm) {
@@ -234,6 +268,15 @@ __device__ __forceinline__ ulonglong2 ld_hint(const ulonglong2* p, uint64_t pol)
 struct Pols {
   uint64_t probe, gather;
 };
+__device__ __forceinline__ uint32_t ld_probe(const uint32_t* p, const Pols& pol) {
+  return HX_PROBE_HINT ? ld_hint(p, pol.probe) : __ldg(p);
+}
+__device__ __forceinline__ ulonglong2 ld_probe(const ulonglong2* p, const Pols& pol) {
+  return HX_PROBE_HINT ? ld_hint(p, pol.probe) : __ldg(p);
+}
+__device__ __forceinline__ int32_t ld_gather(const int32_t* p, const Pols& pol) {
+  return HX_GATHER_HINT ? ld_hint(p, pol.gather) : __ldg(p);
+}
 __device__ __forceinline__ void consumer_sync() {
   asm volatile("bar.sync 1, %0;" ::"n"(kConsumers) : "memory");
 }
@@ -435,7 +478,7 @@ __device__ __forceinline__ void stage_c_row(const K1Params& p, const JoinState (
     const JoinDev& d = p.joins[jx];
     wdm[jx] = 0u;
     if (dm_l2<DM>(p, jx) && alive && dm_in(d, e.key[jx]))
-      wdm[jx] = ld_hint(d.dm + (dm_bit(d, e.key[jx]) >> 5), pol.probe);
+      wdm[jx] = ld_probe(d.dm + (dm_bit(d, e.key[jx]) >> 5), pol);
   }
 #pragma unroll
   for (int jx = 0; jx < NJ; ++jx) {
@@ -465,7 +508,7 @@ __device__ __forceinline__ void stage_c_row(const K1Params& p, const JoinState (
     ulonglong2 v[NJ > 0 ? NJ : 1];
 #pragma unroll
     for (int jx = 0; jx < NJ; ++jx)
-      if ((pend >> jx) & 1u) v[jx] = ld_hint(js[jx].buckets + b[jx], pol.probe);
+      if ((pend >> jx) & 1u) v[jx] = ld_probe(js[jx].buckets + b[jx], pol);
 #pragma unroll
     for (int jx = 0; jx < NJ; ++jx) {
       if (!((pend >> jx) & 1u)) continue;
@@ -481,8 +524,8 @@ __device__ __forceinline__ void stage_c_row(const K1Params& p, const JoinState (
   }
   Pending cur{gg, e.a, e.b, alive};
   if (alive) {  // issue the gathers now, consume them one batch later
-    if (p.ga) cur.a = ld_hint(p.gat_a + e.row, pol.gather);
-    if (p.gb) cur.b = ld_hint(p.gat_b + e.row, pol.gather);
+    if (p.ga) cur.a = ld_gather(p.gat_a + e.row, pol);
+    if (p.gb) cur.b = ld_gather(p.gat_b + e.row, pol);
   }
   if (pd.alive)
     accumulate<GROUPED>(p, smem_table, s_sum, s_cnt, pd.g, measure(p.agg_op, pd.a, pd.b), acc_sum,
@@ -523,8 +566,8 @@ __device__ __forceinline__ void process_tile(const K1Params& p, const JoinState 
   const int r0 = wbase + lane * R;
   const int32_t* tb[2] = {sbase0 + r0, sbase1 + r0};
   uint32_t m = 0;
-  if (rows_valid0 == kTileRows) {  // full tiles (all but the last): no per-row bound checks
-    m = rows_valid1 == kTileRows ? (1u << (2 * R)) - 1u : rows_valid1 == 0 ? (1u << R) - 1u : 0u;
+  if (rows_valid0 == kHalfRows) {  // full halves (all but the last): no per-row bound checks
+    m = rows_valid1 == kHalfRows ? (1u << (2 * R)) - 1u : rows_valid1 == 0 ? (1u << R) - 1u : 0u;
   }
   if (m == 0u) {
 #pragma unroll
@@ -617,7 +660,7 @@ __device__ __forceinline__ void process_tile(const K1Params& p, const JoinState 
       uint32_t w[2 * R];
 #pragma unroll
       for (int k = 0; k < 2 * R; ++k)
-        w[k] = ((m >> k) & 1u) && dm_in(d, key[k]) ? ld_hint(d.dm + (dm_bit(d, key[k]) >> 5), pol.probe) : 0u;
+        w[k] = ((m >> k) & 1u) && dm_in(d, key[k]) ? ld_probe(d.dm + (dm_bit(d, key[k]) >> 5), pol) : 0u;
 #pragma unroll
       for (int k = 0; k < 2 * R; ++k) {
         const uint32_t v = dm_entry(d, w[k], dm_bit(d, key[k]));
@@ -646,7 +689,7 @@ __device__ __forceinline__ void process_tile(const K1Params& p, const JoinState 
 #pragma unroll
       for (int k = 0; k < R; ++k) {
         b[k] = bucket_of(key[h * R + k], j.shift);
-        if ((m >> (h * R + k)) & 1u) v[k] = ld_hint(j.buckets + b[k], pol.probe);
+        if ((m >> (h * R + k)) & 1u) v[k] = ld_probe(j.buckets + b[k], pol);
       }
 #pragma unroll
       for (int k = 0; k < R; ++k) {
@@ -665,15 +708,26 @@ __device__ __forceinline__ void process_tile(const K1Params& p, const JoinState 
     int32_t a8[2 * R] = {}, b8[2 * R] = {};
     if (!p.ga) load8(p.agg_a, a8);
     if (!p.gb) load8(p.agg_b, b8);
-    if (p.ga | p.gb) {  // gathers of every passing row first (all in flight together)
+    if (p.ga | p.gb) {
+      // late materialisation: the gathers of a passing row are issued now and consumed at the
+      // lane's NEXT passing row (the one-deep Pending slot stage C uses), so their latency
+      // overlaps the following chunks instead of stalling this one (gathers are planned only
+      // when at most 1/16 of the rows pass: mostly one pending row per lane at a time)
+      for (uint32_t bits = m; bits; bits &= bits - 1u) {
+        const int k = __ffs(bits) - 1;
+        int32_t gk = g0, ak = 0, bk = 0;
 #pragma unroll
-      for (int k = 0; k < 2 * R; ++k) {
+        for (int kk = 0; kk < 2 * R; ++kk)
+          if (kk == k) gk = g[kk], ak = a8[kk], bk = b8[kk];
         const uint32_t row = (k < R ? frow0 : frow1) + r0 + (k & 3);
-        if ((m >> k) & 1u) {
-          if (p.ga) a8[k] = ld_hint(p.gat_a + row, pol.gather);
-          if (p.gb) b8[k] = ld_hint(p.gat_b + row, pol.gather);
-        }
+        Pending cur{gk, p.ga ? ld_gather(p.gat_a + row, pol) : ak,
+                    p.gb ? ld_gather(p.gat_b + row, pol) : bk, true};
+        if (pd.alive)
+          accumulate<GROUPED>(p, smem_table, s_sum, s_cnt, pd.g, measure(p.agg_op, pd.a, pd.b),
+                              acc_sum, acc_cnt);
+        pd = cur;
       }
+      return;
     }
     if (!GROUPED) {  // branch-free: predicated adds, one population count
       long long sum = 0;
@@ -794,8 +848,9 @@ __global__ void __launch_bounds__(kThreads, kCtasPerSm) k1_probe_agg(const __gri
   extern __shared__ __align__(128) unsigned char smem[];
   uint64_t* full = reinterpret_cast<uint64_t*>(smem);
   uint64_t* empty = full + p.stages;
-  long long* red = reinterpret_cast<long long*>(smem + 128);                // 2 x 8 warps
-  int32_t* headbuf = reinterpret_cast<int32_t*>(smem + 128 + 256);           // 8 cols x 4
+  int32_t* headbuf = reinterpret_cast<int32_t*>(smem + kSmemHeadOff);        // 8 cols x 4
+  int* next_chunk = reinterpret_cast<int*>(smem + kSmemCtlOff);
+  volatile int* slot_tile = reinterpret_cast<volatile int*>(smem + kSmemCtlOff) + 1;
   const int kSmemFixed = p.smem_fixed;
   uint8_t* q_rows = smem + kSmemQueueOff;
   int32_t* q_gs = DM ? nullptr
@@ -817,8 +872,10 @@ __global__ void __launch_bounds__(kThreads, kCtasPerSm) k1_probe_agg(const __gri
   if (tid == kConsumers) {
     for (int s = 0; s < p.stages; ++s) {
       mbar_init(full + s, 1);
-      mbar_init(empty + s, kConsumerWarps);
+      mbar_init(empty + s, kChunksPerTile);  // every chunk of the tile arrives once
+      slot_tile[s] = -1;
     }
+    *next_chunk = 0;
     asm volatile("fence.mbarrier_init.release.cluster;" ::: "memory");
   }
   __syncthreads();
@@ -830,8 +887,10 @@ __global__ void __launch_bounds__(kThreads, kCtasPerSm) k1_probe_agg(const __gri
       int s = 0;
       uint32_t ph = 0;
       bool wrapped = false;
-      for (int64_t t = blockIdx.x; t < p.n_tiles; t += gridDim.x) {
+      int i = 0;  // this CTA's i-th tile
+      for (int64_t t = blockIdx.x; t < p.n_tiles; t += gridDim.x, ++i) {
         if (wrapped) mbar_wait_sleep(empty + s, ph ^ 1u);
+        slot_tile[s] = i;  // slot s now holds (is being filled with) tile i: see the consumers
         const int64_t r0 = t * kTileRows;
         const int64_t rows = std::min<int64_t>(kTileRows, p.n_rows - r0);
         const uint32_t bytes = (uint32_t)(rows & ~int64_t(3)) * 4u;
@@ -946,73 +1005,67 @@ __global__ void __launch_bounds__(kThreads, kCtasPerSm) k1_probe_agg(const __gri
   }
   long long acc_sum = 0, acc_cnt = 0;
   Pending pd{0, 0, 0, false};
-  // misaligned head rows (views at a row offset): CTA 0 reads them directly
-  if (blockIdx.x == 0 && p.head_rows > 0) {
-    if (ctid < p.head_rows)
-      for (int c = 0; c < p.n_cols; ++c) headbuf[c * 4 + ctid] = p.head_col[c][ctid];
-    consumer_sync();
-    process_tile<NJ, GROUPED, DM>(p, js, sdm, headbuf, headbuf, 0u, 0u, 4, p.head_rows, 0, warp, lane,
+  // misaligned head rows (views at a row offset): CTA 0's warp 0 reads them directly
+  if (blockIdx.x == 0 && p.head_rows > 0 && warp == 0) {
+    if (lane < p.head_rows)
+      for (int c = 0; c < p.n_cols; ++c) headbuf[c * 4 + lane] = p.head_col[c][lane];
+    __syncwarp();
+    process_tile<NJ, GROUPED, DM>(p, js, sdm, headbuf, headbuf, 0u, 0u, 4, p.head_rows, 0, 0, lane,
                                   smem_table, s_sum, s_cnt, q_row, q_g, cb, n_carry, acc_sum,
                                   acc_cnt, pd, pol);
   }
   consumer_sync();
 
-  // this CTA's tiles t = blockIdx.x + i * gridDim.x arrive in ring slots i mod stages; the
-  // consumers take them two at a time
-  int s = 0;
-  uint32_t ph = 0;
-  auto acquire = [&](int64_t t, int slot, uint32_t phase) -> int {
+  // This CTA's i-th tile (t = blockIdx.x + i * gridDim.x) arrives in ring slot i mod stages.
+  // Warps claim chunks c = 0, 1, 2, ... (tile i = c / kChunksPerTile) from a shared counter;
+  // a stage is released when all of its chunks are done (empty barrier count =
+  // kChunksPerTile). Before waiting on slot s's full barrier for tile i, a warp waits until
+  // the producer has tagged the slot with i: the barrier's previous phase (tile i - stages)
+  // is then complete, so the parity wait cannot match it.
+  const int64_t my_tiles = p.n_tiles > blockIdx.x ? (p.n_tiles - 1 - blockIdx.x) / gridDim.x + 1 : 0;
+  const int64_t my_chunks = my_tiles * kChunksPerTile;
+  int claimed = 0;
+  if (HX_CLAIM_AHEAD && lane == 0) claimed = atomicAdd(next_chunk, 1);
+  while (true) {
+    int c = 0;
+    if (HX_CLAIM_AHEAD) {
+      // the claim of the next chunk is issued now and read after this chunk: the shared
+      // atomic's latency overlaps the work
+      c = __shfl_sync(kFull, claimed, 0);
+      if (c < my_chunks && lane == 0) claimed = atomicAdd(next_chunk, 1);
+    } else {
+      if (lane == 0) c = atomicAdd(next_chunk, 1);
+      c = __shfl_sync(kFull, c, 0);
+    }
+    if (c >= my_chunks) break;
+    const int i = c / kChunksPerTile, ch = c - i * kChunksPerTile;
+    const int slot = i % p.stages;
+    const uint32_t phase = (uint32_t)(i / p.stages) & 1u;
+    while (slot_tile[slot] != i)
+      if (HX_TAG_SLEEP) __nanosleep(HX_TAG_SLEEP);
     mbar_wait(full + slot, phase);
     int32_t* st = stage0 + (size_t)slot * stage_elems;
+    const int64_t t = blockIdx.x + (int64_t)i * gridDim.x;
     const int64_t r0 = t * kTileRows;
     const int rows = (int)std::min<int64_t>(kTileRows, p.n_rows - r0);
+    const int crows = max(0, min(kChunkRows, rows - ch * kChunkRows));
     const int copied = rows & ~3;
-    if (copied != rows) {  // ragged tail: the last <= 3 rows are not 16-byte multiples
-      if (ctid < rows - copied)
-        for (int c = 0; c < p.n_cols; ++c)
-          st[c * kTileRows + copied + ctid] = p.col[c][r0 + copied + ctid];
-      consumer_sync();
+    if (copied != rows && copied / kChunkRows == ch) {
+      // ragged tail: the last <= 3 rows of the table are not a 16-byte multiple (not copied
+      // by the bulk engine); the warp owning their chunk reads them directly
+      if (lane < rows - copied)
+        for (int cc = 0; cc < p.n_cols; ++cc)
+          st[cc * kTileRows + copied + lane] = p.col[cc][r0 + copied + lane];
+      __syncwarp();
     }
-    return rows;
-  };
-  // (pairs need >= 4 ring slots so that two more tiles stream in while a pair is processed;
-  // a shallower ring takes the tiles one at a time)
-  const bool pairs = p.stages >= 4;
-  for (int64_t t = blockIdx.x; t < p.n_tiles;) {
-    const int64_t t0 = t, t1 = t + gridDim.x;
-    const bool two = pairs && t1 < p.n_tiles;
-    t = two ? t1 + gridDim.x : t1;
-    int s1 = s + 1;
-    uint32_t ph1 = ph;
-    if (s1 == p.stages) {
-      s1 = 0;
-      ph1 ^= 1u;
-    }
-    const int rows0 = acquire(t0, s, ph);
-    const int rows1 = two ? acquire(t1, s1, ph1) : 0;
-    const int32_t* st0 = stage0 + (size_t)s * stage_elems;
-    const int32_t* st1 = two ? stage0 + (size_t)s1 * stage_elems : st0;
-    const uint32_t frow0 = (uint32_t)(p.head_rows + t0 * kTileRows);
-    const uint32_t frow1 = (uint32_t)(p.head_rows + t1 * kTileRows);
-    process_tile<NJ, GROUPED, DM>(p, js, sdm, st0, st1, frow0, frow1, kTileRows, rows0, rows1, warp, lane,
-                                  smem_table, s_sum, s_cnt, q_row, q_g, cb, n_carry, acc_sum,
-                                  acc_cnt, pd, pol);
+    const int32_t* cb0 = st + ch * kChunkRows;
+    const uint32_t frow0 = (uint32_t)(p.head_rows + r0 + ch * kChunkRows);
+    process_tile<NJ, GROUPED, DM>(p, js, sdm, cb0, cb0 + kHalfRows, frow0, frow0 + kHalfRows,
+                                  kTileRows, min(crows, kHalfRows),
+                                  max(0, crows - kHalfRows), 0, lane, smem_table, s_sum,
+                                  s_cnt, q_row, q_g, cb, n_carry, acc_sum, acc_cnt, pd, pol);
     __syncwarp();
-    if (lane == 0) {
-      mbar_arrive(empty + s);
-      if (two) mbar_arrive(empty + s1);
-    }
-    if (two) {  // advance by two slots
-      s = s1 + 1;
-      ph = ph1;
-      if (s == p.stages) {
-        s = 0;
-        ph ^= 1u;
-      }
-    } else {
-      s = s1;
-      ph = ph1;
-    }
+    if (lane == 0) mbar_arrive(empty + slot);
   }
 
   // the rows this warp still carries
@@ -1046,16 +1099,20 @@ __global__ void __launch_bounds__(kThreads, kCtasPerSm) k1_probe_agg(const __gri
       acc_sum += __shfl_xor_sync(kFull, acc_sum, o);
       acc_cnt += __shfl_xor_sync(kFull, acc_cnt, o);
     }
+    // every consumer is done with the queues, maps and ring (and no bulk copy is in flight:
+    // every tile was consumed): the partials go at kSmemQueueOff, {sum, count} per warp
+    consumer_sync();
+    long long* red = reinterpret_cast<long long*>(smem + kSmemQueueOff);
     if (lane == 0) {
-      red[warp] = acc_sum;
-      red[kConsumerWarps + warp] = acc_cnt;
+      red[2 * warp] = acc_sum;
+      red[2 * warp + 1] = acc_cnt;
     }
     consumer_sync();
     if (ctid == 0) {
       long long s = 0, c = 0;
       for (int w = 0; w < kConsumerWarps; ++w) {
-        s += red[w];
-        c += red[kConsumerWarps + w];
+        s += red[2 * w];
+        c += red[2 * w + 1];
       }
       if (c) {
         atomicAdd(p.g_sum, (unsigned long long)s);
