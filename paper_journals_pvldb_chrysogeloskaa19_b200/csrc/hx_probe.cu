@@ -40,9 +40,11 @@ namespace hx {
 namespace {
 
 constexpr unsigned kFull = 0xFFFFFFFFu;
-#ifndef HX_K1_WARPS
-#define HX_K1_WARPS 20  // consumer warps per CTA (tuned: 16 -> 20 is -6% K1 time, 24 spills)
-#endif
+// Consumer warps per CTA: every K1 instance is compiled for two counts and k1_setup picks one
+// per pipeline. More warps hide more latency (L2 map reads) but their per-warp queues and carry
+// buffers take shared memory from the filters and maps (measured at SF100: 26 warps 4.5%
+// faster than 20 in sum; SF10 Q4.1 loses its customer bitmap with 26 and is 30% slower).
+constexpr int kWarpsLo = 20, kWarpsHi = 26;
 #ifndef HX_K1_STAGE_KB
 #define HX_K1_STAGE_KB 160  // max shared memory for the tile ring (the rest: Bloom filters)
 #endif
@@ -57,6 +59,12 @@ constexpr unsigned kFull = 0xFFFFFFFFu;
 #define HX_CLAIM_AHEAD 0  // claim the next chunk before processing the current one (measured:
                           // a reserved chunk waits for its warp and delays its stage, -5%)
 #endif
+#ifndef HX_BALLOT_COMPACT
+#define HX_BALLOT_COMPACT 0  // survivors' queue slots from 8 ballots instead of a shuffle scan
+#endif
+#ifndef HX_CLAIM_EARLY
+#define HX_CLAIM_EARLY 0  // claim the next chunk after stage S of the current one
+#endif
 #ifndef HX_TAG_SLEEP
 #define HX_TAG_SLEEP 20   // ns slept between polls of a ring slot's tile tag (0: spin)
 #endif
@@ -64,11 +72,14 @@ constexpr unsigned kFull = 0xFFFFFFFFu;
 #define HX_K1_CTAS 1    // resident CTAs per SM the launch bounds / smem budget target
                         // (one CTA per SM shares one copy of the Bloom filters)
 #endif
-constexpr int kConsumerWarps = HX_K1_WARPS;
-constexpr int kConsumers = kConsumerWarps * 32;
-constexpr int kThreads = kConsumers + 32;  // + one producer warp
+constexpr int k1_threads(int warps) { return warps * 32 + 32; }  // + one producer warp
 constexpr int kRowsPerThread = 4;          // R
-constexpr int kTileRows = kConsumers * kRowsPerThread;  // T = 2560 rows
+#ifndef HX_K1_TILE_ROWS
+#define HX_K1_TILE_ROWS 2560
+#endif
+// rows per ring stage (one bulk copy per column); independent of the warp count since warps
+// claim chunks dynamically
+constexpr int kTileRows = HX_K1_TILE_ROWS;  // T = 2560 rows
 // A CHUNK is one consumer warp's unit of work: 256 consecutive rows of a tile, two halves of
 // 128 (lane l holds rows 4l..4l+3 of each half: one conflict-free 128-bit shared-memory load
 // per column and half). Warps claim chunks dynamically (a shared counter), so a warp that
@@ -100,10 +111,12 @@ static_assert(kSmemCtlBytes >= 4 * (1 + 8), "counter + 8 slot tags");
 static_assert(kSmemQueueOff % 64 == 0, "queues / carry buffers / group table alignment");
 constexpr int kQueueRows = 2 * kRowsPerThread * 32;       // per warp: one tile pair's rows
 constexpr int kCarryBytes = (HX_MAX_JOINS + 4) * 32 * 4;  // one CarryBuf per consumer warp
-constexpr int smem_carry_off(bool dm) {
-  return kSmemQueueOff + kConsumerWarps * kQueueRows * (dm ? 1 : 5);
+constexpr int smem_carry_off(bool dm, int warps) {
+  return kSmemQueueOff + warps * kQueueRows * (dm ? 1 : 5);
 }
-constexpr int smem_fixed(bool dm) { return smem_carry_off(dm) + kConsumerWarps * kCarryBytes; }
+constexpr int smem_fixed(bool dm, int warps) {
+  return smem_carry_off(dm, warps) + warps * kCarryBytes;
+}
 
 struct JoinDev {
   int32_t c;                               // staged column of the FK
@@ -277,8 +290,9 @@ __device__ __forceinline__ ulonglong2 ld_probe(const ulonglong2* p, const Pols& 
 __device__ __forceinline__ int32_t ld_gather(const int32_t* p, const Pols& pol) {
   return HX_GATHER_HINT ? ld_hint(p, pol.gather) : __ldg(p);
 }
+template <int W>
 __device__ __forceinline__ void consumer_sync() {
-  asm volatile("bar.sync 1, %0;" ::"n"(kConsumers) : "memory");
+  asm volatile("bar.sync 1, %0;" ::"n"(W * 32) : "memory");
 }
 
 __device__ __forceinline__ long long measure(int op, int32_t a, int32_t b) {
@@ -560,7 +574,8 @@ __device__ __forceinline__ void process_tile(const K1Params& p, const JoinState 
                                              unsigned long long* s_sum, uint32_t* s_cnt,
                                              uint8_t* q_row, int32_t* q_g, CarryBuf* cb,
                                              int& n_carry, long long& acc_sum,
-                                             long long& acc_cnt, Pending& pd, const Pols& pol) {
+                                             long long& acc_cnt, Pending& pd, const Pols& pol,
+                                             int* claim = nullptr, int* next_chunk = nullptr) {
   constexpr int R = kRowsPerThread;  // rows per lane per tile
   const int wbase = warp * (32 * R);
   const int r0 = wbase + lane * R;
@@ -576,7 +591,10 @@ __device__ __forceinline__ void process_tile(const K1Params& p, const JoinState 
       m |= (uint32_t)(r0 + k < rows_valid1) << (R + k);
     }
   }
-  if (__ballot_sync(kFull, m) == 0) return;
+  if (__ballot_sync(kFull, m) == 0) {
+    if (claim && lane == 0) *claim = atomicAdd(next_chunk, 1);
+    return;
+  }
   // the 8 values of staged column c for this lane
   auto load8 = [&](int c, int32_t (&v)[2 * R]) {
 #pragma unroll
@@ -673,6 +691,8 @@ __device__ __forceinline__ void process_tile(const K1Params& p, const JoinState 
     }
   }
 
+  // (HX_CLAIM_EARLY) the warp's next chunk is claimed here, its latency overlapping the rest
+  if (claim && lane == 0) *claim = atomicAdd(next_chunk, 1);
   const int j0 = first_join_in_place<NJ, DM>(p, js);
   if (j0) {
     // stage B (hash tables): ONE probe step of the first join per row, 4 independent 128-bit
@@ -748,6 +768,22 @@ __device__ __forceinline__ void process_tile(const K1Params& p, const JoinState 
 
   // compaction: append this warp's survivors to its queue — a warp prefix sum of the lanes'
   // survivor counts gives each lane its slots; a lane then writes only its surviving rows
+  const bool carry_g = j0;
+#if HX_BALLOT_COMPACT
+  // row k of every lane: one ballot; its slot = the rows before it (earlier k, lower lanes)
+  const uint32_t lt = (1u << lane) - 1u;
+  int qn = 0;
+#pragma unroll
+  for (int k = 0; k < 2 * R; ++k) {
+    const uint32_t b = __ballot_sync(kFull, (m >> k) & 1u);
+    if ((m >> k) & 1u) {
+      const int pos = qn + __popc(b & lt);
+      q_row[pos] = (uint8_t)(((k >> 2) << 7) | (lane * R + (k & 3)));
+      if (carry_g) q_g[pos] = g[k];
+    }
+    qn += __popc(b);
+  }
+#else
   const int cnt = __popc(m);
   int incl = cnt;
 #pragma unroll
@@ -757,7 +793,6 @@ __device__ __forceinline__ void process_tile(const K1Params& p, const JoinState 
   }
   const int qn = __shfl_sync(kFull, incl, 31);
   int pos = incl - cnt;
-  const bool carry_g = j0;
   for (uint32_t bits = m; bits; bits &= bits - 1u, ++pos) {
     const int k = __ffs(bits) - 1;
     q_row[pos] = (uint8_t)(((k >> 2) << 7) | (lane * R + (k & 3)));
@@ -768,6 +803,7 @@ __device__ __forceinline__ void process_tile(const K1Params& p, const JoinState 
       q_g[pos] = gv;
     }
   }
+#endif
   __syncwarp();
 
   // stage C in full batches of 32: the warp's queue of this pair is appended to the rows
@@ -843,8 +879,15 @@ __device__ __forceinline__ void mbar_wait_sleep(uint64_t* bar, uint32_t parity) 
   }
 }
 
-template <int NJ, bool GROUPED, bool DM>
-__global__ void __launch_bounds__(kThreads, kCtasPerSm) k1_probe_agg(const __grid_constant__ K1Params p) {
+template <int NJ, bool GROUPED, bool DM, int W>
+#ifndef HX_K1_LB_LO
+#define HX_K1_LB_LO 896  // launch-bound thread count of the 20-warp instances (0: exact):
+                         // 896 caps them at 72 registers, measured 0.3-3% faster than 80
+#endif
+__global__ void __launch_bounds__((W == kWarpsLo && HX_K1_LB_LO) ? HX_K1_LB_LO : k1_threads(W), kCtasPerSm)
+    k1_probe_agg(const __grid_constant__ K1Params p) {
+  constexpr int kConsumerWarps = W;
+  constexpr int kConsumers = W * 32;
   extern __shared__ __align__(128) unsigned char smem[];
   uint64_t* full = reinterpret_cast<uint64_t*>(smem);
   uint64_t* empty = full + p.stages;
@@ -854,7 +897,7 @@ __global__ void __launch_bounds__(kThreads, kCtasPerSm) k1_probe_agg(const __gri
   const int kSmemFixed = p.smem_fixed;
   uint8_t* q_rows = smem + kSmemQueueOff;
   int32_t* q_gs = DM ? nullptr
-                     : reinterpret_cast<int32_t*>(smem + kSmemQueueOff + kConsumerWarps * kQueueRows);
+                     : reinterpret_cast<int32_t*>(smem + kSmemQueueOff + W * kQueueRows);
   unsigned long long* s_sum = reinterpret_cast<unsigned long long*>(smem + kSmemFixed);
   uint32_t* s_cnt = reinterpret_cast<uint32_t*>(s_sum + p.smem_groups);
   const size_t table_bytes = ((size_t)p.smem_groups * 12 + 127) & ~size_t(127);
@@ -926,7 +969,7 @@ __global__ void __launch_bounds__(kThreads, kCtasPerSm) k1_probe_agg(const __gri
   const Pols pol{p.l2_hint ? policy_evict_last() : policy_evict_normal(), policy_evict_first()};
   uint8_t* q_row = q_rows + warp * kQueueRows;
   int32_t* q_g = DM ? nullptr : q_gs + warp * kQueueRows;
-  CarryBuf* cb = reinterpret_cast<CarryBuf*>(smem + smem_carry_off(DM) + warp * kCarryBytes);
+  CarryBuf* cb = reinterpret_cast<CarryBuf*>(smem + smem_carry_off(DM, W) + warp * kCarryBytes);
   int n_carry = 0;
   JoinState js[HX_MAX_JOINS];
 #pragma unroll
@@ -1014,7 +1057,7 @@ __global__ void __launch_bounds__(kThreads, kCtasPerSm) k1_probe_agg(const __gri
                                   smem_table, s_sum, s_cnt, q_row, q_g, cb, n_carry, acc_sum,
                                   acc_cnt, pd, pol);
   }
-  consumer_sync();
+  consumer_sync<W>();
 
   // This CTA's i-th tile (t = blockIdx.x + i * gridDim.x) arrives in ring slot i mod stages.
   // Warps claim chunks c = 0, 1, 2, ... (tile i = c / kChunksPerTile) from a shared counter;
@@ -1025,10 +1068,12 @@ __global__ void __launch_bounds__(kThreads, kCtasPerSm) k1_probe_agg(const __gri
   const int64_t my_tiles = p.n_tiles > blockIdx.x ? (p.n_tiles - 1 - blockIdx.x) / gridDim.x + 1 : 0;
   const int64_t my_chunks = my_tiles * kChunksPerTile;
   int claimed = 0;
-  if (HX_CLAIM_AHEAD && lane == 0) claimed = atomicAdd(next_chunk, 1);
+  if ((HX_CLAIM_AHEAD || HX_CLAIM_EARLY) && lane == 0) claimed = atomicAdd(next_chunk, 1);
   while (true) {
     int c = 0;
-    if (HX_CLAIM_AHEAD) {
+    if (HX_CLAIM_EARLY) {
+      c = __shfl_sync(kFull, claimed, 0);
+    } else if (HX_CLAIM_AHEAD) {
       // the claim of the next chunk is issued now and read after this chunk: the shared
       // atomic's latency overlaps the work
       c = __shfl_sync(kFull, claimed, 0);
@@ -1039,6 +1084,8 @@ __global__ void __launch_bounds__(kThreads, kCtasPerSm) k1_probe_agg(const __gri
     }
     if (c >= my_chunks) break;
     const int i = c / kChunksPerTile, ch = c - i * kChunksPerTile;
+    // (tracking slot and phase incrementally instead of dividing by the ring depth was
+    // measured 3% slower: the loop-carried registers cost more than the division)
     const int slot = i % p.stages;
     const uint32_t phase = (uint32_t)(i / p.stages) & 1u;
     while (slot_tile[slot] != i)
@@ -1063,7 +1110,8 @@ __global__ void __launch_bounds__(kThreads, kCtasPerSm) k1_probe_agg(const __gri
     process_tile<NJ, GROUPED, DM>(p, js, sdm, cb0, cb0 + kHalfRows, frow0, frow0 + kHalfRows,
                                   kTileRows, min(crows, kHalfRows),
                                   max(0, crows - kHalfRows), 0, lane, smem_table, s_sum,
-                                  s_cnt, q_row, q_g, cb, n_carry, acc_sum, acc_cnt, pd, pol);
+                                  s_cnt, q_row, q_g, cb, n_carry, acc_sum, acc_cnt, pd, pol,
+                                  HX_CLAIM_EARLY ? &claimed : nullptr, next_chunk);
     __syncwarp();
     if (lane == 0) mbar_arrive(empty + slot);
   }
@@ -1081,7 +1129,7 @@ __global__ void __launch_bounds__(kThreads, kCtasPerSm) k1_probe_agg(const __gri
   // ---------------- flush the CTA's partial aggregate ----------------
   if (GROUPED) {
     if (smem_table) {
-      consumer_sync();
+      consumer_sync<W>();
       const uint32_t* s_lo = reinterpret_cast<const uint32_t*>(s_sum);
       for (int g = ctid; g < n_groups; g += kConsumers) {
         const uint32_t c = s_cnt[g];
@@ -1101,13 +1149,13 @@ __global__ void __launch_bounds__(kThreads, kCtasPerSm) k1_probe_agg(const __gri
     }
     // every consumer is done with the queues, maps and ring (and no bulk copy is in flight:
     // every tile was consumed): the partials go at kSmemQueueOff, {sum, count} per warp
-    consumer_sync();
+    consumer_sync<W>();
     long long* red = reinterpret_cast<long long*>(smem + kSmemQueueOff);
     if (lane == 0) {
       red[2 * warp] = acc_sum;
       red[2 * warp + 1] = acc_cnt;
     }
-    consumer_sync();
+    consumer_sync<W>();
     if (ctid == 0) {
       long long s = 0, c = 0;
       for (int w = 0; w < kConsumerWarps; ++w) {
@@ -1367,26 +1415,26 @@ cudaError_t launch_k1(KernelFn fn, int grid, int block, size_t smem, cudaStream_
   return cudaLaunchKernelEx(&cfg, fn, p);
 }
 
-// [direct maps][grouped][joins]; join-less pipelines use the hash-table instances
-const KernelFn kKernels[2][2][HX_MAX_JOINS + 1] = {
-    {{k1_probe_agg<0, false, false>, k1_probe_agg<1, false, false>, k1_probe_agg<2, false, false>,
-      k1_probe_agg<3, false, false>, k1_probe_agg<4, false, false>},
-     {k1_probe_agg<0, true, false>, k1_probe_agg<1, true, false>, k1_probe_agg<2, true, false>,
-      k1_probe_agg<3, true, false>, k1_probe_agg<4, true, false>}},
-    {{k1_probe_agg<0, false, false>, k1_probe_agg<1, false, true>, k1_probe_agg<2, false, true>,
-      k1_probe_agg<3, false, true>, k1_probe_agg<4, false, true>},
-     {k1_probe_agg<0, true, false>, k1_probe_agg<1, true, true>, k1_probe_agg<2, true, true>,
-      k1_probe_agg<3, true, true>, k1_probe_agg<4, true, true>}}};
+// [warps: 20, 26][direct maps][grouped][joins]; join-less pipelines use the hash-table instances
+#define HX_K1_ROW(W, G, D)                                                                      \
+  {k1_probe_agg<0, G, false, W>, k1_probe_agg<1, G, D, W>, k1_probe_agg<2, G, D, W>,             \
+   k1_probe_agg<3, G, D, W>, k1_probe_agg<4, G, D, W>}
+const KernelFn kKernels[2][2][2][HX_MAX_JOINS + 1] = {
+    {{HX_K1_ROW(kWarpsLo, false, false), HX_K1_ROW(kWarpsLo, true, false)},
+     {HX_K1_ROW(kWarpsLo, false, true), HX_K1_ROW(kWarpsLo, true, true)}},
+    {{HX_K1_ROW(kWarpsHi, false, false), HX_K1_ROW(kWarpsHi, true, false)},
+     {HX_K1_ROW(kWarpsHi, false, true), HX_K1_ROW(kWarpsHi, true, true)}}};
+#undef HX_K1_ROW
 
-KernelFn pick_kernel(int nj, bool grouped, bool dm) {
-  return kKernels[dm ? 1 : 0][grouped ? 1 : 0][nj];
+KernelFn pick_kernel(int nj, bool grouped, bool dm, int warps) {
+  return kKernels[warps == kWarpsHi ? 1 : 0][dm ? 1 : 0][grouped ? 1 : 0][nj];
 }
 
-size_t k1_smem_bytes(bool dm, int n_cols, int stages, int smem_groups, int filter_words = 0,
-                     int dm_bytes = 0, bool in_place = false) {
+size_t k1_smem_bytes(int warps, bool dm, int n_cols, int stages, int smem_groups,
+                     int filter_words = 0, int dm_bytes = 0, bool in_place = false) {
   const size_t table_bytes = ((size_t)smem_groups * 12 + 127) & ~size_t(127);
   const size_t filter_bytes = ((size_t)filter_words * 4 + 127) & ~size_t(127);
-  return (in_place ? kSmemQueueOff : smem_fixed(dm)) + table_bytes + filter_bytes + (size_t)dm_bytes +
+  return (in_place ? kSmemQueueOff : smem_fixed(dm, warps)) + table_bytes + filter_bytes + (size_t)dm_bytes +
          (size_t)stages * n_cols * kTileRows * sizeof(int32_t);
 }
 
@@ -1406,10 +1454,10 @@ size_t k1_smem_cap() {
   return cap;
 }
 
-int pick_stages(bool dm, int n_cols, int smem_groups) {
+int pick_stages(int warps, bool dm, int n_cols, int smem_groups) {
   // as many tile stages as fit next to kCtasPerSm CTAs per SM, at least double buffering
   // (at most HX_K1_STAGE_KB of tiles per CTA: the rest is left for filters and maps)
-  const size_t fixed = smem_fixed(dm) + (((size_t)smem_groups * 12 + 127) & ~size_t(127));
+  const size_t fixed = smem_fixed(dm, warps) + (((size_t)smem_groups * 12 + 127) & ~size_t(127));
   const size_t budget = std::min<size_t>(std::min(smem_budget(kCtasPerSm), k1_smem_cap()),
                                          fixed + HX_K1_STAGE_KB * 1024);
   const size_t stage = (size_t)n_cols * kTileRows * 4;
@@ -1556,11 +1604,12 @@ int k1_occupancy(hx_ctx* ctx) {
   std::lock_guard<std::mutex> lock(mu);
   const uint64_t bit = ctx->device < 64 ? (uint64_t(1) << ctx->device) : 0;
   if (!bit || !(done & bit)) {
-    for (int d = 0; d < 2; ++d)
-      for (int g = 0; g < 2; ++g)
-        for (int j = 0; j <= HX_MAX_JOINS; ++j)
-          cudaFuncSetAttribute(kKernels[d][g][j], cudaFuncAttributeMaxDynamicSharedMemorySize,
-                               227 * 1024);
+    for (int w = 0; w < 2; ++w)
+      for (int d = 0; d < 2; ++d)
+        for (int g = 0; g < 2; ++g)
+          for (int j = 0; j <= HX_MAX_JOINS; ++j)
+            cudaFuncSetAttribute(kKernels[w][d][g][j], cudaFuncAttributeMaxDynamicSharedMemorySize,
+                                 227 * 1024);
     cudaFuncSetAttribute(k1_scan_agg<1>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)scan_smem(1));
     cudaFuncSetAttribute(k1_scan_agg<2>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)scan_smem(2));
     cudaFuncSetAttribute(k1_scan_agg<3>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)scan_smem(3));
@@ -1569,8 +1618,8 @@ int k1_occupancy(hx_ctx* ctx) {
   }
   int occ = 0;
   cudaOccupancyMaxActiveBlocksPerMultiprocessor(
-      &occ, k1_probe_agg<3, true, false>, kThreads,
-      k1_smem_bytes(false, 4, pick_stages(false, 4, kSmemGroups), kSmemGroups));
+      &occ, k1_probe_agg<3, true, false, kWarpsLo>, k1_threads(kWarpsLo),
+      k1_smem_bytes(kWarpsLo, false, 4, pick_stages(kWarpsLo, false, 4, kSmemGroups), kSmemGroups));
   return occ;
 }
 
@@ -1599,6 +1648,8 @@ struct K1Prepared {
   int occ = 1;
   int64_t seg_rows = kSegRows;  // rows per launch (HX_K1_SEG_TILES overrides, for tests)
   int carveout = 100;           // preferred shared-memory carveout (% of 228 KB)
+  int warps = kWarpsLo;         // consumer warps of the chosen instance
+  double cost = -1.0;           // plan cost (direct maps; -1: hash tables)
   L2Window win;                 // persisting window over the largest L2-read probe structure
 };
 
@@ -1789,190 +1840,215 @@ int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht*
   // more filters lost 6% at SF100); the rest of the CTA's shared memory holds per-join
   // structures: hash-table pipelines get Bloom filters greedily (plan_ht below); direct-map
   // pipelines are planned by a cost model over every combination (plan_dm).
-  p.stages = pick_stages(dm_mode, n_cols, p.smem_groups);
-  int kind[HX_MAX_JOINS] = {kStNone, kStNone, kStNone, kStNone};
-  int bloom_w[HX_MAX_JOINS] = {0, 0, 0, 0};
-  int in_s[HX_MAX_JOINS] = {0, 0, 0, 0};
-  double pass[HX_MAX_JOINS] = {1, 1, 1, 1};
-  bool known[HX_MAX_JOINS] = {false, false, false, false};
-  int bloom_w0[HX_MAX_JOINS] = {0, 0, 0, 0};
-  int64_t keys[HX_MAX_JOINS] = {0, 0, 0, 0};
-  for (int j = 0; j < sh->n_joins; ++j) {
-    const hx_ht* ht = hts[sh->join_ht[j]];
-    if (ht->known_keys < 0) continue;
-    known[j] = true;
-    keys[j] = ht->known_keys;
-    pass[j] = (double)ht->known_keys / (double)std::max<int64_t>(1, ht->dim_rows);
-    bloom_w0[j] = std::max(4, 1 << std::min(ht->max_bloom_log2w, bloom_log2w_for(ht->known_keys)));
-  }
-  auto fits_sizes = [&](const int* kd, const int* bw) {
-    int fw = 0, db = 0;
+  // The shared-memory plan, for one consumer-warp count W (both instances are planned and the
+  // better one launched, see kWarpsHi).
+  auto plan_with = [&](const int W, K1Prepared& k) {
+    K1Params& p = k.p;
+    t_smem_cap = 0;
+    p.stages = pick_stages(W, dm_mode, n_cols, p.smem_groups);
+    int kind[HX_MAX_JOINS] = {kStNone, kStNone, kStNone, kStNone};
+    int bloom_w[HX_MAX_JOINS] = {0, 0, 0, 0};
+    int in_s[HX_MAX_JOINS] = {0, 0, 0, 0};
+    double pass[HX_MAX_JOINS] = {1, 1, 1, 1};
+    bool known[HX_MAX_JOINS] = {false, false, false, false};
+    int bloom_w0[HX_MAX_JOINS] = {0, 0, 0, 0};
+    int64_t keys[HX_MAX_JOINS] = {0, 0, 0, 0};
     for (int j = 0; j < sh->n_joins; ++j) {
-      const JoinDev& d = p.joins[j];
-      if (kd[j] == kStFull) db += d.dm_words * 4;
-      if (kd[j] == kStBitmap) db += d.bm_words * 4;
-      if (kd[j] == kStBloom) fw += bw[j];
-    }
-    return k1_smem_bytes(dm_mode, n_cols, p.stages, p.smem_groups, fw, db) <=
-           k1_smem_cap();
-  };
-  double plan_cost = -1.0;
-  if (dm_mode) {
-    bool grouped_j[HX_MAX_JOINS] = {false, false, false, false};
-    for (int g = 0; g < sh->n_gdims; ++g) grouped_j[sh->gdim_join[g]] = true;
-    plan_cost = plan_dm(sh->n_joins, p.joins, known, pass, keys, bloom_w0, grouped_j, fits_sizes,
-                        kind, bloom_w, in_s);
-    // An L2-lookup-bound plan (SF1000 Q3.1/Q4.1: 2-15 MB maps read for most rows) runs faster
-    // with less shared memory and the freed part of the SM's array as L1 for the map reads:
-    // replan within 164 KB, or within a 4-stage ring (tile pairs) for wide pipelines
-    // (measured at SF1000 per 600 M rows: Q3.1 4.68 -> 3.59 ms, Q4.1 6.55 -> 4.02 ms; a
-    // 3-stage ring (no pairs) gave Q4.1 5.03; plans below the threshold — every SF10/SF100
-    // plan — lose with the cap).
-    if (plan_cost > kL1BoundCost && !std::getenv("HX_K1_SMEM_KB")) {
-      t_smem_cap = std::max<size_t>(164 * 1024, k1_smem_bytes(dm_mode, n_cols, 4, p.smem_groups));
-      p.stages = pick_stages(dm_mode, n_cols, p.smem_groups);
-      for (int j = 0; j < HX_MAX_JOINS; ++j) kind[j] = kStNone, bloom_w[j] = 0, in_s[j] = 0;
-      plan_cost = plan_dm(sh->n_joins, p.joins, known, pass, keys, bloom_w0, grouped_j,
-                          fits_sizes, kind, bloom_w, in_s);
-    }
-    // every join read from L2 in stage S and no shared-memory structure (the §6.4 1:N join):
-    // a 100 KB ring leaves the rest as L1 for the map (measured: 248 -> 273 G rows/s)
-    bool all_l2s = sh->n_joins > 0 && !std::getenv("HX_K1_SMEM_KB");
-    for (int j = 0; j < sh->n_joins; ++j) all_l2s = all_l2s && kind[j] == kStNone && in_s[j];
-    if (all_l2s) t_smem_cap = 100 * 1024;
-  } else {
-    // hash tables: selective joins (at most half the dimension passes), most selective first,
-    // get a Bloom filter (folded to 4 or 2 bits per key when the full one does not fit)
-    int ord[HX_MAX_JOINS] = {0, 1, 2, 3};
-    std::stable_sort(ord, ord + sh->n_joins, [&](int x, int y) { return pass[x] < pass[y]; });
-    for (int i = 0; i < sh->n_joins; ++i) {
-      const int j = ord[i];
-      if (!known[j] || 2 * pass[j] > 1.0) continue;
-      for (int f = 1; f <= 8 && kind[j] == kStNone && bloom_w0[j] / f >= 4; f *= 2) {
-        kind[j] = kStBloom;
-        bloom_w[j] = bloom_w0[j] / f;
-        if (!fits_sizes(kind, bloom_w)) {
-          kind[j] = kStNone;
-          bloom_w[j] = 0;
-        }
-      }
-    }
-  }
-  // offsets: Bloom filters in the filter region, maps and bitmaps in the direct-map region
-  p.filter_words = 0;
-  p.dm_bytes = 0;
-  for (int j = 0; j < sh->n_joins; ++j) {
-    JoinDev& d = p.joins[j];
-    d.bloom_words = 0;
-    d.dm_smem = -1;
-    d.bm_smem = -1;
-    if (kind[j] == kStBloom) {
-      d.bloom_words = bloom_w[j];
-      p.filter_words += bloom_w[j];
-    } else if (kind[j] == kStFull) {
-      d.dm_smem = p.dm_bytes;
-      p.dm_bytes += d.dm_words * 4;
-    } else if (kind[j] == kStBitmap) {
-      d.bm_smem = p.dm_bytes;
-      p.dm_bytes += d.bm_words * 4;
-    }
-    d.in_s = in_s[j];
-  }
-  p.m_dm = p.m_dmsm = p.m_bm = p.m_ins = p.m_l2 = p.m_l2s = p.m_res = 0u;
-  {
-    bool grouped_j[HX_MAX_JOINS] = {false, false, false, false};
-    for (int g = 0; g < sh->n_gdims; ++g) grouped_j[sh->gdim_join[g]] = true;
-    for (int j = 0; j < sh->n_joins; ++j) {
-      const JoinDev& d = p.joins[j];
-      const bool dm = d.dm != nullptr, full = dm && d.dm_smem >= 0, bm = dm && d.bm_smem >= 0;
-      p.m_dm |= (uint32_t)dm << j;
-      p.m_dmsm |= (uint32_t)full << j;
-      p.m_bm |= (uint32_t)bm << j;
-      p.m_ins |= (uint32_t)(d.in_s != 0) << j;
-      const bool l2s = dm && d.in_s && !full && !bm && d.bloom_words == 0;
-      p.m_l2s |= (uint32_t)l2s << j;
-      p.m_res |= (uint32_t)(d.in_s && (full || l2s)) << j;
-      // the L2 map in stage C: for the rank of a grouping join, or for the verdict when no
-      // exact one is known (no structure, or a Bloom filter)
-      p.m_l2 |= (uint32_t)(dm && !full && (grouped_j[j] || !(bm || l2s))) << j;
-    }
-  }
-  // a pipeline whose joins all resolve in stage S aggregates in place: no per-warp queues or
-  // carry buffers. Shared memory the plan left over deepens the tile ring (up to 8 stages:
-  // more bytes in flight per SM while the consumers hold a pair of tiles).
-  const bool in_place = sh->n_joins == 0 ||
-                        (dm_mode && p.m_res == (1u << sh->n_joins) - 1u);
-  p.smem_fixed = in_place ? kSmemQueueOff : smem_fixed(dm_mode);
-  {
-    int max_stages = 8;
-    if (const char* e = std::getenv("HX_K1_MAX_STAGES")) max_stages = std::max(2, std::min(8, std::atoi(e)));
-    while (p.stages < max_stages &&
-           k1_smem_bytes(dm_mode, n_cols, p.stages + 1, p.smem_groups, p.filter_words, p.dm_bytes,
-                         in_place) <= k1_smem_cap())
-      ++p.stages;
-  }
-  // (measured, SF10: a distance of 2 gains 4-7% on the 4-column pipelines whose ring stays at
-  // 4 stages, and loses 3-6% on 3-column ones, whose rings are deeper or whose tiles are
-  // consumed faster)
-  p.prefetch = (n_cols >= 4 && p.stages <= 4 && fact->placement != HX_PLACE_HOST_MAPPED) ? 2 : 0;
-  // L2 residency of the probe structures (north_star; PAPER.md:1016-1022 operator state in
-  // device memory): probe loads carry an evict_last hint, and the largest structure K1 reads
-  // from L2 (a direct map not staged in shared memory, or a hash table's slots) gets a
-  // persisting access-policy window. HX_L2_HINT=0 / hx_ctx_set_option(HX_OPT_L2_PERSIST, 0):
-  // A/B switches.
-  p.l2_hint = 1;
-  if (const char* e = std::getenv("HX_L2_HINT")) p.l2_hint = std::atoi(e) != 0;
-  if (ctx->l2_persist && ctx->l2_persist_max > 0) {
-    for (int j = 0; j < sh->n_joins; ++j) {
-      const JoinDev& d = p.joins[j];
       const hx_ht* ht = hts[sh->join_ht[j]];
-      void* base = nullptr;
-      size_t bytes = 0;
-      if (d.dm) {
-        if (d.dm_smem < 0 && (((p.m_l2 | p.m_l2s) >> j) & 1u)) {
-          base = const_cast<uint32_t*>(d.dm);
-          bytes = (size_t)d.dm_words * 4;
-        }
-      } else {
-        int lg = ht->max_log2cap;
-        if (ht->known_keys >= 0) {
-          lg = kMinLog2Cap;
-          while (lg < ht->max_log2cap && (int64_t(1) << lg) < 4 * ht->known_keys) ++lg;
-        }
-        base = ht->slots;
-        bytes = (size_t(1) << lg) * 8;
+      if (ht->known_keys < 0) continue;
+      known[j] = true;
+      keys[j] = ht->known_keys;
+      pass[j] = (double)ht->known_keys / (double)std::max<int64_t>(1, ht->dim_rows);
+      bloom_w0[j] = std::max(4, 1 << std::min(ht->max_bloom_log2w, bloom_log2w_for(ht->known_keys)));
+    }
+    auto fits_sizes = [&](const int* kd, const int* bw) {
+      int fw = 0, db = 0;
+      for (int j = 0; j < sh->n_joins; ++j) {
+        const JoinDev& d = p.joins[j];
+        if (kd[j] == kStFull) db += d.dm_words * 4;
+        if (kd[j] == kStBitmap) db += d.bm_words * 4;
+        if (kd[j] == kStBloom) fw += bw[j];
       }
-      if (bytes > k.win.bytes) {
-        k.win.base = base;
-        k.win.bytes = std::min<size_t>(bytes, (size_t)ctx->l2_window_max);
+      return k1_smem_bytes(W, dm_mode, n_cols, p.stages, p.smem_groups, fw, db) <=
+             k1_smem_cap();
+    };
+    double plan_cost = -1.0;
+    if (dm_mode) {
+      bool grouped_j[HX_MAX_JOINS] = {false, false, false, false};
+      for (int g = 0; g < sh->n_gdims; ++g) grouped_j[sh->gdim_join[g]] = true;
+      plan_cost = plan_dm(sh->n_joins, p.joins, known, pass, keys, bloom_w0, grouped_j, fits_sizes,
+                          kind, bloom_w, in_s);
+      // An L2-lookup-bound plan (SF1000 Q3.1/Q4.1: 2-15 MB maps read for most rows) runs faster
+      // with less shared memory and the freed part of the SM's array as L1 for the map reads:
+      // replan within 164 KB, or within a 4-stage ring (tile pairs) for wide pipelines
+      // (measured at SF1000 per 600 M rows: Q3.1 4.68 -> 3.59 ms, Q4.1 6.55 -> 4.02 ms; a
+      // 3-stage ring (no pairs) gave Q4.1 5.03; plans below the threshold — every SF10/SF100
+      // plan — lose with the cap).
+      if (plan_cost > kL1BoundCost && !std::getenv("HX_K1_SMEM_KB")) {
+        t_smem_cap = std::max<size_t>(164 * 1024, k1_smem_bytes(W, dm_mode, n_cols, 4, p.smem_groups));
+        p.stages = pick_stages(W, dm_mode, n_cols, p.smem_groups);
+        for (int j = 0; j < HX_MAX_JOINS; ++j) kind[j] = kStNone, bloom_w[j] = 0, in_s[j] = 0;
+        plan_cost = plan_dm(sh->n_joins, p.joins, known, pass, keys, bloom_w0, grouped_j,
+                            fits_sizes, kind, bloom_w, in_s);
+      }
+      // every join read from L2 in stage S and no shared-memory structure (the §6.4 1:N join):
+      // a 100 KB ring leaves the rest as L1 for the map (measured: 248 -> 273 G rows/s)
+      bool all_l2s = sh->n_joins > 0 && !std::getenv("HX_K1_SMEM_KB");
+      for (int j = 0; j < sh->n_joins; ++j) all_l2s = all_l2s && kind[j] == kStNone && in_s[j];
+      if (all_l2s) t_smem_cap = 100 * 1024;
+    } else {
+      // hash tables: selective joins (at most half the dimension passes), most selective first,
+      // get a Bloom filter (folded to 4 or 2 bits per key when the full one does not fit)
+      int ord[HX_MAX_JOINS] = {0, 1, 2, 3};
+      std::stable_sort(ord, ord + sh->n_joins, [&](int x, int y) { return pass[x] < pass[y]; });
+      for (int i = 0; i < sh->n_joins; ++i) {
+        const int j = ord[i];
+        if (!known[j] || 2 * pass[j] > 1.0) continue;
+        for (int f = 1; f <= 8 && kind[j] == kStNone && bloom_w0[j] / f >= 4; f *= 2) {
+          kind[j] = kStBloom;
+          bloom_w[j] = bloom_w0[j] / f;
+          if (!fits_sizes(kind, bloom_w)) {
+            kind[j] = kStNone;
+            bloom_w[j] = 0;
+          }
+        }
       }
     }
-    if (k.win.bytes)
-      k.win.hit_ratio = (float)std::min(1.0, (double)ctx->l2_persist_max / (double)k.win.bytes);
-  }
-  if (const char* e = std::getenv("HX_K1_PREFETCH")) p.prefetch = std::max(0, std::min(64, std::atoi(e)));
-  if (std::getenv("HX_DEBUG")) {  // launch plan of this K1 (tuning aid)
-    std::fprintf(stderr, "[hx] K1 joins=%d cols=%d gather=%d%d stages=%d groups=%d filters:",
-                 sh->n_joins, n_cols, p.ga, p.gb, p.stages, p.smem_groups);
-    for (int j = 0; j < sh->n_joins; ++j) std::fprintf(stderr, " %d", p.joins[j].bloom_words);
-    std::fprintf(stderr, " dm(words@smem/bitmap@smem):");
-    for (int j = 0; j < sh->n_joins; ++j)
-      std::fprintf(stderr, " %d@%d/%d@%d", p.joins[j].dm ? p.joins[j].dm_words : 0,
-                   p.joins[j].dm_smem, p.joins[j].bm_words, p.joins[j].bm_smem);
-    std::fprintf(stderr, " in_s:");
-    for (int j = 0; j < sh->n_joins; ++j) std::fprintf(stderr, "%d", p.joins[j].in_s);
-    std::fprintf(stderr, " l2:%x l2s:%x cost=%.2f stages=%d smem=%zu\n", p.m_l2, p.m_l2s, plan_cost, p.stages,
-                 k1_smem_bytes(dm_mode, n_cols, p.stages, p.smem_groups, p.filter_words, p.dm_bytes,
-                               in_place));
-  }
-  k.fn = pick_kernel(sh->n_joins, grouped, p.m_dm != 0u);
-  k.smem = k1_smem_bytes(dm_mode, n_cols, p.stages, p.smem_groups, p.filter_words, p.dm_bytes,
-                         in_place);
-  // the smallest shared-memory carveout that holds the plan: the rest of the SM's L1/shared
-  // array caches the maps read from L2
-  k.carveout = (int)std::min<size_t>(100, ((k.smem + 1024) * 100 + 228 * 1024 - 1) / (228 * 1024));
+    // offsets: Bloom filters in the filter region, maps and bitmaps in the direct-map region
+    p.filter_words = 0;
+    p.dm_bytes = 0;
+    for (int j = 0; j < sh->n_joins; ++j) {
+      JoinDev& d = p.joins[j];
+      d.bloom_words = 0;
+      d.dm_smem = -1;
+      d.bm_smem = -1;
+      if (kind[j] == kStBloom) {
+        d.bloom_words = bloom_w[j];
+        p.filter_words += bloom_w[j];
+      } else if (kind[j] == kStFull) {
+        d.dm_smem = p.dm_bytes;
+        p.dm_bytes += d.dm_words * 4;
+      } else if (kind[j] == kStBitmap) {
+        d.bm_smem = p.dm_bytes;
+        p.dm_bytes += d.bm_words * 4;
+      }
+      d.in_s = in_s[j];
+    }
+    p.m_dm = p.m_dmsm = p.m_bm = p.m_ins = p.m_l2 = p.m_l2s = p.m_res = 0u;
+    {
+      bool grouped_j[HX_MAX_JOINS] = {false, false, false, false};
+      for (int g = 0; g < sh->n_gdims; ++g) grouped_j[sh->gdim_join[g]] = true;
+      for (int j = 0; j < sh->n_joins; ++j) {
+        const JoinDev& d = p.joins[j];
+        const bool dm = d.dm != nullptr, full = dm && d.dm_smem >= 0, bm = dm && d.bm_smem >= 0;
+        p.m_dm |= (uint32_t)dm << j;
+        p.m_dmsm |= (uint32_t)full << j;
+        p.m_bm |= (uint32_t)bm << j;
+        p.m_ins |= (uint32_t)(d.in_s != 0) << j;
+        const bool l2s = dm && d.in_s && !full && !bm && d.bloom_words == 0;
+        p.m_l2s |= (uint32_t)l2s << j;
+        p.m_res |= (uint32_t)(d.in_s && (full || l2s)) << j;
+        // the L2 map in stage C: for the rank of a grouping join, or for the verdict when no
+        // exact one is known (no structure, or a Bloom filter)
+        p.m_l2 |= (uint32_t)(dm && !full && (grouped_j[j] || !(bm || l2s))) << j;
+      }
+    }
+    // a pipeline whose joins all resolve in stage S aggregates in place: no per-warp queues or
+    // carry buffers. Shared memory the plan left over deepens the tile ring (up to 8 stages:
+    // more bytes in flight per SM while the consumers hold a pair of tiles).
+    const bool in_place = sh->n_joins == 0 ||
+                          (dm_mode && p.m_res == (1u << sh->n_joins) - 1u);
+    p.smem_fixed = in_place ? kSmemQueueOff : smem_fixed(dm_mode, W);
+    {
+      int max_stages = 8;
+      if (const char* e = std::getenv("HX_K1_MAX_STAGES")) max_stages = std::max(2, std::min(8, std::atoi(e)));
+      while (p.stages < max_stages &&
+             k1_smem_bytes(W, dm_mode, n_cols, p.stages + 1, p.smem_groups, p.filter_words, p.dm_bytes,
+                           in_place) <= k1_smem_cap())
+        ++p.stages;
+    }
+    // (measured, SF10: a distance of 2 gains 4-7% on the 4-column pipelines whose ring stays at
+    // 4 stages, and loses 3-6% on 3-column ones, whose rings are deeper or whose tiles are
+    // consumed faster)
+    p.prefetch = (n_cols >= 4 && p.stages <= 4 && fact->placement != HX_PLACE_HOST_MAPPED) ? 2 : 0;
+    // L2 residency of the probe structures (north_star; PAPER.md:1016-1022 operator state in
+    // device memory): probe loads carry an evict_last hint, and the largest structure K1 reads
+    // from L2 (a direct map not staged in shared memory, or a hash table's slots) gets a
+    // persisting access-policy window. HX_L2_HINT=0 / hx_ctx_set_option(HX_OPT_L2_PERSIST, 0):
+    // A/B switches.
+    p.l2_hint = 1;
+    if (const char* e = std::getenv("HX_L2_HINT")) p.l2_hint = std::atoi(e) != 0;
+    if (ctx->l2_persist && ctx->l2_persist_max > 0) {
+      for (int j = 0; j < sh->n_joins; ++j) {
+        const JoinDev& d = p.joins[j];
+        const hx_ht* ht = hts[sh->join_ht[j]];
+        void* base = nullptr;
+        size_t bytes = 0;
+        if (d.dm) {
+          if (d.dm_smem < 0 && (((p.m_l2 | p.m_l2s) >> j) & 1u)) {
+            base = const_cast<uint32_t*>(d.dm);
+            bytes = (size_t)d.dm_words * 4;
+          }
+        } else {
+          int lg = ht->max_log2cap;
+          if (ht->known_keys >= 0) {
+            lg = kMinLog2Cap;
+            while (lg < ht->max_log2cap && (int64_t(1) << lg) < 4 * ht->known_keys) ++lg;
+          }
+          base = ht->slots;
+          bytes = (size_t(1) << lg) * 8;
+        }
+        if (bytes > k.win.bytes) {
+          k.win.base = base;
+          k.win.bytes = std::min<size_t>(bytes, (size_t)ctx->l2_window_max);
+        }
+      }
+      if (k.win.bytes)
+        k.win.hit_ratio = (float)std::min(1.0, (double)ctx->l2_persist_max / (double)k.win.bytes);
+    }
+    if (const char* e = std::getenv("HX_K1_PREFETCH")) p.prefetch = std::max(0, std::min(64, std::atoi(e)));
+    if (std::getenv("HX_DEBUG")) {  // launch plan of this K1 (tuning aid)
+      std::fprintf(stderr, "[hx] K1 warps=%d joins=%d cols=%d gather=%d%d stages=%d groups=%d filters:",
+                   W, sh->n_joins, n_cols, p.ga, p.gb, p.stages, p.smem_groups);
+      for (int j = 0; j < sh->n_joins; ++j) std::fprintf(stderr, " %d", p.joins[j].bloom_words);
+      std::fprintf(stderr, " dm(words@smem/bitmap@smem):");
+      for (int j = 0; j < sh->n_joins; ++j)
+        std::fprintf(stderr, " %d@%d/%d@%d", p.joins[j].dm ? p.joins[j].dm_words : 0,
+                     p.joins[j].dm_smem, p.joins[j].bm_words, p.joins[j].bm_smem);
+      std::fprintf(stderr, " in_s:");
+      for (int j = 0; j < sh->n_joins; ++j) std::fprintf(stderr, "%d", p.joins[j].in_s);
+      std::fprintf(stderr, " l2:%x l2s:%x cost=%.2f stages=%d smem=%zu\n", p.m_l2, p.m_l2s, plan_cost, p.stages,
+                   k1_smem_bytes(W, dm_mode, n_cols, p.stages, p.smem_groups, p.filter_words, p.dm_bytes,
+                                 in_place));
+    }
+    k.fn = pick_kernel(sh->n_joins, grouped, p.m_dm != 0u, W);
+    k.smem = k1_smem_bytes(W, dm_mode, n_cols, p.stages, p.smem_groups, p.filter_words, p.dm_bytes,
+                           in_place);
+    // the smallest shared-memory carveout that holds the plan: the rest of the SM's L1/shared
+    // array caches the maps read from L2
+    k.carveout = (int)std::min<size_t>(100, ((k.smem + 1024) * 100 + 228 * 1024 - 1) / (228 * 1024));
+    k.warps = W;
+    k.cost = plan_cost;
+  };
+  K1Prepared k_lo = k, k_hi = k;
+  plan_with(kWarpsLo, k_lo);
+  plan_with(kWarpsHi, k_hi);
+  // more warps unless the plan they leave room for is costlier by more than kWarpsTol (the
+  // cost model's per-row issue cost; tolerance measured) or the ring is shallower
+  double tol = 1.10;
+  if (const char* e = std::getenv("HX_K1_W_TOL")) tol = std::atof(e);
+  bool hi = k_hi.p.stages >= std::min(k_lo.p.stages, 4) &&
+            (dm_mode ? k_hi.cost <= k_lo.cost * tol + 1e-9
+                     : k_hi.p.filter_words >= k_lo.p.filter_words);
+  // (an L2-lookup-bound plan runs with a reduced carveout so that L1 caches its map reads:
+  // the extra warps' queues take from that L1 and their misses thrash it — SF1000 Q4.1
+  // measured 6.16 ms with 26 warps vs 4.11 with 20, same plan)
+  if (dm_mode && k_lo.cost > kL1BoundCost) hi = false;
+  if (const char* e = std::getenv("HX_K1_W")) hi = std::atoi(e) == kWarpsHi;
+  k = hi ? k_hi : k_lo;
+  t_smem_cap = 0;
   int occ = 0;
-  HX_CK(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, k.fn, kThreads, k.smem));
+  HX_CK(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, k.fn, k1_threads(k.warps), k.smem));
   occ = std::max(1, occ);
   k.occ = occ;
   k.grid = (int)std::max<int64_t>(1, std::min<int64_t>(p.n_tiles, (int64_t)ctx->n_sms * occ));
@@ -2055,7 +2131,7 @@ static int k1_enqueue_host(hx_ctx* ctx, const K1Prepared* k, StageRing* ring, cu
     p.n_rows = rows;
     p.n_tiles = (rows + kTileRows - 1) / kTileRows;
     const int grid = (int)std::max<int64_t>(1, std::min<int64_t>(p.n_tiles, (int64_t)ctx->n_sms * k->occ));
-    HX_CK(launch_k1(k->fn, grid, kThreads, k->smem, ctx->stream, p, ctx->k1_priority));
+    HX_CK(launch_k1(k->fn, grid, k1_threads(k->warps), k->smem, ctx->stream, p, ctx->k1_priority));
     ctx->launches += 1;
     HX_CK(cudaEventRecord(ring->freed[s], ctx->stream));
   }
@@ -2106,7 +2182,7 @@ int k1_enqueue(hx_ctx* ctx, const K1Prepared* k, bool fresh, cudaEvent_t e0, cud
       q.n_rows = std::min<int64_t>(k->seg_rows, p.n_rows - s0);
       q.n_tiles = (q.n_rows + kTileRows - 1) / kTileRows;
       const int grid = (int)std::max<int64_t>(1, std::min<int64_t>(q.n_tiles, (int64_t)k->grid));
-      HX_CK(launch_k1(k->fn, grid, kThreads, k->smem, ctx->stream, q, ctx->k1_priority, k->carveout,
+      HX_CK(launch_k1(k->fn, grid, k1_threads(k->warps), k->smem, ctx->stream, q, ctx->k1_priority, k->carveout,
                       &k->win));
       ctx->launches += 1;
     }
