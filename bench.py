@@ -394,6 +394,82 @@ def run_micro(args, world, rank, local, ctx, stream, torch, dist, hx):
     build.close()
 
 
+def run_sizeup(args, world, rank, local, ctx, stream, torch, dist, hx):
+    """--workload sum|join --sizeup: the §6.4 size-up sweep (Fig. 8):
+    the same prepared plan over the first 0.125 ... 16 GB of the column(s), one JSON line per
+    size. Reported beside rows/s: the step's fixed part (step - K1: graph launch, builds,
+    merge, finalize, D2H) and the overhead against the ideal scan at the read-stream ceiling
+    (the paper: <= 10% above 512 MB, up to 50% at 64 MB for its GPU sum)."""
+    from paper_journals_pvldb_chrysogeloskaa19_b200 import micro
+    sizes_gb = [0.125, 0.25, 0.5, 1, 2, 4, 8, 16]
+    n_max = int(sizes_gb[-1] * 1e9) // 4
+    sz = ssbgen.micro_sizes(n_max * world, ssbgen.MICRO_PAPER_BUILD)
+    C = ssbgen.COLS
+    keep = []
+
+    def gen(c, row_begin, n):
+        t = torch.empty(max(n, 1), dtype=torch.int32, device="cuda")
+        ssbgen.column_device(SEED, sz, c, t.data_ptr(), row_begin, n, stream.cuda_stream)
+        keep.append(t)
+        return t
+
+    cols = ["mb_value"] if args.workload == "sum" else ["mb_value", "mb_probekey"]
+    full = {c: gen(c, rank * n_max, n_max) for c in cols}
+    bt = gen("mb_buildkey", 0, sz["n_part"])
+    build = hx.load_columns(ctx, [(C["mb_buildkey"], bt.data_ptr(), sz["n_part"])],
+                            placement=hx._hx.HX_PLACE_VIEW)
+    torch.cuda.synchronize()
+    peak, _ = peaks()
+    read_ceiling = 7100.0  # GB/s, tools/stream_roofline.cu (DESIGN.md 7)
+    for gb in sizes_gb:
+        n = (int(gb * 1e9) // 4) & ~3
+        fact = hx.load_columns(ctx, [(C[c], full[c].data_ptr(), n) for c in cols],
+                               placement=hx._hx.HX_PLACE_VIEW)
+        eng = micro.MicroEngine(ctx, fact, build)
+        plan = eng.plan_sum() if args.workload == "sum" else eng.plan_join()
+        graph = hx.capture(ctx, lambda: hx.plans_enqueue(ctx, [plan]))
+        for _ in range(max(3, args.warmup)):
+            graph.launch()
+            eng.plan_value(plan, args.workload)
+        if world > 1:
+            dist.barrier()
+        torch.cuda.synchronize()
+        evs = [torch.cuda.Event(enable_timing=True) for _ in range(args.steps + 1)]
+        k1 = 0.0
+        evs[0].record(stream)
+        for i in range(args.steps):
+            graph.launch()
+            evs[i + 1].record(stream)
+            eng.plan_value(plan, args.workload)
+            k1 += plan.k1_time()[0]
+        torch.cuda.synchronize()
+        steps = sorted(a.elapsed_time(b) for a, b in zip(evs, evs[1:]))
+        ms = steps[len(steps) // 2]
+        if world > 1:
+            t = torch.tensor([ms], device="cuda", dtype=torch.float64)
+            dist.all_reduce(t, op=dist.ReduceOp.MAX)
+            ms = float(t[0])
+        k1_ms = k1 / args.steps
+        bytes_ = n * 4 * len(cols)
+        ideal_ms = bytes_ / (read_ceiling * 1e9) * 1e3
+        if rank == 0:
+            print(json.dumps({
+                "metric": f"micro-benchmark size-up ({args.workload})", "size_gb_per_column": gb,
+                "fact_rows_per_gpu": n, "n_gpus": world, "steps": args.steps,
+                "ms_per_step_median": ms, "k1_ms": k1_ms, "fixed_ms": ms - k1_ms,
+                "value": n * world / (ms / 1e3), "unit": "fact rows/s",
+                "gbps_step": bytes_ / (ms / 1e3) / 1e9, "gbps_k1": bytes_ / (k1_ms / 1e3) / 1e9,
+                "frac_of_peak_step": bytes_ / (ms / 1e3) / 1e9 / peak,
+                "overhead_vs_ideal_scan": ms / ideal_ms - 1.0,
+                "ideal_definition": f"bytes / {read_ceiling:.0f} GB/s read-stream ceiling",
+                "step": "one CUDA graph launch of the prepared plan (builds + K1 + merge + "
+                        "finalize + D2H) + the host read of the result"}), flush=True)
+        graph.close()
+        plan.close()
+        fact.close()
+    build.close()
+
+
 def main():
     args = parse()
     how, what = launch_plan(args.gpus, os.environ, sys.argv[1:])
@@ -437,6 +513,12 @@ def main():
     elif args.force_collectives:
         os.environ["HX_FORCE_COLLECTIVES"] = "1"
         ctx.comm_init(1, 0, hx.comm_unique_id())
+    if args.workload != "ssb" and args.sizeup:
+        run_sizeup(args, world, rank, local, ctx, stream, torch, dist, hx)
+        ctx.close()
+        if world > 1:
+            dist.destroy_process_group()
+        return
     if args.workload != "ssb":
         run_micro(args, world, rank, local, ctx, stream, torch, dist, hx)
         ctx.close()

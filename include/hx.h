@@ -271,6 +271,21 @@ int hx_pipeline_probe_agg_into(hx_ctx* ctx, const hx_table* fact, const hx_query
 int hx_merge_aggregates(hx_ctx* ctx, hx_agg* agg, int root, int64_t* sums, int64_t* counts,
                         int32_t* keys, int64_t cap, int64_t* n_rows);
 int hx_agg_free(hx_agg* agg);
+/* The union router's group layout and the host finalize, callable without a GPU (host
+   logic only; the multi-rank CPU tests use them with a gloo all-reduce in place of NCCL).
+   hx_group_layout: a group of rank tuple (r_0 .. r_{n-1}) over n_gdims grouping dimensions
+   with n_ranks[g] dense ranks each (>= 1) sits at index sum_g r_g * strides[g], strides[n-1]
+   = 1, strides[g] = strides[g+1] * n_ranks[g+1]; *n_groups = prod n_ranks (1 for n_gdims 0).
+   This is the layout K1 accumulates into (k1_prepare) and the merge reduces: {sums[n_groups],
+   counts[n_groups]}, 2 * n_groups int64 per rank. HX_ECAPACITY above HX_MAX_GROUPS.
+   hx_group_decode (a7): from merged sums/counts in that layout and each grouping dimension's
+   rank -> code map (rank_to_code[g][r], caller-owned), writes the groups with count > 0 (an
+   ungrouped query: its one row) in index order: keys[i * n_gdims + g], out_sums[i],
+   out_counts[i]; at most `cap` rows; *n_rows = rows produced (HX_ECAPACITY if > cap). */
+int hx_group_layout(int n_gdims, const int32_t* n_ranks, int64_t* strides, int64_t* n_groups);
+int hx_group_decode(int n_gdims, const int32_t* n_ranks, const int32_t* const* rank_to_code,
+                    const int64_t* sums, const int64_t* counts, int64_t n_groups, int32_t* keys,
+                    int64_t* out_sums, int64_t* out_counts, int64_t cap, int64_t* n_rows);
 
 /* ---- prepared plans and CUDA graphs (the native runtime around K1/K2) ----------------
  * PAPER.md:769-790 §4.1 (pipelines are generated and compiled once per query, then run),

@@ -620,27 +620,65 @@ int hx_merge_aggregates(hx_ctx* ctx, hx_agg* agg, int root, int64_t* sums, int64
   ctx->d2h_bytes += (int64_t)sizeof(m) + 16 * ng;
   for (int g = 0; g < agg->n_gdims; ++g) ctx->d2h_bytes += 4 * (int64_t)r2c[g].size();
   // finalize (a7): drop empty groups (an ungrouped query keeps its one row), decode codes
-  int64_t rows = 0;
-  for (int64_t i = 0; i < ng; ++i) {
-    if (agg->n_gdims > 0 && hc[i] == 0) continue;
-    if (rows < cap) {
-      sums[rows] = hs[i];
-      counts[rows] = hc[i];
-      int64_t rem = i;
-      for (int g = agg->n_gdims - 1; g >= 0; --g) {
-        const int64_t nr = std::max(1, m.n_ranks[g]);
-        keys[rows * agg->n_gdims + g] = r2c[g][rem % nr];
-        rem /= nr;
-      }
-    }
-    ++rows;
+  int32_t nrk[HX_MAX_GDIMS];
+  const int32_t* maps[HX_MAX_GDIMS];
+  for (int g = 0; g < agg->n_gdims; ++g) {
+    nrk[g] = std::max(1, m.n_ranks[g]);
+    maps[g] = r2c[g].data();
   }
+  int64_t rows = 0;
   if (agg->n_gdims == 0 && ng == 0) {  // unreachable (n_groups >= 1), kept for safety
     if (cap > 0) sums[0] = counts[0] = 0;
     rows = 1;
+  } else {
+    const int rc = hx_group_decode(agg->n_gdims, nrk, maps, hs.data(), hc.data(), ng, keys, sums,
+                                   counts, cap, &rows);
+    if (rc != HX_OK && rc != HX_ECAPACITY) return rc;
   }
   *n_rows = rows;
   if (rows > cap) return fail(HX_ECAPACITY, "hx_merge_aggregates: output buffer too small");
+  return HX_OK;
+}
+
+int hx_group_layout(int n_gdims, const int32_t* n_ranks, int64_t* strides, int64_t* n_groups) {
+  HX_REQUIRE(n_gdims >= 0 && n_gdims <= HX_MAX_GDIMS && n_groups && (n_gdims == 0 || (n_ranks && strides)),
+             HX_EINVAL, "hx_group_layout: bad argument");
+  int64_t stride = 1;
+  for (int g = n_gdims - 1; g >= 0; --g) {
+    HX_REQUIRE(n_ranks[g] >= 1, HX_EINVAL, "hx_group_layout: a dimension needs >= 1 rank");
+    strides[g] = stride;
+    stride *= n_ranks[g];
+    HX_REQUIRE(stride <= HX_MAX_GROUPS, HX_ECAPACITY, "hx_group_layout: too many groups");
+  }
+  *n_groups = stride;
+  return HX_OK;
+}
+
+int hx_group_decode(int n_gdims, const int32_t* n_ranks, const int32_t* const* rank_to_code,
+                    const int64_t* sums, const int64_t* counts, int64_t n_groups, int32_t* keys,
+                    int64_t* out_sums, int64_t* out_counts, int64_t cap, int64_t* n_rows) {
+  HX_REQUIRE(n_rows && n_groups >= 0 && (n_groups == 0 || (sums && counts)) && cap >= 0 &&
+                 (cap == 0 || (out_sums && out_counts && (n_gdims == 0 || keys))),
+             HX_EINVAL, "hx_group_decode: bad argument");
+  int64_t strides[HX_MAX_GDIMS], ng = 0;
+  const int rc = hx_group_layout(n_gdims, n_ranks, strides, &ng);
+  if (rc != HX_OK) return rc;
+  HX_REQUIRE(ng == n_groups, HX_EINVAL, "hx_group_decode: n_groups differs from the layout");
+  for (int g = 0; g < n_gdims; ++g)
+    HX_REQUIRE(rank_to_code && rank_to_code[g], HX_EINVAL, "hx_group_decode: missing rank map");
+  int64_t rows = 0;
+  for (int64_t i = 0; i < n_groups; ++i) {
+    if (n_gdims > 0 && counts[i] == 0) continue;
+    if (rows < cap) {
+      out_sums[rows] = sums[i];
+      out_counts[rows] = counts[i];
+      for (int g = 0; g < n_gdims; ++g)
+        keys[rows * n_gdims + g] = rank_to_code[g][(i / strides[g]) % n_ranks[g]];
+    }
+    ++rows;
+  }
+  *n_rows = rows;
+  if (rows > cap) return fail(HX_ECAPACITY, "hx_group_decode: output buffer too small");
   return HX_OK;
 }
 

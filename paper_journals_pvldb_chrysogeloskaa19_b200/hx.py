@@ -447,3 +447,36 @@ def merge_aggregates(ctx: Context, agg: Agg, root: int = -1, cap: int = 4096):
             raise _hx.HxError(rc, "hx_merge_aggregates", _hx.lib().hx_last_error().decode())
         k = n.value
         return keys[: k * agg.n_gdims].reshape(k, agg.n_gdims), sums[:k], cnts[:k]
+
+
+# ---- the union router's group layout and host finalize (no GPU needed) --------------------
+def group_layout(n_ranks: Sequence[int]) -> Tuple[List[int], int]:
+    """hx_group_layout: (strides per grouping dimension, n_groups)."""
+    n = len(n_ranks)
+    nr = (ctypes.c_int32 * max(1, n))(*n_ranks)
+    st = (ctypes.c_int64 * max(1, n))()
+    ng = ctypes.c_int64()
+    call("hx_group_layout", n, nr, st, ctypes.byref(ng))
+    return list(st)[:n], ng.value
+
+
+def group_decode(n_ranks: Sequence[int], rank_to_code: Sequence[Sequence[int]],
+                 sums: np.ndarray, counts: np.ndarray):
+    """hx_group_decode: (keys [rows x n_gdims] int32, sums int64, counts int64)."""
+    n = len(n_ranks)
+    nr = (ctypes.c_int32 * max(1, n))(*n_ranks)
+    maps = [np.ascontiguousarray(m, dtype=np.int32) for m in rank_to_code]
+    mp = (ctypes.POINTER(ctypes.c_int32) * max(1, n))(
+        *[m.ctypes.data_as(ctypes.POINTER(ctypes.c_int32)) for m in maps])
+    s = np.ascontiguousarray(sums, dtype=np.int64)
+    c = np.ascontiguousarray(counts, dtype=np.int64)
+    cap = max(1, len(s))
+    keys = np.zeros((cap, max(1, n)), dtype=np.int32)
+    os_, oc = np.zeros(cap, dtype=np.int64), np.zeros(cap, dtype=np.int64)
+    rows = ctypes.c_int64()
+    P64 = ctypes.POINTER(ctypes.c_int64)
+    call("hx_group_decode", n, nr, mp, s.ctypes.data_as(P64), c.ctypes.data_as(P64), len(s),
+         keys.ctypes.data_as(ctypes.POINTER(ctypes.c_int32)), os_.ctypes.data_as(P64),
+         oc.ctypes.data_as(P64), cap, ctypes.byref(rows))
+    r = rows.value
+    return keys[:r, :n], os_[:r], oc[:r]

@@ -229,12 +229,17 @@ class SsbEngine:
         dparts.close()
         return rows
 
-    def run_hash_routed(self, q: str, dim: str, root: int = -1) -> List[Tuple]:
+    def run_hash_routed(self, q: str, dim: str, root: int = -1,
+                        dim_local: Optional[hx.Table] = None) -> List[Tuple]:
         """The multi-GPU form: every rank hash-packs its lineorder rows into nranks parts and
         the hash-routing exchange (hx_exchange_partitions, NCCL send/recv over NVLink) gives
-        rank r part r of everyone's rows; rank r joins them with part r of the (replicated)
-        dimension (identity ranks; the other dimensions broadcast), and the union router
-        merges the partials (allreduce). With one rank: a copy of itself."""
+        rank r part r of everyone's rows; rank r joins them with part r of the dimension
+        (identity ranks; the other dimensions broadcast), and the union router merges the
+        partials (allreduce). With one rank: a copy of itself.
+        The dimension is replicated (self.dims[dim]: part r is taken locally) unless
+        `dim_local` gives this rank's share of a PARTITIONED dimension (each row on exactly
+        one rank): then it is hash-packed and exchanged too, both inputs of the join going
+        through the hash-routing router (Fig. 1d/e)."""
         plan = PLANS[q]
         j = self._join_of(plan, dim)
         fk, b = plan.joins[j]
@@ -242,11 +247,15 @@ class SsbEngine:
         fparts, foffs = hx.hash_partition(self.ctx, self.fact, C[fk], nr)
         f_in = hx.exchange_partitions(self.ctx, fparts, foffs)
         fparts.close()
-        # the dimension tables are replicated on every GPU (§8(a) a1), so rank r's part of the
-        # dimension is already local: hash-pack it and keep part r (exchanging it too would
-        # deliver nranks copies of every key)
-        dparts, doffs = hx.hash_partition(self.ctx, self.dims[dim], C[b.key], nr)
-        d_in = dparts.slice(doffs[rank], doffs[rank + 1])
+        if dim_local is None:
+            # a replicated dimension (§8(a) a1): rank r's part is already local — hash-pack
+            # it and keep part r (exchanging it would deliver nranks copies of every key)
+            dparts, doffs = hx.hash_partition(self.ctx, self.dims[dim], C[b.key], nr)
+            d_in = dparts.slice(doffs[rank], doffs[rank + 1])
+        else:
+            # a partitioned dimension: its rows hashed to part p go to rank p
+            dparts, doffs = hx.hash_partition(self.ctx, dim_local, C[b.key], nr)
+            d_in = hx.exchange_partitions(self.ctx, dparts, doffs)
         hts = [self.build(bb) if i != j else self._partitioned_build(bb, d_in)
                for i, (_, bb) in enumerate(plan.joins)]
         agg = hx.pipeline_probe_agg(self.ctx, f_in, self.shape(plan), hts)

@@ -5,7 +5,8 @@ communicator carries every data-path collective (gloo only ships the NCCL unique
   * hx_merge_aggregates allreduce (every rank) and reduce (root 0) of the 13 queries;
   * prepared plans with their per-plan allreduce, plain and replayed from a CUDA graph;
   * hx_ht_broadcast from rank 0 into tables the other ranks built with a different filter;
-  * the hash-routing exchange (NCCL send/recv) of the hash-partitioned join.
+  * the hash-routing exchange (NCCL send/recv) of the hash-partitioned join, with the
+    dimension replicated and with it partitioned across the ranks (both inputs exchanged).
 Results are compared bit-exactly with the oracle over the WHOLE table."""
 import os
 import sys
@@ -80,6 +81,12 @@ def main():
         check("ht_broadcast", eng.finish(ssb.Pending(plan, hts, agg)), q)
     for q, dim in (("q2.1", "part"), ("q3.1", "customer"), ("q4.3", "supplier")):
         check(f"hash_routed[{dim}]", eng.run_hash_routed(q, dim), q)
+        # the dimension partitioned too (rows r, r + world, ... on rank r): both inputs are
+        # hash-packed and exchanged
+        mine = {c: v[rank::world] for c, v in db[dim].items()}
+        local = hx.load_numpy(ctx, {ssbgen.COLS[c]: v for c, v in mine.items()})
+        check(f"hash_routed_partitioned[{dim}]", eng.run_hash_routed(q, dim, dim_local=local), q)
+        local.close()
     for t in list(dims.values()) + [fact]:
         t.close()
     ctx.close()

@@ -84,10 +84,18 @@ def test_no_gpu_fails_loudly():
 
 # ---- world_size 2 over gloo: router partition -> partials -> union-router merge -------------
 def _rank_main(rank, world, port, out):
+    """One rank of the union-router merge, driven through libhx's host logic: the router
+    partition (hx_router_partition) gives this rank its blocks; its partial aggregate (the
+    oracle over those rows, standing in for K1, which needs a GPU) is laid out in libhx's
+    dense group layout (hx_group_layout: {sums[n_groups], counts[n_groups]}, the 2 x n_groups
+    int64 the merge all-reduces), all-reduced over gloo in place of NCCL, and finalized by
+    libhx (hx_group_decode). The rank -> code maps come from the tables (tests/ssb_groups.py),
+    not from libhx."""
     import torch
     import torch.distributed as dist
 
     import oracle
+    from ssb_groups import rank_maps
     from ssb_tiny import tiny_db
 
     os.environ.update(MASTER_ADDR="127.0.0.1", MASTER_PORT=str(port))
@@ -96,19 +104,23 @@ def _rank_main(rank, world, port, out):
     n = len(db["lineorder"]["lo_orderdate"])
     part = hx.router_partition(n, world, 1000, _hx.HX_POLICY_ROUND_ROBIN)
     mine = [(b, e) for b, e, p in part.blocks() if p == rank]
+    assert sum(e - b for b, e in mine) == part.rows(rank)
     results = {}
-    for q in ("q2.1", "q3.1", "q4.2"):
-        partial = {}
+    for q in ("q1.1", "q2.1", "q3.1", "q4.2", "q4.3"):
+        maps = rank_maps(db, q)
+        strides, ng = hx.group_layout([len(m) for m in maps])
+        arr = torch.zeros(2 * ng, dtype=torch.int64)
         for b, e in mine:
-            for k, (s, c) in oracle.as_dict(oracle.run_query(q, db, b, e)).items():
-                s0, c0 = partial.get(k, (0, 0))
-                partial[k] = (s0 + s, c0 + c)
-        # dense group arrays over the union of keys (as the device arrays are dense)
-        keys = sorted(set().union(*[set(oracle.as_dict(oracle.run_query(q, db)).keys())]))
-        arr = torch.tensor([[partial.get(k, (0, 0))[0], partial.get(k, (0, 0))[1]] for k in keys],
-                           dtype=torch.int64)
-        dist.all_reduce(arr)  # the union router's global aggregation
-        results[q] = {k: (int(arr[i, 0]), int(arr[i, 1])) for i, k in enumerate(keys)}
+            for k, (s_, c_) in oracle.as_dict(oracle.run_query(q, db, b, e)).items():
+                i = sum(int(np.searchsorted(m, code)) * st for m, code, st in zip(maps, k, strides))
+                arr[i] += s_
+                arr[ng + i] += c_
+        dist.all_reduce(arr)  # the union router's global aggregation (NCCL on GPUs)
+        keys, sums, cnts = hx.group_decode([len(m) for m in maps], maps, arr[:ng].numpy(),
+                                           arr[ng:].numpy())
+        results[q] = {tuple(int(x) for x in keys[i]): (int(sums[i]), int(cnts[i]))
+                      for i in range(len(sums))}
+        results[q + ":elements"] = int(arr.numel())
     out.put((rank, results))
     dist.destroy_process_group()
 
@@ -135,11 +147,18 @@ def test_two_rank_partition_merge_gloo():
     for p in procs:
         p.join(timeout=60)
         assert p.exitcode == 0
+    from ssb_groups import n_groups
     db = tiny_db(17, n_lo=12007)
     for rank, res in got:
         for qq, merged in res.items():
+            if qq.endswith(":elements"):  # the merge moves 2 x n_groups int64 per rank
+                assert merged == 2 * n_groups(db, qq.split(":")[0]), (rank, qq)
+                continue
             want = oracle.as_dict(oracle.run_query(qq, db))
-            assert {k: v for k, v in merged.items() if v[1] > 0} == want, (rank, qq)
+            if not oracle.N_KEYS[qq]:  # ungrouped: one row, also when empty
+                assert merged == want, (rank, qq)
+            else:
+                assert merged == {k: v for k, v in want.items() if v[1] > 0}, (rank, qq)
 
 
 # ---- world_size 2 over gloo: the hash-partitioned join's exchange (§8(f) NEXT-1) ----------

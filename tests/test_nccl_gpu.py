@@ -92,43 +92,28 @@ def test_hash_routing_exchange(nctx, db):
         assert eng.run_hash_routed(q, dim) == oracle.run_query(q, db), (q, dim)
 
 
+def test_hash_routing_exchange_partitioned_dimension(nctx, db):
+    """Both join inputs through the hash-routing router: the dimension is NOT replicated for
+    the routed join (dim_local = this rank's rows, here all of them), so it is hash-packed
+    and exchanged like lineorder."""
+    dims, fact = ssb.load_db_numpy(nctx, db)
+    eng = ssb.SsbEngine(nctx, dims, fact)
+    for q, dim in (("q2.1", "part"), ("q3.1", "customer"), ("q4.3", "supplier"), ("q4.1", "date")):
+        local = hx.load_numpy(nctx, {ssbgen.COLS[c]: v for c, v in db[dim].items()})
+        nctx.comm_trace(reset=True)
+        assert eng.run_hash_routed(q, dim, dim_local=local) == oracle.run_query(q, db), (q, dim)
+        ops = [r["op"] for r in nctx.comm_trace(reset=True)]
+        assert ops.count("allgather") == 2, ops  # lineorder's and the dimension's part sizes
+        local.close()
+
+
 # ---- the sizes of the collectives, from the collective trace (hx_comm_trace) ----------------
 # A 1-rank allreduce / broadcast is an identity whatever its count, so the counts libhx
 # issues are checked here against values computed independently from the generated tables
 # with numpy, following the query texts (SURVEY.md 8(c)): a grouping dimension contributes the
 # number of distinct group codes among its rows that pass the dimension's filter (the dense
 # ranks, DESIGN.md R17), and the group array is their product.
-AMERICA, ASIA, US, KI = 1, 2, 23, (221, 225)
-
-
-def _groups(db, q):
-    d, c, s, p = db["date"], db["customer"], db["supplier"], db["part"]
-    year = d["d_year"]
-    y9297 = (year >= 1992) & (year <= 1997)
-    y9798 = (year == 1997) | (year == 1998)
-    brand, cat = p["p_brand1"], p["p_category"]
-    spec = {
-        "q1.1": [], "q1.2": [], "q1.3": [],
-        "q2.1": [(year, year == year), (brand, cat == 1)],
-        "q2.2": [(year, year == year), (brand, (brand >= 260) & (brand <= 267))],
-        "q2.3": [(year, year == year), (brand, brand == 278)],
-        "q3.1": [(c["c_nation"], c["c_region"] == ASIA), (s["s_nation"], s["s_region"] == ASIA),
-                 (year, y9297)],
-        "q3.2": [(c["c_city"], c["c_nation"] == US), (s["s_city"], s["s_nation"] == US),
-                 (year, y9297)],
-        "q3.3": [(c["c_city"], np.isin(c["c_city"], KI)), (s["s_city"], np.isin(s["s_city"], KI)),
-                 (year, y9297)],
-        "q3.4": [(c["c_city"], np.isin(c["c_city"], KI)), (s["s_city"], np.isin(s["s_city"], KI)),
-                 (year, d["d_yearmonthnum"] == 199712)],
-        "q4.1": [(year, year == year), (c["c_nation"], c["c_region"] == AMERICA)],
-        "q4.2": [(year, y9798), (s["s_nation"], s["s_region"] == AMERICA),
-                 (cat, np.isin(p["p_mfgr"], (0, 1)))],
-        "q4.3": [(year, y9798), (s["s_city"], s["s_nation"] == US), (brand, cat == 3)],
-    }[q]
-    n = 1
-    for col, mask in spec:
-        n *= max(1, len(np.unique(col[mask])))
-    return n
+from ssb_groups import n_groups as _groups  # noqa: E402
 
 
 def test_trace_merge_counts(nctx, db):
@@ -175,9 +160,9 @@ def test_trace_ht_broadcast_sizes(nctx, db):
     dims, fact = ssb.load_db_numpy(nctx, db)
     eng = ssb.SsbEngine(nctx, dims, fact)
     c, s = db["customer"], db["supplier"]
-    cases = [("q3.1", "customer", int(np.sum(c["c_region"] == ASIA))),
-             ("q3.2", "supplier", int(np.sum(s["s_nation"] == US))),
-             ("q4.1", "customer", int(np.sum(c["c_region"] == AMERICA)))]
+    cases = [("q3.1", "customer", int(np.sum(c["c_region"] == 2))),     # ASIA
+             ("q3.2", "supplier", int(np.sum(s["s_nation"] == 23))),    # UNITED STATES
+             ("q4.1", "customer", int(np.sum(c["c_region"] == 1)))]     # AMERICA
     for q, dim, n_pass in cases:
         plan = ssb.PLANS[q]
         (b,) = [b for _, b in plan.joins if b.table == dim]
