@@ -257,6 +257,32 @@ int hx_pipeline_probe_agg(hx_ctx* ctx, const hx_table* fact, const hx_query_shap
 int hx_pipeline_probe_agg_into(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* shape,
                                hx_ht* const* hts, int n_hts, hx_agg* agg);
 
+/* ---- the router's dynamic load balancing across processes (§8(e) host-resident) --------
+ * PAPER.md:469-473 §3.1 (the router routes block handles to consumers "while load-balancing"),
+ * PAPER.md:1214-1233 §6.2 (SF1000 stays in CPU memory, streamed to the GPUs). One process per
+ * GPU: the block counter is a POSIX shared-memory segment `name` ("/word") every process of
+ * the node opens. hx_shared_router_next hands out the block indices 0 .. n_blocks-1, each
+ * exactly once over all processes (atomic fetch-add), then -1. create = 1 creates the segment
+ * (or re-initialises an existing one) with the counter at 0; create = 0 opens a segment created
+ * for the same n_blocks (HX_EINVAL otherwise). reset puts the counter back to 0 (between runs,
+ * by one process, while no other draws). close(unlink = 1) also removes the name. Host only. */
+typedef struct hx_shared_router hx_shared_router;
+int hx_shared_router_open(const char* name, int64_t n_blocks, int create, hx_shared_router** out);
+int hx_shared_router_next(hx_shared_router* r, int64_t* block);
+int hx_shared_router_reset(hx_shared_router* r);
+int hx_shared_router_close(hx_shared_router* r, int unlink_name);
+/* The host-resident pipeline fed by a shared router: `fact` is HX_PLACE_HOST_PINNED over the
+   WHOLE table (every process maps the same pinned host memory); block b is rows
+   [b * block_rows, min((b + 1) * block_rows, n_rows)). This GPU draws a block whenever one of
+   its staging-ring slots is free (the host waits for that slot's previous K1), copies it H2D
+   on the ctx's copy stream and runs K1 on it, accumulating into a NEW agg; blocks beyond the
+   table end the loop. *n_blocks = blocks this process ran. Returns once the router is
+   exhausted (the last K1s still run on the ctx stream; hx_merge_aggregates then merges over
+   the ranks). Not capturable in a CUDA graph. */
+int hx_pipeline_probe_agg_routed(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* shape,
+                                 hx_ht* const* hts, int n_hts, hx_shared_router* router,
+                                 int64_t block_rows, hx_agg** out, int64_t* n_blocks);
+
 /* ---- merge partial aggregates + finalize (§8(a) a6, a7) ----------------------------
  * PAPER.md:485-488 §3.1 (a local reduction per device, then the union router gathers the
  * partial results into one global aggregation), PAPER.md:927-936 (pipelines 8, 3 → 2).

@@ -111,6 +111,12 @@ _SIGS = {
     "hx_pipeline_probe_agg_into": ([_P, _P, ctypes.POINTER(hx_query_shape), _PP, _I, _P], _I),
     "hx_merge_aggregates": ([_P, _P, _I, _PI64, _PI64, _PI32, _I64, _PI64], _I),
     "hx_agg_free": ([_P], _I),
+    "hx_shared_router_open": ([ctypes.c_char_p, _I64, _I, _PP], _I),
+    "hx_shared_router_next": ([_P, _PI64], _I),
+    "hx_shared_router_reset": ([_P], _I),
+    "hx_shared_router_close": ([_P, _I], _I),
+    "hx_pipeline_probe_agg_routed": ([_P, _P, ctypes.POINTER(hx_query_shape), _PP, _I, _P, _I64, _PP,
+                                      _PI64], _I),
     "hx_group_layout": ([_I, _PI32, _PI64, _PI64], _I),
     "hx_group_decode": ([_I, _PI32, ctypes.POINTER(_PI32), _PI64, _PI64, _I64, _PI32, _PI64, _PI64,
                          _I64, _PI64], _I),

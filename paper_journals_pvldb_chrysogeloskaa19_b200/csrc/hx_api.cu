@@ -541,6 +541,23 @@ int hx_pipeline_probe_agg_into(hx_ctx* ctx, const hx_table* fact, const hx_query
   return probe_agg(ctx, fact, shape, hts, n_hts, agg, false);
 }
 
+int hx_pipeline_probe_agg_routed(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* shape,
+                                 hx_ht* const* hts, int n_hts, hx_shared_router* router,
+                                 int64_t block_rows, hx_agg** out, int64_t* n_blocks) {
+  HX_REQUIRE(ctx && out, HX_EINVAL, "hx_pipeline_probe_agg_routed: null argument");
+  HX_CK(cudaSetDevice(ctx->device));
+  hx_agg* agg = new hx_agg();
+  agg->ctx = ctx;
+  int rc = probe_agg_routed(ctx, fact, shape, hts, n_hts, agg, router, block_rows, n_blocks);
+  if (rc != HX_OK) {
+    if (agg->base) cudaFreeAsync(agg->base, ctx->stream);
+    delete agg;
+    return rc;
+  }
+  *out = agg;
+  return HX_OK;
+}
+
 // ---- union-router merge + finalize ------------------------------------------------------------
 int hx_merge_aggregates(hx_ctx* ctx, hx_agg* agg, int root, int64_t* sums, int64_t* counts,
                         int32_t* keys, int64_t cap, int64_t* n_rows) {

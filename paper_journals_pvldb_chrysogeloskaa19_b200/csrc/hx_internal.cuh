@@ -257,6 +257,10 @@ int ht_enable_direct(hx_ctx* ctx, hx_ht* ht, int32_t kmin, uint32_t span, int lw
 int probe_agg(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* shape,
               hx_ht* const* hts, int n_hts, hx_agg* agg, bool fresh);
 int k1_occupancy(hx_ctx* ctx);
+// host-resident K1 over the blocks a shared router hands out (hx_pipeline_probe_agg_routed)
+int probe_agg_routed(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht* const* hts,
+                     int n_hts, hx_agg* agg, hx_shared_router* router, int64_t block_rows,
+                     int64_t* n_blocks);
 struct K1Prepared;  // a resolved K1 launch (hx_probe.cu)
 long long k1_group_bound(const hx_query_shape* sh, hx_ht* const* hts, int n_hts);
 int agg_alloc(hx_ctx* ctx, hx_agg* agg, long long cap_groups, const hx_query_shape* sh,

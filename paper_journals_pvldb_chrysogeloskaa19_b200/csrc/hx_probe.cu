@@ -2142,6 +2142,77 @@ static int k1_enqueue_host(hx_ctx* ctx, const K1Prepared* k, StageRing* ring, cu
   return HX_OK;
 }
 
+// K1 over a host-resident fact table whose blocks are handed out by a shared router (dynamic
+// load balancing across the processes of a node): the host draws a block only when a staging
+// slot is free (it waits for the slot's previous K1 with cudaEventSynchronize), so each GPU
+// takes blocks at the rate it consumes them. Not capturable (host-driven).
+int k1_enqueue_routed(hx_ctx* ctx, const K1Prepared* k, StageRing* ring, hx_shared_router* router,
+                      int64_t* n_blocks) {
+  HX_REQUIRE(ring && ring->n_cols == k->n_cols && k->host, HX_EINVAL,
+             "routed K1 needs a host-resident table and a staging ring");
+  const int64_t B = ring->block_rows;
+  int64_t mine = 0;
+  HX_CK(cudaEventRecord(ctx->fork_ev, ctx->stream));
+  HX_CK(cudaStreamWaitEvent(ctx->copy_stream, ctx->fork_ev, 0));
+  for (int64_t used = 0;; ++used) {
+    const int s = (int)(used % kRingStages);
+    if (used >= kRingStages) HX_CK(cudaEventSynchronize(ring->freed[s]));  // slot free: ask for work
+    int64_t b = -1;
+    int rc = hx_shared_router_next(router, &b);
+    if (rc != HX_OK) return rc;
+    const int64_t r0 = b * B;
+    if (b < 0 || r0 >= k->rows) break;
+    const int64_t rows = std::min<int64_t>(B, k->rows - r0);
+    if (used >= kRingStages) HX_CK(cudaStreamWaitEvent(ctx->copy_stream, ring->freed[s], 0));
+    for (int c = 0; c < k->n_cols; ++c)
+      HX_CK(cudaMemcpyAsync(ring->buf[s][c], k->host_col[c] + r0, (size_t)rows * 4,
+                            cudaMemcpyHostToDevice, ctx->copy_stream));
+    ctx->h2d_bytes += rows * 4 * k->n_cols;
+    HX_CK(cudaEventRecord(ring->full[s], ctx->copy_stream));
+    HX_CK(cudaStreamWaitEvent(ctx->stream, ring->full[s], 0));
+    K1Params p = k->p;
+    for (int c = 0; c < k->n_cols; ++c) p.col[c] = p.head_col[c] = ring->buf[s][c];
+    p.head_rows = 0;
+    p.n_rows = rows;
+    p.n_tiles = (rows + kTileRows - 1) / kTileRows;
+    const int grid = (int)std::max<int64_t>(1, std::min<int64_t>(p.n_tiles, (int64_t)ctx->n_sms * k->occ));
+    HX_CK(launch_k1(k->fn, grid, k1_threads(k->warps), k->smem, ctx->stream, p, ctx->k1_priority));
+    ctx->launches += 1;
+    HX_CK(cudaEventRecord(ring->freed[s], ctx->stream));
+    ++mine;
+  }
+  HX_CK(cudaEventRecord(ctx->fork_ev, ctx->copy_stream));
+  HX_CK(cudaStreamWaitEvent(ctx->stream, ctx->fork_ev, 0));
+  if (n_blocks) *n_blocks = mine;
+  return HX_OK;
+}
+
+int probe_agg_routed(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht* const* hts,
+                     int n_hts, hx_agg* agg, hx_shared_router* router, int64_t block_rows,
+                     int64_t* n_blocks) {
+  HX_REQUIRE(ctx && fact && sh && agg && router, HX_EINVAL, "hx_pipeline_probe_agg_routed: null argument");
+  HX_REQUIRE(fact->placement == HX_PLACE_HOST_PINNED, HX_EINVAL,
+             "hx_pipeline_probe_agg_routed: the fact table must be HX_PLACE_HOST_PINNED");
+  HX_REQUIRE(block_rows > 0 && block_rows % 4 == 0, HX_EINVAL,
+             "hx_pipeline_probe_agg_routed: block_rows must be a positive multiple of 4");
+  const long long bound = k1_group_bound(sh, hts, n_hts);
+  HX_REQUIRE(bound >= 1, HX_EINVAL, "hx_pipeline_probe_agg_routed: bad gdim_join / join_ht");
+  int rc = agg_alloc(ctx, agg, bound, sh, hts);
+  if (rc != HX_OK) return rc;
+  K1Prepared* k = nullptr;
+  rc = k1_setup(ctx, fact, sh, hts, n_hts, agg, &k);
+  if (rc != HX_OK) return rc;
+  for (int j = 0; j < sh->n_joins; ++j) agg->deps.push_back(hts[sh->join_ht[j]]);
+  StageRing* ring = nullptr;
+  rc = k1_enqueue_prepare(ctx, k, true, ctx->stream);
+  if (rc == HX_OK && k->rows > 0) rc = ring_create(ctx, k, block_rows, &ring);
+  if (rc == HX_OK && k->rows > 0) rc = k1_enqueue_routed(ctx, k, ring, router, n_blocks);
+  else if (n_blocks) *n_blocks = 0;
+  ring_destroy(ctx, ring);
+  k1_free(k);
+  return rc;
+}
+
 // prepare (group layout + zeroing when `fresh`) then K1; optional timing events around K1.
 int k1_enqueue_prepare(hx_ctx* ctx, const K1Prepared* k, bool fresh, cudaStream_t s) {
   const K1Params& p = k->p;

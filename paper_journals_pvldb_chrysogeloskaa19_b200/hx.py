@@ -480,3 +480,38 @@ def group_decode(n_ranks: Sequence[int], rank_to_code: Sequence[Sequence[int]],
          oc.ctypes.data_as(P64), cap, ctypes.byref(rows))
     r = rows.value
     return keys[:r, :n], os_[:r], oc[:r]
+
+
+# ---- the router's dynamic load balancing across processes (hx_shared_router_*) --------------
+class SharedRouter:
+    """A block counter in POSIX shared memory drawn from by every process of the node."""
+
+    def __init__(self, name: str, n_blocks: int, create: bool):
+        h = ctypes.c_void_p()
+        call("hx_shared_router_open", name.encode(), n_blocks, 1 if create else 0, ctypes.byref(h))
+        self.h, self.name, self.n_blocks = h, name, n_blocks
+
+    def next(self) -> int:
+        b = ctypes.c_int64()
+        call("hx_shared_router_next", self.h, ctypes.byref(b))
+        return b.value
+
+    def reset(self) -> None:
+        call("hx_shared_router_reset", self.h)
+
+    def close(self, unlink: bool = False) -> None:
+        if self.h:
+            call("hx_shared_router_close", self.h, 1 if unlink else 0)
+            self.h = None
+
+
+def pipeline_probe_agg_routed(ctx: Context, fact: Table, shape: hx_query_shape,
+                              hts: Sequence[HashTable], router: SharedRouter,
+                              block_rows: int) -> Tuple["Agg", int]:
+    """hx_pipeline_probe_agg_routed -> (agg, blocks this process ran)."""
+    arr = _hts_array(hts)
+    h = ctypes.c_void_p()
+    nb = ctypes.c_int64()
+    call("hx_pipeline_probe_agg_routed", ctx.h, fact.h, ctypes.byref(shape), arr, len(hts),
+         router.h, block_rows, ctypes.byref(h), ctypes.byref(nb))
+    return Agg(ctx, h, shape.n_gdims, (fact, list(hts))), nb.value

@@ -229,6 +229,18 @@ class SsbEngine:
         dparts.close()
         return rows
 
+    def run_routed(self, q: str, router: hx.SharedRouter, block_rows: int,
+                   root: int = -1) -> Tuple[List[Tuple], int]:
+        """Host-resident lineorder (self.fact: HX_PLACE_HOST_PINNED over the WHOLE table)
+        streamed in the blocks a shared router hands out — every process of the node draws
+        from the same counter, so each GPU takes blocks as fast as it consumes them
+         — then the union-router merge. -> (rows, blocks this rank ran)."""
+        plan = PLANS[q]
+        hts = [self.build(b) for _, b in plan.joins]
+        agg, nb = hx.pipeline_probe_agg_routed(self.ctx, self.fact, self.shape(plan), hts, router,
+                                               block_rows)
+        return self.finish(Pending(plan, hts, agg), root), nb
+
     def run_hash_routed(self, q: str, dim: str, root: int = -1,
                         dim_local: Optional[hx.Table] = None) -> List[Tuple]:
         """The multi-GPU form: every rank hash-packs its lineorder rows into nranks parts and

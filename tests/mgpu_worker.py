@@ -6,7 +6,9 @@ communicator carries every data-path collective (gloo only ships the NCCL unique
   * prepared plans with their per-plan allreduce, plain and replayed from a CUDA graph;
   * hx_ht_broadcast from rank 0 into tables the other ranks built with a different filter;
   * the hash-routing exchange (NCCL send/recv) of the hash-partitioned join, with the
-    dimension replicated and with it partitioned across the ranks (both inputs exchanged).
+    dimension replicated and with it partitioned across the ranks (both inputs exchanged);
+  * host-resident lineorder in one shared pinned buffer, blocks drawn from a shared router
+    (dynamic load balancing across the ranks).
 Results are compared bit-exactly with the oracle over the WHOLE table."""
 import os
 import sys
@@ -87,6 +89,50 @@ def main():
         local = hx.load_numpy(ctx, {ssbgen.COLS[c]: v for c, v in mine.items()})
         check(f"hash_routed_partitioned[{dim}]", eng.run_hash_routed(q, dim, dim_local=local), q)
         local.close()
+    # host-resident lineorder in ONE shared pinned buffer (every rank maps it), blocks handed
+    # out by the shared router: each block runs on exactly one GPU, whichever drew it
+    from multiprocessing import shared_memory
+
+    import numpy as np
+    lo = db["lineorder"]
+    n = len(lo["lo_orderdate"])
+    names = list(lo)
+    shm_name = f"hx_mgpu_lo_{os.environ.get('MASTER_PORT', '0')}"
+    if rank == 0:
+        shm = shared_memory.SharedMemory(name=shm_name, create=True, size=4 * n * len(names))
+        buf = np.ndarray((len(names), n), dtype=np.int32, buffer=shm.buf)
+        for i, c in enumerate(names):
+            buf[i] = lo[c]
+        router = hx.SharedRouter(f"/{shm_name}_r", (n + 8191) // 8192, create=True)
+    dist.barrier()
+    if rank != 0:
+        shm = shared_memory.SharedMemory(name=shm_name)
+        buf = np.ndarray((len(names), n), dtype=np.int32, buffer=shm.buf)
+        router = hx.SharedRouter(f"/{shm_name}_r", (n + 8191) // 8192, create=False)
+    ptr = buf.ctypes.data
+    assert torch.cuda.cudart().cudaHostRegister(ptr, buf.nbytes, 1) == 0  # portable
+    hfact = hx.load_columns(ctx, [(ssbgen.COLS[c], ptr + 4 * n * i, n) for i, c in enumerate(names)],
+                            placement=hx._hx.HX_PLACE_HOST_PINNED)
+    heng = ssb.SsbEngine(ctx, dims, hfact)
+    for q in ("q1.1", "q2.1", "q3.1", "q4.1"):
+        if rank == 0:
+            router.reset()
+        dist.barrier()
+        rows, nb = heng.run_routed(q, router, 8192)
+        check("shared_router", rows, q)
+        tot = torch.tensor([nb], dtype=torch.int64)
+        dist.all_reduce(tot)
+        if int(tot[0]) != (n + 8191) // 8192:
+            fails.append(f"rank {rank} shared_router {q}: {int(tot[0])} blocks ran")
+        dist.barrier()
+    hfact.close()
+    torch.cuda.cudart().cudaHostUnregister(ptr)
+    router.close(unlink=(rank == 0))
+    dist.barrier()
+    del buf
+    shm.close()
+    if rank == 0:
+        shm.unlink()
     for t in list(dims.values()) + [fact]:
         t.close()
     ctx.close()

@@ -250,3 +250,54 @@ def test_two_rank_hash_partitioned_join_gloo():
     for rank, res in got:
         for qq, merged in res.items():
             assert merged == oracle.as_dict(oracle.run_query(qq, db)), (rank, qq)
+
+
+# ---- the router's dynamic load balancing across processes (hx_shared_router) ---------------
+def _router_worker(name, n_blocks, out):
+    from paper_journals_pvldb_chrysogeloskaa19_b200 import hx as hx_
+    r = hx_.SharedRouter(name, n_blocks, create=False)
+    got = []
+    while True:
+        b = r.next()
+        if b < 0:
+            break
+        got.append(b)
+    r.close()
+    out.put(got)
+
+
+def test_shared_router_hands_out_every_block_once_across_processes():
+    """Four processes draw from one counter in POSIX shared memory: the blocks they get are
+    disjoint and cover 0 .. n_blocks-1 (dynamic routing to consumers)."""
+    import multiprocessing as mp
+    name, n = f"/hx_test_router_{os.getpid()}", 20011
+    r = hx.SharedRouter(name, n, create=True)
+    ctx = mp.get_context("spawn")
+    q = ctx.Queue()
+    procs = [ctx.Process(target=_router_worker, args=(name, n, q)) for _ in range(4)]
+    for p in procs:
+        p.start()
+    parts = [q.get(timeout=120) for _ in procs]
+    for p in procs:
+        p.join(timeout=60)
+        assert p.exitcode == 0
+    allb = sorted(b for part in parts for b in part)
+    assert allb == list(range(n))
+    assert all(part == sorted(part) for part in parts)  # each draws in increasing order
+    assert r.next() == -1
+    r.reset()
+    assert r.next() == 0
+    r.close(unlink=True)
+
+
+def test_shared_router_rejects_bad_arguments():
+    with pytest.raises(_hx.HxError):
+        hx.SharedRouter("no_slash", 4, create=True)
+    name = f"/hx_test_router_b{os.getpid()}"
+    r = hx.SharedRouter(name, 8, create=True)
+    with pytest.raises(_hx.HxError) as e:
+        hx.SharedRouter(name, 9, create=False)  # created for another block count
+    assert e.value.code == _hx.HX_EINVAL
+    with pytest.raises(_hx.HxError):
+        hx.SharedRouter("/hx_test_router_missing_x", 8, create=False)
+    r.close(unlink=True)

@@ -495,3 +495,23 @@ def test_reserved_key_minus_one_rejected(ctx, table, col):
     with pytest.raises(_hx.HxError) as ei:
         eng.plan(q)
     assert ei.value.code == _hx.HX_EINVAL
+
+
+def test_host_resident_shared_router(ctx):
+    """Host-resident lineorder streamed in the blocks a shared router hands out
+    (hx_pipeline_probe_agg_routed): every block once, bit-exact."""
+    import os
+    db = ssbgen.database(21, ssbgen.sizes(0.05))  # 300 K rows
+    n = len(db["lineorder"]["lo_orderdate"])
+    pin = lambda k: torch.empty(k, dtype=torch.int32, pin_memory=True)
+    dims, fact = ssb.load_db_host_resident(ctx, db, pin)
+    eng = ssb.SsbEngine(ctx, dims, fact)
+    block = 4096 * 3 + 4  # ragged blocks; the last one partial
+    n_blocks = (n + block - 1) // block
+    r = hx.SharedRouter(f"/hx_test_routed_{os.getpid()}", n_blocks, create=True)
+    for q in ("q1.1", "q2.1", "q3.1", "q4.3"):
+        r.reset()
+        rows, nb = eng.run_routed(q, r, block)
+        assert nb == n_blocks, (q, nb)
+        assert rows == oracle.run_query(q, db), q
+    r.close(unlink=True)
