@@ -69,6 +69,11 @@ def parse(argv=None):
                          "step includes the union-router allreduce a multi-GPU step issues")
     ap.add_argument("--micro-rows", type=int, default=0,
                     help="fact rows per GPU of the micro-benchmarks (default: the paper's 23 GB)")
+    ap.add_argument("--router", default="static", choices=["static", "shared"],
+                    help="--variant host: static = each rank streams its own router blocks (plans, "
+                         "CUDA graph); shared = ONE pinned copy of lineorder in shared memory, blocks "
+                         "drawn from a shared counter by whichever GPU is free (dynamic load "
+                         "balancing, PAPER.md:469-473)")
     ap.add_argument("--sizeup", action="store_true",
                     help="with --workload sum|join: the §6.4 size-up sweep (0.125-16 GB per "
                          "column), one JSON line per size")
@@ -394,6 +399,158 @@ def run_micro(args, world, rank, local, ctx, stream, torch, dist, hx):
     build.close()
 
 
+def run_host_routed(args, world, rank, local, ctx, stream, torch, dist, hx, ssb, queries):
+    """--variant host --router shared: lineorder (the referenced columns of the whole table)
+    lives ONCE in shared pinned host memory that every rank maps (cudaHostRegister); each
+    query's blocks are drawn from a shared counter (hx_shared_router) as GPUs free a staging
+    slot — the paper's router with dynamic load balancing over the consumers (PAPER.md:469-473,
+    1214-1233) — then merged by the union router (NCCL allreduce). Not a CUDA graph (the host
+    draws blocks). value = queries x rows / step time (max over ranks)."""
+    from multiprocessing import shared_memory
+    C = ssbgen.COLS
+    sz = ssbgen.sizes(args.sf * world)
+    n = sz["n_lineorder"]
+    need = set().union(*(ssb.FACT_COLS[q] for q in queries))
+    lo_cols = [c for c in ssbgen.TABLE_COLS["lineorder"] if C[c] in need]
+    tag = os.environ.get("MASTER_PORT", str(os.getpid()))
+    shm_name = f"hx_bench_lo_{tag}"
+    if rank == 0:
+        shm = shared_memory.SharedMemory(name=shm_name, create=True, size=4 * n * len(lo_cols))
+    if world > 1:
+        dist.barrier()
+    if rank != 0:
+        shm = shared_memory.SharedMemory(name=shm_name)
+    buf = np.ndarray((len(lo_cols), n), dtype=np.int32, buffer=shm.buf)
+    if rank == 0:  # fill from the seeded generator (in HBM, copied down in pieces)
+        piece = 1 << 27
+        tmp = torch.empty(piece, dtype=torch.int32, device="cuda")
+        for i, c in enumerate(lo_cols):
+            for b in range(0, n, piece):
+                k = min(piece, n - b)
+                ssbgen.column_device(SEED, sz, c, tmp.data_ptr(), b, k, stream.cuda_stream)
+                torch.cuda.synchronize()
+                buf[i, b:b + k] = tmp[:k].cpu().numpy()
+        del tmp
+    if world > 1:
+        dist.barrier()
+    ptr = buf.ctypes.data
+    assert torch.cuda.cudart().cudaHostRegister(ptr, buf.nbytes, 1) == 0  # portable pinning
+    keep = []
+
+    def dev_table(cols, nrows):
+        spec = []
+        for c in cols:
+            t = torch.empty(max(nrows, 1), dtype=torch.int32, device="cuda")
+            ssbgen.column_device(SEED, sz, c, t.data_ptr(), 0, nrows, stream.cuda_stream)
+            keep.append(t)
+            spec.append((C[c], t.data_ptr(), nrows))
+        return hx.load_columns(ctx, spec, placement=hx._hx.HX_PLACE_VIEW)
+
+    dims = {t: dev_table(ssbgen.TABLE_COLS[t], ssbgen.table_rows(sz, ssbgen.TABLE_COLS[t][0]))
+            for t in ("date", "customer", "supplier", "part")}
+    fact = hx.load_columns(ctx, [(C[c], ptr + 4 * n * i, n) for i, c in enumerate(lo_cols)],
+                           placement=hx._hx.HX_PLACE_HOST_PINNED)
+    torch.cuda.synchronize()
+    block = 1 << 21
+    n_blocks = (n + block - 1) // block
+    rname = f"/{shm_name}_r"
+    router = hx.SharedRouter(rname, n_blocks, create=True) if rank == 0 else None
+    if world > 1:
+        dist.barrier()
+    if rank != 0:
+        router = hx.SharedRouter(rname, n_blocks, create=False)
+    eng = ssb.SsbEngine(ctx, dims, fact)
+    mine_blocks = [0]
+
+    def step():
+        for q in queries:
+            if rank == 0:
+                router.reset()
+            if world > 1:
+                dist.barrier()
+            _, nb = eng.run_routed(q, router, block)
+            mine_blocks[0] += nb
+
+    for _ in range(args.warmup):
+        step()
+    ctx.stats(reset=True)
+    mine_blocks[0] = 0
+    clocks = Clocks(local)
+    if world > 1:
+        dist.barrier()
+    torch.cuda.synchronize()
+    clocks.start()
+    e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+    e0.record(stream)
+    for _ in range(args.steps):
+        step()
+    e1.record(stream)
+    torch.cuda.synchronize()
+    if world > 1:
+        dist.barrier()
+    clk = clocks.stop()
+    ms = e0.elapsed_time(e1)
+    launches, h2d, d2h = ctx.stats(reset=True)
+    share = float(mine_blocks[0]) / max(1, args.steps * len(queries) * n_blocks)
+    if world > 1:
+        t = torch.tensor([ms, float(launches), share, share], device="cuda", dtype=torch.float64)
+        dist.all_reduce(t[:1], op=dist.ReduceOp.MAX)
+        dist.all_reduce(t[1:2], op=dist.ReduceOp.SUM)
+        dist.all_reduce(t[2:3], op=dist.ReduceOp.MIN)
+        dist.all_reduce(t[3:4], op=dist.ReduceOp.MAX)
+        ms, launches, smin, smax = float(t[0]), int(t[1]), float(t[2]), float(t[3])
+    else:
+        smin = smax = share
+    ms_step = ms / args.steps
+    value = len(queries) * n / (ms_step / 1e3)
+    # the host link's own ceiling, measured in this run (pinned H2D, 1 GiB, best of 3)
+    hb = torch.empty(1 << 28, dtype=torch.int32, pin_memory=True)
+    dbf = torch.empty(1 << 28, dtype=torch.int32, device="cuda")
+    best = 0.0
+    for _ in range(3):
+        c0, c1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+        c0.record(stream)
+        dbf.copy_(hb, non_blocking=True)
+        c1.record(stream)
+        torch.cuda.synchronize()
+        best = max(best, hb.numel() * 4 / (c0.elapsed_time(c1) / 1e3) / 1e9)
+    del hb, dbf
+    streamed = sum(4 * len(ssb.FACT_COLS[q]) * n for q in queries) / (ms_step / 1e3) / 1e9
+    if rank == 0:
+        print(json.dumps({
+            "metric": METRIC, "value": value, "unit": UNIT, "n_gpus": world, "steps": args.steps,
+            "warmup": args.warmup, "ms_per_step": ms_step, "higher_is_better": True,
+            "scaling": "weak", "vs_baseline": None, "dtype": "int32 columns, int64 accumulate",
+            "data": f"synthetic (ssbgen dbgen-shaped SSB, seed {SEED}), lineorder in shared pinned "
+                    "host memory",
+            "config": dict(config(args, world, n // world, queries), router="shared counter "
+                           "(hx_shared_router): blocks of 2^21 rows to whichever GPU frees a "
+                           "staging slot", block_rows=block, n_blocks=n_blocks),
+            "roofline": {"bound": "pcie", "achieved": streamed, "peak": best * world,
+                         "unit": "GB/s", "frac": streamed / (best * world),
+                         "peak_source": "measured in this run: pinned H2D cudaMemcpyAsync, 1 GiB, "
+                                        "best of 3, x GPUs",
+                         "kernel": "mem-move H2D ring + k1_probe_agg per drawn block",
+                         "traffic": None},
+            "load_balance": {"min_share": smin, "max_share": smax,
+                             "ideal_share": 1.0 / world},
+            "e2e": {"value": value, "unit": UNIT, "h2d_bytes_per_step": h2d // args.steps,
+                    "d2h_bytes_per_step": d2h // args.steps, "ms_per_step": ms_step,
+                    "path": "builds + hx_pipeline_probe_agg_routed + hx_merge_aggregates per query"},
+            "cpu_baseline": None, "clocks": clk, "gpu_launches": launches}), flush=True)
+    fact.close()
+    for t in dims.values():
+        t.close()
+    torch.cuda.cudart().cudaHostUnregister(ptr)
+    router.close(unlink=(rank == 0))
+    if world > 1:
+        dist.barrier()
+    del buf
+    shm.close()
+    if rank == 0:
+        shm.unlink()
+
+
 def run_sizeup(args, world, rank, local, ctx, stream, torch, dist, hx):
     """--workload sum|join --sizeup: the §6.4 size-up sweep (Fig. 8):
     the same prepared plan over the first 0.125 ... 16 GB of the column(s), one JSON line per
@@ -529,6 +686,12 @@ def main():
         queries = ["q2.1", "q3.1", "q4.1"] if args.variant in ("host", "uva") else ssb.QUERIES
     else:
         queries = args.queries.split(",")
+    if args.variant == "host" and args.router == "shared":
+        run_host_routed(args, world, rank, local, ctx, stream, torch, dist, hx, ssb, queries)
+        ctx.close()
+        if world > 1:
+            dist.destroy_process_group()
+        return
     C = ssbgen.COLS
     # only the lineorder columns the selected queries reference are placed (SF1000 on one
     # GPU: the 6 columns of Q2-Q4 = 144 GB or the 4 of Q1 = 96 GB fit HBM; all 9 do not)
