@@ -55,18 +55,15 @@ constexpr int kWarpsLo = 20, kWarpsHi = 26;
 #ifndef HX_GATHER_HINT
 #define HX_GATHER_HINT 0  // gathered measures with an L2 evict_first hint (0: plain)
 #endif
-#ifndef HX_CLAIM_AHEAD
-#define HX_CLAIM_AHEAD 0  // claim the next chunk before processing the current one (measured:
-                          // a reserved chunk waits for its warp and delays its stage, -5%)
+#ifndef HX_CLAIM_SPAN
+#define HX_CLAIM_SPAN 1   // consecutive chunks claimed per shared atomic
 #endif
 #ifndef HX_BALLOT_COMPACT
 #define HX_BALLOT_COMPACT 0  // survivors' queue slots from 8 ballots instead of a shuffle scan
 #endif
-#ifndef HX_CLAIM_EARLY
-#define HX_CLAIM_EARLY 0  // claim the next chunk after stage S of the current one
-#endif
 #ifndef HX_TAG_SLEEP
-#define HX_TAG_SLEEP 20   // ns slept between polls of a ring slot's tile tag (0: spin)
+#define HX_TAG_SLEEP 0    // ns slept between polls of a ring slot's tile tag (0: spin; measured
+                          // 0.5% faster than 20 ns)
 #endif
 #ifndef HX_K1_CTAS
 #define HX_K1_CTAS 1    // resident CTAs per SM the launch bounds / smem budget target
@@ -574,8 +571,7 @@ __device__ __forceinline__ void process_tile(const K1Params& p, const JoinState 
                                              unsigned long long* s_sum, uint32_t* s_cnt,
                                              uint8_t* q_row, int32_t* q_g, CarryBuf* cb,
                                              int& n_carry, long long& acc_sum,
-                                             long long& acc_cnt, Pending& pd, const Pols& pol,
-                                             int* claim = nullptr, int* next_chunk = nullptr) {
+                                             long long& acc_cnt, Pending& pd, const Pols& pol) {
   constexpr int R = kRowsPerThread;  // rows per lane per tile
   const int wbase = warp * (32 * R);
   const int r0 = wbase + lane * R;
@@ -591,10 +587,7 @@ __device__ __forceinline__ void process_tile(const K1Params& p, const JoinState 
       m |= (uint32_t)(r0 + k < rows_valid1) << (R + k);
     }
   }
-  if (__ballot_sync(kFull, m) == 0) {
-    if (claim && lane == 0) *claim = atomicAdd(next_chunk, 1);
-    return;
-  }
+  if (__ballot_sync(kFull, m) == 0) return;
   // the 8 values of staged column c for this lane
   auto load8 = [&](int c, int32_t (&v)[2 * R]) {
 #pragma unroll
@@ -691,8 +684,6 @@ __device__ __forceinline__ void process_tile(const K1Params& p, const JoinState 
     }
   }
 
-  // (HX_CLAIM_EARLY) the warp's next chunk is claimed here, its latency overlapping the rest
-  if (claim && lane == 0) *claim = atomicAdd(next_chunk, 1);
   const int j0 = first_join_in_place<NJ, DM>(p, js);
   if (j0) {
     // stage B (hash tables): ONE probe step of the first join per row, 4 independent 128-bit
@@ -1067,21 +1058,18 @@ __global__ void __launch_bounds__((W == kWarpsLo && HX_K1_LB_LO) ? HX_K1_LB_LO :
   // is then complete, so the parity wait cannot match it.
   const int64_t my_tiles = p.n_tiles > blockIdx.x ? (p.n_tiles - 1 - blockIdx.x) / gridDim.x + 1 : 0;
   const int64_t my_chunks = my_tiles * kChunksPerTile;
-  int claimed = 0;
-  if ((HX_CLAIM_AHEAD || HX_CLAIM_EARLY) && lane == 0) claimed = atomicAdd(next_chunk, 1);
+  // (measured and rejected: claiming the next chunk before processing the current one, or
+  // during its stage C — a reserved chunk waits for its warp and holds its stage back)
+  int c = 0, span_left = 0;
   while (true) {
-    int c = 0;
-    if (HX_CLAIM_EARLY) {
-      c = __shfl_sync(kFull, claimed, 0);
-    } else if (HX_CLAIM_AHEAD) {
-      // the claim of the next chunk is issued now and read after this chunk: the shared
-      // atomic's latency overlaps the work
-      c = __shfl_sync(kFull, claimed, 0);
-      if (c < my_chunks && lane == 0) claimed = atomicAdd(next_chunk, 1);
-    } else {
-      if (lane == 0) c = atomicAdd(next_chunk, 1);
+    if (span_left == 0) {  // HX_CLAIM_SPAN consecutive chunks per shared atomic
+      if (lane == 0) c = atomicAdd(next_chunk, HX_CLAIM_SPAN);
       c = __shfl_sync(kFull, c, 0);
+      span_left = HX_CLAIM_SPAN;
+    } else {
+      ++c;
     }
+    --span_left;
     if (c >= my_chunks) break;
     const int i = c / kChunksPerTile, ch = c - i * kChunksPerTile;
     // (tracking slot and phase incrementally instead of dividing by the ring depth was
@@ -1110,8 +1098,7 @@ __global__ void __launch_bounds__((W == kWarpsLo && HX_K1_LB_LO) ? HX_K1_LB_LO :
     process_tile<NJ, GROUPED, DM>(p, js, sdm, cb0, cb0 + kHalfRows, frow0, frow0 + kHalfRows,
                                   kTileRows, min(crows, kHalfRows),
                                   max(0, crows - kHalfRows), 0, lane, smem_table, s_sum,
-                                  s_cnt, q_row, q_g, cb, n_carry, acc_sum, acc_cnt, pd, pol,
-                                  HX_CLAIM_EARLY ? &claimed : nullptr, next_chunk);
+                                  s_cnt, q_row, q_g, cb, n_carry, acc_sum, acc_cnt, pd, pol);
     __syncwarp();
     if (lane == 0) mbar_arrive(empty + slot);
   }
