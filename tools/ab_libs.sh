@@ -3,5 +3,5 @@
 sf=$1; shift
 for lib in "$@"; do
   echo "== $lib"
-  HX_LIB=$PWD/$lib HX_L2_PERSIST_MB=${HX_L2_PERSIST_MB:-0} timeout 600 python tools/time_queries.py --sf $sf --reps 5 2>&1 | awk '{printf "%s %s  ", $1, $6} END {print ""}'
+  HX_LIB=$PWD/$lib timeout 600 python tools/time_queries.py --sf $sf --reps 5 2>&1 | awk '{printf "%s %s  ", $1, $6} END {print ""}'
 done
