@@ -98,7 +98,14 @@ int hx_init(int device, void* stream, hx_ctx** out) {
   }
   ctx->k1_ctas_per_sm = std::max(1, k1_occupancy(ctx));
   // (the persisting L2 set-aside is reserved only when HX_OPT_L2_PERSIST is enabled: reserving
-  // it, even with no access-policy window in use, measured 2-5% slower K1 and a 2x slower K3)
+  // it, even with no access-policy window in use, measured 2-5% slower K1 and a 2x slower K3;
+  // HX_L2_PERSIST=1 enables it at init, for A/B measurements)
+  if (const char* e = std::getenv("HX_L2_PERSIST")) {
+    if (std::atoi(e) != 0) {
+      const int rc = hx_ctx_set_option(ctx, HX_OPT_L2_PERSIST, 1);
+      if (rc != HX_OK) return rc;
+    }
+  }
   {
     int least = 0, greatest = 0;
     if (cudaDeviceGetStreamPriorityRange(&least, &greatest) == cudaSuccess &&
