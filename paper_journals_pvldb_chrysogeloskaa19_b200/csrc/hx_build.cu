@@ -84,8 +84,12 @@ __device__ void rank_codes(const BuildParams& p) {
   }
   if (threadIdx.x == 0) {
     const int n = __ldcg(&p.hdr->n_keys);
+    // load factor <= 1/4, or <= 1/2 for a table that would exceed kBigTableBytes at 1/4 (a
+    // large table's L2 footprint costs more than its slightly longer probe chains; measured
+    // at SF100: customer 600 K keys, 32 -> 16 MB, HT-path Q4.1 -33%, Q3.1 -9%)
+    const long long inv = (long long)n * kLoadInv * 8 > kBigTableBytes ? 2 : kLoadInv;
     int lg = kMinLog2Cap;
-    while (lg < p.max_log2cap && (1ll << lg) < (long long)kLoadInv * n) ++lg;
+    while (lg < p.max_log2cap && (1ll << lg) < inv * n) ++lg;
     p.hdr->log2cap = lg;
     p.hdr->bloom_log2w = min(p.max_bloom_log2w, bloom_log2w_for(n));
     p.hdr->n_ranks = p.group ? running : 1;

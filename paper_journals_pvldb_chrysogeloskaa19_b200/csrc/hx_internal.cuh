@@ -89,7 +89,11 @@ __host__ __device__ __forceinline__ uint32_t bloom_mask(int32_t key) {
 // slot from there, so within a bucket slot 1 is filled only after slot 0 and "slot 1 of the
 // bucket is empty" proves a miss. Load factor <= 1/kLoadInv.
 constexpr int kBucketSlots = 2;
-constexpr int kLoadInv = 4;
+#ifndef HX_LOAD_INV
+#define HX_LOAD_INV 4
+#endif
+constexpr int kLoadInv = HX_LOAD_INV;
+constexpr long long kBigTableBytes = 8ll << 20;  // above: load factor <= 1/2 (hx_build.cu)
 constexpr int32_t kEmptyKey = -1;  // keys must differ from -1 (checked by the build)
 
 // Multiplicative (Fibonacci) hashing: the top log2(cap/2) bits of key * 2^32/phi.

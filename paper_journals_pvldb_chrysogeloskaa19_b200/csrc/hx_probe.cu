@@ -61,6 +61,9 @@ constexpr int kWarpsLo = 20, kWarpsHi = 26;
 #ifndef HX_BALLOT_COMPACT
 #define HX_BALLOT_COMPACT 0  // survivors' queue slots from 8 ballots instead of a shuffle scan
 #endif
+#ifndef HX_HT_SEQ
+#define HX_HT_SEQ 0       // hash-table joins probed one round trip per join in stage C
+#endif
 #ifndef HX_TAG_SLEEP
 #define HX_TAG_SLEEP 0    // ns slept between polls of a ring slot's tile tag (0: spin; measured
                           // 0.5% faster than 20 ns)
@@ -173,6 +176,8 @@ struct K1Params {
                                            // shared-memory structure: exact verdict + rank)
   uint32_t m_res;                          // resolved in stage S (full map staged, or m_l2s)
   int32_t l2_hint;                         // 1: probe loads evict_last (0: evict_normal; A/B)
+  int32_t ht_seq;                          // hash tables: stage C probes the first remaining
+                                           // join alone, the others only for its hits
 };
 
 // join kinds (uniform per launch: read from the kernel parameters)
@@ -515,6 +520,14 @@ __device__ __forceinline__ void stage_c_row(const K1Params& p, const JoinState (
     if (GROUPED) gg += (int32_t)v * js[jx].jstride;
   }
   if (!alive) pend = 0;
+  // (hash tables, HX_HT_SEQ) the first remaining join alone, the others only for its hits:
+  // the open-addressing tables are large and mostly missed, so fewer probes beat one round trip
+  uint32_t later = 0;
+  if ((HX_HT_SEQ || p.ht_seq) && !DM) {
+    const uint32_t first = pend & (0u - pend);
+    later = pend & ~first;
+    pend = first;
+  }
   while (pend) {
     ulonglong2 v[NJ > 0 ? NJ : 1];
 #pragma unroll
@@ -531,7 +544,11 @@ __device__ __forceinline__ void stage_c_row(const K1Params& p, const JoinState (
       pend &= ~((uint32_t)(hit || miss) << jx);
       b[jx] = (b[jx] + 1) & js[jx].bmask;
     }
-    if (!alive) pend = 0;
+    if (!alive) pend = later = 0;
+    if (!pend && later) {
+      pend = later;
+      later = 0;
+    }
   }
   Pending cur{gg, e.a, e.b, alive};
   if (alive) {  // issue the gathers now, consume them one batch later
@@ -1901,7 +1918,17 @@ int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht*
         }
       }
     }
-    // offsets: Bloom filters in the filter region, maps and bitmaps in the direct-map region
+    // hash tables: probe the first stage-C join alone when it is selective and has no Bloom
+  // filter (its misses then save the other probes; with a filter its conditional pass
+  // fraction is high and one round trip for all is cheaper; measured at SF100: HT Q4.1
+  // 15.5 -> 10.2 ms, Q3.1 5.1 -> 4.8, while Q2.1 / Q4.3 lose 5-9% when forced)
+  p.ht_seq = 0;
+  if (!dm_mode && sh->n_joins > 1) {
+    const int j0 = (p.n_preds == 0 && kind[0] != kStBloom) ? 1 : 0;  // stage B probes join 0
+    p.ht_seq = j0 < sh->n_joins && kind[j0] != kStBloom && known[j0] && pass[j0] < 0.5;
+  }
+  if (const char* e = std::getenv("HX_HT_SEQ")) p.ht_seq = std::atoi(e) != 0;
+  // offsets: Bloom filters in the filter region, maps and bitmaps in the direct-map region
     p.filter_words = 0;
     p.dm_bytes = 0;
     for (int j = 0; j < sh->n_joins; ++j) {
