@@ -153,7 +153,8 @@ int hx_table_write(hx_table* t, int32_t col_id, int64_t row_begin, int64_t n, co
  * Rows of `dim` passing the AND of `preds` (range lo <= v <= hi, or v IN in[0..n_in)) are
  * inserted as key -> rank into an open-addressing table in HBM (linear probing, 8-byte
  * slots {int32 key, int32 rank} in 16-byte buckets, capacity the power of two >=
- * 4*n_pass, min 16), built with warp-cooperative CAS inserts. Key -1 is reserved. If group_col >= 0 its values must lie in
+ * 4*n_pass, min 16 — >= 2*n_pass when 4*n_pass slots would exceed 8 MB), built with
+ * warp-cooperative CAS inserts. Key -1 is reserved. If group_col >= 0 its values must lie in
  * [group_lo, group_hi]; rank = position of the row's group code among the DISTINCT codes
  * of the passing rows in ascending order (dense ranks; rank_to_code recovers the code).
  * group_col < 0: membership only, rank 0, one rank.
