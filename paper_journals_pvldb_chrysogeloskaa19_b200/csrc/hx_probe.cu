@@ -1445,9 +1445,10 @@ size_t k1_smem_bytes(int warps, bool dm, int n_cols, int stages, int smem_groups
 // Per-CTA shared memory for `ctas` resident CTAs per SM (228 KB per SM, 1 KB reserved each).
 constexpr size_t smem_budget(int ctas) { return (228 * 1024) / ctas - 1024; }
 // The shared memory K1 may plan with per CTA: the rest of the SM's 256 KB L1/shared array
-// becomes L1 cache for the L2 map reads. HX_K1_SMEM_KB lowers it (tuning aid).
+// becomes L1 cache for the L2 map reads. t_smem_cap lowers it while k1_setup replans an
+// L2-lookup-bound pipeline; HX_K1_SMEM_KB lowers it (tuning aid).
 thread_local size_t t_smem_cap = 0;
-constexpr double kL1BoundCost = 50.0;  // plan cost above which K1 is L2-lookup-bound  // set while k1_setup replans an L2-lookup-bound pipeline
+constexpr double kL1BoundCost = 50.0;  // plan cost above which K1 is L2-lookup-bound
 size_t k1_smem_cap() {
   size_t cap = smem_budget(std::min(kCtasPerSm, 2));
   if (t_smem_cap) cap = std::min(cap, t_smem_cap);
