@@ -15,6 +15,7 @@
 #include <cub/block/block_scan.cuh>
 
 #include <algorithm>
+#include <cstdlib>
 #include <vector>
 
 #include "hx_internal.cuh"
@@ -172,6 +173,149 @@ __global__ void __launch_bounds__(kK3Threads) k3_scatter(K3Params p) {
   }
 }
 
+// ---- k3_scatter_tma: the same scatter with the tiles staged by the bulk-copy engine --------
+// r02: each CTA's next tile (every column, the key among them) is copied HBM -> shared memory
+// with cp.async.bulk while the current one is regrouped, so no thread waits on a global load;
+// the regroup is a permutation (src_of: the tile row of each part-sorted position) applied
+// column by column while writing, instead of copying every column into a second buffer.
+// Requires 16-byte aligned column bases and CTA chunks of whole tiles (checked by the host).
+__device__ __forceinline__ uint32_t k3_smem_u32(const void* p) {
+  return (uint32_t)__cvta_generic_to_shared(p);
+}
+__device__ __forceinline__ void k3_mbar_init(uint64_t* bar, uint32_t count) {
+  asm volatile("mbarrier.init.shared::cta.b64 [%0], %1;" ::"r"(k3_smem_u32(bar)), "r"(count));
+}
+__device__ __forceinline__ void k3_mbar_expect_tx(uint64_t* bar, uint32_t bytes) {
+  asm volatile("mbarrier.arrive.expect_tx.shared::cta.b64 _, [%0], %1;" ::"r"(k3_smem_u32(bar)),
+               "r"(bytes)
+               : "memory");
+}
+__device__ __forceinline__ void k3_mbar_wait(uint64_t* bar, uint32_t parity) {
+  asm volatile(
+      "{\n"
+      ".reg .pred p;\n"
+      "K3WAIT_%=:\n"
+      "mbarrier.try_wait.parity.shared::cta.b64 p, [%0], %1;\n"
+      "@!p bra K3WAIT_%=;\n"
+      "}\n" ::"r"(k3_smem_u32(bar)),
+      "r"(parity)
+      : "memory");
+}
+__device__ __forceinline__ void k3_bulk_g2s(void* dst, const void* src, uint32_t bytes, uint64_t* bar) {
+  asm volatile(
+      "cp.async.bulk.shared::cluster.global.mbarrier::complete_tx::bytes [%0], [%1], %2, [%3];" ::"r"(
+          k3_smem_u32(dst)),
+      "l"(src), "r"(bytes), "r"(k3_smem_u32(bar))
+      : "memory");
+}
+
+constexpr int kK3MaxTmaCols = 12;
+constexpr size_t k3_tma_smem(int n_cols) { return 2 * (size_t)n_cols * kK3Tile * 4; }
+
+__global__ void __launch_bounds__(kK3Threads) k3_scatter_tma(K3Params p, int key_c) {
+  __shared__ unsigned long long cur[HX_MAX_PARTS];
+  __shared__ unsigned tcnt[HX_MAX_PARTS], tstart[HX_MAX_PARTS];
+  __shared__ uint16_t src_of[kK3Tile];
+  __shared__ uint8_t psorted[kK3Tile];
+  __shared__ __align__(8) uint64_t full[2];
+  extern __shared__ __align__(128) int32_t stage[];  // [2][n_cols][kK3Tile]
+  const int tid = threadIdx.x, lane = tid & 31;
+  for (int i = tid; i < p.n_parts; i += blockDim.x) {
+    cur[i] = (unsigned long long)p.counts[(int64_t)i * gridDim.x + blockIdx.x];
+    tcnt[i] = 0;
+  }
+  if (tid == 0) {
+    k3_mbar_init(full + 0, 1);
+    k3_mbar_init(full + 1, 1);
+    asm volatile("fence.mbarrier_init.release.cluster;" ::: "memory");
+  }
+  __syncthreads();
+  const int64_t r0 = (int64_t)blockIdx.x * p.chunk;
+  const int64_t r1 = min(p.n_rows, r0 + p.chunk);
+  const size_t stage_elems = (size_t)p.n_cols * kK3Tile;
+  auto issue = [&](int64_t t0, int s) {  // one thread: every column of the tile at t0
+    const int rows = (int)(r1 - t0 < kK3Tile ? r1 - t0 : (int64_t)kK3Tile);
+    const uint32_t bytes = (uint32_t)(rows & ~3) * 4u;
+    k3_mbar_expect_tx(full + s, bytes * p.n_cols);
+    if (bytes)
+      for (int c = 0; c < p.n_cols; ++c)
+        k3_bulk_g2s(stage + s * stage_elems + (size_t)c * kK3Tile, p.src[c] + t0, bytes, full + s);
+  };
+  if (tid == 0 && r0 < r1) issue(r0, 0);
+  uint32_t phases = 0u;  // bit s: the parity the next wait on stage s expects
+  int s = 0;
+  for (int64_t t0 = r0; t0 < r1; t0 += kK3Tile, s ^= 1) {
+    const int rows = (int)(r1 - t0 < kK3Tile ? r1 - t0 : (int64_t)kK3Tile);
+    // the other stage was last used by the previous tile, finished at the barrier below
+    if (tid == 0 && t0 + kK3Tile < r1) issue(t0 + kK3Tile, s ^ 1);
+    k3_mbar_wait(full + s, (phases >> s) & 1u);
+    phases ^= 1u << s;
+    int32_t* st = stage + s * stage_elems;
+    const int copied = rows & ~3;
+    if (copied != rows) {  // the chunk's last <= 3 rows: not a 16-byte multiple
+      if (tid < rows - copied)
+        for (int c = 0; c < p.n_cols; ++c) st[(size_t)c * kK3Tile + copied + tid] = p.src[c][t0 + copied + tid];
+      __syncthreads();
+    }
+    const int32_t* keys = st + (size_t)key_c * kK3Tile;
+    int mypart[kK3PerThread], myslot[kK3PerThread];
+#pragma unroll
+    for (int k = 0; k < kK3PerThread; ++k) {
+      const int j = tid + k * kK3Threads;
+      const bool live = j < rows;
+      const int part = live ? part_of(keys[j], p.n_parts) : 0;
+      const unsigned act = __ballot_sync(0xFFFFFFFFu, live);
+      int slot = 0;
+      if (live) {  // warp-aggregated slot within the tile's part
+        const unsigned same = __match_any_sync(act, part);
+        const int leader = __ffs(same) - 1;
+        unsigned base = 0;
+        if (lane == leader) base = atomicAdd(&tcnt[part], (unsigned)__popc(same));
+        base = __shfl_sync(same, base, leader);
+        slot = (int)(base + __popc(same & ((1u << lane) - 1u)));
+      }
+      mypart[k] = part;
+      myslot[k] = live ? slot : -1;
+    }
+    __syncthreads();
+    if (tid < 32) {  // exclusive scan of the (<= 64) tile counts
+      const unsigned a = lane < p.n_parts ? tcnt[lane] : 0u;
+      const unsigned b = lane + 32 < p.n_parts ? tcnt[lane + 32] : 0u;
+      unsigned ia = a, ib = b;
+#pragma unroll
+      for (int o = 1; o < 32; o <<= 1) {
+        const unsigned va = __shfl_up_sync(0xFFFFFFFFu, ia, o);
+        const unsigned vb = __shfl_up_sync(0xFFFFFFFFu, ib, o);
+        if (lane >= o) ia += va, ib += vb;
+      }
+      const unsigned tot_a = __shfl_sync(0xFFFFFFFFu, ia, 31);
+      if (lane < p.n_parts) tstart[lane] = ia - a;
+      if (lane + 32 < p.n_parts) tstart[lane + 32] = tot_a + ib - b;
+    }
+    __syncthreads();
+#pragma unroll
+    for (int k = 0; k < kK3PerThread; ++k)
+      if (myslot[k] >= 0) {
+        const int pos = (int)tstart[mypart[k]] + myslot[k];
+        src_of[pos] = (uint16_t)(tid + k * kK3Threads);
+        psorted[pos] = (uint8_t)mypart[k];
+      }
+    __syncthreads();
+    for (int i = tid; i < rows; i += kK3Threads) {  // part-sorted position i: one run per part
+      const int part = psorted[i];
+      const unsigned long long o = cur[part] + (unsigned)(i - (int)tstart[part]);
+      const int j = src_of[i];
+      for (int c = 0; c < p.n_cols; ++c) p.dst[c][o] = st[(size_t)c * kK3Tile + j];
+    }
+    __syncthreads();
+    for (int i = tid; i < p.n_parts; i += blockDim.x) {
+      cur[i] += tcnt[i];
+      tcnt[i] = 0;
+    }
+    __syncthreads();
+  }
+}
+
 int table_alloc_like(hx_ctx* ctx, const hx_table* t, int64_t n_rows, hx_table** out) {
   hx_table* o = new hx_table();
   o->ctx = ctx;
@@ -217,11 +361,19 @@ int hx_hash_partition(hx_ctx* ctx, const hx_table* t, int32_t key_col, int n_par
     *out = o;
     return HX_OK;
   }
-  // one wave of the scatter kernel (its shared memory grows with the column count)
-  const size_t scatter_smem = (size_t)t->n_cols * kK3Tile * sizeof(int32_t);
-  cudaFuncSetAttribute(k3_scatter, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)scatter_smem);
+  // the bulk-copy scatter when every column base is 16-byte aligned (CTA chunks are whole
+  // tiles), else the load-based one; one wave of either (shared memory grows with the columns)
+  int key_c = 0;
+  bool tma = t->n_cols <= kK3MaxTmaCols && std::getenv("HX_K3_LDG") == nullptr;
+  for (int c = 0; c < t->n_cols; ++c) {
+    tma = tma && (reinterpret_cast<uintptr_t>(t->dev[c]) & 15u) == 0;
+    if (t->col_id[c] == key_col) key_c = c;
+  }
+  const size_t scatter_smem = tma ? k3_tma_smem(t->n_cols) : (size_t)t->n_cols * kK3Tile * sizeof(int32_t);
+  const void* scatter_fn = tma ? (const void*)k3_scatter_tma : (const void*)k3_scatter;
+  cudaFuncSetAttribute(scatter_fn, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)scatter_smem);
   int occ = 1;
-  cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, k3_scatter, kK3Threads, scatter_smem);
+  cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, scatter_fn, kK3Threads, scatter_smem);
   const int64_t grid = std::max<int64_t>(1, std::min<int64_t>((int64_t)ctx->n_sms * std::max(1, occ),
                                                              (t->n_rows + 4095) / 4096));
   K3Params p{};
@@ -234,6 +386,7 @@ int hx_hash_partition(hx_ctx* ctx, const hx_table* t, int32_t key_col, int n_par
   p.n_parts = n_parts;
   p.n_rows = t->n_rows;
   p.chunk = (t->n_rows + grid - 1) / grid;
+  if (tma) p.chunk = (p.chunk + kK3Tile - 1) / kK3Tile * kK3Tile;  // whole (aligned) tiles
   void* scratch = nullptr;
   const size_t sbytes = sizeof(int64_t) * ((size_t)n_parts * grid + n_parts + 1);
   cudaError_t e = cudaMallocAsync(&scratch, sbytes, ctx->stream);
@@ -245,7 +398,10 @@ int hx_hash_partition(hx_ctx* ctx, const hx_table* t, int32_t key_col, int n_par
   p.part_offsets = p.counts + (size_t)n_parts * grid;
   k3_count<<<(unsigned)grid, kK3Threads, 0, ctx->stream>>>(p);
   k3_scan<<<1, 1024, 0, ctx->stream>>>(p, (int)grid);
-  k3_scatter<<<(unsigned)grid, kK3Threads, scatter_smem, ctx->stream>>>(p);
+  if (tma)
+    k3_scatter_tma<<<(unsigned)grid, kK3Threads, scatter_smem, ctx->stream>>>(p, key_c);
+  else
+    k3_scatter<<<(unsigned)grid, kK3Threads, scatter_smem, ctx->stream>>>(p);
   ctx->launches += 3;
   e = cudaGetLastError();
   if (e == cudaSuccess)

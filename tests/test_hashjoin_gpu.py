@@ -46,15 +46,26 @@ def part_of(keys: np.ndarray, n_parts: int) -> np.ndarray:
     return ((h * np.uint64(n_parts)) >> np.uint64(32)).astype(np.int64)
 
 
+@pytest.mark.parametrize("kernel", ["tma", "ldg", "misaligned"])
 @pytest.mark.parametrize("n_rows", [0, 1, 1000, 300_001])
 @pytest.mark.parametrize("n_parts", [1, 3, 8, 64])
-def test_hash_partition_is_a_grouped_permutation(ctx, n_rows, n_parts):
+def test_hash_partition_is_a_grouped_permutation(ctx, monkeypatch, n_rows, n_parts, kernel):
+    """Both K3 scatters: the bulk-copy one (aligned columns), the load-based one (HX_K3_LDG=1,
+    and automatically for a view at an odd row offset)."""
+    if kernel == "ldg":
+        monkeypatch.setenv("HX_K3_LDG", "1")
     rng = np.random.default_rng(n_rows * 7 + n_parts)
     key = rng.integers(-2**31, 2**31 - 1, n_rows, dtype=np.int64).astype(np.int32)
     key[: n_rows // 3] = rng.integers(0, 50, n_rows // 3)  # heavy duplicates too
     a = rng.integers(-1000, 1000, n_rows).astype(np.int32)
     b = np.arange(n_rows, dtype=np.int32)
-    t = hx.load_numpy(ctx, {10: key, 11: a, 12: b})
+    full = None
+    if kernel == "misaligned":  # the same rows behind one leading row: 4-byte aligned only
+        pad = lambda v: np.concatenate([np.zeros(1, np.int32), v])
+        full = hx.load_numpy(ctx, {10: pad(key), 11: pad(a), 12: pad(b)})
+        t = full.slice(1, n_rows + 1)
+    else:
+        t = hx.load_numpy(ctx, {10: key, 11: a, 12: b})
     out, offs = hx.hash_partition(ctx, t, 10, n_parts)
     assert len(offs) == n_parts + 1 and offs[0] == 0 and offs[-1] == n_rows
     assert all(x <= y for x, y in zip(offs, offs[1:]))
@@ -68,6 +79,8 @@ def test_hash_partition_is_a_grouped_permutation(ctx, n_rows, n_parts):
     assert np.array_equal(k2, key[b2]) and np.array_equal(a2, a[b2])
     out.close()
     t.close()
+    if full is not None:
+        full.close()
 
 
 def test_identity_ranks(ctx):
