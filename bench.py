@@ -43,6 +43,7 @@ with open(os.path.join(ROOT, "BASELINE.json")) as _f:
 UNIT = "lineorder rows/s"
 SEED = 42
 BLOCK_ROWS = 1 << 22
+SCALING = ["weak"]  # "strong" with --sf-total
 
 
 def parse(argv=None):
@@ -50,7 +51,10 @@ def parse(argv=None):
     ap.add_argument("--gpus", type=int, default=1)
     ap.add_argument("--steps", type=int, default=50)
     ap.add_argument("--warmup", type=int, default=3)
-    ap.add_argument("--sf", type=float, default=100.0, help="SSB scale factor per GPU")
+    ap.add_argument("--sf", type=float, default=100.0, help="SSB scale factor per GPU (weak scaling)")
+    ap.add_argument("--sf-total", type=float, default=0.0,
+                    help="strong scaling: this total scale factor split over the GPUs (e.g. "
+                         "configs[3]: --sf-total 1000 --gpus 2|4|8); overrides --sf")
     ap.add_argument("--impl", default="hx", choices=["hx", "reference"])
     ap.add_argument("--no-cpu-baseline", action="store_true")
     ap.add_argument("--no-e2e", action="store_true")
@@ -258,7 +262,7 @@ def run_reference(args, world, rank):
             f"once outside the clock), {len(queries)} queries, {threads} threads")
     line = {"impl": "reference", "metric": METRIC, "value": value, "unit": UNIT, "n_gpus": world,
             "steps": args.steps, "warmup": args.warmup, "ms_per_step": dt * 1e3,
-            "higher_is_better": True, "scaling": "weak", "vs_baseline": None, "dtype": "int64",
+            "higher_is_better": True, "scaling": SCALING[0], "vs_baseline": None, "dtype": "int64",
             "data": f"synthetic (ssbgen dbgen-shaped SSB, seed {SEED})",
             "config": dict(config(args, world, sz["n_lineorder"] // world, queries),
                            executed_as=f"reference arm: the CPU oracle (oracle/ssb_oracle.cpp) "
@@ -378,7 +382,7 @@ def run_micro(args, world, rank, local, ctx, stream, torch, dist, hx):
         line = {"metric": f"micro-benchmark fact rows/sec & HBM GB/s ({args.workload})",
                 "value": n_gpu * world / (ms_step / 1e3), "unit": "fact rows/s",
                 "n_gpus": world, "steps": args.steps, "warmup": args.warmup,
-                "ms_per_step": ms_step, "higher_is_better": True, "scaling": "weak",
+                "ms_per_step": ms_step, "higher_is_better": True, "scaling": SCALING[0],
                 "vs_baseline": None, "dtype": "int32 columns, int64 accumulate",
                 "data": f"synthetic (ssbgen mb_* columns, seed {SEED}), generated in HBM",
                 "config": {"workload": f"{name}: {n_gpu * 4 / 1e9:.1f} GB per column per GPU, "
@@ -520,7 +524,7 @@ def run_host_routed(args, world, rank, local, ctx, stream, torch, dist, hx, ssb,
         print(json.dumps({
             "metric": METRIC, "value": value, "unit": UNIT, "n_gpus": world, "steps": args.steps,
             "warmup": args.warmup, "ms_per_step": ms_step, "higher_is_better": True,
-            "scaling": "weak", "vs_baseline": None, "dtype": "int32 columns, int64 accumulate",
+            "scaling": SCALING[0], "vs_baseline": None, "dtype": "int32 columns, int64 accumulate",
             "data": f"synthetic (ssbgen dbgen-shaped SSB, seed {SEED}), lineorder in shared pinned "
                     "host memory",
             "config": dict(config(args, world, n // world, queries), router="shared counter "
@@ -639,6 +643,9 @@ def main():
         env.setdefault("NCCL_DEBUG_SUBSYS", "INIT")
         sys.exit(subprocess.run(what, env=env).returncode)
     world, rank, local = dist_env()
+    if args.sf_total > 0:
+        args.sf = args.sf_total / world
+    SCALING[0] = "strong" if args.sf_total > 0 else "weak"
     if world > 1:
         os.environ.setdefault("NCCL_DEBUG", "INFO")
         os.environ.setdefault("NCCL_DEBUG_SUBSYS", "INIT")
@@ -1105,7 +1112,7 @@ def main():
         line = {"metric": METRIC, "value": value, "unit": UNIT, "n_gpus": world,
                 "steps": args.steps, "warmup": args.warmup, "ms_per_step": ms_step,
                 "ms_per_step_median": statistics.median(per_step), "ms_per_step_min": min(per_step),
-                "higher_is_better": True, "scaling": "weak", "vs_baseline": None,
+                "higher_is_better": True, "scaling": SCALING[0], "vs_baseline": None,
                 "dtype": "int32 columns, int64 accumulate",
                 "data": f"synthetic (ssbgen dbgen-shaped SSB distributions, seed {SEED}), "
                         "generated in HBM",
