@@ -281,15 +281,24 @@ def cpu_baseline(args, world):
     sample = min(sz["n_lineorder"], 12_000_000)  # ~10 s of single-threaded oracle work
     db = ssbgen.database(SEED, sz, 0, sample)
     idx = oracle.DimIndex(db)  # the dimension maps, built once (not timed: SURVEY.md 8(d))
-    t0 = time.perf_counter()
-    for q in oracle.QUERIES:
-        idx.query(q, db["lineorder"])
-    dt = time.perf_counter() - t0
+    # pinned to one core for the timed evaluation (taskset to one core)
+    aff = os.sched_getaffinity(0) if hasattr(os, "sched_getaffinity") else None
+    core = min(aff) if aff else None
+    if core is not None:
+        os.sched_setaffinity(0, {core})
+    try:
+        t0 = time.perf_counter()
+        for q in oracle.QUERIES:
+            idx.query(q, db["lineorder"])
+        dt = time.perf_counter() - t0
+    finally:
+        if aff:
+            os.sched_setaffinity(0, aff)
     idx.close()
     return {"value": 13 * sample / dt, "unit": UNIT, "cores": 1, "kind": "oracle",
             "sample": f"13 queries over lineorder rows [0, {sample}) of SF{args.sf * world:g} "
-                      f"(full dims, maps built once outside the clock), single-threaded, "
-                      f"{dt:.1f} s"}
+                      f"(full dims, maps built once outside the clock), single-threaded, pinned "
+                      f"to core {core}, {dt:.1f} s"}
 
 
 def run_micro(args, world, rank, local, ctx, stream, torch, dist, hx):
