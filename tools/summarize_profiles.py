@@ -23,7 +23,8 @@ BROW = {"1": 16, "2": 16, "3": 16, "4": 24}
 def main(tag, rep, launches, sf="10", probe_csv=None):
     global N
     N = int(6_000_000 * float(sf))
-    raw = subprocess.run(["ncu", "-i", rep, "--page", "raw", "--csv"], capture_output=True, text=True).stdout
+    raw = (open(rep).read() if rep.endswith(".csv") else  # a saved `--page raw --csv` export
+           subprocess.run(["ncu", "-i", rep, "--page", "raw", "--csv"], capture_output=True, text=True).stdout)
     rows = list(csv.reader(io.StringIO(raw)))
     hdr, data = rows[0], rows[2:]
     c = hdr.index
