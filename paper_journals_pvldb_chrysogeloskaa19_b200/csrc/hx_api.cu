@@ -101,9 +101,9 @@ int hx_init(int device, void* stream, hx_ctx** out) {
   // it, even with no access-policy window in use, measured 2-5% slower K1 and a 2x slower K3;
   // HX_L2_PERSIST=1 enables it at init, for A/B measurements)
   if (const char* e = std::getenv("HX_L2_PERSIST")) {
-    if (std::atoi(e) != 0) {
-      const int rc = hx_ctx_set_option(ctx, HX_OPT_L2_PERSIST, 1);
-      if (rc != HX_OK) return rc;
+    if (std::atoi(e) != 0 && hx_ctx_set_option(ctx, HX_OPT_L2_PERSIST, 1) != HX_OK) {
+      ctx->l2_persist = 0;  // (an A/B switch: without it the context still works, unpinned)
+      cudaGetLastError();
     }
   }
   {
