@@ -504,6 +504,12 @@ class SharedRouter:
             call("hx_shared_router_close", self.h, 1 if unlink else 0)
             self.h = None
 
+    def __del__(self):
+        try:
+            self.close()
+        except Exception:
+            pass
+
 
 def pipeline_probe_agg_routed(ctx: Context, fact: Table, shape: hx_query_shape,
                               hts: Sequence[HashTable], router: SharedRouter,
