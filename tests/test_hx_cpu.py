@@ -301,3 +301,42 @@ def test_shared_router_rejects_bad_arguments():
     with pytest.raises(_hx.HxError):
         hx.SharedRouter("/hx_test_router_missing_x", 8, create=False)
     r.close(unlink=True)
+
+
+# ---- the union router's host layout and finalize (hx_group_layout / hx_group_decode) -------
+def test_group_layout_is_row_major_mixed_radix():
+    """Independent restatement: index = sum_g r_g * prod_{h > g} n_h (the last dimension
+    fastest), n_groups = prod n_g."""
+    n = [7, 5, 3]
+    strides, ng = hx.group_layout(n)
+    assert ng == 105 and strides == [15, 3, 1]
+    seen = set()
+    for r0 in range(7):
+        for r1 in range(5):
+            for r2 in range(3):
+                seen.add(r0 * strides[0] + r1 * strides[1] + r2 * strides[2])
+    assert seen == set(range(ng))
+    assert hx.group_layout([]) == ([], 1)
+    with pytest.raises(_hx.HxError) as e:
+        hx.group_layout([1 << 14, 1 << 14])  # 2^28 > HX_MAX_GROUPS
+    assert e.value.code == _hx.HX_ECAPACITY
+    with pytest.raises(_hx.HxError):
+        hx.group_layout([3, 0])
+
+
+def test_group_decode_drops_empty_groups_and_maps_codes():
+    rng = np.random.default_rng(5)
+    n = [4, 6]
+    maps = [np.array([1992, 1993, 1995, 1998]), np.array([3, 7, 11, 12, 40, 41])]
+    ng = 24
+    cnt = rng.integers(0, 3, ng)
+    sums = rng.integers(-50, 50, ng) * (cnt > 0)
+    keys, s, c = hx.group_decode(n, maps, sums, cnt)
+    want = [(int(maps[0][i // 6]), int(maps[1][i % 6]), int(sums[i]), int(cnt[i]))
+            for i in range(ng) if cnt[i] > 0]
+    assert [(int(k[0]), int(k[1]), int(x), int(y)) for k, x, y in zip(keys, s, c)] == want
+    # ungrouped: the one row is kept even with count 0 (SQL NULL sum, DESIGN.md R7)
+    k0, s0, c0 = hx.group_decode([], [], np.array([0]), np.array([0]))
+    assert len(s0) == 1 and int(c0[0]) == 0
+    with pytest.raises(_hx.HxError):  # n_groups must match the layout
+        hx.group_decode(n, maps, sums[:10], cnt[:10])
