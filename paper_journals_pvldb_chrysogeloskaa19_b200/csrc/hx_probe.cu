@@ -1503,19 +1503,19 @@ const KernelFn kKernels[2][2][2][HX_MAX_JOINS + 1] = {
      {HX_K1_ROW(kWarpsHi, false, true), HX_K1_ROW(kWarpsHi, true, true)}}};
 #undef HX_K1_ROW
 
-// instances reading narrow-encoded columns: [warps][grouped][joins] (direct maps; the
-// join-less shape uses its hash-table-free instance)
-#define HX_K1_NWROW(W, G)                                                                         \
-  {k1_probe_agg<0, G, false, W, true>, k1_probe_agg<1, G, true, W, true>,                         \
-   k1_probe_agg<2, G, true, W, true>, k1_probe_agg<3, G, true, W, true>,                          \
-   k1_probe_agg<4, G, true, W, true>}
-const KernelFn kKernelsNarrow[2][2][HX_MAX_JOINS + 1] = {
-    {HX_K1_NWROW(kWarpsLo, false), HX_K1_NWROW(kWarpsLo, true)},
-    {HX_K1_NWROW(kWarpsHi, false), HX_K1_NWROW(kWarpsHi, true)}};
+// instances reading narrow-encoded columns: [warps][direct maps][grouped][joins]
+#define HX_K1_NWROW(W, G, D)                                                                      \
+  {k1_probe_agg<0, G, false, W, true>, k1_probe_agg<1, G, D, W, true>,                            \
+   k1_probe_agg<2, G, D, W, true>, k1_probe_agg<3, G, D, W, true>, k1_probe_agg<4, G, D, W, true>}
+const KernelFn kKernelsNarrow[2][2][2][HX_MAX_JOINS + 1] = {
+    {{HX_K1_NWROW(kWarpsLo, false, false), HX_K1_NWROW(kWarpsLo, true, false)},
+     {HX_K1_NWROW(kWarpsLo, false, true), HX_K1_NWROW(kWarpsLo, true, true)}},
+    {{HX_K1_NWROW(kWarpsHi, false, false), HX_K1_NWROW(kWarpsHi, true, false)},
+     {HX_K1_NWROW(kWarpsHi, false, true), HX_K1_NWROW(kWarpsHi, true, true)}}};
 #undef HX_K1_NWROW
 
 KernelFn pick_kernel(int nj, bool grouped, bool dm, int warps, bool narrow = false) {
-  if (narrow) return kKernelsNarrow[warps == kWarpsHi ? 1 : 0][grouped ? 1 : 0][nj];
+  if (narrow) return kKernelsNarrow[warps == kWarpsHi ? 1 : 0][dm ? 1 : 0][grouped ? 1 : 0][nj];
   return kKernels[warps == kWarpsHi ? 1 : 0][dm ? 1 : 0][grouped ? 1 : 0][nj];
 }
 
@@ -1702,10 +1702,11 @@ int k1_occupancy(hx_ctx* ctx) {
             cudaFuncSetAttribute(kKernels[w][d][g][j], cudaFuncAttributeMaxDynamicSharedMemorySize,
                                  227 * 1024);
     for (int w = 0; w < 2; ++w)
-      for (int g = 0; g < 2; ++g)
-        for (int j = 0; j <= HX_MAX_JOINS; ++j)
-          cudaFuncSetAttribute(kKernelsNarrow[w][g][j], cudaFuncAttributeMaxDynamicSharedMemorySize,
-                               227 * 1024);
+      for (int d = 0; d < 2; ++d)
+        for (int g = 0; g < 2; ++g)
+          for (int j = 0; j <= HX_MAX_JOINS; ++j)
+            cudaFuncSetAttribute(kKernelsNarrow[w][d][g][j],
+                                 cudaFuncAttributeMaxDynamicSharedMemorySize, 227 * 1024);
     cudaFuncSetAttribute(k1_scan_agg<1>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)scan_smem(1));
     cudaFuncSetAttribute(k1_scan_agg<2>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)scan_smem(2));
     cudaFuncSetAttribute(k1_scan_agg<3>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)scan_smem(3));
