@@ -78,10 +78,6 @@ def parse(argv=None):
                          "CUDA graph); shared = ONE pinned copy of lineorder in shared memory, blocks "
                          "drawn from a shared counter by whichever GPU is free (dynamic load "
                          "balancing, PAPER.md:469-473)")
-    ap.add_argument("--encoding", default="int32", choices=["int32", "narrow"],
-                    help="narrow: lineorder columns whose range fits 1 or 2 bytes are stored that "
-                         "way (hx_table_encode, SURVEY.md 8(f) NEXT-4); K1 streams them at their "
-                         "width. The e2e leg stays int32")
     ap.add_argument("--sizeup", action="store_true",
                     help="with --workload sum|join: the §6.4 size-up sweep (0.125-16 GB per "
                          "column), one JSON line per size")
@@ -750,10 +746,6 @@ def main():
                                else hx._hx.HX_PLACE_HOST_MAPPED)
     else:
         fact = dev_table(lo_cols, r0, n_mine)
-    encoded = {}
-    if args.encoding == "narrow" and args.variant == "hbm":
-        torch.cuda.synchronize()
-        encoded = ssb.narrow_fact(fact, lo_cols)
     torch.cuda.synchronize()
     eng = ssb.SsbEngine(ctx, dims, fact)
     # one prepared plan per query (HT + group buffers allocated once, builds sized once);
@@ -1134,8 +1126,6 @@ def main():
                 "data": f"synthetic (ssbgen dbgen-shaped SSB distributions, seed {SEED}), "
                         "generated in HBM",
                 "config": dict(config(args, world, n_mine, queries), plan_sets=n_sets,
-                               encoding=({"narrow (bytes per value; the rest int32)": encoded}
-                                         if encoded else "int32"),
                                step_overlap="host reads step i's results while the device runs "
                                             "step i+1" if n_sets == 2 else "none"),
                 "hbm_gbps_per_gpu": sum(n_mine * B[q] for q in queries) / (ms_step / 1e3) / 1e9,

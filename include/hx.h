@@ -135,17 +135,6 @@ int hx_table_info(const hx_table* t, int64_t* n_rows, int* n_cols);
 /* A view of rows [row_begin, row_end) of `t` (no copy; lifetime bounded by `t`). */
 int hx_table_slice(const hx_table* t, int64_t row_begin, int64_t row_end, hx_table** out);
 int hx_table_free(hx_table* t);
-/* Narrow encoding of one column (§8(f) NEXT-4: "narrower encodings", the
-   columns a pipeline reads cost their bytes): the int32 column `col_id` of a device table
-   (HX_PLACE_COPY / VIEW, not a slice) is replaced by `width` (1 or 2) bytes per value in
-   frame-of-reference form, value = min + stored, into a library-owned buffer (a COPY table's
-   old buffer is freed; a VIEW's caller buffer is left alone). HX_EINVAL if max - min does not
-   fit in `width` bytes (the table is unchanged). Synchronises (reads min/max back).
-   Only the fused pipeline (hx_pipeline_probe_agg*, plans) reads narrow columns — they are
-   staged at their width and widened in registers; the other calls (builds, hash-pack,
-   read/write/slice, host-resident streaming) refuse a table with narrow columns
-   (HX_EUNSUPPORTED). Results are identical (the values are unchanged). */
-int hx_table_encode(hx_table* t, int32_t col_id, int width);
 /* Copies rows [row_begin, row_begin + n) of column `col_id` of `t` (device or host resident)
    into caller host memory `dst` (n int32). Synchronises the ctx stream. */
 int hx_table_read(const hx_table* t, int32_t col_id, int64_t row_begin, int64_t n, int32_t* dst);

@@ -98,7 +98,6 @@ _SIGS = {
     "hx_table_info": ([_P, _PI64, ctypes.POINTER(_I)], _I),
     "hx_table_slice": ([_P, _I64, _I64, _PP], _I),
     "hx_table_free": ([_P], _I),
-    "hx_table_encode": ([_P, _I32, _I], _I),
     "hx_table_read": ([_P, _I32, _I64, _I64, _PI32], _I),
     "hx_table_write": ([_P, _I32, _I64, _I64, _P], _I),
     "hx_build_dim_ht": ([_P, _P, _I32, ctypes.POINTER(hx_pred), _I, _I32, _I32, _I32, _PP], _I),

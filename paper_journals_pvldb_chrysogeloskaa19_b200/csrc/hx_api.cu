@@ -366,10 +366,8 @@ int hx_table_info(const hx_table* t, int64_t* n_rows, int* n_cols) {
 int hx_table_slice(const hx_table* t, int64_t row_begin, int64_t row_end, hx_table** out) {
   HX_REQUIRE(t && out && row_begin >= 0 && row_end >= row_begin && row_end <= t->n_rows,
              HX_EINVAL, "hx_table_slice: bad range");
-  HX_REQUIRE(!table_narrow(t), HX_EUNSUPPORTED, "hx_table_slice: the table has narrow-encoded columns");
   hx_table* s = new hx_table(*t);
   s->owned = false;
-  s->own_mask = 0;
   s->parent = t;
   s->n_rows = row_end - row_begin;
   for (int c = 0; c < t->n_cols; ++c) s->dev[c] = t->dev[c] ? t->dev[c] + row_begin : nullptr;
@@ -381,7 +379,6 @@ int hx_table_read(const hx_table* t, int32_t col_id, int64_t row_begin, int64_t 
   HX_REQUIRE(t && (dst || n == 0) && row_begin >= 0 && n >= 0 && row_begin + n <= t->n_rows,
              HX_EINVAL, "hx_table_read: bad argument");
   HX_REQUIRE(table_has_col(t, col_id), HX_EINVAL, "hx_table_read: column not in table");
-  HX_REQUIRE(!table_narrow(t), HX_EUNSUPPORTED, "hx_table_read: the table has narrow-encoded columns");
   if (n == 0) return HX_OK;
   HX_CK(cudaSetDevice(t->ctx->device));
   HX_CK(cudaMemcpyAsync(dst, table_col(t, col_id) + row_begin, (size_t)n * 4, cudaMemcpyDefault,
@@ -397,7 +394,6 @@ int hx_table_write(hx_table* t, int32_t col_id, int64_t row_begin, int64_t n, co
   HX_REQUIRE(t->placement == HX_PLACE_COPY || t->placement == HX_PLACE_VIEW, HX_EUNSUPPORTED,
              "hx_table_write: the table must be device resident");
   HX_REQUIRE(table_has_col(t, col_id), HX_EINVAL, "hx_table_write: column not in table");
-  HX_REQUIRE(!table_narrow(t), HX_EUNSUPPORTED, "hx_table_write: the table has narrow-encoded columns");
   if (n == 0) return HX_OK;
   HX_CK(cudaSetDevice(t->ctx->device));
   cudaPointerAttributes pa{};
@@ -413,45 +409,12 @@ int hx_table_write(hx_table* t, int32_t col_id, int64_t row_begin, int64_t n, co
 
 int hx_table_free(hx_table* t) {
   HX_REQUIRE(t, HX_EINVAL, "hx_table_free: null table");
-  if (t->owned || t->own_mask) {
+  if (t->owned) {
     cudaSetDevice(t->ctx->device);
     for (int c = 0; c < t->n_cols; ++c)
-      if (t->dev[c] && (t->owned || ((t->own_mask >> c) & 1u))) cudaFreeAsync(t->dev[c], t->ctx->stream);
+      if (t->dev[c]) cudaFreeAsync(t->dev[c], t->ctx->stream);
   }
   delete t;
-  return HX_OK;
-}
-
-int hx_table_encode(hx_table* t, int32_t col_id, int width) {
-  HX_REQUIRE(t && (width == 1 || width == 2), HX_EINVAL, "hx_table_encode: width must be 1 or 2");
-  HX_REQUIRE(t->placement == HX_PLACE_COPY || t->placement == HX_PLACE_VIEW, HX_EUNSUPPORTED,
-             "hx_table_encode: the table must be device resident");
-  HX_REQUIRE(!t->parent, HX_EUNSUPPORTED, "hx_table_encode: not on a slice");
-  int c = -1;
-  for (int i = 0; i < t->n_cols; ++i)
-    if (t->col_id[i] == col_id) c = i;
-  HX_REQUIRE(c >= 0, HX_EINVAL, "hx_table_encode: column not in table");
-  HX_REQUIRE(t->width[c] == 4, HX_EINVAL, "hx_table_encode: column already encoded");
-  hx_ctx* ctx = t->ctx;
-  HX_CK(cudaSetDevice(ctx->device));
-  int32_t lo = 0, hi = 0;
-  int rc = column_min_max(ctx, t->dev[c], t->n_rows, &lo, &hi);
-  if (rc != HX_OK) return rc;
-  HX_REQUIRE(t->n_rows == 0 || (int64_t)hi - (int64_t)lo < (int64_t(1) << (8 * width)), HX_EINVAL,
-             "hx_table_encode: the column's value range does not fit the width");
-  void* nb = nullptr;
-  HX_CK(cudaMallocAsync(&nb, (((size_t)t->n_rows * width + 255) & ~size_t(255)) + 256, ctx->stream));
-  rc = column_narrow(ctx, t->dev[c], t->n_rows, lo, width, nb);
-  if (rc != HX_OK) {
-    cudaFreeAsync(nb, ctx->stream);
-    return rc;
-  }
-  if (t->owned || ((t->own_mask >> c) & 1u)) cudaFreeAsync(t->dev[c], ctx->stream);
-  t->dev[c] = static_cast<int32_t*>(nb);
-  t->width[c] = (int8_t)width;
-  t->base[c] = t->n_rows ? lo : 0;
-  t->own_mask |= 1u << c;
-  HX_CK(cudaStreamSynchronize(ctx->stream));
   return HX_OK;
 }
 

@@ -306,8 +306,6 @@ int ceil_log2(int64_t x) {
 int ht_create(hx_ctx* ctx, const hx_table* dim, int32_t key_col, const hx_pred* preds,
               int n_preds, int32_t group_col, int32_t group_lo, int32_t group_hi, hx_ht** out,
               int flags) {
-  HX_REQUIRE(dim && !table_narrow(dim), dim ? HX_EUNSUPPORTED : HX_EINVAL,
-             "hx_build_dim_ht: the dimension has narrow-encoded columns (only K1 reads them)");
   HX_REQUIRE(ctx && dim && out, HX_EINVAL, "hx_build_dim_ht: null argument");
   HX_REQUIRE(n_preds >= 0 && n_preds <= HX_MAX_PREDS && (n_preds == 0 || preds), HX_EINVAL,
              "hx_build_dim_ht: bad predicate list");

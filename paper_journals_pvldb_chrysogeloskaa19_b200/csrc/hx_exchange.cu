@@ -351,7 +351,6 @@ int hx_hash_partition(hx_ctx* ctx, const hx_table* t, int32_t key_col, int n_par
   HX_REQUIRE(n_parts >= 1 && n_parts <= HX_MAX_PARTS, HX_EINVAL, "hx_hash_partition: bad n_parts");
   HX_REQUIRE(t->placement == HX_PLACE_COPY || t->placement == HX_PLACE_VIEW, HX_EUNSUPPORTED,
              "hx_hash_partition: the table must be device resident");
-  HX_REQUIRE(!table_narrow(t), HX_EUNSUPPORTED, "hx_hash_partition: the table has narrow-encoded columns");
   HX_REQUIRE(table_has_col(t, key_col), HX_EINVAL, "hx_hash_partition: key column not in table");
   HX_CK(cudaSetDevice(ctx->device));
   hx_table* o = nullptr;

@@ -191,22 +191,7 @@ struct hx_table {
   int placement = HX_PLACE_COPY;
   bool owned = false;              // columns allocated by the library
   const hx_table* parent = nullptr;
-  // narrow encodings (hx_table_encode, §8(f) NEXT-4): bytes per value (4 = plain int32, 2 or
-  // 1 = frame of reference: value = base + unsigned stored value) and the columns the encode
-  // allocated (freed with the table)
-  int8_t width[HX_MAX_COLS];
-  int32_t base[HX_MAX_COLS];
-  uint32_t own_mask = 0;
-  hx_table() {
-    for (int c = 0; c < HX_MAX_COLS; ++c) width[c] = 4, base[c] = 0;
-  }
 };
-// any narrow-encoded column (only K1 reads them; other operators require int32 columns)
-inline bool table_narrow(const hx_table* t) {
-  for (int c = 0; c < t->n_cols; ++c)
-    if (t->width[c] != 4) return true;
-  return false;
-}
 
 struct hx_ht {
   hx_ctx* ctx = nullptr;
@@ -276,9 +261,6 @@ int ht_enable_direct(hx_ctx* ctx, hx_ht* ht, int32_t kmin, uint32_t span, int lw
 int probe_agg(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* shape,
               hx_ht* const* hts, int n_hts, hx_agg* agg, bool fresh);
 int k1_occupancy(hx_ctx* ctx);
-// narrow encodings (hx_encode.cu): the column's [min, max]; (v - base) as width-byte unsigned
-int column_min_max(hx_ctx* ctx, const int32_t* v, int64_t n, int32_t* lo, int32_t* hi);
-int column_narrow(hx_ctx* ctx, const int32_t* v, int64_t n, int32_t base, int width, void* out);
 // host-resident K1 over the blocks a shared router hands out (hx_pipeline_probe_agg_routed)
 int probe_agg_routed(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht* const* hts,
                      int n_hts, hx_agg* agg, hx_shared_router* router, int64_t block_rows,

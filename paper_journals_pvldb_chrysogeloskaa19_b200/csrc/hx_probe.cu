@@ -178,14 +178,6 @@ struct K1Params {
   int32_t l2_hint;                         // 1: probe loads evict_last (0: evict_normal; A/B)
   int32_t ht_seq;                          // hash tables: stage C probes the first remaining
                                            // join alone, the others only for its hits
-  // narrow encodings (hx_table_encode; NW instances): bytes per value, frame-of-reference
-  // base and byte offset in a ring stage of each staged column; bytes of one stage; the row
-  // multiple a bulk copy of every column covers (16 / narrowest width)
-  int8_t col_w[kMaxStageCols];
-  int32_t col_base[kMaxStageCols];
-  int32_t col_off[kMaxStageCols];
-  int32_t stage_bytes;
-  int32_t align_rows;
 };
 
 // join kinds (uniform per launch: read from the kernel parameters)
@@ -425,29 +417,14 @@ struct CarryBuf {
 };
 
 // Entry idx of the combined sequence [carried rows..., this tile's queue...].
-// Staged value of column c at row r of a chunk half whose row 0 is at `half` (NW: the column's
-// bytes at p.col_off[c], widened from p.col_w[c] bytes plus the base; else int32 at c*stride).
-// (NW: `half` is the ring slot's base and hoff the half's first row within the tile.)
-template <bool NW>
-__device__ __forceinline__ int32_t staged_val(const K1Params& p, const int32_t* half, int hoff,
-                                              int stride, int c, int r) {
-  if (!NW) return half[c * stride + r];
-  const unsigned char* cp = reinterpret_cast<const unsigned char*>(half) + p.col_off[c];
-  const int w = p.col_w[c];
-  if (w == 4) return reinterpret_cast<const int32_t*>(cp)[hoff + r];
-  if (w == 2) return p.col_base[c] + (int32_t)reinterpret_cast<const uint16_t*>(cp)[hoff + r];
-  return p.col_base[c] + (int32_t)cp[hoff + r];
-}
-
-template <int NJ, bool DM, bool NW>
+template <int NJ, bool DM>
 __device__ __forceinline__ CarryEntry load_entry(const K1Params& p,
                                                  const JoinState (&js)[HX_MAX_JOINS],
                                                  const CarryBuf* cb, int n_carry,
                                                  const uint8_t* q_row, const int32_t* q_g,
                                                  bool carry_g, const int32_t* wcol0,
                                                  const int32_t* wcol1, uint32_t wrow0,
-                                                 uint32_t wrow1, int stride, int idx,
-                                                 int hoff0 = 0, int hoff1 = 0) {
+                                                 uint32_t wrow1, int stride, int idx) {
   CarryEntry e;
   if (idx < n_carry) {
 #pragma unroll
@@ -460,13 +437,12 @@ __device__ __forceinline__ CarryEntry load_entry(const K1Params& p,
     const int i = idx - n_carry;
     const int q = q_row[i];  // bit 7: which tile of the pair; bits 0-6: row in the warp's slice
     const int32_t* wcol = (q & 128) ? wcol1 : wcol0;
-    const int hoff = (q & 128) ? hoff1 : hoff0;
     const int r = q & 127;
 #pragma unroll
     for (int jx = 0; jx < NJ; ++jx)
-      e.key[jx] = staged_val<NW>(p, wcol, hoff, stride, js[jx].c, r);
-    e.a = p.ga ? 0 : staged_val<NW>(p, wcol, hoff, stride, p.agg_a, r);
-    e.b = p.gb ? 0 : staged_val<NW>(p, wcol, hoff, stride, p.agg_b, r);
+      e.key[jx] = wcol[js[jx].c * stride + r];
+    e.a = p.ga ? 0 : wcol[p.agg_a * stride + r];
+    e.b = p.gb ? 0 : wcol[p.agg_b * stride + r];
     e.g = carry_g ? q_g[i] : 0;
     e.row = ((q & 128) ? wrow1 : wrow0) + (uint32_t)r;
   }
@@ -602,7 +578,7 @@ __device__ __forceinline__ void stage_c_row(const K1Params& p, const JoinState (
 //   stage C  in full batches of 32 queued rows, one row per lane: the remaining filters,
 //            then the lookups / probes of ALL remaining joins issued together (one L2 round
 //            trip), the measure and the group-table atomic.
-template <int NJ, bool GROUPED, bool DM, bool NW = false>
+template <int NJ, bool GROUPED, bool DM>
 __device__ __forceinline__ void process_tile(const K1Params& p, const JoinState (&js)[HX_MAX_JOINS],
                                              const unsigned char* sdm, const int32_t* sbase0,
                                              const int32_t* sbase1, uint32_t frow0,
@@ -612,8 +588,7 @@ __device__ __forceinline__ void process_tile(const K1Params& p, const JoinState 
                                              unsigned long long* s_sum, uint32_t* s_cnt,
                                              uint8_t* q_row, int32_t* q_g, CarryBuf* cb,
                                              int& n_carry, long long& acc_sum,
-                                             long long& acc_cnt, Pending& pd, const Pols& pol,
-                                             int hoff0 = 0, int hoff1 = 0) {
+                                             long long& acc_cnt, Pending& pd, const Pols& pol) {
   constexpr int R = kRowsPerThread;  // rows per lane per tile
   const int wbase = warp * (32 * R);
   const int r0 = wbase + lane * R;
@@ -632,33 +607,6 @@ __device__ __forceinline__ void process_tile(const K1Params& p, const JoinState 
   if (__ballot_sync(kFull, m) == 0) return;
   // the 8 values of staged column c for this lane
   auto load8 = [&](int c, int32_t (&v)[2 * R]) {
-    if (NW) {  // the column at its width: 16, 8 or 4 bytes for the lane's 4 rows of a half
-      const int w = p.col_w[c];
-      const int32_t b = p.col_base[c];
-#pragma unroll
-      for (int h = 0; h < 2; ++h) {
-        const unsigned char* cp = reinterpret_cast<const unsigned char*>(h ? sbase1 : sbase0) +
-                                  p.col_off[c] + (h ? hoff1 : hoff0) * w;
-        if (w == 4) {
-          const int4 x = *reinterpret_cast<const int4*>(cp + r0 * 4);
-          v[h * R + 0] = x.x;
-          v[h * R + 1] = x.y;
-          v[h * R + 2] = x.z;
-          v[h * R + 3] = x.w;
-        } else if (w == 2) {
-          const uint2 x = *reinterpret_cast<const uint2*>(cp + r0 * 2);
-          v[h * R + 0] = b + (int32_t)(x.x & 0xFFFFu);
-          v[h * R + 1] = b + (int32_t)(x.x >> 16);
-          v[h * R + 2] = b + (int32_t)(x.y & 0xFFFFu);
-          v[h * R + 3] = b + (int32_t)(x.y >> 16);
-        } else {
-          const uint32_t x = *reinterpret_cast<const uint32_t*>(cp + r0);
-#pragma unroll
-          for (int k = 0; k < R; ++k) v[h * R + k] = b + (int32_t)((x >> (8 * k)) & 0xFFu);
-        }
-      }
-      return;
-    }
 #pragma unroll
     for (int h = 0; h < 2; ++h) {
       const int4 x = *reinterpret_cast<const int4*>(tb[h] + c * stride);
@@ -876,8 +824,8 @@ __device__ __forceinline__ void process_tile(const K1Params& p, const JoinState 
   const int total = n_carry + qn;
   const int full_end = total & ~31;
   for (int base = 0; base < full_end; base += 32) {
-    CarryEntry e = load_entry<NJ, DM, NW>(p, js, cb, n_carry, q_row, q_g, carry_g, wcol0, wcol1,
-                                          wrow0, wrow1, stride, base + lane, hoff0, hoff1);
+    CarryEntry e = load_entry<NJ, DM>(p, js, cb, n_carry, q_row, q_g, carry_g, wcol0, wcol1,
+                                      wrow0, wrow1, stride, base + lane);
     stage_c_row<NJ, GROUPED, DM>(p, js, sdm, e, j0, jf, smem_table, s_sum, s_cnt, acc_sum, acc_cnt, pd,
                                  pol);
   }
@@ -886,8 +834,8 @@ __device__ __forceinline__ void process_tile(const K1Params& p, const JoinState 
     const bool has = idx < total;
     CarryEntry e{};
     if (has)
-      e = load_entry<NJ, DM, NW>(p, js, cb, n_carry, q_row, q_g, carry_g, wcol0, wcol1, wrow0,
-                                 wrow1, stride, idx, hoff0, hoff1);
+      e = load_entry<NJ, DM>(p, js, cb, n_carry, q_row, q_g, carry_g, wcol0, wcol1, wrow0, wrow1,
+                             stride, idx);
     __syncwarp();
     if (has) {
 #pragma unroll
@@ -939,7 +887,7 @@ __device__ __forceinline__ void mbar_wait_sleep(uint64_t* bar, uint32_t parity) 
   }
 }
 
-template <int NJ, bool GROUPED, bool DM, int W, bool NW = false>
+template <int NJ, bool GROUPED, bool DM, int W>
 #ifndef HX_K1_LB_LO
 #define HX_K1_LB_LO 896  // launch-bound thread count of the 20-warp instances (0: exact):
                          // 896 caps them at 72 registers, measured 0.3-3% faster than 80
@@ -964,7 +912,8 @@ __global__ void __launch_bounds__((W == kWarpsLo && HX_K1_LB_LO) ? HX_K1_LB_LO :
   uint32_t* s_filters = reinterpret_cast<uint32_t*>(smem + kSmemFixed + table_bytes);
   const size_t filter_bytes = ((size_t)p.filter_words * 4 + 127) & ~size_t(127);
   unsigned char* sdm = smem + kSmemFixed + table_bytes + filter_bytes;  // staged direct maps
-  unsigned char* stage0 = sdm + p.dm_bytes;  // ring slot s at stage0 + s * p.stage_bytes
+  int32_t* stage0 = reinterpret_cast<int32_t*>(sdm + p.dm_bytes);
+  const int stage_elems = p.n_cols * kTileRows;
 
   // a failed group layout (capacity, or a plan whose dimensions changed) disables the pass
   if (GROUPED && p.meta->error) return;
@@ -995,34 +944,23 @@ __global__ void __launch_bounds__((W == kWarpsLo && HX_K1_LB_LO) ? HX_K1_LB_LO :
         slot_tile[s] = i;  // slot s now holds (is being filled with) tile i: see the consumers
         const int64_t r0 = t * kTileRows;
         const int64_t rows = std::min<int64_t>(kTileRows, p.n_rows - r0);
-        // every column's bulk copy covers the same whole multiple of align_rows rows (each a
-        // 16-byte multiple at every width); the < align_rows left are read by the consumers
-        const uint32_t crows = (uint32_t)(rows & ~(int64_t)(p.align_rows - 1));
-        uint32_t tx = 0;
-        for (int c = 0; c < p.n_cols; ++c) tx += crows * (NW ? (uint32_t)p.col_w[c] : 4u);
-        mbar_arrive_expect_tx(full + s, tx);
+        const uint32_t bytes = (uint32_t)(rows & ~int64_t(3)) * 4u;
+        mbar_arrive_expect_tx(full + s, bytes * p.n_cols);
         // L2 prefetch of the tile `prefetch` ring refills ahead: its bulk copy then hits L2,
         // so the ring's bytes in flight are not bounded by its free slots alone
         if (p.prefetch) {
           const int64_t tp = t + (int64_t)p.prefetch * gridDim.x;
           if (tp < p.n_tiles) {
             const int64_t rp = tp * kTileRows;
-            const uint32_t pr = (uint32_t)(std::min<int64_t>(kTileRows, p.n_rows - rp) &
-                                           ~(int64_t)(p.align_rows - 1));
-            if (pr)
-              for (int c = 0; c < p.n_cols; ++c) {
-                const uint32_t w = NW ? (uint32_t)p.col_w[c] : 4u;
-                bulk_prefetch_l2(reinterpret_cast<const char*>(p.col[c]) + rp * w, pr * w);
-              }
+            const uint32_t pb = (uint32_t)(std::min<int64_t>(kTileRows, p.n_rows - rp) & ~int64_t(3)) * 4u;
+            if (pb)
+              for (int c = 0; c < p.n_cols; ++c) bulk_prefetch_l2(p.col[c] + rp, pb);
           }
         }
-        if (crows) {
-          unsigned char* dst = stage0 + (size_t)s * p.stage_bytes;
-          for (int c = 0; c < p.n_cols; ++c) {
-            const uint32_t w = NW ? (uint32_t)p.col_w[c] : 4u;
-            bulk_g2s(dst + (NW ? p.col_off[c] : c * kTileRows * 4),
-                     reinterpret_cast<const char*>(p.col[c]) + r0 * w, crows * w, full + s, pol);
-          }
+        if (bytes) {
+          int32_t* dst = stage0 + (size_t)s * stage_elems;
+          for (int c = 0; c < p.n_cols; ++c)
+            bulk_g2s(dst + c * kTileRows, p.col[c] + r0, bytes, full + s, pol);
         }
         if (++s == p.stages) {
           s = 0;
@@ -1158,37 +1096,26 @@ __global__ void __launch_bounds__((W == kWarpsLo && HX_K1_LB_LO) ? HX_K1_LB_LO :
     while (slot_tile[slot] != i)
       if (HX_TAG_SLEEP) __nanosleep(HX_TAG_SLEEP);
     mbar_wait(full + slot, phase);
-    unsigned char* stb = stage0 + (size_t)slot * p.stage_bytes;
-    int32_t* st = reinterpret_cast<int32_t*>(stb);
+    int32_t* st = stage0 + (size_t)slot * stage_elems;
     const int64_t t = blockIdx.x + (int64_t)i * gridDim.x;
     const int64_t r0 = t * kTileRows;
     const int rows = (int)std::min<int64_t>(kTileRows, p.n_rows - r0);
     const int crows = max(0, min(kChunkRows, rows - ch * kChunkRows));
-    const int copied = rows & ~(p.align_rows - 1);
+    const int copied = rows & ~3;
     if (copied != rows && copied / kChunkRows == ch) {
-      // ragged tail: the last < align_rows rows of the table are not a 16-byte multiple at
-      // every width (not copied by the bulk engine); the warp owning their chunk reads them
+      // ragged tail: the last <= 3 rows of the table are not a 16-byte multiple (not copied
+      // by the bulk engine); the warp owning their chunk reads them directly
       if (lane < rows - copied)
-        for (int cc = 0; cc < p.n_cols; ++cc) {
-          if (NW) {
-            const int w = p.col_w[cc];
-            const char* src = reinterpret_cast<const char*>(p.col[cc]) + (r0 + copied + lane) * w;
-            unsigned char* dst = stb + p.col_off[cc] + (copied + lane) * w;
-            for (int b = 0; b < w; ++b) dst[b] = (unsigned char)src[b];
-          } else {
-            st[cc * kTileRows + copied + lane] = p.col[cc][r0 + copied + lane];
-          }
-        }
+        for (int cc = 0; cc < p.n_cols; ++cc)
+          st[cc * kTileRows + copied + lane] = p.col[cc][r0 + copied + lane];
       __syncwarp();
     }
-    // (NW: byte offsets; a chunk's rows are ch * kChunkRows * width bytes into each column)
-    const int32_t* cb0 = NW ? reinterpret_cast<const int32_t*>(stb) : st + ch * kChunkRows;
+    const int32_t* cb0 = st + ch * kChunkRows;
     const uint32_t frow0 = (uint32_t)(p.head_rows + r0 + ch * kChunkRows);
-    process_tile<NJ, GROUPED, DM, NW>(p, js, sdm, cb0, NW ? cb0 : cb0 + kHalfRows, frow0,
-                                      frow0 + kHalfRows, kTileRows, min(crows, kHalfRows),
-                                      max(0, crows - kHalfRows), 0, lane, smem_table, s_sum, s_cnt,
-                                      q_row, q_g, cb, n_carry, acc_sum, acc_cnt, pd, pol,
-                                      ch * kChunkRows, ch * kChunkRows + kHalfRows);
+    process_tile<NJ, GROUPED, DM>(p, js, sdm, cb0, cb0 + kHalfRows, frow0, frow0 + kHalfRows,
+                                  kTileRows, min(crows, kHalfRows),
+                                  max(0, crows - kHalfRows), 0, lane, smem_table, s_sum,
+                                  s_cnt, q_row, q_g, cb, n_carry, acc_sum, acc_cnt, pd, pol);
     __syncwarp();
     if (lane == 0) mbar_arrive(empty + slot);
   }
@@ -1503,29 +1430,16 @@ const KernelFn kKernels[2][2][2][HX_MAX_JOINS + 1] = {
      {HX_K1_ROW(kWarpsHi, false, true), HX_K1_ROW(kWarpsHi, true, true)}}};
 #undef HX_K1_ROW
 
-// instances reading narrow-encoded columns: [warps][direct maps][grouped][joins]
-#define HX_K1_NWROW(W, G, D)                                                                      \
-  {k1_probe_agg<0, G, false, W, true>, k1_probe_agg<1, G, D, W, true>,                            \
-   k1_probe_agg<2, G, D, W, true>, k1_probe_agg<3, G, D, W, true>, k1_probe_agg<4, G, D, W, true>}
-const KernelFn kKernelsNarrow[2][2][2][HX_MAX_JOINS + 1] = {
-    {{HX_K1_NWROW(kWarpsLo, false, false), HX_K1_NWROW(kWarpsLo, true, false)},
-     {HX_K1_NWROW(kWarpsLo, false, true), HX_K1_NWROW(kWarpsLo, true, true)}},
-    {{HX_K1_NWROW(kWarpsHi, false, false), HX_K1_NWROW(kWarpsHi, true, false)},
-     {HX_K1_NWROW(kWarpsHi, false, true), HX_K1_NWROW(kWarpsHi, true, true)}}};
-#undef HX_K1_NWROW
-
-KernelFn pick_kernel(int nj, bool grouped, bool dm, int warps, bool narrow = false) {
-  if (narrow) return kKernelsNarrow[warps == kWarpsHi ? 1 : 0][dm ? 1 : 0][grouped ? 1 : 0][nj];
+KernelFn pick_kernel(int nj, bool grouped, bool dm, int warps) {
   return kKernels[warps == kWarpsHi ? 1 : 0][dm ? 1 : 0][grouped ? 1 : 0][nj];
 }
 
-// (row_bytes: the staged columns' bytes per row, 4 per int32 column)
-size_t k1_smem_bytes(int warps, bool dm, int row_bytes, int stages, int smem_groups,
+size_t k1_smem_bytes(int warps, bool dm, int n_cols, int stages, int smem_groups,
                      int filter_words = 0, int dm_bytes = 0, bool in_place = false) {
   const size_t table_bytes = ((size_t)smem_groups * 12 + 127) & ~size_t(127);
   const size_t filter_bytes = ((size_t)filter_words * 4 + 127) & ~size_t(127);
   return (in_place ? kSmemQueueOff : smem_fixed(dm, warps)) + table_bytes + filter_bytes + (size_t)dm_bytes +
-         (size_t)stages * row_bytes * kTileRows;
+         (size_t)stages * n_cols * kTileRows * sizeof(int32_t);
 }
 
 // Per-CTA shared memory for `ctas` resident CTAs per SM (228 KB per SM, 1 KB reserved each).
@@ -1545,13 +1459,13 @@ size_t k1_smem_cap() {
   return cap;
 }
 
-int pick_stages(int warps, bool dm, int row_bytes, int smem_groups) {
+int pick_stages(int warps, bool dm, int n_cols, int smem_groups) {
   // as many tile stages as fit next to kCtasPerSm CTAs per SM, at least double buffering
   // (at most HX_K1_STAGE_KB of tiles per CTA: the rest is left for filters and maps)
   const size_t fixed = smem_fixed(dm, warps) + (((size_t)smem_groups * 12 + 127) & ~size_t(127));
   const size_t budget = std::min<size_t>(std::min(smem_budget(kCtasPerSm), k1_smem_cap()),
                                          fixed + HX_K1_STAGE_KB * 1024);
-  const size_t stage = (size_t)row_bytes * kTileRows;
+  const size_t stage = (size_t)n_cols * kTileRows * 4;
   const int s = budget > fixed ? (int)((budget - fixed) / stage) : 0;
   return std::max(2, std::min(4, s));
 }
@@ -1701,12 +1615,6 @@ int k1_occupancy(hx_ctx* ctx) {
           for (int j = 0; j <= HX_MAX_JOINS; ++j)
             cudaFuncSetAttribute(kKernels[w][d][g][j], cudaFuncAttributeMaxDynamicSharedMemorySize,
                                  227 * 1024);
-    for (int w = 0; w < 2; ++w)
-      for (int d = 0; d < 2; ++d)
-        for (int g = 0; g < 2; ++g)
-          for (int j = 0; j <= HX_MAX_JOINS; ++j)
-            cudaFuncSetAttribute(kKernelsNarrow[w][d][g][j],
-                                 cudaFuncAttributeMaxDynamicSharedMemorySize, 227 * 1024);
     cudaFuncSetAttribute(k1_scan_agg<1>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)scan_smem(1));
     cudaFuncSetAttribute(k1_scan_agg<2>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)scan_smem(2));
     cudaFuncSetAttribute(k1_scan_agg<3>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)scan_smem(3));
@@ -1716,7 +1624,7 @@ int k1_occupancy(hx_ctx* ctx) {
   int occ = 0;
   cudaOccupancyMaxActiveBlocksPerMultiprocessor(
       &occ, k1_probe_agg<3, true, false, kWarpsLo>, k1_threads(kWarpsLo),
-      k1_smem_bytes(kWarpsLo, false, 16, pick_stages(kWarpsLo, false, 16, kSmemGroups), kSmemGroups));
+      k1_smem_bytes(kWarpsLo, false, 4, pick_stages(kWarpsLo, false, 4, kSmemGroups), kSmemGroups));
   return occ;
 }
 
@@ -1746,7 +1654,6 @@ struct K1Prepared {
   int64_t seg_rows = kSegRows;  // rows per launch (HX_K1_SEG_TILES overrides, for tests)
   int carveout = 100;           // preferred shared-memory carveout (% of 228 KB)
   int warps = kWarpsLo;         // consumer warps of the chosen instance
-  int row_bytes = 0;            // staged bytes per row (4 per int32 column; less when narrow)
   double cost = -1.0;           // plan cost (direct maps; -1: hash tables)
   L2Window win;                 // persisting window over the largest L2-read probe structure
 };
@@ -1892,14 +1799,8 @@ int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht*
     HX_REQUIRE(table_has_col(fact, sh->agg_a) &&
                    (sh->agg_op == HX_AGG_SUM || table_has_col(fact, sh->agg_b)),
                HX_EINVAL, "hx_pipeline_probe_agg: measure column not in fact table");
-    auto int32_col = [&](int32_t col) {  // (gathers read plain int32 columns)
-      for (int i = 0; i < fact->n_cols; ++i)
-        if (fact->col_id[i] == col) return fact->width[i] == 4;
-      return false;
-    };
-    p.ga = ok && !read_by_stages(sh->agg_a) && int32_col(sh->agg_a);
-    p.gb = sh->agg_op == HX_AGG_SUM ? p.ga
-                                    : (ok && !read_by_stages(sh->agg_b) && int32_col(sh->agg_b));
+    p.ga = ok && !read_by_stages(sh->agg_a);
+    p.gb = sh->agg_op == HX_AGG_SUM ? p.ga : (ok && !read_by_stages(sh->agg_b));
     p.gat_a = p.ga ? table_col(fact, sh->agg_a) : nullptr;
     p.gat_b = p.gb ? table_col(fact, sh->agg_op == HX_AGG_SUM ? sh->agg_a : sh->agg_b) : nullptr;
   }
@@ -1932,26 +1833,6 @@ int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht*
     p.head_col[c] = table_col(fact, ids[c]);
     p.col[c] = p.head_col[c] + head;
   }
-  // staged column widths (narrow encodings, hx_table_encode): byte offsets within a ring stage,
-  // the stage's bytes and the row multiple every column's bulk copy covers
-  bool narrow = false;
-  int row_bytes = 0, min_w = 4;
-  for (int c = 0; c < n_cols; ++c) {
-    int w = 4, b = 0;
-    for (int i = 0; i < fact->n_cols; ++i)
-      if (fact->col_id[i] == ids[c]) w = fact->width[i], b = fact->base[i];
-    p.col_w[c] = (int8_t)w;
-    p.col_base[c] = b;
-    p.col_off[c] = row_bytes * kTileRows;
-    row_bytes += w;
-    min_w = std::min(min_w, w);
-    narrow = narrow || w != 4;
-  }
-  p.stage_bytes = row_bytes * kTileRows;
-  p.align_rows = 16 / min_w;
-  HX_REQUIRE(!narrow || (head == 0 && !k.host && !k.mapped), HX_EUNSUPPORTED,
-             "hx_pipeline_probe_agg: narrow-encoded columns must be device resident and aligned");
-  k.row_bytes = row_bytes;
   p.head_rows = (int32_t)head;
   p.n_rows = fact->n_rows - head;
   p.n_tiles = (p.n_rows + kTileRows - 1) / kTileRows;
@@ -1969,7 +1850,7 @@ int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht*
   auto plan_with = [&](const int W, K1Prepared& k) {
     K1Params& p = k.p;
     t_smem_cap = 0;
-    p.stages = pick_stages(W, dm_mode, row_bytes, p.smem_groups);
+    p.stages = pick_stages(W, dm_mode, n_cols, p.smem_groups);
     int kind[HX_MAX_JOINS] = {kStNone, kStNone, kStNone, kStNone};
     int bloom_w[HX_MAX_JOINS] = {0, 0, 0, 0};
     int in_s[HX_MAX_JOINS] = {0, 0, 0, 0};
@@ -1993,7 +1874,7 @@ int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht*
         if (kd[j] == kStBitmap) db += d.bm_words * 4;
         if (kd[j] == kStBloom) fw += bw[j];
       }
-      return k1_smem_bytes(W, dm_mode, row_bytes, p.stages, p.smem_groups, fw, db) <=
+      return k1_smem_bytes(W, dm_mode, n_cols, p.stages, p.smem_groups, fw, db) <=
              k1_smem_cap();
     };
     double plan_cost = -1.0;
@@ -2009,8 +1890,8 @@ int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht*
       // 3-stage ring (no pairs) gave Q4.1 5.03; plans below the threshold — every SF10/SF100
       // plan — lose with the cap).
       if (plan_cost > kL1BoundCost && !std::getenv("HX_K1_SMEM_KB")) {
-        t_smem_cap = std::max<size_t>(164 * 1024, k1_smem_bytes(W, dm_mode, row_bytes, 4, p.smem_groups));
-        p.stages = pick_stages(W, dm_mode, row_bytes, p.smem_groups);
+        t_smem_cap = std::max<size_t>(164 * 1024, k1_smem_bytes(W, dm_mode, n_cols, 4, p.smem_groups));
+        p.stages = pick_stages(W, dm_mode, n_cols, p.smem_groups);
         for (int j = 0; j < HX_MAX_JOINS; ++j) kind[j] = kStNone, bloom_w[j] = 0, in_s[j] = 0;
         plan_cost = plan_dm(sh->n_joins, p.joins, known, pass, keys, bloom_w0, grouped_j,
                             fits_sizes, kind, bloom_w, in_s);
@@ -2097,7 +1978,7 @@ int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht*
       int max_stages = 8;
       if (const char* e = std::getenv("HX_K1_MAX_STAGES")) max_stages = std::max(2, std::min(8, std::atoi(e)));
       while (p.stages < max_stages &&
-             k1_smem_bytes(W, dm_mode, row_bytes, p.stages + 1, p.smem_groups, p.filter_words, p.dm_bytes,
+             k1_smem_bytes(W, dm_mode, n_cols, p.stages + 1, p.smem_groups, p.filter_words, p.dm_bytes,
                            in_place) <= k1_smem_cap())
         ++p.stages;
     }
@@ -2152,11 +2033,11 @@ int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht*
       std::fprintf(stderr, " in_s:");
       for (int j = 0; j < sh->n_joins; ++j) std::fprintf(stderr, "%d", p.joins[j].in_s);
       std::fprintf(stderr, " l2:%x l2s:%x cost=%.2f stages=%d smem=%zu\n", p.m_l2, p.m_l2s, plan_cost, p.stages,
-                   k1_smem_bytes(W, dm_mode, row_bytes, p.stages, p.smem_groups, p.filter_words, p.dm_bytes,
+                   k1_smem_bytes(W, dm_mode, n_cols, p.stages, p.smem_groups, p.filter_words, p.dm_bytes,
                                  in_place));
     }
-    k.fn = pick_kernel(sh->n_joins, grouped, p.m_dm != 0u, W, narrow);
-    k.smem = k1_smem_bytes(W, dm_mode, row_bytes, p.stages, p.smem_groups, p.filter_words, p.dm_bytes,
+    k.fn = pick_kernel(sh->n_joins, grouped, p.m_dm != 0u, W);
+    k.smem = k1_smem_bytes(W, dm_mode, n_cols, p.stages, p.smem_groups, p.filter_words, p.dm_bytes,
                            in_place);
     // the smallest shared-memory carveout that holds the plan: the rest of the SM's L1/shared
     // array caches the maps read from L2
@@ -2192,7 +2073,7 @@ int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht*
     const long long t = std::atoll(e);
     if (t > 0 && t <= (1LL << 20)) k.seg_rows = t * kTileRows;
   }
-  if (sh->n_joins == 0 && n_cols >= 1 && n_cols <= 4 && !k.host && !narrow &&
+  if (sh->n_joins == 0 && n_cols >= 1 && n_cols <= 4 && !k.host &&
       std::getenv("HX_NO_SCAN") == nullptr) {
     const KernelFn scans[4] = {k1_scan_agg<1>, k1_scan_agg<2>, k1_scan_agg<3>, k1_scan_agg<4>};
     k.scan = scans[n_cols - 1];
@@ -2398,7 +2279,7 @@ int k1_enqueue(hx_ctx* ctx, const K1Prepared* k, bool fresh, cudaEvent_t e0, cud
 }
 
 void k1_free(K1Prepared* k) { delete k; }
-int64_t k1_bytes(const K1Prepared* k) { return k->rows * k->row_bytes; }
+int64_t k1_bytes(const K1Prepared* k) { return k->rows * 4 * k->n_cols; }
 int k1_gathered_cols(const K1Prepared* k) {
   return k->p.ga + (k->p.agg_op != HX_AGG_SUM && k->p.gb ? 1 : 0);
 }

@@ -161,10 +161,6 @@ class Table:
         call("hx_table_slice", self.h, row_begin, row_end, ctypes.byref(h))
         return Table(self.ctx, h, parent=self)
 
-    def encode(self, col_id: int, width: int) -> None:
-        """hx_table_encode: store the column in `width` (1 or 2) bytes, frame of reference."""
-        call("hx_table_encode", self.h, col_id, width)
-
     def read(self, col_id: int, row_begin: int = 0, n: Optional[int] = None) -> np.ndarray:
         """Rows of one column, copied to the host (synchronous)."""
         if n is None:

@@ -325,23 +325,6 @@ def order_by(plan: Plan, rows: List[Tuple]) -> List[Tuple]:
     return sorted(rows, key=lambda r: r[:-2])
 
 
-# ---- narrow encodings ------------------------------------------------
-def narrow_fact(fact: hx.Table, cols=None) -> Dict[str, int]:
-    """Encode every lineorder column whose value range fits 1 or 2 bytes (hx_table_encode:
-    frame of reference; only K1 reads them). -> {column: width} of the encoded columns."""
-    done = {}
-    for c in cols or ssbgen.TABLE_COLS["lineorder"]:
-        for w in (1, 2):
-            try:
-                fact.encode(C[c], w)
-                done[c] = w
-                break
-            except hx._hx.HxError as e:
-                if e.code != _hx.HX_EINVAL:
-                    raise
-    return done
-
-
 # ---- loading an SSB database onto one GPU --------------------------------------------------
 def load_db_numpy(ctx: hx.Context, db: Dict[str, Dict[str, np.ndarray]],
                   part: Optional[hx.Partition] = None, part_index: int = 0):
