@@ -1903,19 +1903,40 @@ int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht*
       if (all_l2s) t_smem_cap = 100 * 1024;
     } else {
       // hash tables: selective joins (at most half the dimension passes), most selective first,
-      // get a Bloom filter (folded to 4 or 2 bits per key when the full one does not fit)
+      // get a Bloom filter (folded to 4 or 2 bits per key when the full one does not fit).
+      // The ring gives up a stage when that lets more selective joins carry a filter of >= 4
+      // bits per key (measured at SF100: Q2.1 3.10 -> 2.55 ms, Q4.1 10.3 -> 8.5, Q4.2 5.3 ->
+      // 4.4; plans that already had their filters lose 5-15% with the shallower ring)
       int ord[HX_MAX_JOINS] = {0, 1, 2, 3};
       std::stable_sort(ord, ord + sh->n_joins, [&](int x, int y) { return pass[x] < pass[y]; });
-      for (int i = 0; i < sh->n_joins; ++i) {
-        const int j = ord[i];
-        if (!known[j] || 2 * pass[j] > 1.0) continue;
-        for (int f = 1; f <= 8 && kind[j] == kStNone && bloom_w0[j] / f >= 4; f *= 2) {
-          kind[j] = kStBloom;
-          bloom_w[j] = bloom_w0[j] / f;
-          if (!fits_sizes(kind, bloom_w)) {
-            kind[j] = kStNone;
-            bloom_w[j] = 0;
+      auto allocate = [&]() {  // greedy Bloom budget at the current ring depth -> good filters
+        int good = 0;
+        for (int j = 0; j < HX_MAX_JOINS; ++j) kind[j] = kStNone, bloom_w[j] = 0;
+        for (int i = 0; i < sh->n_joins; ++i) {
+          const int j = ord[i];
+          if (!known[j] || 2 * pass[j] > 1.0) continue;
+          for (int f = 1; f <= 8 && kind[j] == kStNone && bloom_w0[j] / f >= 4; f *= 2) {
+            kind[j] = kStBloom;
+            bloom_w[j] = bloom_w0[j] / f;
+            if (!fits_sizes(kind, bloom_w)) {
+              kind[j] = kStNone;
+              bloom_w[j] = 0;
+            }
           }
+          good += kind[j] == kStBloom && 32.0 * bloom_w[j] >= 4.0 * (double)keys[j];
+        }
+        return good;
+      };
+      const int stages0 = p.stages;
+      const int good0 = allocate();
+      int ht_stages = stages0 > 3 ? 3 : stages0;
+      if (const char* e = std::getenv("HX_HT_STAGES")) ht_stages = std::max(2, std::min(stages0, std::atoi(e)));
+      if (ht_stages < stages0) {
+        p.stages = ht_stages;
+        const int good1 = allocate();
+        if (good1 <= good0 && !std::getenv("HX_HT_STAGES")) {  // no better: keep the deeper ring
+          p.stages = stages0;
+          allocate();
         }
       }
     }
