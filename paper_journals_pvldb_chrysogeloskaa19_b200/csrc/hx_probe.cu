@@ -1077,8 +1077,18 @@ __global__ void __launch_bounds__((W == kWarpsLo && HX_K1_LB_LO) ? HX_K1_LB_LO :
   const int64_t my_chunks = my_tiles * kChunksPerTile;
   // (measured and rejected: claiming the next chunk before processing the current one, or
   // during its stage C — a reserved chunk waits for its warp and holds its stage back)
-  int c = 0, span_left = 0;
+#ifndef HX_DYNAMIC_CHUNKS
+  // warp w takes chunks w, w + W, w + 2W, ... of the CTA's range: no claim atomic on a
+  // chunk's critical path (SF100 step 19.77 -> 19.47 ms); the tile tags still
+  // release each ring slot when its last chunk is done
+  int c = warp - kConsumerWarps;
+#else
+  int c = 0, span_left = 0;  // A/B: chunks claimed from a shared counter
+#endif
   while (true) {
+#ifndef HX_DYNAMIC_CHUNKS
+    c += kConsumerWarps;
+#else
     if (span_left == 0) {  // HX_CLAIM_SPAN consecutive chunks per shared atomic
       if (lane == 0) c = atomicAdd(next_chunk, HX_CLAIM_SPAN);
       c = __shfl_sync(kFull, c, 0);
@@ -1087,6 +1097,7 @@ __global__ void __launch_bounds__((W == kWarpsLo && HX_K1_LB_LO) ? HX_K1_LB_LO :
       ++c;
     }
     --span_left;
+#endif
     if (c >= my_chunks) break;
     const int i = c / kChunksPerTile, ch = c - i * kChunksPerTile;
     // (tracking slot and phase incrementally instead of dividing by the ring depth was
@@ -2043,6 +2054,7 @@ int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht*
         k.win.hit_ratio = (float)std::min(1.0, (double)ctx->l2_persist_max / (double)k.win.bytes);
     }
     if (const char* e = std::getenv("HX_K1_PREFETCH")) p.prefetch = std::max(0, std::min(64, std::atoi(e)));
+
     if (std::getenv("HX_DEBUG")) {  // launch plan of this K1 (tuning aid)
       std::fprintf(stderr, "[hx] K1 warps=%d joins=%d cols=%d gather=%d%d stages=%d groups=%d filters:",
                    W, sh->n_joins, n_cols, p.ga, p.gb, p.stages, p.smem_groups);

@@ -20,9 +20,12 @@ ap = argparse.ArgumentParser()
 ap.add_argument("--sf", type=float, default=10)
 ap.add_argument("--queries", default="all")
 ap.add_argument("--reps", type=int, default=5)
+ap.add_argument("--join", default="auto", choices=["auto", "hash"], help="HX_OPT_JOIN_LAYOUT")
 ap.add_argument("--lo-rows", type=int, default=0, help="first rows of lineorder only (SF1000 dims)")
 a = ap.parse_args()
 ctx = hx.Context(0)
+if a.join == "hash":
+    ctx.set_option(hx._hx.HX_OPT_JOIN_LAYOUT, hx._hx.HX_JOIN_HASH)
 qs = ssb.QUERIES if a.queries == "all" else a.queries.split(",")
 need = set().union(*(ssb.FACT_COLS[q] for q in qs))
 dims, fact = device_db(ctx, ssbgen.sizes(a.sf), lo_rows=a.lo_rows or None,
