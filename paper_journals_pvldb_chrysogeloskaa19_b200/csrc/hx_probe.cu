@@ -176,8 +176,10 @@ struct K1Params {
                                            // shared-memory structure: exact verdict + rank)
   uint32_t m_res;                          // resolved in stage S (full map staged, or m_l2s)
   int32_t l2_hint;                         // 1: probe loads evict_last (0: evict_normal; A/B)
-  int32_t ht_seq;                          // hash tables: stage C probes the first remaining
-                                           // join alone, the others only for its hits
+  int32_t ht_seq;                          // hash tables: stage C probes one join alone (ht_first
+                                           // if still pending, else the first), the others
+                                           // only for its hits
+  int32_t ht_first;
 };
 
 // join kinds (uniform per launch: read from the kernel parameters)
@@ -520,11 +522,12 @@ __device__ __forceinline__ void stage_c_row(const K1Params& p, const JoinState (
     if (GROUPED) gg += (int32_t)v * js[jx].jstride;
   }
   if (!alive) pend = 0;
-  // (hash tables, HX_HT_SEQ) the first remaining join alone, the others only for its hits:
+  // (hash tables, p.ht_seq) one join alone (p.ht_first, the likeliest miss), the others only for its hits:
   // the open-addressing tables are large and mostly missed, so fewer probes beat one round trip
   uint32_t later = 0;
   if ((HX_HT_SEQ || p.ht_seq) && !DM) {
-    const uint32_t first = pend & (0u - pend);
+    const uint32_t fb = 1u << p.ht_first;
+    const uint32_t first = (pend & fb) ? fb : pend & (0u - pend);
     later = pend & ~first;
     pend = first;
   }
@@ -1951,14 +1954,34 @@ int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht*
         }
       }
     }
-    // hash tables: probe the first stage-C join alone when it is selective and has no Bloom
-  // filter (its misses then save the other probes; with a filter its conditional pass
-  // fraction is high and one round trip for all is cheaper; measured at SF100: HT Q4.1
-  // 15.5 -> 10.2 ms, Q3.1 5.1 -> 4.8, while Q2.1 / Q4.3 lose 5-9% when forced)
+    // hash tables: stage C probes the join a row most likely fails (given that it passed
+  // every Bloom filter) alone, and the others only for its hits, when that saves at least
+  // kHtSeqMin probes per row (the second round trip costs one L2 latency per batch).
+  // Measured at SF100 (saved -> K1 ms): Q4.1 0.62: 8.74 -> 5.97, Q3.1 0.42: 4.70 -> 3.78;
+  // Q4.2 0.18: 4.67 -> 5.09 and Q2.1 0.09: 2.93 -> 3.18 lose.
+  constexpr double kHtSeqMin = 0.3;
   p.ht_seq = 0;
+  p.ht_first = 0;
+  double ht_saved = 0.0;
   if (!dm_mode && sh->n_joins > 1) {
     const int j0 = (p.n_preds == 0 && kind[0] != kStBloom) ? 1 : 0;  // stage B probes join 0
-    p.ht_seq = j0 < sh->n_joins && kind[j0] != kStBloom && known[j0] && pass[j0] < 0.5;
+    double f_c = 1.0, cmin = 2.0;
+    int ht_first_c = j0;
+    for (int j = j0; j < sh->n_joins; ++j) {
+      double c = known[j] ? pass[j] : 1.0;
+      if (kind[j] == kStBloom) {
+        const double fp = bloom_fp(32.0 * bloom_w[j] / (double)std::max<int64_t>(1, keys[j]));
+        f_c *= c + (1.0 - c) * fp;
+        c = c / std::max(1e-9, c + (1.0 - c) * fp);
+      }
+      if (c < cmin) cmin = c, ht_first_c = j;
+    }
+    // probes per row saved by probing it alone: (stage-C joins - 1) x its miss fraction
+    ht_saved = f_c * (sh->n_joins - j0 - 1) * (1.0 - cmin);
+    double min_saved = kHtSeqMin;
+    if (const char* e = std::getenv("HX_HT_FIRST_MIN")) min_saved = std::atof(e);
+    p.ht_seq = ht_saved >= min_saved;
+    p.ht_first = ht_first_c;
   }
   if (const char* e = std::getenv("HX_HT_SEQ")) p.ht_seq = std::atoi(e) != 0;
   // offsets: Bloom filters in the filter region, maps and bitmaps in the direct-map region
@@ -2065,6 +2088,7 @@ int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht*
                      p.joins[j].dm_smem, p.joins[j].bm_words, p.joins[j].bm_smem);
       std::fprintf(stderr, " in_s:");
       for (int j = 0; j < sh->n_joins; ++j) std::fprintf(stderr, "%d", p.joins[j].in_s);
+      std::fprintf(stderr, " ht_seq=%d first=%d saved=%.3f", p.ht_seq, p.ht_first, ht_saved);
       std::fprintf(stderr, " l2:%x l2s:%x cost=%.2f stages=%d smem=%zu\n", p.m_l2, p.m_l2s, plan_cost, p.stages,
                    k1_smem_bytes(W, dm_mode, n_cols, p.stages, p.smem_groups, p.filter_words, p.dm_bytes,
                                  in_place));

@@ -44,6 +44,41 @@ def test_parity_small_sf(ctx, sf, seed):
         assert got[q] == oracle.run_query(q, db), q
 
 
+@pytest.fixture(scope="module")
+def sf005():
+    db = ssbgen.database(7, ssbgen.sizes(0.05))
+    return db, {q: oracle.run_query(q, db) for q in QUERIES}
+
+
+@pytest.mark.parametrize("seq_min", [None, "0", "99"])
+@pytest.mark.parametrize("layout", ["auto", "hash"])
+@pytest.mark.parametrize("warps", ["20", "26"])
+def test_k1_instances_and_probe_schedules(sf005, monkeypatch, warps, layout, seq_min):
+    """Both consumer-warp instances (HX_K1_W), the direct maps and the hash tables
+    (HX_OPT_JOIN_LAYOUT, prepared plans), and the hash-table stage-C schedules: the planner's choice, every
+    plan probing its likeliest-miss join alone first (HX_HT_FIRST_MIN=0), and all joins in one
+    round trip (=99) — all bit-exact against the oracle over 30 K1 tiles plus a ragged tail."""
+    db, want = sf005
+    monkeypatch.setenv("HX_K1_W", warps)
+    if seq_min is not None:
+        monkeypatch.setenv("HX_HT_FIRST_MIN", seq_min)
+    c = hx.Context(0)
+    try:
+        if layout == "hash":
+            c.set_option(_hx.HX_OPT_JOIN_LAYOUT, _hx.HX_JOIN_HASH)
+        dims, fact = ssb.load_db_numpy(c, db)
+        eng = ssb.SsbEngine(c, dims, fact)
+        for q in QUERIES:  # prepared plans (the bench's path; they pick direct maps under auto)
+            pl = eng.plan(q)
+            pl.enqueue()
+            assert pl.rows() == want[q], (q, warps, layout, seq_min)
+            pl.close()
+        for q in QUERIES:  # the unprepared calls (hash tables)
+            assert eng.run(q) == want[q], (q, warps, layout, seq_min)
+    finally:
+        c.close()
+
+
 def test_parity_handcrafted(ctx, handcrafted):
     db, expect = handcrafted
     got = run_all(ctx, db)

@@ -3,5 +3,5 @@
 sf=$1; shift
 for e in "$@"; do
   echo "== $e"
-  env $e timeout 600 python tools/time_queries.py --sf $sf --reps 5 2>&1 | awk '{printf "%s %s  ", $1, $6} END {print ""}'
+  env $e timeout 600 python tools/time_queries.py --sf $sf --reps 5 --join ${JOIN:-auto} 2>&1 | awk '{printf "%s %s  ", $1, $6} END {print ""}'
 done

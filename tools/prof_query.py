@@ -41,8 +41,11 @@ def main():
     ap.add_argument("--queries", default="q1.1,q2.1,q3.1,q4.1")
     ap.add_argument("--reps", type=int, default=2)
     ap.add_argument("--lo-rows", type=int, default=0, help="first rows of lineorder only")
+    ap.add_argument("--join", default="auto", choices=["auto", "hash"], help="HX_OPT_JOIN_LAYOUT")
     a = ap.parse_args()
     ctx = hx.Context(0, torch.cuda.current_stream().cuda_stream)
+    if a.join == "hash":
+        ctx.set_option(_hx.HX_OPT_JOIN_LAYOUT, _hx.HX_JOIN_HASH)
     qs = ssb.QUERIES if a.queries == "all" else a.queries.split(",")
     need = set().union(*(ssb.FACT_COLS[q] for q in qs))
     dims, fact = device_db(ctx, ssbgen.sizes(a.sf), lo_rows=a.lo_rows or None,
