@@ -61,6 +61,12 @@ constexpr int kWarpsLo = 20, kWarpsHi = 26;
 #ifndef HX_BALLOT_COMPACT
 #define HX_BALLOT_COMPACT 0  // survivors' queue slots from 8 ballots instead of a shuffle scan
 #endif
+#ifndef HX_DM_STATIC_CHUNKS
+#define HX_DM_STATIC_CHUNKS 1  // chunk assignment of the direct-map instances (0: claimed)
+#endif
+#ifndef HX_HT_STATIC_CHUNKS
+#define HX_HT_STATIC_CHUNKS 1  // ... of the hash-table instances
+#endif
 #ifndef HX_HT_SEQ
 #define HX_HT_SEQ 0       // hash-table joins probed one round trip per join in stage C
 #endif
@@ -1080,27 +1086,27 @@ __global__ void __launch_bounds__((W == kWarpsLo && HX_K1_LB_LO) ? HX_K1_LB_LO :
   const int64_t my_chunks = my_tiles * kChunksPerTile;
   // (measured and rejected: claiming the next chunk before processing the current one, or
   // during its stage C — a reserved chunk waits for its warp and holds its stage back)
-#ifndef HX_DYNAMIC_CHUNKS
-  // warp w takes chunks w, w + W, w + 2W, ... of the CTA's range: no claim atomic on a
-  // chunk's critical path (SF100 step 19.77 -> 19.47 ms); the tile tags still
-  // release each ring slot when its last chunk is done
-  int c = warp - kConsumerWarps;
-#else
-  int c = 0, span_left = 0;  // A/B: chunks claimed from a shared counter
-#endif
+  // Direct-map instances: warp w takes chunks w, w + W, w + 2W, ... of the CTA's range, no
+  // claim atomic on a chunk's critical path (SF100 step 19.77 -> 19.47 ms); the
+  // tile tags still release each ring slot when its last chunk is done. Hash-table instances:
+  // the same for up to 3 joins; with 4 (Q4.x: the most variable stage C) chunks are claimed
+  // from a shared counter, in order (measured at SF100: HT Q4.1 5.98 -> 5.62 ms, Q4.2 4.68 ->
+  // 4.44, Q4.3 2.61 -> 2.48; Q2.x/Q3.x lose 2-6% with claims).
+  constexpr bool kStatic = DM ? HX_DM_STATIC_CHUNKS : (HX_HT_STATIC_CHUNKS && NJ < 4);
+  int c = kStatic ? warp - kConsumerWarps : 0, span_left = 0;
   while (true) {
-#ifndef HX_DYNAMIC_CHUNKS
-    c += kConsumerWarps;
-#else
-    if (span_left == 0) {  // HX_CLAIM_SPAN consecutive chunks per shared atomic
-      if (lane == 0) c = atomicAdd(next_chunk, HX_CLAIM_SPAN);
-      c = __shfl_sync(kFull, c, 0);
-      span_left = HX_CLAIM_SPAN;
+    if constexpr (kStatic) {
+      c += kConsumerWarps;
     } else {
-      ++c;
+      if (span_left == 0) {  // HX_CLAIM_SPAN consecutive chunks per shared atomic
+        if (lane == 0) c = atomicAdd(next_chunk, HX_CLAIM_SPAN);
+        c = __shfl_sync(kFull, c, 0);
+        span_left = HX_CLAIM_SPAN;
+      } else {
+        ++c;
+      }
+      --span_left;
     }
-    --span_left;
-#endif
     if (c >= my_chunks) break;
     const int i = c / kChunksPerTile, ch = c - i * kChunksPerTile;
     // (tracking slot and phase incrementally instead of dividing by the ring depth was
