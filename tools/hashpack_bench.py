@@ -26,6 +26,7 @@ ap = argparse.ArgumentParser()
 ap.add_argument("--sf", type=float, default=10)
 ap.add_argument("--parts", type=int, default=8)
 ap.add_argument("--reps", type=int, default=5)
+ap.add_argument("--no-join", action="store_true", help="time the hash-pack only")
 a = ap.parse_args()
 s = torch.cuda.Stream()
 torch.cuda.set_stream(s)
@@ -46,7 +47,7 @@ out["hashpack_ms"] = best * 1e3
 out["hashpack_gbps"] = alg / best / 1e9
 out["hashpack_alg_bytes"] = alg
 eng = ssb.SsbEngine(ctx, dims, fact)
-for q in ("q3.1", "q4.1"):
+for q in (() if a.no_join else ("q3.1", "q4.1")):
     for mode in ("broadcast", "partitioned"):
         ts = []
         for _ in range(a.reps):
