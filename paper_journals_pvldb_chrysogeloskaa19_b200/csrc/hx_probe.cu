@@ -74,6 +74,9 @@ constexpr int kWarpsLo = 20, kWarpsHi = 26;
 #define HX_TAG_SLEEP 0    // ns slept between polls of a ring slot's tile tag (0: spin; measured
                           // 0.5% faster than 20 ns)
 #endif
+#ifndef HX_PROD_SLEEP
+#define HX_PROD_SLEEP 128  // ns the producer sleeps between polls of a slot's empty barrier
+#endif
 #ifndef HX_K1_CTAS
 #define HX_K1_CTAS 1    // resident CTAs per SM the launch bounds / smem budget target
                         // (one CTA per SM shares one copy of the Bloom filters)
@@ -104,16 +107,22 @@ constexpr int kSmemGroups = 1024;          // per-CTA group table capacity
 // Bloom filters | direct maps | tile ring]. (The ungrouped final reduce writes the warps' partials
 // at kSmemQueueOff once every consumer is done — all of those regions are dead by then — so it
 // needs no region of its own.)
-constexpr int kSmemBarOff = 0;                                    // 2 x 8 stages x 8 B
-constexpr int kSmemHeadOff = 128;
+// ring depth cap and the depth pick_stages starts from, in tiles: the same bytes (4 x 2560 rows)
+// whatever the tile size
+constexpr int kMaxStages = 8 * 2560 / kTileRows;  // 80 KB per column
+static_assert(kMaxStages >= 2 && kMaxStages <= 16, "ring depth");
+constexpr int kBaseStages = (4 * 2560 + kTileRows - 1) / kTileRows;
+static_assert(kBaseStages <= kMaxStages, "ring");
+constexpr int kSmemBarOff = 0;                                    // 2 x kMaxStages x 8 B
+constexpr int kSmemHeadOff = 2 * kMaxStages * 8;
 constexpr int kSmemHeadBytes = 128;                               // kMaxStageCols x 4 x 4 B
 // chunk scheduling: [next chunk counter | ring slot tags (the tile each slot was last filled
 // with) x 8]
 constexpr int kSmemCtlOff = kSmemHeadOff + kSmemHeadBytes;
-constexpr int kSmemCtlBytes = 64;
-constexpr int kSmemQueueOff = kSmemCtlOff + kSmemCtlBytes;       // 320
-static_assert(kSmemHeadOff - kSmemBarOff >= 2 * 8 * 8, "barriers overlap the head rows");
-static_assert(kSmemCtlBytes >= 4 * (1 + 8), "counter + 8 slot tags");
+constexpr int kSmemCtlBytes = (4 * (1 + kMaxStages) + 63) & ~63;
+constexpr int kSmemQueueOff = kSmemCtlOff + kSmemCtlBytes;       // 320 (2560-row tiles)
+static_assert(kSmemHeadOff - kSmemBarOff >= 2 * kMaxStages * 8, "barriers overlap the head rows");
+static_assert(kSmemCtlBytes >= 4 * (1 + kMaxStages), "counter + slot tags");
 static_assert(kSmemQueueOff % 64 == 0, "queues / carry buffers / group table alignment");
 constexpr int kQueueRows = 2 * kRowsPerThread * 32;       // per warp: one tile pair's rows
 constexpr int kCarryBytes = (HX_MAX_JOINS + 4) * 32 * 4;  // one CarryBuf per consumer warp
@@ -147,7 +156,9 @@ struct JoinDev {
 struct K1Params {
   const int32_t* col[kMaxStageCols];       // staged fact columns (table base + head offset)
   int32_t n_cols;
-  int32_t stages;                          // tile ring depth (4..8)
+  int32_t stages;                          // tile ring depth (kBaseStages..kMaxStages)
+  uint32_t stage_magic;                    // floor(2^32 / stages) + 1: i / stages = umulhi(i, magic)
+                                           // exactly for i < 2^32 / stages (a CTA has < 2^21 tiles)
   int32_t prefetch;                        // L2 prefetch distance in tiles of this CTA (0: off)
   int32_t smem_fixed;                      // bytes before the group table (no per-warp queues
                                            // when every join resolves in stage S)
@@ -892,7 +903,7 @@ __device__ __forceinline__ void mbar_wait_sleep(uint64_t* bar, uint32_t parity) 
         : "r"(smem_u32(bar)), "r"(parity)
         : "memory");
     if (ok) return;
-    __nanosleep(128);
+    if (HX_PROD_SLEEP) __nanosleep(HX_PROD_SLEEP);
   }
 }
 
@@ -1110,9 +1121,11 @@ __global__ void __launch_bounds__((W == kWarpsLo && HX_K1_LB_LO) ? HX_K1_LB_LO :
     if (c >= my_chunks) break;
     const int i = c / kChunksPerTile, ch = c - i * kChunksPerTile;
     // (tracking slot and phase incrementally instead of dividing by the ring depth was
-    // measured 3% slower: the loop-carried registers cost more than the division)
-    const int slot = i % p.stages;
-    const uint32_t phase = (uint32_t)(i / p.stages) & 1u;
+    // measured 3% slower: the loop-carried registers cost more than the division; the division
+    // is a multiply-high by the ring depth's reciprocal, not the ~20-instruction runtime divide)
+    const uint32_t lap = __umulhi((uint32_t)i, p.stage_magic);
+    const int slot = i - (int)lap * p.stages;
+    const uint32_t phase = lap & 1u;
     while (slot_tile[slot] != i)
       if (HX_TAG_SLEEP) __nanosleep(HX_TAG_SLEEP);
     mbar_wait(full + slot, phase);
@@ -1487,7 +1500,7 @@ int pick_stages(int warps, bool dm, int n_cols, int smem_groups) {
                                          fixed + HX_K1_STAGE_KB * 1024);
   const size_t stage = (size_t)n_cols * kTileRows * 4;
   const int s = budget > fixed ? (int)((budget - fixed) / stage) : 0;
-  return std::max(2, std::min(4, s));
+  return std::max(2, std::min(kBaseStages, s));
 }
 
 enum { kStNone = 0, kStFull, kStBitmap, kStBloom };
@@ -1568,7 +1581,10 @@ double plan_dm(int nj, const JoinDev* joins, const bool* known, const double* pa
       kd[j] = opts[j][idx[j]].kind;
       bw[j] = opts[j][idx[j]].bw;
     }
-    if (fits(kd, bw)) {
+    // a plan that resolves every join in stage S aggregates in place and needs no per-warp
+    // queues or carry buffers: it is checked against that smaller footprint
+    const bool fits_q = fits(kd, bw, false), fits_ip = fits_q || fits(kd, bw, true);
+    if (fits_ip) {
       // every subset of the joins may run in stage S: a join with a shared-memory structure
       // applies it there; one without reads its map from L2 there (exact, like a full map)
       const uint32_t has = (1u << nj) - 1u;
@@ -1583,6 +1599,10 @@ double plan_dm(int nj, const JoinDev* joins, const bool* known, const double* pa
             fS *= kd[j] == kStNone ? (known[j] ? pass[j] : 1.0) : opts[j][idx[j]].e;
           }
           all_res = all_res && ((S >> j) & 1u) && (kd[j] == kStFull || kd[j] == kStNone);
+        }
+        if (!all_res && !fits_q) {
+          if (S == 0) break;
+          continue;
         }
         if (!all_res) {
           cost += K.c * fS;
@@ -1886,7 +1906,7 @@ int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht*
       pass[j] = (double)ht->known_keys / (double)std::max<int64_t>(1, ht->dim_rows);
       bloom_w0[j] = std::max(4, 1 << std::min(ht->max_bloom_log2w, bloom_log2w_for(ht->known_keys)));
     }
-    auto fits_sizes = [&](const int* kd, const int* bw) {
+    auto fits_sizes = [&](const int* kd, const int* bw, bool in_place) {
       int fw = 0, db = 0;
       for (int j = 0; j < sh->n_joins; ++j) {
         const JoinDev& d = p.joins[j];
@@ -1894,7 +1914,7 @@ int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht*
         if (kd[j] == kStBitmap) db += d.bm_words * 4;
         if (kd[j] == kStBloom) fw += bw[j];
       }
-      return k1_smem_bytes(W, dm_mode, n_cols, p.stages, p.smem_groups, fw, db) <=
+      return k1_smem_bytes(W, dm_mode, n_cols, p.stages, p.smem_groups, fw, db, in_place) <=
              k1_smem_cap();
     };
     double plan_cost = -1.0;
@@ -1910,7 +1930,7 @@ int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht*
       // 3-stage ring (no pairs) gave Q4.1 5.03; plans below the threshold — every SF10/SF100
       // plan — lose with the cap).
       if (plan_cost > kL1BoundCost && !std::getenv("HX_K1_SMEM_KB")) {
-        t_smem_cap = std::max<size_t>(164 * 1024, k1_smem_bytes(W, dm_mode, n_cols, 4, p.smem_groups));
+        t_smem_cap = std::max<size_t>(164 * 1024, k1_smem_bytes(W, dm_mode, n_cols, kBaseStages, p.smem_groups));
         p.stages = pick_stages(W, dm_mode, n_cols, p.smem_groups);
         for (int j = 0; j < HX_MAX_JOINS; ++j) kind[j] = kStNone, bloom_w[j] = 0, in_s[j] = 0;
         plan_cost = plan_dm(sh->n_joins, p.joins, known, pass, keys, bloom_w0, grouped_j,
@@ -1938,7 +1958,7 @@ int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht*
           for (int f = 1; f <= 8 && kind[j] == kStNone && bloom_w0[j] / f >= 4; f *= 2) {
             kind[j] = kStBloom;
             bloom_w[j] = bloom_w0[j] / f;
-            if (!fits_sizes(kind, bloom_w)) {
+            if (!fits_sizes(kind, bloom_w, false)) {
               kind[j] = kStNone;
               bloom_w[j] = 0;
             }
@@ -1949,7 +1969,8 @@ int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht*
       };
       const int stages0 = p.stages;
       const int good0 = allocate();
-      int ht_stages = stages0 > 3 ? 3 : stages0;
+      const int ht3 = (3 * kBaseStages + 3) / 4;  // 3/4 of the base ring
+      int ht_stages = stages0 > ht3 ? ht3 : stages0;
       if (const char* e = std::getenv("HX_HT_STAGES")) ht_stages = std::max(2, std::min(stages0, std::atoi(e)));
       if (ht_stages < stages0) {
         p.stages = ht_stages;
@@ -2030,23 +2051,25 @@ int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht*
       }
     }
     // a pipeline whose joins all resolve in stage S aggregates in place: no per-warp queues or
-    // carry buffers. Shared memory the plan left over deepens the tile ring (up to 8 stages:
+    // carry buffers. Shared memory the plan left over deepens the tile ring (up to 80 KB per column:
     // more bytes in flight per SM while the consumers hold a pair of tiles).
     const bool in_place = sh->n_joins == 0 ||
                           (dm_mode && p.m_res == (1u << sh->n_joins) - 1u);
     p.smem_fixed = in_place ? kSmemQueueOff : smem_fixed(dm_mode, W);
     {
-      int max_stages = 8;
-      if (const char* e = std::getenv("HX_K1_MAX_STAGES")) max_stages = std::max(2, std::min(8, std::atoi(e)));
+      int max_stages = kMaxStages;
+      if (const char* e = std::getenv("HX_K1_MAX_STAGES")) max_stages = std::max(2, std::min(kMaxStages, std::atoi(e)));
       while (p.stages < max_stages &&
              k1_smem_bytes(W, dm_mode, n_cols, p.stages + 1, p.smem_groups, p.filter_words, p.dm_bytes,
                            in_place) <= k1_smem_cap())
         ++p.stages;
     }
+    p.stage_magic = (uint32_t)((uint64_t(1) << 32) / (uint64_t)p.stages + 1);
     // (measured, SF10: a distance of 2 gains 4-7% on the 4-column pipelines whose ring stays at
     // 4 stages, and loses 3-6% on 3-column ones, whose rings are deeper or whose tiles are
     // consumed faster)
-    p.prefetch = (n_cols >= 4 && p.stages <= 4 && fact->placement != HX_PLACE_HOST_MAPPED) ? 2 : 0;
+    p.prefetch = (n_cols >= 4 && p.stages <= kBaseStages && fact->placement != HX_PLACE_HOST_MAPPED)
+                     ? 2 * kBaseStages / 4 : 0;
     // L2 residency of the probe structures (north_star; PAPER.md:1016-1022 operator state in
     // device memory): probe loads carry an evict_last hint, and the largest structure K1 reads
     // from L2 (a direct map not staged in shared memory, or a hash table's slots) gets a
@@ -2115,7 +2138,7 @@ int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht*
   // cost model's per-row issue cost; tolerance measured) or the ring is shallower
   double tol = 1.10;
   if (const char* e = std::getenv("HX_K1_W_TOL")) tol = std::atof(e);
-  bool hi = k_hi.p.stages >= std::min(k_lo.p.stages, 4) &&
+  bool hi = k_hi.p.stages >= std::min(k_lo.p.stages, kBaseStages) &&
             (dm_mode ? k_hi.cost <= k_lo.cost * tol + 1e-9
                      : k_hi.p.filter_words >= k_lo.p.filter_words);
   // (an L2-lookup-bound plan runs with a reduced carveout so that L1 caches its map reads:
