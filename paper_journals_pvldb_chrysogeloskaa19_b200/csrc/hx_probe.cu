@@ -70,9 +70,12 @@ constexpr int kWarpsLo = 20, kWarpsHi = 26;
 #ifndef HX_HT_SEQ
 #define HX_HT_SEQ 0       // hash-table joins probed one round trip per join in stage C
 #endif
-#ifndef HX_TAG_SLEEP
-#define HX_TAG_SLEEP 0    // ns slept between polls of a ring slot's tile tag (0: spin; measured
-                          // 0.5% faster than 20 ns)
+#ifndef HX_TAG_SLEEP_DM
+#define HX_TAG_SLEEP_DM 32  // ns slept between polls of a ring slot's tile tag, direct-map
+                            // instances (measured at SF100: K1 sum -0.55% vs spinning)
+#endif
+#ifndef HX_TAG_SLEEP_HT
+#define HX_TAG_SLEEP_HT 0   // ... hash-table instances (0: spin; 32 ns measured +1.9%)
 #endif
 #ifndef HX_PROD_SLEEP
 #define HX_PROD_SLEEP 128  // ns the producer sleeps between polls of a slot's empty barrier
@@ -1126,8 +1129,9 @@ __global__ void __launch_bounds__((W == kWarpsLo && HX_K1_LB_LO) ? HX_K1_LB_LO :
     const uint32_t lap = __umulhi((uint32_t)i, p.stage_magic);
     const int slot = i - (int)lap * p.stages;
     const uint32_t phase = lap & 1u;
+    constexpr int kTagSleep = DM ? HX_TAG_SLEEP_DM : HX_TAG_SLEEP_HT;
     while (slot_tile[slot] != i)
-      if (HX_TAG_SLEEP) __nanosleep(HX_TAG_SLEEP);
+      if (kTagSleep) __nanosleep(kTagSleep);
     mbar_wait(full + slot, phase);
     int32_t* st = stage0 + (size_t)slot * stage_elems;
     const int64_t t = blockIdx.x + (int64_t)i * gridDim.x;
@@ -1528,7 +1532,12 @@ struct K1Cost {
   // 16 per row (fitted at SF10-SF100, where such reads follow a selective shared-memory
   // filter) made SF1000 plans read 2-15 MB maps for every row; charging the live fraction
   // keeps the SF100 plans and picks the Bloom-filtered plans at SF1000 (Q2.1 2.2x, Q3.2 2.2x).
-  double s = 8.0, c = 60.0, sc = 8.0, l2 = 20.0, s2 = 40.0;
+  // c: 60 fitted at SF10 (r01); 120 measured better or equal at SF10, SF100 and SF1000
+  // dimensions (profiles/r02_cost_model_sweep.txt: SF100 K1 sum 19.29 -> 19.23 ms, SF1000 dims
+  // 24.76 -> 24.53; Q2.1 then filters with the supplier bitmap in stage S as well: 1.80 -> 1.70
+  // ms at SF100, 2.00 -> 1.77 at SF1000). (90 and 150 lose on Q4.2/Q4.3: the landscape is not
+  // smooth — the constants rank discrete plans.)
+  double s = 8.0, c = 120.0, sc = 8.0, l2 = 20.0, s2 = 40.0;
 };
 K1Cost k1_cost() {
   K1Cost k;

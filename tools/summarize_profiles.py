@@ -55,6 +55,24 @@ def main(tag, rep, launches, sf="10", probe_csv=None):
                    f"{d[c('launch__registers_per_thread')]} |")
     out += ["", f"Sum over the 13 launches: {tt:.0f} us; algorithmic {ta/1e9:.2f} GB; DRAM {tr/1e9:.2f} GB "
                 f"(traffic/algorithmic {tr/ta:.3f}; below 1 where late materialisation gathers measure columns for passing rows only)."]
+    # speed of light per unit: which resource bounds each launch (ncu % of peak; a launch with no
+    # unit near 100% is latency-bound: too few loads in flight for its request pattern)
+    sol = [("issue", "smsp__issue_active.avg.pct_of_peak_sustained_active"),
+           ("SM", "sm__throughput.avg.pct_of_peak_sustained_elapsed"),
+           ("L1TEX", "l1tex__throughput.avg.pct_of_peak_sustained_active"),
+           ("L2", "lts__throughput.avg.pct_of_peak_sustained_elapsed"),
+           ("DRAM", "gpu__dram_throughput.avg.pct_of_peak_sustained_elapsed")]
+    out += ["", "Speed of light (ncu, % of each unit's peak) and the instruction mix per lineorder row:", "",
+            "| query | " + " | ".join(n + " %" for n, _ in sol) + " | top unit | warp instr / row | global-load sectors / row | shared wavefronts / row |",
+            "|---|" + "---|" * (len(sol) + 4)]
+    for q, d in zip(QS, data):
+        v = [float(d[c(m)] or 0) for _, m in sol]
+        top = max(range(len(sol)), key=lambda i: v[i])
+        inst = float(d[c("smsp__inst_executed.sum")] or 0)
+        gld = float(d[c("l1tex__t_sectors_pipe_lsu_mem_global_op_ld.sum")] or 0)
+        shw = float(d[c("l1tex__data_pipe_lsu_wavefronts_mem_shared.sum")] or 0)
+        out.append(f"| {q} | " + " | ".join(f"{x:.1f}" for x in v) +
+                   f" | {sol[top][0]} | {inst / N:.2f} | {gld / N:.3f} | {shw / N:.3f} |")
     with open(os.path.join(ROOT, "profiles", f"{tag}_k1_ncu_summary.md"), "w") as f:
         f.write("\n".join(out) + "\n")
     with open(os.path.join(ROOT, "profiles", "k1_traffic.json"), "w") as f:
