@@ -2020,6 +2020,25 @@ int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht*
     p.ht_first = ht_first_c;
   }
   if (const char* e = std::getenv("HX_HT_SEQ")) p.ht_seq = std::atoi(e) != 0;
+  // hash tables: stage B probes join 0 in place for the rows the stage-F Bloom filter passed
+  // (no lineorder predicate, join 0 unfiltered). When join 0 carries the filter instead, the
+  // join stage C would probe alone (rule 1) — or the most selective unfiltered join passing
+  // at most half the rows (rule 2, HX_HT_INPLACE=2) — is moved to the front of the probe order
+  // (results do not depend on it; the group layout follows the grouping joins wherever they
+  // sit), so that it is probed in place, 4 loads in flight per lane, instead of in stage C.
+  // Measured at SF100 (profiles/r02_ab_reentry.txt): 3 joins, Q3.1 3.79 -> 3.00 ms; with 4
+  // joins (Q4.1 5.58 -> 7.04, rule 2 also Q4.2/Q4.3) it loses, so it is limited to <= 3 joins.
+  int ht_inplace = -1;
+  if (!dm_mode && sh->n_joins > 1 && sh->n_joins <= 3 && p.n_preds == 0 && kind[0] == kStBloom) {
+    int rule = 1;
+    if (const char* e = std::getenv("HX_HT_INPLACE")) rule = std::atoi(e);
+    if (rule == 1 && p.ht_seq && kind[p.ht_first] != kStBloom) ht_inplace = p.ht_first;
+    if (rule == 2) {
+      double best = 0.5 + 1e-9;
+      for (int j = 0; j < sh->n_joins; ++j)
+        if (kind[j] != kStBloom && known[j] && pass[j] < best) best = pass[j], ht_inplace = j;
+    }
+  }
   // offsets: Bloom filters in the filter region, maps and bitmaps in the direct-map region
     p.filter_words = 0;
     p.dm_bytes = 0;
@@ -2126,11 +2145,21 @@ int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht*
                      p.joins[j].dm_smem, p.joins[j].bm_words, p.joins[j].bm_smem);
       std::fprintf(stderr, " in_s:");
       for (int j = 0; j < sh->n_joins; ++j) std::fprintf(stderr, "%d", p.joins[j].in_s);
-      std::fprintf(stderr, " ht_seq=%d first=%d saved=%.3f", p.ht_seq, p.ht_first, ht_saved);
+      std::fprintf(stderr, " ht_seq=%d first=%d saved=%.3f inplace=%d", p.ht_seq, p.ht_first, ht_saved, ht_inplace);
       std::fprintf(stderr, " l2:%x l2s:%x cost=%.2f stages=%d smem=%zu\n", p.m_l2, p.m_l2s, plan_cost, p.stages,
                    k1_smem_bytes(W, dm_mode, n_cols, p.stages, p.smem_groups, p.filter_words, p.dm_bytes,
                                  in_place));
     }
+    if (ht_inplace > 0) {  // rotate join ht_inplace to the front (hash-table plans: no masks)
+      const int jb = ht_inplace;
+      auto mapj = [jb](int j) { return j == jb ? 0 : (j < jb ? j + 1 : j); };
+      const JoinDev moved = p.joins[jb];
+      for (int j = jb; j > 0; --j) p.joins[j] = p.joins[j - 1];
+      p.joins[0] = moved;
+      for (int g = 0; g < sh->n_gdims; ++g) (&k.gj.x)[g] = mapj((&k.gj.x)[g]);
+      p.ht_first = mapj(p.ht_first);
+    }
+    if (ht_inplace >= 0) p.ht_seq = 0;
     k.fn = pick_kernel(sh->n_joins, grouped, p.m_dm != 0u, W);
     k.smem = k1_smem_bytes(W, dm_mode, n_cols, p.stages, p.smem_groups, p.filter_words, p.dm_bytes,
                            in_place);

@@ -79,6 +79,34 @@ def test_k1_instances_and_probe_schedules(sf005, monkeypatch, warps, layout, seq
         c.close()
 
 
+@pytest.mark.parametrize("rule", ["1", "2"])
+def test_hash_plans_join_probed_in_place(sf005, monkeypatch, capfd, rule):
+    """Hash-table plans that move a selective unfiltered join to the front of the probe order
+    so that stage B probes it in place after the stage-F Bloom filter (HX_HT_INPLACE; with
+    HX_HT_FIRST_MIN=0 every multi-join plan qualifies for rule 1): under rule 1 the rotation must
+    happen for some plan (HX_DEBUG prints it); every query stays bit-exact against the oracle."""
+    db, want = sf005
+    monkeypatch.setenv("HX_HT_INPLACE", rule)
+    monkeypatch.setenv("HX_HT_FIRST_MIN", "0")
+    monkeypatch.setenv("HX_DEBUG", "1")
+    c = hx.Context(0)
+    try:
+        c.set_option(_hx.HX_OPT_JOIN_LAYOUT, _hx.HX_JOIN_HASH)
+        dims, fact = ssb.load_db_numpy(c, db)
+        eng = ssb.SsbEngine(c, dims, fact)
+        for q in QUERIES:
+            pl = eng.plan(q)
+            pl.enqueue()
+            assert pl.rows() == want[q], (q, rule)
+            pl.close()
+    finally:
+        c.close()
+    err = capfd.readouterr().err
+    moved = [ln for ln in err.splitlines() if "inplace=" in ln and "inplace=-1" not in ln]
+    if rule == "1":  # (rule 2 needs a selective join too large for a Bloom filter: SF100-sized)
+        assert moved, "no plan probed a moved join in place"
+
+
 def test_parity_handcrafted(ctx, handcrafted):
     db, expect = handcrafted
     got = run_all(ctx, db)
