@@ -915,7 +915,14 @@ template <int NJ, bool GROUPED, bool DM, int W>
 #define HX_K1_LB_LO 896  // launch-bound thread count of the 20-warp instances (0: exact):
                          // 896 caps them at 72 registers, measured 0.3-3% faster than 80
 #endif
-__global__ void __launch_bounds__((W == kWarpsLo && HX_K1_LB_LO) ? HX_K1_LB_LO : k1_threads(W), kCtasPerSm)
+#ifndef HX_K1_LB_LO_HT
+#define HX_K1_LB_LO_HT 0  // ... of the 20-warp hash-table instances (0: exact, 80 registers:
+                          // no spills with 3 joins; see kWarpsHi's choice in k1_setup)
+#endif
+__global__ void __launch_bounds__((W == kWarpsLo && (DM ? HX_K1_LB_LO : HX_K1_LB_LO_HT))
+                                      ? (DM ? HX_K1_LB_LO : HX_K1_LB_LO_HT)
+                                      : k1_threads(W),
+                                  kCtasPerSm)
     k1_probe_agg(const __grid_constant__ K1Params p) {
   constexpr int kConsumerWarps = W;
   constexpr int kConsumers = W * 32;
@@ -2029,7 +2036,10 @@ int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht*
   // Measured at SF100 (profiles/r02_ab_reentry.txt): 3 joins, Q3.1 3.79 -> 3.00 ms; with 4
   // joins (Q4.1 5.58 -> 7.04, rule 2 also Q4.2/Q4.3) it loses, so it is limited to <= 3 joins.
   int ht_inplace = -1;
-  if (!dm_mode && sh->n_joins > 1 && sh->n_joins <= 3 && p.n_preds == 0 && kind[0] == kStBloom) {
+  int ht_inplace_maxj = 3;
+  if (const char* e = std::getenv("HX_HT_INPLACE_MAXJ")) ht_inplace_maxj = std::atoi(e);
+  if (!dm_mode && sh->n_joins > 1 && sh->n_joins <= ht_inplace_maxj && p.n_preds == 0 &&
+      kind[0] == kStBloom) {
     int rule = 1;
     if (const char* e = std::getenv("HX_HT_INPLACE")) rule = std::atoi(e);
     if (rule == 1 && p.ht_seq && kind[p.ht_first] != kStBloom) ht_inplace = p.ht_first;
@@ -2183,6 +2193,15 @@ int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht*
   // the extra warps' queues take from that L1 and their misses thrash it — SF1000 Q4.1
   // measured 6.16 ms with 26 warps vs 4.11 with 20, same plan)
   if (dm_mode && k_lo.cost > kL1BoundCost) hi = false;
+  // hash tables: the 20-warp instances run at 80 registers (the 26-warp ones at 72, spilling
+  // with 3-4 joins); 26 warps pay where latency hiding dominates — stage B probing a join in
+  // place for most rows, or 4 joins — and 20 where stage C's per-row work does (measured at
+  // SF100, profiles/r02_ab_reentry.txt: Q2.1 3.26 -> 2.61 ms, Q3.2 2.92 -> 1.95 with 20;
+  // Q3.1 in place 2.97 vs 3.03, Q4.1 5.56 vs 5.71 with 26)
+  if (!dm_mode && sh->n_joins >= 2 && sh->n_joins <= 3) {
+    const bool stage_b = k_hi.p.n_preds == 0 && k_hi.p.joins[0].bloom_words == 0;
+    if (!stage_b) hi = false;
+  }
   if (const char* e = std::getenv("HX_K1_W")) hi = std::atoi(e) == kWarpsHi;
   k = hi ? k_hi : k_lo;
   t_smem_cap = 0;
