@@ -45,6 +45,10 @@ constexpr unsigned kFull = 0xFFFFFFFFu;
 // buffers take shared memory from the filters and maps (measured at SF100: 26 warps 4.5%
 // faster than 20 in sum; SF10 Q4.1 loses its customer bitmap with 26 and is 30% slower).
 constexpr int kWarpsLo = 20, kWarpsHi = 26;
+#ifndef HX_WARPS_HI_HT
+#define HX_WARPS_HI_HT 26
+#endif
+constexpr int kWarpsHiHt = HX_WARPS_HI_HT;  // the hash-table instances' larger warp count
 #ifndef HX_K1_STAGE_KB
 #define HX_K1_STAGE_KB 160  // max shared memory for the tile ring (the rest: Bloom filters)
 #endif
@@ -1470,12 +1474,12 @@ cudaError_t launch_k1(KernelFn fn, int grid, int block, size_t smem, cudaStream_
 const KernelFn kKernels[2][2][2][HX_MAX_JOINS + 1] = {
     {{HX_K1_ROW(kWarpsLo, false, false), HX_K1_ROW(kWarpsLo, true, false)},
      {HX_K1_ROW(kWarpsLo, false, true), HX_K1_ROW(kWarpsLo, true, true)}},
-    {{HX_K1_ROW(kWarpsHi, false, false), HX_K1_ROW(kWarpsHi, true, false)},
+    {{HX_K1_ROW(kWarpsHiHt, false, false), HX_K1_ROW(kWarpsHiHt, true, false)},
      {HX_K1_ROW(kWarpsHi, false, true), HX_K1_ROW(kWarpsHi, true, true)}}};
 #undef HX_K1_ROW
 
 KernelFn pick_kernel(int nj, bool grouped, bool dm, int warps) {
-  return kKernels[warps == kWarpsHi ? 1 : 0][dm ? 1 : 0][grouped ? 1 : 0][nj];
+  return kKernels[warps == kWarpsLo ? 0 : 1][dm ? 1 : 0][grouped ? 1 : 0][nj];
 }
 
 size_t k1_smem_bytes(int warps, bool dm, int n_cols, int stages, int smem_groups,
@@ -2181,7 +2185,7 @@ int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht*
   };
   K1Prepared k_lo = k, k_hi = k;
   plan_with(kWarpsLo, k_lo);
-  plan_with(kWarpsHi, k_hi);
+  plan_with(dm_mode ? kWarpsHi : kWarpsHiHt, k_hi);
   // more warps unless the plan they leave room for is costlier by more than kWarpsTol (the
   // cost model's per-row issue cost; tolerance measured) or the ring is shallower
   double tol = 1.10;
@@ -2202,7 +2206,7 @@ int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht*
     const bool stage_b = k_hi.p.n_preds == 0 && k_hi.p.joins[0].bloom_words == 0;
     if (!stage_b) hi = false;
   }
-  if (const char* e = std::getenv("HX_K1_W")) hi = std::atoi(e) == kWarpsHi;
+  if (const char* e = std::getenv("HX_K1_W")) hi = std::atoi(e) != kWarpsLo;
   k = hi ? k_hi : k_lo;
   t_smem_cap = 0;
   int occ = 0;
