@@ -71,6 +71,9 @@ constexpr int kWarpsHiHt = HX_WARPS_HI_HT;  // the hash-table instances' larger 
 #ifndef HX_HT_STATIC_CHUNKS
 #define HX_HT_STATIC_CHUNKS 1  // ... of the hash-table instances
 #endif
+#ifndef HX_HT_CLAIM_NJ
+#define HX_HT_CLAIM_NJ 4  // hash-table instances with at least this many joins claim chunks
+#endif
 #ifndef HX_HT_SEQ
 #define HX_HT_SEQ 0       // hash-table joins probed one round trip per join in stage C
 #endif
@@ -1117,7 +1120,10 @@ __global__ void __launch_bounds__((W == kWarpsLo && (DM ? HX_K1_LB_LO : HX_K1_LB
   // the same for up to 3 joins; with 4 (Q4.x: the most variable stage C) chunks are claimed
   // from a shared counter, in order (measured at SF100: HT Q4.1 5.98 -> 5.62 ms, Q4.2 4.68 ->
   // 4.44, Q4.3 2.61 -> 2.48; Q2.x/Q3.x lose 2-6% with claims).
-  constexpr bool kStatic = DM ? HX_DM_STATIC_CHUNKS : (HX_HT_STATIC_CHUNKS && NJ < 4);
+  // (hash tables with 4 joins: the 26-warp instance claims, the 20-warp one is static — the
+  // planner launches the latter when stage B probes a join in place: SF100 Q4.1 5.61 -> 4.95 ms)
+  constexpr bool kStatic =
+      DM ? HX_DM_STATIC_CHUNKS : (HX_HT_STATIC_CHUNKS && (NJ < HX_HT_CLAIM_NJ || W == kWarpsLo));
   int c = kStatic ? warp - kConsumerWarps : 0, span_left = 0;
   while (true) {
     if constexpr (kStatic) {
@@ -2037,10 +2043,10 @@ int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht*
   // at most half the rows (rule 2, HX_HT_INPLACE=2) — is moved to the front of the probe order
   // (results do not depend on it; the group layout follows the grouping joins wherever they
   // sit), so that it is probed in place, 4 loads in flight per lane, instead of in stage C.
-  // Measured at SF100 (profiles/r02_ab_reentry.txt): 3 joins, Q3.1 3.79 -> 3.00 ms; with 4
-  // joins (Q4.1 5.58 -> 7.04, rule 2 also Q4.2/Q4.3) it loses, so it is limited to <= 3 joins.
+  // Measured at SF100 (profiles/r02_ab_reentry.txt): 3 joins, Q3.1 3.79 -> 3.00 ms; 4 joins,
+  // Q4.1 5.61 -> 4.95 with the 20-warp static-chunk instance (7.04 with the claiming one).
   int ht_inplace = -1;
-  int ht_inplace_maxj = 3;
+  int ht_inplace_maxj = 4;
   if (const char* e = std::getenv("HX_HT_INPLACE_MAXJ")) ht_inplace_maxj = std::atoi(e);
   if (!dm_mode && sh->n_joins > 1 && sh->n_joins <= ht_inplace_maxj && p.n_preds == 0 &&
       kind[0] == kStBloom) {
@@ -2206,6 +2212,10 @@ int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht*
     const bool stage_b = k_hi.p.n_preds == 0 && k_hi.p.joins[0].bloom_words == 0;
     if (!stage_b) hi = false;
   }
+  // (4 joins: the claiming 26-warp instance unless stage B probes in place, which the static
+  // 20-warp one does best)
+  if (!dm_mode && sh->n_joins == 4 && k_lo.p.n_preds == 0 && k_lo.p.joins[0].bloom_words == 0)
+    hi = false;
   if (const char* e = std::getenv("HX_K1_W")) hi = std::atoi(e) != kWarpsLo;
   k = hi ? k_hi : k_lo;
   t_smem_cap = 0;
