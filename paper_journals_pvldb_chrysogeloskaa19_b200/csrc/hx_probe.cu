@@ -2039,8 +2039,9 @@ int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht*
   if (const char* e = std::getenv("HX_HT_SEQ")) p.ht_seq = std::atoi(e) != 0;
   // hash tables: stage B probes join 0 in place for the rows the stage-F Bloom filter passed
   // (no lineorder predicate, join 0 unfiltered). When join 0 carries the filter instead, the
-  // join stage C would probe alone (rule 1) — or the most selective unfiltered join passing
-  // at most half the rows (rule 2, HX_HT_INPLACE=2) — is moved to the front of the probe order
+  // join stage C would probe alone (rule 1) — or else the most selective unfiltered join
+  // passing at most half the rows (rule 2; HX_HT_INPLACE = 0 off, 1, 2, 3 both: default) — is
+  // moved to the front of the probe order
   // (results do not depend on it; the group layout follows the grouping joins wherever they
   // sit), so that it is probed in place, 4 loads in flight per lane, instead of in stage C.
   // Measured at SF100 (profiles/r02_ab_reentry.txt): 3 joins, Q3.1 3.79 -> 3.00 ms; 4 joins,
@@ -2050,13 +2051,23 @@ int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht*
   if (const char* e = std::getenv("HX_HT_INPLACE_MAXJ")) ht_inplace_maxj = std::atoi(e);
   if (!dm_mode && sh->n_joins > 1 && sh->n_joins <= ht_inplace_maxj && p.n_preds == 0 &&
       kind[0] == kStBloom) {
-    int rule = 1;
+    int rule = 3;
     if (const char* e = std::getenv("HX_HT_INPLACE")) rule = std::atoi(e);
-    if (rule == 1 && p.ht_seq && kind[p.ht_first] != kStBloom) ht_inplace = p.ht_first;
-    if (rule == 2) {
+    if ((rule & 1) && p.ht_seq && kind[p.ht_first] != kStBloom) ht_inplace = p.ht_first;
+    // rule 2: the most selective unfiltered join (pass <= 1/2) — when the stage-C Bloom
+    // filters of the other joins keep at least 1/10 of the rows stage F passed (else stage C
+    // would probe that join for far fewer rows than stage B: Q4.3 2.40 -> 2.91 ms; Q4.2, whose
+    // stage-C filters keep 0.29, 4.38 -> 3.72)
+    if ((rule & 2) && ht_inplace < 0) {
+      double keep = 1.0;
+      for (int j = 1; j < sh->n_joins; ++j)
+        if (kind[j] == kStBloom && known[j])
+          keep *= pass[j] + (1.0 - pass[j]) *
+                                bloom_fp(32.0 * bloom_w[j] / (double)std::max<int64_t>(1, keys[j]));
       double best = 0.5 + 1e-9;
-      for (int j = 0; j < sh->n_joins; ++j)
-        if (kind[j] != kStBloom && known[j] && pass[j] < best) best = pass[j], ht_inplace = j;
+      if (keep >= 0.1)
+        for (int j = 0; j < sh->n_joins; ++j)
+          if (kind[j] != kStBloom && known[j] && pass[j] < best) best = pass[j], ht_inplace = j;
     }
   }
   // offsets: Bloom filters in the filter region, maps and bitmaps in the direct-map region
