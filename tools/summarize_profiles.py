@@ -22,13 +22,15 @@ BROW = {"1": 16, "2": 16, "3": 16, "4": 24}
 
 def main(tag, rep, launches, sf="10", probe_csv=None):
     global N
+    launches = None if launches == "-" else launches
     N = int(6_000_000 * float(sf))
     raw = (open(rep).read() if rep.endswith(".csv") else  # a saved `--page raw --csv` export
            subprocess.run(["ncu", "-i", rep, "--page", "raw", "--csv"], capture_output=True, text=True).stdout)
     rows = list(csv.reader(io.StringIO(raw)))
     hdr, data = rows[0], rows[2:]
     c = hdr.index
-    out = [f"# {tag} — ncu --set full of K1 (k1_probe_agg), SSB SF{sf}, 1 B200", "",
+    layout = " on open-addressing hash tables (HX_JOIN_HASH: the bench's ht_path)" if launches is None else ""
+    out = [f"# {tag} — ncu --set full of K1 (k1_probe_agg){layout}, SSB SF{sf}, 1 B200", "",
            "Captured with `ncu --set full --clock-control none --import-source on -k regex:k1_probe_agg "
            f"-s 13 -c 13 python tools/prof_query.py --sf {sf} --queries all --reps 2` (the second, "
            "planned execution of each query). ncu times are cold-cache and serialised: compare shares.", "",
@@ -75,6 +77,9 @@ def main(tag, rep, launches, sf="10", probe_csv=None):
                    f" | {sol[top][0]} | {inst / N:.2f} | {gld / N:.3f} | {shw / N:.3f} |")
     with open(os.path.join(ROOT, "profiles", f"{tag}_k1_ncu_summary.md"), "w") as f:
         f.write("\n".join(out) + "\n")
+    if launches is None:  # (a capture of another layout: no traffic file, no launch list)
+        print("\n".join(out[-20:]))
+        return
     with open(os.path.join(ROOT, "profiles", "k1_traffic.json"), "w") as f:
         json.dump({"dram_bytes_per_launch": tr / 13, "algorithmic_bytes_per_launch": ta / 13,
                    "launches": 13, "source": f"profiles/{tag}_k1_ncu_summary.md (ncu --set full, "
