@@ -2220,8 +2220,10 @@ int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht*
   // SF100, profiles/r02_ab_reentry.txt: Q2.1 3.26 -> 2.61 ms, Q3.2 2.92 -> 1.95 with 20;
   // Q3.1 in place 2.97 vs 3.03, Q4.1 5.56 vs 5.71 with 26)
   if (!dm_mode && sh->n_joins >= 2 && sh->n_joins <= 3) {
+    // (a 26-warp plan that probes in place beats a 20-warp one with one more Bloom filter:
+    // Q2.1 2.62 -> 2.42 ms)
     const bool stage_b = k_hi.p.n_preds == 0 && k_hi.p.joins[0].bloom_words == 0;
-    if (!stage_b) hi = false;
+    hi = stage_b && k_hi.p.stages >= std::min(k_lo.p.stages, kBaseStages);
   }
   // (4 joins: the claiming 26-warp instance unless stage B probes in place, which the static
   // 20-warp one does best)
