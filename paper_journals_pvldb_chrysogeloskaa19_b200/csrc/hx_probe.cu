@@ -74,6 +74,9 @@ constexpr int kWarpsHiHt = HX_WARPS_HI_HT;  // the hash-table instances' larger 
 #ifndef HX_HT_CLAIM_NJ
 #define HX_HT_CLAIM_NJ 4  // hash-table instances with at least this many joins claim chunks
 #endif
+#ifndef HX_STAGE_B_ROWS
+#define HX_STAGE_B_ROWS 4  // hash-table stage B: probes in flight per lane (4 or 8)
+#endif
 #ifndef HX_HT_SEQ
 #define HX_HT_SEQ 0       // hash-table joins probed one round trip per join in stage C
 #endif
@@ -740,18 +743,20 @@ __device__ __forceinline__ void process_tile(const K1Params& p, const JoinState 
     const JoinState& j = js[0];
     int32_t key[2 * R];
     load8(j.c, key);
+    // HX_STAGE_B_ROWS rows' probes in flight per lane (4: one tile half at a time)
+    constexpr int RB = HX_STAGE_B_ROWS;
 #pragma unroll
-    for (int h = 0; h < 2; ++h) {
-      ulonglong2 v[R];
-      uint32_t b[R];
+    for (int h = 0; h < 2 * R / RB; ++h) {
+      ulonglong2 v[RB];
+      uint32_t b[RB];
 #pragma unroll
-      for (int k = 0; k < R; ++k) {
-        b[k] = bucket_of(key[h * R + k], j.shift);
-        if ((m >> (h * R + k)) & 1u) v[k] = ld_probe(j.buckets + b[k], pol);
+      for (int k = 0; k < RB; ++k) {
+        b[k] = bucket_of(key[h * RB + k], j.shift);
+        if ((m >> (h * RB + k)) & 1u) v[k] = ld_probe(j.buckets + b[k], pol);
       }
 #pragma unroll
-      for (int k = 0; k < R; ++k) {
-        const int kk = h * R + k;
+      for (int k = 0; k < RB; ++k) {
+        const int kk = h * RB + k;
         if (!((m >> kk) & 1u)) continue;
         bool hit, miss;
         int32_t rank;
