@@ -340,3 +340,16 @@ def test_group_decode_drops_empty_groups_and_maps_codes():
     assert len(s0) == 1 and int(c0[0]) == 0
     with pytest.raises(_hx.HxError):  # n_groups must match the layout
         hx.group_decode(n, maps, sums[:10], cnt[:10])
+
+
+def test_ring_slot_reciprocal_is_exact():
+    """K1 finds the ring slot and phase of a CTA's i-th tile with a multiply-high by
+    floor(2^32 / stages) + 1 (hx_probe.cu, K1Params::stage_magic) instead of a runtime divide:
+    exact for every ring depth K1 plans (2..16) over more tiles than one CTA ever gets
+    (a launch is at most 2^20 tiles; checked to 2^22 and at the top of 32 bits / stages)."""
+    for stages in range(2, 17):
+        magic = (1 << 32) // stages + 1
+        i = np.concatenate([np.arange(1 << 22, dtype=np.uint64),
+                            np.arange((1 << 32) // stages - 4096, (1 << 32) // stages, dtype=np.uint64)])
+        q = (i * np.uint64(magic)) >> np.uint64(32)
+        assert np.array_equal(q, i // np.uint64(stages)), stages
