@@ -640,6 +640,16 @@ def run_sizeup(args, world, rank, local, ctx, stream, torch, dist, hx):
     build.close()
 
 
+def nccl_log_env(env):
+    """NCCL's communicator log on (INFO, INIT subsystem: it shows nranks = N) and written to
+    stderr, so that stdout carries only the one JSON line. The image sets NCCL_DEBUG=VERSION,
+    which prints a bare version line on stdout: anything below INFO is raised to INFO."""
+    if env.get("NCCL_DEBUG", "").upper() not in ("INFO", "TRACE"):
+        env["NCCL_DEBUG"] = "INFO"
+    env.setdefault("NCCL_DEBUG_SUBSYS", "INIT")
+    env.setdefault("NCCL_DEBUG_FILE", "/dev/stderr")
+
+
 def main():
     args = parse()
     how, what = launch_plan(args.gpus, os.environ, sys.argv[1:])
@@ -648,16 +658,14 @@ def main():
         sys.exit(2)
     if how == "relaunch":
         env = dict(os.environ)
-        env.setdefault("NCCL_DEBUG", "INFO")  # the communicator log shows nranks = N
-        env.setdefault("NCCL_DEBUG_SUBSYS", "INIT")
+        nccl_log_env(env)
         sys.exit(subprocess.run(what, env=env).returncode)
     world, rank, local = dist_env()
     if args.sf_total > 0:
         args.sf = args.sf_total / world
     SCALING[0] = "strong" if args.sf_total > 0 else "weak"
-    if world > 1:
-        os.environ.setdefault("NCCL_DEBUG", "INFO")
-        os.environ.setdefault("NCCL_DEBUG_SUBSYS", "INIT")
+    if world > 1 or args.force_collectives:
+        nccl_log_env(os.environ)
     if args.impl == "reference":
         run_reference(args, world, rank)
         return
