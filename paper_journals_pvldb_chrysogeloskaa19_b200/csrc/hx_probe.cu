@@ -1518,6 +1518,8 @@ size_t k1_smem_cap() {
   return cap;
 }
 
+// ring depth the plan starts from (0: kBaseStages); k1_setup also plans one stage deeper
+thread_local int t_base_stages = 0;
 int pick_stages(int warps, bool dm, int n_cols, int smem_groups) {
   // as many tile stages as fit next to kCtasPerSm CTAs per SM, at least double buffering
   // (at most HX_K1_STAGE_KB of tiles per CTA: the rest is left for filters and maps)
@@ -1526,7 +1528,9 @@ int pick_stages(int warps, bool dm, int n_cols, int smem_groups) {
                                          fixed + HX_K1_STAGE_KB * 1024);
   const size_t stage = (size_t)n_cols * kTileRows * 4;
   const int s = budget > fixed ? (int)((budget - fixed) / stage) : 0;
-  return std::max(2, std::min(kBaseStages, s));
+  int base = t_base_stages ? t_base_stages : kBaseStages;
+  if (const char* e = std::getenv("HX_K1_MIN_STAGES")) base = std::max(2, std::min(kMaxStages, std::atoi(e)));
+  return std::max(2, std::min(base, s));
 }
 
 enum { kStNone = 0, kStFull, kStBitmap, kStBloom };
@@ -1775,7 +1779,10 @@ int agg_alloc(hx_ctx* ctx, hx_agg* agg, long long cap_groups, const hx_query_sha
 int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht* const* hts,
              int n_hts, const hx_agg* agg, K1Prepared** out) {
   struct CapReset {
-    ~CapReset() { t_smem_cap = 0; }
+    ~CapReset() {
+      t_smem_cap = 0;
+      t_base_stages = 0;
+    }
   } cap_reset;
   t_smem_cap = 0;
   HX_REQUIRE(ctx && fact && sh && agg && out, HX_EINVAL, "hx_pipeline_probe_agg: null argument");
@@ -2205,9 +2212,24 @@ int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht*
     k.warps = W;
     k.cost = plan_cost;
   };
+  // Direct maps: the plan is also made around a ring one stage deeper, and taken when the cost
+  // model charges that at most kDeepTol more (a deeper ring keeps more bytes in flight while
+  // the consumers hold their chunks; the model does not see it). Measured at SF100
+  // (profiles/r02_ab_reentry.txt): Q2.2 1.45 -> 1.29 ms (+5% cost), Q3.2 1.48 -> 1.36 (+8%),
+  // Q3.3 1.28 -> 1.15 (+0.3%), Q3.1 2.07 -> 2.03; Q2.1 (+29% cost) 1.69 -> 1.74 keeps 4.
+  auto plan_deeper = [&](const int W, K1Prepared& kk) {
+    plan_with(W, kk);
+    if (!dm_mode || std::getenv("HX_K1_MIN_STAGES")) return;
+    constexpr double kDeepTol = 1.10;
+    K1Prepared deep = k;
+    t_base_stages = kBaseStages + 1;
+    plan_with(W, deep);
+    t_base_stages = 0;
+    if (deep.p.stages > kk.p.stages && deep.cost <= kk.cost * kDeepTol + 1e-9) kk = deep;
+  };
   K1Prepared k_lo = k, k_hi = k;
-  plan_with(kWarpsLo, k_lo);
-  plan_with(dm_mode ? kWarpsHi : kWarpsHiHt, k_hi);
+  plan_deeper(kWarpsLo, k_lo);
+  plan_deeper(dm_mode ? kWarpsHi : kWarpsHiHt, k_hi);
   // more warps unless the plan they leave room for is costlier by more than kWarpsTol (the
   // cost model's per-row issue cost; tolerance measured) or the ring is shallower
   double tol = 1.10;
