@@ -77,6 +77,10 @@ constexpr int kWarpsHiHt = HX_WARPS_HI_HT;  // the hash-table instances' larger 
 #ifndef HX_STAGE_B_ROWS
 #define HX_STAGE_B_ROWS 4  // hash-table stage B: probes in flight per lane (4 or 8)
 #endif
+#ifndef HX_HT_GIVEUP_MINCOLS
+#define HX_HT_GIVEUP_MINCOLS 4  // hash tables: narrower pipelines never give up a ring stage
+                                // for filters (SF100 HT K1 sum -0.45%: Q3.2 -9%, Q2.2 +3%)
+#endif
 #ifndef HX_HT_SEQ
 #define HX_HT_SEQ 0       // hash-table joins probed one round trip per join in stage C
 #endif
@@ -2009,6 +2013,9 @@ int k1_setup(hx_ctx* ctx, const hx_table* fact, const hx_query_shape* sh, hx_ht*
       const int good0 = allocate();
       const int ht3 = (3 * kBaseStages + 3) / 4;  // 3/4 of the base ring
       int ht_stages = stages0 > ht3 ? ht3 : stages0;
+#if HX_HT_GIVEUP_MINCOLS
+      if (n_cols < HX_HT_GIVEUP_MINCOLS) ht_stages = stages0;
+#endif
       if (const char* e = std::getenv("HX_HT_STAGES")) ht_stages = std::max(2, std::min(stages0, std::atoi(e)));
       if (ht_stages < stages0) {
         p.stages = ht_stages;
